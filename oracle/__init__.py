@@ -1,0 +1,160 @@
+"""CPU oracle -- TEST INFRASTRUCTURE ONLY.
+
+Only ``tests/``, ``__graft_entry__.smoke()`` and ``bench.py`` (its
+``cpu_baseline`` leg and ``--impl reference``) may import this package.  The
+product package ``paper_conf_asplos_ginsbachrsbdo18_b200`` never imports it
+and shares no code with it; the only shared module is the seeded input
+generator ``gen`` (which holds none of the method's arithmetic).
+
+The arithmetic lives in ``oracle_spmv.c`` (plain sequential fp64 C, each
+function citing the PAPER.md passage it follows); this file only compiles it
+with gcc (``-O3 -march=native -ffp-contract=off``) and marshals numpy arrays
+through ctypes.
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+import subprocess
+
+import numpy as np
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+_SRC = os.path.join(_HERE, "oracle_spmv.c")
+_LIB = os.path.join(_HERE, "liboracle_spmv.so")
+_lib = None
+
+_P = ctypes.c_void_p
+_I64 = ctypes.c_int64
+_I32 = ctypes.c_int32
+_D = ctypes.c_double
+
+
+def build(force: bool = False) -> str:
+    """Compile the oracle (gcc, no FMA contraction).  Returns the .so path."""
+    if force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < os.path.getmtime(_SRC):
+        tmp = _LIB + f".tmp{os.getpid()}"
+        subprocess.check_call(
+            ["gcc", "-O3", "-march=native", "-ffp-contract=off", "-std=c11", "-fPIC",
+             "-shared", "-o", tmp, _SRC, "-lm"])
+        os.replace(tmp, _LIB)
+    return _LIB
+
+
+def lib():
+    global _lib
+    if _lib is None:
+        build()
+        L = ctypes.CDLL(_LIB)
+        L.oracle_spmv_f64.argtypes = [_I64, _P, _P, _P, _P, _P, _D, _D, _P, _P]
+        L.oracle_spmv_f64.restype = None
+        L.oracle_spmv_f32.argtypes = [_I64, _P, _P, _P, _P, _P, _D, _D, _P, _P]
+        L.oracle_spmv_f32.restype = None
+        L.oracle_cg.argtypes = [_I64, _P, _P, _P, _P, _P, _I32, _D, _P, _P]
+        L.oracle_cg.restype = ctypes.c_int
+        L.oracle_npb_outer.argtypes = [_I64, _P, _P, _P, _P, _P, _I32, _D, _P, _P]
+        L.oracle_npb_outer.restype = ctypes.c_int
+        L.oracle_partition.argtypes = [_P, _I64, _I32, _P]
+        L.oracle_partition.restype = None
+        L.oracle_merge_path.argtypes = [_P, _I64, _I64, _P, _P]
+        L.oracle_merge_path.restype = None
+        _lib = L
+    return _lib
+
+
+def _ptr(a):
+    return a.ctypes.data_as(ctypes.c_void_p) if a is not None else None
+
+
+def _c(a, dt):
+    return np.ascontiguousarray(a, dtype=dt)
+
+
+def spmv(rowptr, colidx, vals, x, y_old=None, alpha=1.0, beta=0.0):
+    """y_ref, bound = alpha*A@x + beta*y_old with fp64 accumulation.
+
+    vals/x/y_old may be float64 or float32 (then products are formed in double
+    from the fp32 inputs, alpha/beta rounded to float first).
+    """
+    rowptr = _c(rowptr, np.int32)
+    colidx = _c(colidx, np.int32)
+    m = rowptr.shape[0] - 1
+    f32 = np.asarray(vals).dtype == np.float32
+    dt = np.float32 if f32 else np.float64
+    vals = _c(vals, dt)
+    x = _c(x, dt)
+    yo = _c(y_old, dt) if y_old is not None else np.zeros(max(m, 1), dtype=dt)
+    y_ref = np.empty(max(m, 1), dtype=np.float64)
+    bound = np.empty(max(m, 1), dtype=np.float64)
+    fn = lib().oracle_spmv_f32 if f32 else lib().oracle_spmv_f64
+    fn(m, _ptr(rowptr), _ptr(colidx), _ptr(vals), _ptr(x), _ptr(yo), float(alpha),
+       float(beta), _ptr(y_ref), _ptr(bound))
+    return y_ref[:m], bound[:m]
+
+
+def cg(rowptr, colidx, vals, b, max_iter, tol=0.0):
+    """Textbook CG from x0=0 (NPB conj_grad).  Returns (z, iters, rnorm, status)."""
+    rowptr = _c(rowptr, np.int32)
+    colidx = _c(colidx, np.int32)
+    vals = _c(vals, np.float64)
+    b = _c(b, np.float64)
+    n = rowptr.shape[0] - 1
+    z = np.zeros(max(n, 1))
+    its = ctypes.c_int32(0)
+    rn = ctypes.c_double(0.0)
+    st = lib().oracle_cg(n, _ptr(rowptr), _ptr(colidx), _ptr(vals), _ptr(b), _ptr(z),
+                         int(max_iter), float(tol), ctypes.byref(its), ctypes.byref(rn))
+    return z[:n], its.value, rn.value, st
+
+
+def npb_outer(rowptr, colidx, vals, x, cgitmax, shift):
+    """One NAS CG outer iteration; x (float64, contiguous) updated in place.
+
+    Returns (z, zeta, rnorm).
+    """
+    assert x.dtype == np.float64 and x.flags.c_contiguous
+    rowptr = _c(rowptr, np.int32)
+    colidx = _c(colidx, np.int32)
+    vals = _c(vals, np.float64)
+    n = rowptr.shape[0] - 1
+    z = np.zeros(n)
+    zeta = ctypes.c_double(0.0)
+    rn = ctypes.c_double(0.0)
+    lib().oracle_npb_outer(n, _ptr(rowptr), _ptr(colidx), _ptr(vals), _ptr(x), _ptr(z),
+                           int(cgitmax), float(shift), ctypes.byref(zeta), ctypes.byref(rn))
+    return z, zeta.value, rn.value
+
+
+def npb_run(rowptr, colidx, vals, niter, shift, cgitmax=25, on_iter=None):
+    """NPB CG benchmark driver: x=1; NITER outer iterations; returns zetas, rnorms.
+
+    (The untimed warm-up iteration of NPB resets x=1 afterwards and so does not
+    change any zeta; it is not repeated here.)
+    """
+    n = len(rowptr) - 1
+    x = np.ones(n)
+    zetas, rnorms = [], []
+    for it in range(niter):
+        _, zeta, rn = npb_outer(rowptr, colidx, vals, x, cgitmax, shift)
+        zetas.append(zeta)
+        rnorms.append(rn)
+        if on_iter:
+            on_iter(it, zeta, rn)
+    return np.array(zetas), np.array(rnorms)
+
+
+def partition(rowptr, nranks):
+    rowptr = _c(rowptr, np.int32)
+    m = rowptr.shape[0] - 1
+    bounds = np.zeros(nranks + 1, dtype=np.int64)
+    lib().oracle_partition(_ptr(rowptr), m, int(nranks), _ptr(bounds))
+    return bounds
+
+
+def merge_path(rowptr, pieces):
+    rowptr = _c(rowptr, np.int32)
+    m = rowptr.shape[0] - 1
+    sr = np.zeros(pieces + 1, dtype=np.int64)
+    sn = np.zeros(pieces + 1, dtype=np.int64)
+    lib().oracle_merge_path(_ptr(rowptr), m, int(pieces), _ptr(sr), _ptr(sn))
+    return sr, sn

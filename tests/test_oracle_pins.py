@@ -1,0 +1,246 @@
+"""Pins for the CPU oracle (oracle/oracle_spmv.c) against facts that do not come
+from the oracle itself: closed forms, exact integer brute force, published NPB
+verification values, and characterising properties of the partition and
+merge-path splits.  All CPU (-m "not gpu").
+
+Each pin is chosen so a plausible oracle bug fails it: a dropped term (dense
+brute force, Laplacian closed forms), a wrong sign/index (permutation, j and j^2
+Laplacian forms), transposed operands (non-square and non-symmetric brute
+force), beta/alpha mix-ups (alpha/beta tests), a wrong CG update (Laplacian CG
+closed form, NPB zeta).
+"""
+import os
+
+import numpy as np
+import pytest
+
+import gen
+import oracle
+
+GOLD = os.path.join(os.path.dirname(__file__), "golden")
+
+
+def _read_golden(name):
+    rows = []
+    with open(os.path.join(GOLD, name)) as f:
+        for line in f:
+            if line.startswith("#") or not line.strip():
+                continue
+            rows.append(line.split())
+    return rows
+
+
+# ---------------------------------------------------------------- SpMV pins
+def test_identity_exact():
+    n = 257
+    A = gen.from_dense(np.eye(n))
+    x = gen.uniform(n, seed=1)
+    y, b = oracle.spmv(A.rowptr, A.colidx, A.vals, x)
+    assert np.array_equal(y, x)
+    assert np.array_equal(b, np.abs(x))
+
+
+def test_permutation_exact():
+    n = 300
+    rng = np.random.default_rng(3)
+    pi = rng.permutation(n)
+    A = gen.from_coo(n, n, np.arange(n), pi, np.ones(n))
+    x = gen.uniform(n, seed=2)
+    y, _ = oracle.spmv(A.rowptr, A.colidx, A.vals, x)
+    assert np.array_equal(y, x[pi])
+
+
+def test_diagonal_exact():
+    n = 123
+    d = gen.uniform(n, seed=5)
+    x = gen.uniform(n, seed=6)
+    A = gen.from_coo(n, n, np.arange(n), np.arange(n), d)
+    y, _ = oracle.spmv(A.rowptr, A.colidx, A.vals, x)
+    assert np.array_equal(y, d * x)  # one correctly rounded product per row
+
+
+@pytest.mark.parametrize("density", [0.0, 0.05, 0.3, 1.0])
+@pytest.mark.parametrize("shape", [(1, 1), (7, 13), (64, 64), (40, 3)])
+def test_dense_bruteforce_exact(density, shape):
+    """Small-integer A, x: every partial sum is an exact integer in fp64."""
+    m, n = shape
+    rng = np.random.default_rng(int(density * 100) + m * 7 + n)
+    A = rng.integers(-9, 10, size=(m, n)) * (rng.random((m, n)) < density)
+    x = rng.integers(-9, 10, size=n)
+    ref = A.astype(np.int64) @ x.astype(np.int64)
+    C = gen.from_dense(A.astype(np.float64))
+    y, b = oracle.spmv(C.rowptr, C.colidx, C.vals, x.astype(np.float64))
+    assert np.array_equal(y, ref.astype(np.float64))
+    assert np.array_equal(b, (np.abs(A) @ np.abs(x)).astype(np.float64))
+    # fp32 variant: same exact integers
+    y32, _ = oracle.spmv(C.rowptr, C.colidx, C.vals.astype(np.float32), x.astype(np.float32))
+    assert np.array_equal(y32, ref.astype(np.float64))
+
+
+def test_duplicates_unsorted_offset_rowptr_empty_rows():
+    """Reading R10 (duplicates/unsorted summed), R2 (rowptr[0] != 0), R7 (empty rows written)."""
+    m, n = 6, 5
+    rows = [0, 0, 0, 2, 2, 2, 2, 5]
+    cols = [4, 1, 4, 0, 3, 0, 3, 2]
+    vals = [1, 2, 3, 4, 5, 6, 7, 8]
+    C = gen.from_coo(m, n, rows, cols, vals)
+    dense = np.zeros((m, n), np.int64)
+    for r, c, v in zip(rows, cols, vals):
+        dense[r, c] += v
+    x = np.array([1.0, -2.0, 3.0, 5.0, 7.0])
+    ref = dense @ x.astype(np.int64)
+    # shift the arrays: rowptr[0] = 11, arrays carry 11 junk leading entries
+    off = 11
+    colidx = np.concatenate([np.full(off, 10**6, np.int32), C.colidx])
+    v = np.concatenate([np.full(off, np.nan), C.vals])
+    y, _ = oracle.spmv(C.rowptr + off, colidx, v, x)
+    assert np.array_equal(y, ref.astype(np.float64))
+    assert y[1] == 0.0 and y[3] == 0.0 and y[4] == 0.0
+
+
+def test_alpha_beta_conventions():
+    rng = np.random.default_rng(11)
+    m, n = 17, 9
+    A = rng.integers(-5, 6, size=(m, n)) * (rng.random((m, n)) < 0.5)
+    x = rng.integers(-5, 6, size=n).astype(np.float64)
+    yo = rng.integers(-5, 6, size=m).astype(np.float64)
+    C = gen.from_dense(A.astype(np.float64))
+    y, _ = oracle.spmv(C.rowptr, C.colidx, C.vals, x, yo, alpha=2.0, beta=-3.0)
+    assert np.array_equal(y, 2.0 * (A @ x) - 3.0 * yo)
+    # beta == 0: y_old is not read (NaN must not propagate)
+    y, _ = oracle.spmv(C.rowptr, C.colidx, C.vals, x, np.full(m, np.nan), alpha=1.0, beta=0.0)
+    assert np.array_equal(y, A @ x)
+    # alpha == 0: A and x are not read
+    xn = np.full(n, np.nan)
+    y, _ = oracle.spmv(C.rowptr, C.colidx, C.vals, xn, yo, alpha=0.0, beta=2.0)
+    assert np.array_equal(y, 2.0 * yo)
+
+
+@pytest.mark.parametrize("n", [2, 3, 10, 1000, 65537])
+def test_laplace1d_closed_forms(n):
+    A = gen.laplace1d(n)
+    j = np.arange(n, dtype=np.float64)
+    y, _ = oracle.spmv(A.rowptr, A.colidx, A.vals, np.ones(n))
+    e = np.zeros(n); e[0] += 1; e[-1] += 1
+    assert np.array_equal(y, e)
+    y, _ = oracle.spmv(A.rowptr, A.colidx, A.vals, j)
+    ref = np.zeros(n); ref[0] = -1; ref[-1] = n
+    assert np.array_equal(y, ref)
+    y, _ = oracle.spmv(A.rowptr, A.colidx, A.vals, j * j)
+    ref = np.full(n, -2.0); ref[0] = -1; ref[-1] = float(n) * n - 2
+    assert np.array_equal(y, ref)
+
+
+def test_nonsymmetric_orientation():
+    """Transposed operand check: a strictly upper-triangular shift matrix."""
+    n = 50
+    A = gen.from_coo(n, n, np.arange(n - 1), np.arange(1, n), np.ones(n - 1))
+    x = np.arange(n, dtype=np.float64)
+    y, _ = oracle.spmv(A.rowptr, A.colidx, A.vals, x)
+    assert np.array_equal(y[:-1], x[1:]) and y[-1] == 0.0
+
+
+# ------------------------------------------------------------------ CG pins
+@pytest.mark.parametrize("n", [1, 2, 5, 16, 64])
+def test_cg_laplace1d_closed_form(n):
+    """A=tridiag(-1,2,-1), b=1: z_j=(j+1)(n-j)/2; CG terminates in <= n steps."""
+    A = gen.laplace1d(n)
+    z, its, rn, st = oracle.cg(A.rowptr, A.colidx, A.vals, np.ones(n), max_iter=n, tol=1e-14)
+    j = np.arange(n)
+    ref = (j + 1) * (n - j) / 2.0
+    assert st == 0
+    assert np.allclose(z, ref, rtol=1e-10, atol=0)
+    assert rn <= 1e-10 * np.sqrt(n) * ref.max()
+
+
+def test_cg_diagonal_one_step():
+    """Diagonal c*I: CG reaches b/c after one iteration exactly (up to one rounding)."""
+    n = 40
+    A = gen.from_coo(n, n, np.arange(n), np.arange(n), np.full(n, 4.0))
+    b = gen.uniform(n, seed=9)
+    z, its, rn, st = oracle.cg(A.rowptr, A.colidx, A.vals, b, max_iter=1)
+    assert st == 0 and its == 1
+    assert np.allclose(z, b / 4.0, rtol=1e-15, atol=0)
+
+
+def test_cg_breakdown_zero_rhs():
+    A = gen.laplace1d(8)
+    z, its, rn, st = oracle.cg(A.rowptr, A.colidx, A.vals, np.zeros(8), max_iter=5)
+    assert st == 7 and its == 0
+
+
+def test_randlc_against_bigint():
+    """NPB randlc: x <- 5^13 x mod 2^46 (exact integer recurrence)."""
+    vals = gen.randlc_stream(2000)
+    x, a = 314159265, 1220703125
+    for i in range(2000):
+        x = (a * x) % (1 << 46)
+        assert vals[i] == x / float(1 << 46)
+
+
+@pytest.mark.parametrize("cls", ["S", "W", "A"])
+def test_makea_nnz_golden(cls):
+    g = {r[0]: r[1:] for r in _read_golden("npb_nnz.txt")}[cls]
+    A = gen.makea(cls)
+    L = A.row_lengths()
+    assert A.nnz == int(g[0]) and L.min() == int(g[1]) and L.max() == int(g[2])
+    # pattern symmetric, columns ascending, diagonal present (reading R16)
+    assert np.all(np.diff(A.colidx.astype(np.int64))[np.diff(np.repeat(np.arange(A.m), L)) == 0] > 0)
+
+
+@pytest.mark.parametrize("cls", ["S", "W", "A"])
+def test_npb_zeta_published(cls):
+    """The oracle's NAS CG run reproduces the published zeta within 1e-10 and
+    keeps rnorm <= 1e-11 at every outer iteration."""
+    g = {r[0]: r[1:] for r in _read_golden("npb_zeta.txt")}[cls]
+    na, nonzer, niter, shift, zeta_ref = int(g[0]), int(g[1]), int(g[2]), float(g[3]), float(g[4])
+    A = gen.makea(cls)
+    assert A.m == na
+    zetas, rnorms = oracle.npb_run(A.rowptr, A.colidx, A.vals, niter, shift)
+    assert abs(zetas[-1] - zeta_ref) / zeta_ref <= 1e-10
+    assert rnorms.max() <= 1e-11
+
+
+# ------------------------------------------------------- partition / merge
+def _rowptr_cases():
+    rng = np.random.default_rng(5)
+    cases = [np.array([0], np.int32), np.array([0, 0, 0], np.int32), np.array([0, 5], np.int32),
+             np.array([3, 3, 10, 10, 11], np.int32)]
+    for m in [1, 2, 7, 33]:
+        L = rng.integers(0, 9, size=m)
+        L[rng.random(m) < 0.2] = 0
+        cases.append((np.concatenate([[0], np.cumsum(L)]) + rng.integers(0, 4)).astype(np.int32))
+    skew = np.zeros(20, np.int64); skew[3] = 100
+    cases.append(np.concatenate([[0], np.cumsum(skew)]).astype(np.int32))
+    return cases
+
+
+@pytest.mark.parametrize("P", [1, 2, 3, 4, 8])
+def test_partition_characterisation(P):
+    """b_r is the unique i with prefix(i) >= t_r and (i == 0 or prefix(i-1) < t_r)."""
+    for rp in _rowptr_cases():
+        m = len(rp) - 1
+        b = oracle.partition(rp, P)
+        pre = rp.astype(np.int64) - rp[0]
+        nnz = int(pre[-1])
+        assert b[0] == 0 and b[P] == m and np.all(np.diff(b) >= 0)
+        for r in range(1, P):
+            t = (r * nnz) // P
+            cands = [i for i in range(m + 1) if pre[i] >= t and (i == 0 or pre[i - 1] < t)]
+            assert cands == [b[r]]
+
+
+@pytest.mark.parametrize("C", [1, 2, 5, 16])
+def test_merge_path_characterisation(C):
+    for rp in _rowptr_cases():
+        m = len(rp) - 1
+        A = rp[1:].astype(np.int64) - rp[0]
+        nnz = int(rp[-1]) - int(rp[0])
+        sr, sn = oracle.merge_path(rp, C)
+        for c in range(C + 1):
+            d = (c * (m + nnz)) // C
+            cands = [(i, d - i) for i in range(0, min(d, m) + 1)
+                     if 0 <= d - i <= nnz
+                     and (i == 0 or A[i - 1] <= d - i)
+                     and (i == m or d - i == 0 or A[i] > d - i - 1)]
+            assert cands == [(sr[c], sn[c])], (rp, c, cands, sr[c], sn[c])
