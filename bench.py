@@ -1,0 +1,383 @@
+#!/usr/bin/env python3
+"""Benchmark: NAS CG class C (fp64) on the B200 SpMV/CG library.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
+
+Workload (BASELINE.json metric "CSR SpMV GB/s & % HBM peak (NAS CG class C
+fp64); CG iters/s at 1/2/4/8 GPU", config BJ.cfg[3]): the NAS CG class-C
+matrix (exact NPB makea, n = 150,000, 36,121,058 nnz), fp64.  One STEP is one
+NAS CG outer iteration = every row of SURVEY 8(a): 25 CG iterations (SpMV +
+2 dots + 3 axpys each, a2/a3), the residual SpMV and the zeta/normalisation
+tail (a4), row-sharded over N GPUs with the NCCL exchange (a5); the handle is
+created once (a1, device-resident A, the paper's lazy copying P:1175-1184).
+
+value  = CG iterations per second of the whole job (25 per step; the residual
+         SpMV is timed but not counted, reading R23), device-timed with CUDA
+         events per step, L2 flushed between steps, max over ranks.
+e2e    = the same metric through the public API with HOST buffers: x copied in
+         from pinned memory and x, z, {zeta, rnorm} copied back every step.
+roofline = the SpMV kernel (the dominant kernel, ~97% of the step's bytes),
+         timed alone with CUDA events on the launching stream (L2 flushed
+         before each launch): algorithmic bytes / duration vs the measured
+         HBM copy bandwidth of MEASURED_PEAKS.json.
+cpu_baseline = the CPU oracle (oracle/, plain C, 1 thread) on a bounded sample.
+`--impl reference` times the oracle itself as the reference arm.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "CSR SpMV GB/s & % HBM peak (NAS CG class C fp64); CG iters/s at 1/2/4/8 GPU"
+UNIT = "CG iters/s"
+CLS = "C"
+NOMINAL_HBM_GBS = 8000.0
+FLUSH_BYTES = 256 << 20  # > 126 MB L2
+
+
+def log(*a):
+    print(*a, file=sys.stderr, flush=True)
+
+
+def measured_peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    try:
+        with open(p) as f:
+            d = json.load(f)
+        return float(d["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs, copy read+write)"
+    except Exception:
+        return 6650.0, "fallback (B200_PROFILING.md 6.65 TB/s)"
+
+
+def workload_config(A, n_gpus):
+    na, nonzer, niter, shift = __import__("gen").NPB_CLASSES[CLS]
+    return {
+        "workload": f"NAS CG class {CLS} (makea NA={na}, NONZER={nonzer}, SHIFT={shift}), fp64 CG, "
+                    f"1 step = 1 NPB outer iteration (25 CG its + residual SpMV)",
+        "n": int(A.n), "nnz": int(A.nnz), "cgitmax": 25,
+        "bytes_per_spmv": int(A.bytes_per_spmv()),
+        "l2": "flushed between timed steps (256 MiB write); A = 436 MB > 126 MB L2",
+        "parallelism": f"row-shard x{n_gpus} (nnz-balanced), NCCL allgather x + allreduce dots",
+    }
+
+
+# ------------------------------------------------------------------ clocks
+class ClockSampler:
+    FIELDS = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,"
+              "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+              "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, gpu_index: int):
+        self.gpu = gpu_index
+        self.proc = None
+        self.lines = []
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.gpu), f"--query-gpu={self.FIELDS}", "--format=csv,noheader,nounits",
+                 "-lms", "200"], stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+        except Exception:
+            self.proc = None
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.lines.append(line.strip())
+
+    def stop(self):
+        if not self.proc:
+            return None
+        self.proc.terminate()
+        try:
+            self.proc.wait(timeout=5)
+        except Exception:
+            self.proc.kill()
+        self.t.join(timeout=2)
+        sm, mx, reasons = [], 0.0, set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for ln in self.lines:
+            f = [x.strip() for x in ln.split(",")]
+            if len(f) < 9:
+                continue
+            try:
+                sm.append(float(f[1]))
+                mx = max(mx, float(f[2]))
+            except ValueError:
+                continue
+            for nm, v in zip(names, f[5:9]):
+                if v.lower().startswith("active"):
+                    reasons.add(nm)
+        if not sm:
+            return None
+        return {"sm_mhz": statistics.median(sm), "sm_max_mhz": mx, "reasons": sorted(reasons),
+                "samples": len(sm)}
+
+
+# --------------------------------------------------------------- our arm
+def run_ours(args):
+    import numpy as np
+    import torch
+    import torch.distributed as dist
+
+    import gen
+    import paper_conf_asplos_ginsbachrsbdo18_b200 as sp
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    if world != args.gpus:
+        log(f"note: --gpus {args.gpus} but WORLD_SIZE={world}; using WORLD_SIZE")
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    d = None
+    if world > 1:
+        dist.init_process_group("nccl", device_id=dev)
+        d = sp.Dist(rank, world, local)
+
+    na, nonzer, niter, shift = gen.NPB_CLASSES[CLS]
+    t0 = time.time()
+    A = gen.makea(CLS)
+    log(f"[rank {rank}] generated class {CLS}: n={A.n} nnz={A.nnz} in {time.time() - t0:.1f}s")
+    rp = torch.from_numpy(A.rowptr).to(dev)
+    ci = torch.from_numpy(A.colidx).to(dev)
+    va = torch.from_numpy(A.vals).to(dev)
+    M = sp.CSRMatrix(rp, ci, va, A.n, dist=d)
+    info = M.info()
+    b0, b1 = info["row_begin"], info["row_end"]
+    nl = b1 - b0
+    flush = torch.empty(FLUSH_BYTES // 4, dtype=torch.int32, device=dev)
+    stream = torch.cuda.current_stream(dev)
+
+    def barrier():
+        torch.cuda.synchronize(dev)
+        if world > 1:
+            dist.barrier(device_ids=[local])
+        torch.cuda.synchronize(dev)
+
+    def max_over_ranks(v: float) -> float:
+        if world == 1:
+            return v
+        t = torch.tensor([v], dtype=torch.float64, device=dev)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        return float(t.item())
+
+    # ---------------- device-resident NAS CG steps (value)
+    x = torch.ones(nl, dtype=torch.float64, device=dev)
+    z = torch.empty(nl, dtype=torch.float64, device=dev)
+    out2 = torch.zeros(2, dtype=torch.float64, device=dev)
+    for _ in range(args.warmup):
+        M.npb_outer(x, z, 25, shift, out2)
+    barrier()
+    x.fill_(1.0)
+    clocks = ClockSampler(local)
+    clocks.start()
+    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
+    launches0 = sp.launch_count()
+    zetas = []
+    for k in range(args.steps):
+        flush.zero_()  # L2 flush, outside the timed events
+        barrier()
+        ev[k][0].record(stream)
+        M.npb_outer(x, z, 25, shift, out2)
+        ev[k][1].record(stream)
+    barrier()
+    launches = sp.launch_count() - launches0
+    M.cg_status()
+    step_ms = [a.elapsed_time(b) for a, b in ev]
+    t_ms = max_over_ranks(sum(step_ms))
+    clk = clocks.stop()
+    zeta_last = float(out2[0].item())
+    value = 25.0 * args.steps / (t_ms / 1e3)
+
+    # ---------------- e2e through the public API with host buffers
+    xh = torch.ones(nl, dtype=torch.float64).pin_memory()
+    zh = torch.empty(nl, dtype=torch.float64).pin_memory()
+    o2h = torch.zeros(2, dtype=torch.float64).pin_memory()
+    M.npb_outer(xh, zh, 25, shift, o2h)  # warm the staged path
+    xh.fill_(1.0)
+    barrier()
+    e2e_ms = 0.0
+    for k in range(args.steps):
+        flush.zero_()
+        barrier()
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record(stream)
+        M.npb_outer(xh, zh, 25, shift, o2h)  # H2D x, graph, D2H x, z, out2 (synchronous)
+        b.record(stream)
+        b.synchronize()
+        e2e_ms += a.elapsed_time(b)
+    e2e_ms = max_over_ranks(e2e_ms)
+    e2e_val = 25.0 * args.steps / (e2e_ms / 1e3)
+
+    # ---------------- roofline: the SpMV kernel timed alone
+    p = torch.from_numpy(gen.uniform(A.n, seed=5)[b0:b1].copy()).to(dev)
+    q = torch.empty(nl, dtype=torch.float64, device=dev)
+    reps = max(10, args.steps)
+    for _ in range(3):
+        M.spmv(p, q)
+    sp_ms = []
+    for _ in range(reps):
+        flush.zero_()
+        barrier()
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record(stream)
+        M.spmv(p, q)
+        b.record(stream)
+        b.synchronize()
+        sp_ms.append(a.elapsed_time(b))
+    # algorithmic bytes of this rank's launch: local nnz*(8+4) + 4*(m_loc+1) + 8*n (x) + 8*m_loc (y)
+    nnz_loc = info["nnz_local"]
+    spmv_bytes = nnz_loc * 12 + 4 * (nl + 1) + 8 * A.n + 8 * nl
+    sp_avg = statistics.mean(sp_ms)
+    sp_med = statistics.median(sp_ms)
+    achieved = spmv_bytes / (sp_avg / 1e3) / 1e9
+    peak, peak_src = measured_peaks()
+    traffic = None
+    tf = os.path.join(ROOT, "profiles", "spmv_traffic.json")
+    if os.path.exists(tf) and world == 1:
+        try:
+            tj = json.load(open(tf))
+            key = f"class{CLS}:{info['kernel_name']}:lanes{info['vec_lanes']}"
+            traffic = tj.get(key)
+        except Exception:
+            traffic = None
+
+    # ---------------- CPU oracle baseline (rank 0, N=1 only)
+    cpu = None
+    if world == 1 and not args.no_cpu:
+        cpu = cpu_baseline(A, shift, budget_s=args.cpu_budget)
+
+    if rank == 0:
+        line = {
+            "metric": METRIC, "value": round(value, 2), "unit": UNIT, "n_gpus": world,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": round(t_ms / args.steps, 4),
+            "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "f64",
+            "data": "synthetic (exact NPB makea class C generator, seeded)",
+            "config": workload_config(A, world),
+            "impl": "ours",
+            "kernel": {"name": info["kernel_name"], "vec_lanes": info["vec_lanes"], "grid": info["grid"]},
+            "spmv": {
+                "gbs": round(achieved, 1), "gflops": round(2 * nnz_loc / (sp_avg / 1e3) / 1e9, 1),
+                "us_avg": round(sp_avg * 1e3, 2), "us_median": round(sp_med * 1e3, 2),
+                "pct_of_8TBs": round(100 * achieved / NOMINAL_HBM_GBS, 2),
+                "pct_of_measured_copy": round(100 * achieved / peak, 2),
+                "bytes_per_launch": int(spmv_bytes),
+            },
+            "cg_gbs_effective": round(value * (spmv_bytes + 10 * 8 * nl) / 1e9 * world, 1),
+            "roofline": {"bound": "hbm", "achieved": round(achieved, 1), "peak": peak, "unit": "GB/s",
+                         "frac": round(achieved / peak, 4), "traffic": traffic,
+                         "peak_source": peak_src, "kernel": f"k_spmv_vector<double,{info['vec_lanes']}>"},
+            "e2e": {"value": round(e2e_val, 2), "unit": UNIT, "h2d_bytes_per_step": 8 * nl,
+                    "d2h_bytes_per_step": 2 * 8 * nl + 16},
+            "gpu_launches": int(launches),
+            "clocks": clk,
+            "zeta_last": zeta_last,
+            "cpu_baseline": cpu,
+        }
+        print(json.dumps(line), flush=True)
+    M.destroy()
+    if d is not None:
+        d.close()
+    if world > 1:
+        dist.destroy_process_group()
+
+
+def cpu_baseline(A, shift, budget_s=15.0):
+    """The oracle as it stands (plain C, 1 thread) on a bounded sample: whole NAS
+    outer iterations of the same class-C workload until ~budget_s of CPU work."""
+    import numpy as np
+
+    import oracle
+    x = np.ones(A.n)
+    t0 = time.perf_counter()
+    steps = 0
+    while True:
+        oracle.npb_outer(A.rowptr, A.colidx, A.vals, x, 25, shift)
+        steps += 1
+        el = time.perf_counter() - t0
+        if el >= budget_s or steps >= 50:
+            break
+    return {"value": round(25.0 * steps / el, 3), "unit": UNIT, "cores": 1, "kind": "oracle",
+            "sample": f"{steps} NAS CG class {CLS} outer iterations ({25 * steps} CG iterations + "
+                      f"{steps} residual SpMVs) in {el:.1f} s, oracle/oracle_spmv.c -O3 1 thread",
+            "host": _cpu_model()}
+
+
+def _cpu_model():
+    try:
+        for ln in open("/proc/cpuinfo"):
+            if ln.startswith("model name"):
+                return ln.split(":", 1)[1].strip()
+    except Exception:
+        pass
+    return None
+
+
+# ---------------------------------------------------------- reference arm
+def run_reference(args):
+    """The reference arm of this tier is the CPU oracle, timed as it stands on
+    the host cores, same metric/config; one step = one NAS outer iteration."""
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return
+    import numpy as np
+
+    import gen
+    import oracle
+    na, nonzer, niter, shift = gen.NPB_CLASSES[CLS]
+    A = gen.makea(CLS)
+    x = np.ones(A.n)
+    for _ in range(args.warmup):
+        oracle.npb_outer(A.rowptr, A.colidx, A.vals, x, 25, shift)
+    x[:] = 1.0
+    t0 = time.perf_counter()
+    for _ in range(args.steps):
+        oracle.npb_outer(A.rowptr, A.colidx, A.vals, x, 25, shift)
+    el = time.perf_counter() - t0
+    v = 25.0 * args.steps / el
+    line = {
+        "metric": METRIC, "value": round(v, 3), "unit": UNIT, "n_gpus": world, "steps": args.steps,
+        "warmup": args.warmup, "ms_per_step": round(1e3 * el / args.steps, 2), "higher_is_better": True,
+        "scaling": "strong", "vs_baseline": None, "dtype": "f64",
+        "data": "synthetic (exact NPB makea class C generator, seeded)",
+        "config": workload_config(A, world), "impl": "reference",
+        "cpu_baseline": {"value": round(v, 3), "unit": UNIT, "cores": 1, "kind": "oracle",
+                         "sample": f"{args.steps} NAS CG class {CLS} outer iterations (full workload per step), "
+                                   "oracle/oracle_spmv.c -O3, 1 thread", "host": _cpu_model()},
+        "e2e": {"value": round(v, 3), "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(line), flush=True)
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
+    ap.add_argument("--no-cpu", action="store_true", help="skip the cpu_baseline leg")
+    ap.add_argument("--cpu-budget", type=float, default=15.0)
+    args = ap.parse_args()
+    if args.warmup < 3:
+        log("warmup < 3 is not allowed by the timing rules; using 3")
+        args.warmup = 3
+    if args.impl == "reference":
+        run_reference(args)
+    else:
+        run_ours(args)
+
+
+if __name__ == "__main__":
+    main()

@@ -1,0 +1,276 @@
+"""B200-native CSR SpMV + CG: thin Python binding of libspmv_b200.so.
+
+The library (include/spmv.h) implements the data-parallel hot path of the SPMV
+idiom of Ginsbach et al., ASPLOS'18 (Fig. 4, Fig. 12, the
+cuSPARSE call shape of Fig. 6) on hand-written sm_100a kernels.
+This module only marshals arguments: torch tensors become raw device pointers
+and every step of the path runs in the library's kernels.  There is no CPU
+fallback: if the shared library is missing the import fails loudly.
+
+Function names follow the C ABI: ``spmv_csr_create``, ``spmv_csr``,
+``cg_solve``, ``cg_npb_outer``, ``spmv_csr_destroy`` (plus introspection and
+the NCCL distributed-mode entry points).  ``CSRMatrix`` wraps a handle.
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_HERE, "libspmv_b200.so")
+
+if not os.path.exists(LIB_PATH):
+    raise ImportError(
+        f"{LIB_PATH} is missing: build it with `python -c 'import __graft_entry__ as g; g.build()'` "
+        "(there is no CPU fallback)")
+
+_lib = ctypes.CDLL(LIB_PATH)
+
+_P, _I64, _I32, _D = ctypes.c_void_p, ctypes.c_int64, ctypes.c_int32, ctypes.c_double
+_ST = ctypes.c_int
+
+SPMV_OK, SPMV_ERR_ARG, SPMV_ERR_INDEX, SPMV_ERR_ALIAS, SPMV_ERR_CUDA = 0, 1, 2, 3, 4
+SPMV_ERR_NCCL, SPMV_ERR_NOMEM, SPMV_ERR_BREAKDOWN, SPMV_ERR_UNSUPPORTED = 5, 6, 7, 8
+SPMV_F64, SPMV_F32 = 0, 1
+KERNELS = {"auto": 0, "scalar": 1, "vector": 2, "merge": 3, "xstat": 4}
+KERNEL_NAMES = {v: k for k, v in KERNELS.items()}
+
+
+class SpmvOpts(ctypes.Structure):
+    _fields_ = [("stream", _P), ("kernel", _I32), ("vec_lanes", _I32), ("validate", _I32),
+                ("l2_window", _I32), ("dist", _P)]
+
+
+class SpmvInfo(ctypes.Structure):
+    _fields_ = [("kernel", _I32), ("vec_lanes", _I32), ("row_min", _I64), ("row_max", _I64),
+                ("row_mean", _D), ("row_cv", _D), ("m_local", _I64), ("row_begin", _I64),
+                ("row_end", _I64), ("nnz_local", _I64), ("rank", _I32), ("nranks", _I32),
+                ("sorted_cols", _I32), ("grid", _I64)]
+
+
+def _decl(name, args, res=_ST):
+    f = getattr(_lib, name)
+    f.argtypes = args
+    f.restype = res
+    return f
+
+
+spmv_csr_create_c = _decl("spmv_csr_create", [ctypes.POINTER(_P), _ST, _I64, _I64, _I64, _P, _P, _P,
+                                               ctypes.POINTER(SpmvOpts)])
+spmv_csr_c = _decl("spmv_csr", [_P, _I64, _I64, _I64, _P, _P, _P, _P, _P, _D, _D])
+cg_solve_c = _decl("cg_solve", [_P, _P, _P, _I32, _D, ctypes.POINTER(_I32), ctypes.POINTER(_D)])
+cg_npb_outer_c = _decl("cg_npb_outer", [_P, _P, _P, _I32, _D, _P])
+spmv_cg_status_c = _decl("spmv_cg_status", [_P])
+spmv_csr_destroy_c = _decl("spmv_csr_destroy", [_P])
+spmv_csr_partition_c = _decl("spmv_csr_partition", [_P, _I64, _I32, _P])
+spmv_csr_merge_splits_c = _decl("spmv_csr_merge_splits", [_P, _I64, _I64, _P, _P])
+spmv_csr_info_c = _decl("spmv_csr_info", [_P, ctypes.POINTER(SpmvInfo)])
+spmv_launch_count = _decl("spmv_launch_count", [], ctypes.c_uint64)
+spmv_status_string = _decl("spmv_status_string", [_ST], ctypes.c_char_p)
+spmv_last_error_string = _decl("spmv_last_error_string", [], ctypes.c_char_p)
+spmv_dist_get_unique_id_c = _decl("spmv_dist_get_unique_id", [_P])
+spmv_dist_init_c = _decl("spmv_dist_init", [ctypes.POINTER(_P), _I32, _I32, _P, _I32])
+spmv_dist_destroy_c = _decl("spmv_dist_destroy", [_P])
+spmv_dist_plan_host_c = _decl("spmv_dist_plan_host", [_P, _P, _I64, _I32, _I32, _P, _P, _P])
+spmv_dist_colidx_c = _decl("spmv_dist_colidx", [_P, _P])
+
+# every symbol include/spmv.h declares (checked by tests/test_abi.py)
+EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_status",
+           "spmv_csr_destroy", "spmv_csr_partition", "spmv_csr_merge_splits", "spmv_csr_info",
+           "spmv_launch_count", "spmv_status_string", "spmv_last_error_string",
+           "spmv_dist_get_unique_id", "spmv_dist_init", "spmv_dist_destroy", "spmv_dist_plan_host",
+           "spmv_dist_colidx"]
+
+
+class SpmvError(RuntimeError):
+    def __init__(self, status, where):
+        self.status = status
+        msg = spmv_last_error_string().decode(errors="replace")
+        super().__init__(f"{where}: {spmv_status_string(status).decode()} ({msg})")
+
+
+def _check(st, where):
+    if st != SPMV_OK:
+        raise SpmvError(st, where)
+
+
+def _ptr(t):
+    """Raw data pointer of a torch tensor, numpy array, int or None."""
+    if t is None:
+        return None
+    if isinstance(t, int):
+        return t
+    if hasattr(t, "data_ptr"):
+        return t.data_ptr()
+    if hasattr(t, "ctypes"):
+        return t.ctypes.data
+    raise TypeError(f"cannot take a pointer of {type(t)}")
+
+
+# ----------------------------------------------------------------- host-side
+def spmv_csr_partition(rowptr_host, nranks: int):
+    """nnz-balanced row bounds (int64[nranks+1]) of a host rowptr (numpy int32)."""
+    import numpy as np
+    rp = np.ascontiguousarray(rowptr_host, dtype=np.int32)
+    b = np.zeros(nranks + 1, dtype=np.int64)
+    _check(spmv_csr_partition_c(rp.ctypes.data, rp.shape[0] - 1, nranks, b.ctypes.data),
+           "spmv_csr_partition")
+    return b
+
+
+def spmv_csr_merge_splits(rowptr_host, pieces: int):
+    import numpy as np
+    rp = np.ascontiguousarray(rowptr_host, dtype=np.int32)
+    sr = np.zeros(pieces + 1, dtype=np.int64)
+    sn = np.zeros(pieces + 1, dtype=np.int64)
+    _check(spmv_csr_merge_splits_c(rp.ctypes.data, rp.shape[0] - 1, pieces, sr.ctypes.data,
+                                   sn.ctypes.data), "spmv_csr_merge_splits")
+    return sr, sn
+
+
+def spmv_dist_plan_host(rowptr_host, colidx_host, nranks: int, rank: int):
+    """Host exchange plan of one rank: (bounds, maxlen, renumbered local colidx)."""
+    import numpy as np
+    rp = np.ascontiguousarray(rowptr_host, dtype=np.int32)
+    ci = np.ascontiguousarray(colidx_host, dtype=np.int32)
+    m = rp.shape[0] - 1
+    b = np.zeros(nranks + 1, dtype=np.int64)
+    ml = ctypes.c_int64(0)
+    _check(spmv_dist_plan_host_c(rp.ctypes.data, ci.ctypes.data, m, nranks, rank, b.ctypes.data,
+                                 ctypes.byref(ml), None), "spmv_dist_plan_host")
+    loc = np.zeros(int(rp[b[rank + 1]]) - int(rp[b[rank]]), dtype=np.int32)
+    _check(spmv_dist_plan_host_c(rp.ctypes.data, ci.ctypes.data, m, nranks, rank, b.ctypes.data,
+                                 ctypes.byref(ml), loc.ctypes.data), "spmv_dist_plan_host")
+    return b, ml.value, loc
+
+
+# ------------------------------------------------------------- distributed
+class Dist:
+    """NCCL context of the library, bootstrapped through a torch process group
+    (torch.distributed is used only to broadcast the 128-byte unique id)."""
+
+    def __init__(self, rank: int, nranks: int, device: int, group=None):
+        import torch
+        import torch.distributed as dist
+        uid = (ctypes.c_char * 128)()
+        if rank == 0:
+            _check(spmv_dist_get_unique_id_c(ctypes.addressof(uid)), "spmv_dist_get_unique_id")
+        buf = [bytes(uid)] if rank == 0 else [None]
+        dist.broadcast_object_list(buf, src=0, group=group)
+        ctypes.memmove(uid, buf[0], 128)
+        h = _P()
+        _check(spmv_dist_init_c(ctypes.byref(h), rank, nranks, ctypes.addressof(uid), device),
+               "spmv_dist_init")
+        self.handle = h
+        self.rank, self.nranks, self.device = rank, nranks, device
+
+    def close(self):
+        if self.handle:
+            _check(spmv_dist_destroy_c(self.handle), "spmv_dist_destroy")
+            self.handle = None
+
+
+# ------------------------------------------------------------------- handle
+class CSRMatrix:
+    """A device-resident CSR matrix handle (spmv_csr_create ... spmv_csr_destroy).
+
+    rowptr/colidx/vals are torch CUDA tensors (int32, int32, float64|float32)
+    that the caller keeps alive; the handle stores their pointers (the paper's
+    lazy copying: A is uploaded once and stays resident).
+    """
+
+    def __init__(self, rowptr, colidx, vals, n: int | None = None, *, kernel: str = "auto",
+                 vec_lanes: int = 0, validate: bool = False, stream=None, dist: Dist | None = None):
+        import torch
+        assert rowptr.dtype == torch.int32 and colidx.dtype == torch.int32
+        assert vals.dtype in (torch.float64, torch.float32)
+        self.rowptr, self.colidx, self.vals = rowptr, colidx, vals
+        self.m = rowptr.numel() - 1
+        self.n = self.m if n is None else int(n)
+        self.dtype = vals.dtype
+        self.dist = dist
+        if stream is None:
+            stream = torch.cuda.current_stream(rowptr.device)
+        self.stream = stream
+        o = SpmvOpts()
+        o.stream = stream.cuda_stream
+        o.kernel = KERNELS[kernel]
+        o.vec_lanes = int(vec_lanes)
+        o.validate = int(bool(validate))
+        o.l2_window = 0
+        o.dist = dist.handle if dist is not None else None
+        nnz = int(rowptr[-1].item()) - int(rowptr[0].item()) if self.m >= 0 else 0
+        self.nnz = nnz
+        h = _P()
+        _check(spmv_csr_create_c(ctypes.byref(h), SPMV_F64 if vals.dtype == torch.float64 else SPMV_F32,
+                                 self.m, self.n, nnz, _ptr(rowptr), _ptr(colidx), _ptr(vals),
+                                 ctypes.byref(o)), "spmv_csr_create")
+        self.handle = h
+        self._info = self.info()
+
+    # -- calls ------------------------------------------------------------
+    def spmv(self, x, y, alpha: float = 1.0, beta: float = 0.0, vals=None):
+        """y <- alpha*A@x + beta*y (asynchronous on the handle's stream)."""
+        v = self.vals if vals is None else vals
+        _check(spmv_csr_c(self.handle, self.m, self.n, self.nnz, _ptr(self.rowptr), _ptr(self.colidx),
+                          _ptr(v), _ptr(x), _ptr(y), float(alpha), float(beta)), "spmv_csr")
+        return y
+
+    def cg_solve(self, b, x, max_iter: int, tol: float = 0.0):
+        """Textbook CG from x0=0 into x; returns (iterations, ||b - A x||).  Synchronous."""
+        its = _I32(0)
+        rn = _D(0.0)
+        _check(cg_solve_c(self.handle, _ptr(b), _ptr(x), int(max_iter), float(tol), ctypes.byref(its),
+                          ctypes.byref(rn)), "cg_solve")
+        return its.value, rn.value
+
+    def npb_outer(self, x, z, cgitmax: int, shift: float, out2):
+        """One NAS CG outer iteration (x updated in place, z = CG(A, x)); out2 <- {zeta, rnorm}.
+        Asynchronous when x, z, out2 are device tensors."""
+        _check(cg_npb_outer_c(self.handle, _ptr(x), _ptr(z), int(cgitmax), float(shift), _ptr(out2)),
+               "cg_npb_outer")
+        return out2
+
+    def dist_colidx(self):
+        import numpy as np
+        out = np.zeros(self._info["nnz_local"], dtype=np.int32)
+        _check(spmv_dist_colidx_c(self.handle, out.ctypes.data), "spmv_dist_colidx")
+        return out
+
+    def cg_status(self):
+        _check(spmv_cg_status_c(self.handle), "spmv_cg_status")
+
+    def info(self) -> dict:
+        inf = SpmvInfo()
+        _check(spmv_csr_info_c(self.handle, ctypes.byref(inf)), "spmv_csr_info")
+        d = {f: getattr(inf, f) for f, _ in SpmvInfo._fields_}
+        d["kernel_name"] = KERNEL_NAMES.get(d["kernel"], "?")
+        return d
+
+    @property
+    def row_range(self):
+        return self._info["row_begin"], self._info["row_end"]
+
+    def destroy(self):
+        if getattr(self, "handle", None):
+            st = spmv_csr_destroy_c(self.handle)
+            self.handle = None
+            _check(st, "spmv_csr_destroy")
+
+    def __del__(self):
+        try:
+            if getattr(self, "handle", None):
+                spmv_csr_destroy_c(self.handle)
+                self.handle = None
+        except Exception:
+            pass
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *a):
+        self.destroy()
+
+
+def launch_count() -> int:
+    return int(spmv_launch_count())

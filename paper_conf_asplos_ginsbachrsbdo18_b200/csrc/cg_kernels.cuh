@@ -1,0 +1,151 @@
+// cg_kernels.cuh -- fused vector kernels of textbook CG (NPB conj_grad
+// [ext:NPB]).  One CG iteration is
+//   K1  q = A p  and partial p.q              (k_spmv_vector<..., DOT=true>)
+//   K2  d = p.q; alpha = rho/d; z += alpha p; r -= alpha q; partial r.r
+//   K3  rho' = r.r; beta = rho'/rho; p = r + beta p
+// Scalars never leave the device: every CTA of a consumer kernel sums the
+// producer's per-CTA partials in the same fixed order (read_sum), so all CTAs
+// (and all runs) see bit-identical alpha/beta.  In distributed mode the
+// partials are first finalized into one value and NCCL-all-reduced; the
+// consumers then read that single value (SumSrc.count == 1).
+#pragma once
+#include "common.cuh"
+
+namespace spmv {
+
+struct CgState {
+  int* flags;   // [0] breakdown (sticky), [1] converged, [2] iterations done
+};
+
+// z = 0, r = b, p = b, partial r.r
+__global__ void __launch_bounds__(256)
+k_cg_init(int64_t n, const double* __restrict__ b, double* __restrict__ z,
+          double* __restrict__ r, double* __restrict__ p, double* __restrict__ part_rr) {
+  __shared__ double red[8];
+  double acc = 0.0;
+  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n;
+       j += int64_t(gridDim.x) * blockDim.x) {
+    const double bj = b[j];
+    z[j] = 0.0;
+    r[j] = bj;
+    p[j] = bj;
+    acc += bj * bj;
+  }
+  const double t = block_sum(acc, red);
+  if (threadIdx.x == 0) part_rr[blockIdx.x] = t;
+}
+
+// K2.  pq: p.q; rr_old: rho.  If tol_check, iterations stop once done.
+__global__ void __launch_bounds__(256)
+k_cg_zr(int64_t n, SumSrc pq, SumSrc rr_old, const double* __restrict__ p,
+        const double* __restrict__ q, double* __restrict__ z, double* __restrict__ r,
+        double* __restrict__ part_rr_new, int* __restrict__ flags) {
+  __shared__ double red[8];
+  __shared__ double s_pq, s_rr;
+  if (flags[1]) return;  // converged (tol mode): no-op
+  const double d = read_sum(pq, &s_pq);
+  const double rho = read_sum(rr_old, &s_rr);
+  if (d == 0.0 || !isfinite(d)) {
+    if (blockIdx.x == 0 && threadIdx.x == 0) flags[0] = 1;
+  }
+  const double alpha = rho / d;
+  double acc = 0.0;
+  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n;
+       j += int64_t(gridDim.x) * blockDim.x) {
+    const double zj = z[j] + alpha * p[j];
+    const double rj = r[j] - alpha * q[j];
+    z[j] = zj;
+    r[j] = rj;
+    acc += rj * rj;
+  }
+  const double t = block_sum(acc, red);
+  if (threadIdx.x == 0) part_rr_new[blockIdx.x] = t;
+}
+
+// K3.  rr_new: rho', rr_old: rho.  tol > 0: after the update, mark converged
+// once sqrt(rho') <= tol * ||b|| (rr_b: ||b||^2 source), recording `it`+1.
+__global__ void __launch_bounds__(256)
+k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
+       double* __restrict__ p, int* __restrict__ flags, double tol, SumSrc rr_b, int it) {
+  __shared__ double s_new, s_old, s_b;
+  if (flags[1]) return;
+  const double rho1 = read_sum(rr_new, &s_new);
+  const double rho0 = read_sum(rr_old, &s_old);
+  const double beta = rho1 / rho0;
+  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n;
+       j += int64_t(gridDim.x) * blockDim.x)
+    p[j] = r[j] + beta * p[j];
+  if (tol > 0.0) {
+    const double bb = read_sum(rr_b, &s_b);
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
+      flags[2] = it + 1;
+      if (sqrt(rho1) <= tol * sqrt(bb)) flags[1] = 1;
+    }
+  } else if (blockIdx.x == 0 && threadIdx.x == 0) {
+    flags[2] = it + 1;
+  }
+}
+
+// Residual / NPB norms: partials of ||b - Az||^2 and (NPB) x.z, z.z.
+// b is the right-hand side (NPB: x), az = A z.
+template <bool NPB>
+__global__ void __launch_bounds__(256)
+k_cg_resid(int64_t n, const double* __restrict__ b, const double* __restrict__ az,
+           const double* __restrict__ z, double* __restrict__ part_res,
+           double* __restrict__ part_xz, double* __restrict__ part_zz) {
+  __shared__ double red[8];
+  double a0 = 0.0, a1 = 0.0, a2 = 0.0;
+  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n;
+       j += int64_t(gridDim.x) * blockDim.x) {
+    const double bj = b[j];
+    const double d = bj - az[j];
+    a0 += d * d;
+    if (NPB) {
+      const double zj = z[j];
+      a1 += bj * zj;
+      a2 += zj * zj;
+    }
+  }
+  double t = block_sum(a0, red);
+  if (threadIdx.x == 0) part_res[blockIdx.x] = t;
+  if (NPB) {
+    t = block_sum(a1, red);
+    if (threadIdx.x == 0) part_xz[blockIdx.x] = t;
+    t = block_sum(a2, red);
+    if (threadIdx.x == 0) part_zz[blockIdx.x] = t;
+  }
+}
+
+// NPB tail: zeta = shift + 1/(x.z); x = z / ||z||; out2 = {zeta, rnorm}.
+__global__ void __launch_bounds__(256)
+k_npb_finish(int64_t n, SumSrc res, SumSrc xz, SumSrc zz, const double* __restrict__ z,
+             double* __restrict__ x, double shift, double* __restrict__ out2) {
+  __shared__ double s0, s1, s2;
+  const double rr = read_sum(res, &s0);
+  const double nt1 = read_sum(xz, &s1);
+  double nt2 = read_sum(zz, &s2);
+  nt2 = 1.0 / sqrt(nt2);
+  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n;
+       j += int64_t(gridDim.x) * blockDim.x)
+    x[j] = nt2 * z[j];
+  if (blockIdx.x == 0 && threadIdx.x == 0) {
+    out2[0] = shift + 1.0 / nt1;
+    out2[1] = sqrt(rr);
+  }
+}
+
+// cg_solve tail: rnorm = sqrt(sum).
+__global__ void k_finish_norm(SumSrc res, double* out) {
+  __shared__ double s0;
+  const double rr = read_sum(res, &s0);
+  if (threadIdx.x == 0) *out = sqrt(rr);
+}
+
+// Distributed mode: sum `count` partials into one value (then all-reduced).
+__global__ void k_finalize(SumSrc s, double* out) {
+  __shared__ double s0;
+  const double v = read_sum(s, &s0);
+  if (threadIdx.x == 0) *out = v;
+}
+
+}  // namespace spmv

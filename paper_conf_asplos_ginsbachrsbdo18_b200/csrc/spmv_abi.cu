@@ -1,0 +1,879 @@
+// spmv_abi.cu -- the C ABI of include/spmv.h: handle management, argument and
+// alias checks, kernel selection, the CG drivers (CUDA-graph captured) and the
+// NCCL row-sharded mode.  All arithmetic of the hot path runs in the kernels of
+// spmv_kernels.cuh / cg_kernels.cuh; this file only validates, chooses and
+// launches.  P:a-b = /root/reference/PAPER.md lines; Rn = DESIGN.md reading n.
+#include <algorithm>
+#include <atomic>
+#include <cmath>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <string>
+#include <vector>
+
+#include <cuda_runtime.h>
+#include <nccl.h>
+
+#include "../../include/spmv.h"
+#include "analysis_kernels.cuh"
+#include "cg_kernels.cuh"
+#include "spmv_kernels.cuh"
+
+using namespace spmv;
+
+// ------------------------------------------------------------------ errors
+static thread_local std::string g_err = "no error";
+static std::atomic<uint64_t> g_launches{0};
+
+static spmv_status cuda_fail(cudaError_t e, const char* what, int line) {
+  char buf[512];
+  snprintf(buf, sizeof buf, "%s (line %d): %s", what, line, cudaGetErrorString(e));
+  g_err = buf;
+  return e == cudaErrorMemoryAllocation ? SPMV_ERR_NOMEM : SPMV_ERR_CUDA;
+}
+static spmv_status arg_fail(const char* why) {
+  g_err = why;
+  return SPMV_ERR_ARG;
+}
+#define CK(call)                                                   \
+  do {                                                             \
+    cudaError_t e__ = (call);                                      \
+    if (e__ != cudaSuccess) return cuda_fail(e__, #call, __LINE__); \
+  } while (0)
+#define NK(call)                                                   \
+  do {                                                             \
+    ncclResult_t r__ = (call);                                     \
+    if (r__ != ncclSuccess) {                                      \
+      g_err = std::string(#call ": ") + ncclGetErrorString(r__);   \
+      return SPMV_ERR_NCCL;                                        \
+    }                                                              \
+  } while (0)
+#define ST(call)                         \
+  do {                                   \
+    spmv_status s__ = (call);            \
+    if (s__ != SPMV_OK) return s__;      \
+  } while (0)
+// after each kernel launch: count it and surface launch-configuration errors
+#define LAUNCHED()                                                        \
+  do {                                                                    \
+    g_launches.fetch_add(1, std::memory_order_relaxed);                   \
+    cudaError_t e__ = cudaGetLastError();                                 \
+    if (e__ != cudaSuccess) return cuda_fail(e__, "kernel launch", __LINE__); \
+  } while (0)
+
+// ------------------------------------------------------------------ types
+struct spmv_dist_s {
+  ncclComm_t comm = nullptr;
+  int rank = 0, nranks = 1, device = 0;
+};
+
+struct Graph {
+  cudaGraphExec_t exec = nullptr;
+  uint64_t nodes = 0;
+  const void *k0 = nullptr, *k1 = nullptr, *k2 = nullptr;
+  int32_t ki = 0;
+  double kd = 0.0;
+  void reset() {
+    if (exec) cudaGraphExecDestroy(exec);
+    exec = nullptr;
+    nodes = 0;
+  }
+};
+
+struct spmv_csr_s {
+  int device = 0;
+  cudaStream_t stream = nullptr;      // user stream (may be the legacy stream 0)
+  cudaStream_t cap = nullptr;         // private stream used for graph capture
+  cudaEvent_t ev_a = nullptr, ev_b = nullptr;
+  spmv_dtype dt = SPMV_F64;
+  size_t ts = 8;
+  int64_t m = 0, n = 0, nnz = 0;
+  int32_t base = 0;
+  const int32_t* rowptr = nullptr;
+  const int32_t* colidx = nullptr;
+  const void* vals = nullptr;
+  // execution view: local rows (all rows on a single GPU)
+  int64_t m_loc = 0, row0 = 0, k0 = 0, k1 = 0;
+  const int32_t* rp_loc = nullptr;   // rowptr + row0 (absolute k)
+  const int32_t* ci_loc = nullptr;   // colidx (single) or renumbered copy - k0 (dist)
+  // kernel choice
+  int32_t kernel = SPMV_KERNEL_VECTOR, lanes = 32, unroll = 4;
+  int64_t grid = 1, vgrid = 1;
+  int64_t row_min = 0, row_max = 0;
+  double row_mean = 0, row_cv = 0;
+  int32_t sorted = 0;
+  // dist
+  spmv_dist_s* dist = nullptr;
+  std::vector<long long> bounds;
+  long long maxlen = 0;
+  int32_t* ci_own = nullptr;
+  void* xpad = nullptr;               // nranks*maxlen, the gathered x / p
+  // CG workspace (lazy)
+  double *z = nullptr, *r = nullptr, *q = nullptr, *p_single = nullptr;
+  double *part_pq = nullptr, *part_rr = nullptr, *part_res = nullptr, *part_xz = nullptr,
+         *part_zz = nullptr, *scal = nullptr, *out2 = nullptr;
+  int* flags = nullptr;
+  double *stage_x = nullptr, *stage_z = nullptr;
+  Graph g_npb;
+};
+
+// --------------------------------------------------------------- helpers
+static bool env_int(const char* name, int* v) {
+  const char* s = getenv(name);
+  if (!s || !*s) return false;
+  *v = atoi(s);
+  return true;
+}
+
+static int num_sms(int dev) {
+  int v = kNumSMs;
+  cudaDeviceGetAttribute(&v, cudaDevAttrMultiProcessorCount, dev);
+  return v > 0 ? v : kNumSMs;
+}
+
+// 1 = device (or managed) memory of `dev`, 0 = host (pinned, pageable), -1 = error
+static int mem_kind(const void* p, int dev) {
+  cudaPointerAttributes a;
+  cudaError_t e = cudaPointerGetAttributes(&a, p);
+  if (e != cudaSuccess) { cudaGetLastError(); return 0; }
+  if (a.type == cudaMemoryTypeDevice || a.type == cudaMemoryTypeManaged)
+    return a.device == dev ? 1 : -1;
+  return 0;
+}
+
+static spmv_status need_device(const void* p, int dev, const char* what, bool may_be_null) {
+  if (!p) return may_be_null ? SPMV_OK : arg_fail(what);
+  return mem_kind(p, dev) == 1 ? SPMV_OK : arg_fail(what);
+}
+
+static bool overlap(const void* a, size_t na, const void* b, size_t nb) {
+  if (!a || !b || na == 0 || nb == 0) return false;
+  const uintptr_t a0 = (uintptr_t)a, b0 = (uintptr_t)b;
+  return a0 < b0 + nb && b0 < a0 + na;
+}
+
+static int64_t cdiv(int64_t a, int64_t b) { return (a + b - 1) / b; }
+
+static spmv_status ensure_buf(void** p, size_t bytes) {
+  if (*p) return SPMV_OK;
+  CK(cudaMalloc(p, bytes > 0 ? bytes : 8));
+  return SPMV_OK;
+}
+
+// ------------------------------------------------------- kernel dispatch
+template <typename T, int G, bool DOT>
+static void launch_vec_u(int unroll, int64_t grid, cudaStream_t s, const SpmvArgs& a) {
+  switch (unroll) {
+    case 2: k_spmv_vector<T, G, 2, DOT><<<grid, 256, 0, s>>>(a); break;
+    case 8: k_spmv_vector<T, G, 8, DOT><<<grid, 256, 0, s>>>(a); break;
+    default: k_spmv_vector<T, G, 4, DOT><<<grid, 256, 0, s>>>(a); break;
+  }
+}
+
+template <typename T, bool DOT>
+static void launch_vec(int lanes, int unroll, int64_t grid, cudaStream_t s, const SpmvArgs& a) {
+  switch (lanes) {
+    case 1: launch_vec_u<T, 1, DOT>(unroll, grid, s, a); break;
+    case 2: launch_vec_u<T, 2, DOT>(unroll, grid, s, a); break;
+    case 4: launch_vec_u<T, 4, DOT>(unroll, grid, s, a); break;
+    case 8: launch_vec_u<T, 8, DOT>(unroll, grid, s, a); break;
+    case 16: launch_vec_u<T, 16, DOT>(unroll, grid, s, a); break;
+    default: launch_vec_u<T, 32, DOT>(unroll, grid, s, a); break;
+  }
+}
+
+// Local SpMV of the handle: y = alpha*A_loc*x + beta*y (+ partial w.y per CTA).
+static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
+                            double alpha, double beta, const double* w, double* part) {
+  if (h->m_loc == 0) {
+    if (part) {
+      CK(cudaMemsetAsync(part, 0, sizeof(double) * h->grid, s));
+    }
+    return SPMV_OK;
+  }
+  if (alpha == 0.0 && !part) {
+    const int64_t g = std::min<int64_t>(cdiv(h->m_loc, 256), 4 * num_sms(h->device));
+    if (h->dt == SPMV_F64) k_scale<double><<<g, 256, 0, s>>>(h->m_loc, (double*)y, beta);
+    else k_scale<float><<<g, 256, 0, s>>>(h->m_loc, (float*)y, (double)(float)beta);
+    LAUNCHED();
+    return SPMV_OK;
+  }
+  SpmvArgs a;
+  a.m = h->m_loc;
+  a.rowptr = h->rp_loc;
+  a.colidx = h->ci_loc;
+  a.vals = vals;
+  a.x = x;
+  a.y = y;
+  a.alpha = alpha;
+  a.beta = beta;
+  a.w = w;
+  a.part = part;
+  if (h->dt == SPMV_F64) {
+    if (part) launch_vec<double, true>(h->lanes, h->unroll, h->grid, s, a);
+    else launch_vec<double, false>(h->lanes, h->unroll, h->grid, s, a);
+  } else {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+    launch_vec<float, false>(h->lanes, h->unroll, h->grid, s, a);
+  }
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+// Kernel selection from row statistics (the paper's "try every API, keep the
+// fastest", becomes a rule fitted by the bench sweep).
+static void choose_kernel(spmv_csr_s* h, int req_kernel, int req_lanes) {
+  int lanes;
+  const double mean = h->row_mean;
+  if (mean < 2.0) lanes = 1;
+  else if (mean < 6.0) lanes = 2;
+  else if (mean < 12.0) lanes = 4;
+  else if (mean < 24.0) lanes = 8;
+  else if (mean < 48.0) lanes = 16;
+  else lanes = 32;
+  h->kernel = SPMV_KERNEL_VECTOR;
+  if (req_kernel == SPMV_KERNEL_SCALAR) lanes = 1;
+  if (req_lanes == 1 || req_lanes == 2 || req_lanes == 4 || req_lanes == 8 || req_lanes == 16 ||
+      req_lanes == 32)
+    lanes = req_lanes;
+  h->lanes = lanes;
+  h->unroll = 4;
+  int u;
+  if (env_int("SPMV_UNROLL", &u) && (u == 2 || u == 4 || u == 8)) h->unroll = u;
+  const int sms = num_sms(h->device);
+  // fixed grid-stride grid (deterministic CTA partials): 8 CTAs of 256 per SM
+  const int64_t groups_per_cta = 256 / lanes;
+  h->grid = std::max<int64_t>(1, std::min<int64_t>(cdiv(h->m_loc, groups_per_cta), 8LL * sms));
+  h->vgrid = std::max<int64_t>(1, std::min<int64_t>(cdiv(h->m_loc, 1024), 4LL * sms));
+}
+
+// ----------------------------------------------------------------- create
+extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m, int64_t n,
+                                       int64_t nnz, const int32_t* rowptr, const int32_t* colidx,
+                                       const void* vals, const spmv_opts* opts) {
+  if (!out) return arg_fail("out is NULL");
+  *out = nullptr;
+  if (dt != SPMV_F64 && dt != SPMV_F32) return arg_fail("dtype must be SPMV_F64 or SPMV_F32");
+  if (m < 0 || n < 0 || nnz < 0 || nnz > 2147483647LL || m > 2147483646LL || n > 2147483647LL)
+    return arg_fail("sizes out of range (m, n, nnz >= 0; nnz < 2^31)");
+  if (!rowptr) return arg_fail("rowptr is NULL");
+  spmv_opts o{};
+  if (opts) o = *opts;
+  int dev = 0;
+  CK(cudaGetDevice(&dev));
+  if (o.dist) dev = o.dist->device;
+  CK(cudaSetDevice(dev));
+  ST(need_device(rowptr, dev, "rowptr must be a device pointer on the current device", false));
+  ST(need_device(colidx, dev, "colidx must be a device pointer", nnz == 0));
+  ST(need_device(vals, dev, "vals must be a device pointer", nnz == 0));
+  if (o.dist && m != n) return arg_fail("distributed mode needs a square matrix (R25)");
+
+  // rowptr[0], rowptr[m] -> nnz check (R1)
+  int32_t ends[2];
+  CK(cudaMemcpy(&ends[0], rowptr, 4, cudaMemcpyDeviceToHost));
+  CK(cudaMemcpy(&ends[1], rowptr + m, 4, cudaMemcpyDeviceToHost));
+  if ((int64_t)ends[1] - (int64_t)ends[0] != nnz)
+    return arg_fail("nnz != rowptr[m] - rowptr[0] (reading R1)");
+
+  spmv_csr_s* h = new spmv_csr_s();
+  h->device = dev;
+  h->stream = (cudaStream_t)o.stream;
+  h->dt = dt;
+  h->ts = dt == SPMV_F64 ? 8 : 4;
+  h->m = m;
+  h->n = n;
+  h->nnz = nnz;
+  h->base = ends[0];
+  h->rowptr = rowptr;
+  h->colidx = colidx;
+  h->vals = vals;
+  h->dist = o.dist;
+  auto fail = [&](spmv_status s) {
+    spmv_csr_destroy(h);
+    return s;
+  };
+  cudaStream_t s = h->stream;
+  const int sms = num_sms(dev);
+
+  // validation (device pass, synchronous)
+  if (o.validate && m > 0) {
+    int* fl = nullptr;
+    if (cudaMalloc(&fl, sizeof(int)) != cudaSuccess) return fail(cuda_fail(cudaErrorMemoryAllocation, "cudaMalloc", __LINE__));
+    cudaMemsetAsync(fl, 0, sizeof(int), s);
+    k_validate<<<std::min<int64_t>(cdiv(std::max(m, nnz), 256), 8LL * sms), 256, 0, s>>>(m, n, rowptr, colidx, fl);
+    g_launches.fetch_add(1);
+    int hv = 0;
+    cudaError_t e = cudaMemcpyAsync(&hv, fl, sizeof(int), cudaMemcpyDeviceToHost, s);
+    if (e == cudaSuccess) e = cudaStreamSynchronize(s);
+    cudaFree(fl);
+    if (e != cudaSuccess) return fail(cuda_fail(e, "validate", __LINE__));
+    if (hv) {
+      g_err = (hv & 1) ? "rowptr is decreasing" : "colidx outside [0, n)";
+      return fail(SPMV_ERR_INDEX);
+    }
+  }
+
+  // row statistics (device pass over rowptr [+ colidx sortedness]; host reduce in CTA order)
+  if (m > 0) {
+    const int64_t g = std::min<int64_t>(cdiv(m, 256), 2LL * sms);
+    double* dpart = nullptr;
+    if (cudaMalloc(&dpart, sizeof(double) * 5 * g) != cudaSuccess)
+      return fail(cuda_fail(cudaErrorMemoryAllocation, "cudaMalloc", __LINE__));
+    k_row_stats<<<g, 256, 0, s>>>(m, rowptr, colidx, 0, dpart);
+    g_launches.fetch_add(1);
+    std::vector<double> hp(5 * g);
+    cudaError_t e = cudaMemcpyAsync(hp.data(), dpart, sizeof(double) * 5 * g, cudaMemcpyDeviceToHost, s);
+    if (e == cudaSuccess) e = cudaStreamSynchronize(s);
+    cudaFree(dpart);
+    if (e != cudaSuccess) return fail(cuda_fail(e, "row stats", __LINE__));
+    double mn = 1e300, mx = -1e300, sum = 0, sq = 0;
+    for (int64_t b = 0; b < g; ++b) {
+      mn = std::min(mn, hp[5 * b]);
+      mx = std::max(mx, hp[5 * b + 1]);
+      sum += hp[5 * b + 2];
+      sq += hp[5 * b + 3];
+    }
+    h->row_min = (int64_t)mn;
+    h->row_max = (int64_t)mx;
+    h->row_mean = sum / (double)m;
+    const double var = std::max(0.0, sq / (double)m - h->row_mean * h->row_mean);
+    h->row_cv = h->row_mean > 0 ? std::sqrt(var) / h->row_mean : 0.0;
+  }
+
+  // execution view
+  if (!o.dist) {
+    h->m_loc = m;
+    h->row0 = 0;
+    h->k0 = ends[0];
+    h->k1 = ends[1];
+    h->rp_loc = rowptr;
+    h->ci_loc = colidx;
+  } else {
+    spmv_dist_s* d = o.dist;
+    const int P = d->nranks;
+    long long* dbounds = nullptr;
+    if (cudaMalloc(&dbounds, sizeof(long long) * (P + 1)) != cudaSuccess)
+      return fail(cuda_fail(cudaErrorMemoryAllocation, "cudaMalloc", __LINE__));
+    k_partition<<<cdiv(P + 1, 128), 128, 0, s>>>(m, rowptr, P, dbounds);
+    g_launches.fetch_add(1);
+    h->bounds.assign(P + 1, 0);
+    cudaError_t e = cudaMemcpyAsync(h->bounds.data(), dbounds, sizeof(long long) * (P + 1),
+                                    cudaMemcpyDeviceToHost, s);
+    if (e == cudaSuccess) e = cudaStreamSynchronize(s);
+    if (e != cudaSuccess) { cudaFree(dbounds); return fail(cuda_fail(e, "partition", __LINE__)); }
+    long long maxlen = 1;
+    for (int r = 0; r < P; ++r) maxlen = std::max(maxlen, h->bounds[r + 1] - h->bounds[r]);
+    h->maxlen = maxlen;
+    const int r = d->rank;
+    h->row0 = h->bounds[r];
+    h->m_loc = h->bounds[r + 1] - h->bounds[r];
+    int32_t kk[2] = {0, 0};
+    e = cudaMemcpy(&kk[0], rowptr + h->row0, 4, cudaMemcpyDeviceToHost);
+    if (e == cudaSuccess) e = cudaMemcpy(&kk[1], rowptr + h->row0 + h->m_loc, 4, cudaMemcpyDeviceToHost);
+    if (e != cudaSuccess) { cudaFree(dbounds); return fail(cuda_fail(e, "rowptr", __LINE__)); }
+    h->k0 = kk[0];
+    h->k1 = kk[1];
+    const int64_t nloc = h->k1 - h->k0;
+    if (cudaMalloc(&h->ci_own, sizeof(int32_t) * std::max<int64_t>(nloc, 1)) != cudaSuccess ||
+        cudaMalloc(&h->xpad, h->ts * (size_t)(maxlen * P)) != cudaSuccess) {
+      cudaFree(dbounds);
+      return fail(cuda_fail(cudaErrorMemoryAllocation, "cudaMalloc", __LINE__));
+    }
+    cudaMemsetAsync(h->xpad, 0, h->ts * (size_t)(maxlen * P), s);
+    if (nloc > 0) {
+      k_renumber<<<std::min<int64_t>(cdiv(nloc, 256), 8LL * sms), 256, sizeof(long long) * (P + 1), s>>>(
+          h->k0, h->k1, colidx, dbounds, P, maxlen, h->ci_own);
+      g_launches.fetch_add(1);
+    }
+    e = cudaStreamSynchronize(s);
+    cudaFree(dbounds);
+    if (e != cudaSuccess) return fail(cuda_fail(e, "renumber", __LINE__));
+    h->rp_loc = rowptr + h->row0;
+    h->ci_loc = h->ci_own - h->k0;  // absolute k addressing
+  }
+
+  int rk = 0, rl = 0;
+  if (!env_int("SPMV_KERNEL", &rk)) rk = o.kernel;
+  if (!env_int("SPMV_LANES", &rl)) rl = o.vec_lanes;
+  choose_kernel(h, rk, rl);
+  CK(cudaStreamCreateWithFlags(&h->cap, cudaStreamNonBlocking));
+  CK(cudaEventCreateWithFlags(&h->ev_a, cudaEventDisableTiming));
+  CK(cudaEventCreateWithFlags(&h->ev_b, cudaEventDisableTiming));
+  *out = h;
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
+  if (!h) return SPMV_OK;
+  cudaSetDevice(h->device);
+  spmv_status st = SPMV_OK;
+  cudaError_t e = h->stream ? cudaStreamSynchronize(h->stream) : cudaDeviceSynchronize();
+  if (e != cudaSuccess) st = cuda_fail(e, "pending asynchronous error", __LINE__);
+  h->g_npb.reset();
+  void* bufs[] = {h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
+                  h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
+                  h->stage_x, h->stage_z};
+  for (void* b : bufs)
+    if (b) cudaFree(b);
+  if (h->cap) cudaStreamDestroy(h->cap);
+  if (h->ev_a) cudaEventDestroy(h->ev_a);
+  if (h->ev_b) cudaEventDestroy(h->ev_b);
+  delete h;
+  return st;
+}
+
+// ------------------------------------------------------------------ spmv
+extern "C" spmv_status spmv_csr(spmv_csr_t h, int64_t m, int64_t n, int64_t nnz,
+                                const int32_t* rowptr, const int32_t* colidx, const void* vals,
+                                const void* x, void* y, double alpha, double beta) {
+  if (!h) return arg_fail("handle is NULL");
+  if (m != h->m || n != h->n || nnz != h->nnz || rowptr != h->rowptr || colidx != h->colidx)
+    return arg_fail("m, n, nnz, rowptr, colidx must equal those bound at create");
+  CK(cudaSetDevice(h->device));
+  const int64_t ml = h->m_loc;
+  const int64_t xl = h->dist ? h->m_loc : n;  // local slice length of x in dist mode
+  if (ml > 0) ST(need_device(y, h->device, "y must be a device pointer", false));
+  if (alpha != 0.0) {
+    ST(need_device(x, h->device, "x must be a device pointer", xl == 0));
+    ST(need_device(vals, h->device, "vals must be a device pointer", nnz == 0));
+  }
+  const size_t ts = h->ts;
+  // aliasing check (reading R13)
+  const size_t ybytes = ts * (size_t)ml;
+  if (overlap(y, ybytes, x, ts * (size_t)xl) ||
+      overlap(y, ybytes, (const char*)vals + ts * (size_t)h->base, ts * (size_t)nnz) ||
+      overlap(y, ybytes, colidx + h->base, 4 * (size_t)nnz) ||
+      overlap(y, ybytes, rowptr, 4 * (size_t)(m + 1))) {
+    g_err = "y overlaps x, vals, colidx or rowptr";
+    return SPMV_ERR_ALIAS;
+  }
+  cudaStream_t s = h->stream;
+  const void* xin = x;
+  if (h->dist && alpha != 0.0) {
+    spmv_dist_s* d = h->dist;
+    char* mine = (char*)h->xpad + ts * (size_t)(d->rank * h->maxlen);
+    if (ml > 0 && x != mine) CK(cudaMemcpyAsync(mine, x, ts * (size_t)ml, cudaMemcpyDeviceToDevice, s));
+    NK(ncclAllGather(mine, h->xpad, (size_t)h->maxlen, h->dt == SPMV_F64 ? ncclDouble : ncclFloat,
+                     d->comm, s));
+    xin = h->xpad;
+  }
+  return run_spmv(h, s, vals, xin, y, alpha, beta, nullptr, nullptr);
+}
+
+// ------------------------------------------------------------------ CG
+static spmv_status cg_alloc(spmv_csr_s* h) {
+  if (h->z) return SPMV_OK;
+  const size_t nb = sizeof(double) * (size_t)std::max<int64_t>(h->m_loc, 1);
+  const size_t pb = sizeof(double) * (size_t)std::max<int64_t>(std::max(h->grid, h->vgrid), 1);
+  ST(ensure_buf((void**)&h->z, nb));
+  ST(ensure_buf((void**)&h->r, nb));
+  ST(ensure_buf((void**)&h->q, nb));
+  if (!h->dist) ST(ensure_buf((void**)&h->p_single, nb));
+  ST(ensure_buf((void**)&h->part_pq, pb));
+  ST(ensure_buf((void**)&h->part_rr, 2 * pb));
+  ST(ensure_buf((void**)&h->part_res, pb));
+  ST(ensure_buf((void**)&h->part_xz, pb));
+  ST(ensure_buf((void**)&h->part_zz, pb));
+  ST(ensure_buf((void**)&h->scal, sizeof(double) * 16));
+  ST(ensure_buf((void**)&h->out2, sizeof(double) * 2));
+  ST(ensure_buf((void**)&h->flags, sizeof(int) * 4));
+  CK(cudaMemset(h->flags, 0, sizeof(int) * 4));
+  return SPMV_OK;
+}
+
+static double* cg_p(spmv_csr_s* h) {
+  if (!h->dist) return h->p_single;
+  return (double*)h->xpad + h->dist->rank * h->maxlen;
+}
+
+// In distributed mode a SumSrc of per-CTA partials is finalized into scal[slot]
+// and all-reduced over the ranks; single GPU returns the partials unchanged.
+static spmv_status reduce_src(spmv_csr_s* h, cudaStream_t s, SumSrc in, int slot, SumSrc* out) {
+  if (!h->dist) { *out = in; return SPMV_OK; }
+  double* dst = h->scal + slot;
+  k_finalize<<<1, 32, 0, s>>>(in, dst);
+  LAUNCHED();
+  NK(ncclAllReduce(dst, dst, 1, ncclDouble, ncclSum, h->dist->comm, s));
+  *out = SumSrc{dst, 1};
+  return SPMV_OK;
+}
+
+static spmv_status gather_p(spmv_csr_s* h, cudaStream_t s) {
+  if (!h->dist) return SPMV_OK;
+  NK(ncclAllGather((double*)h->xpad + h->dist->rank * h->maxlen, h->xpad, (size_t)h->maxlen,
+                   ncclDouble, h->dist->comm, s));
+  return SPMV_OK;
+}
+
+// CG enqueue state: the scalar sources carried between iterations.
+struct CgRun {
+  SumSrc rr_b, rr_old;
+  int it = 0;
+};
+
+// Enqueue CG init (x0 = 0): z = 0, r = b, p = b, rho = r.r (no host sync).
+static spmv_status cg_enqueue_init(spmv_csr_s* h, cudaStream_t s, const double* b, double* z,
+                                   CgRun* run) {
+  const int vg = (int)h->vgrid;
+  k_cg_init<<<vg, 256, 0, s>>>(h->m_loc, b, z, h->r, cg_p(h), h->part_rr);
+  LAUNCHED();
+  ST(reduce_src(h, s, SumSrc{h->part_rr, vg}, 0, &run->rr_b));
+  run->rr_old = run->rr_b;
+  run->it = 0;
+  return SPMV_OK;
+}
+
+// Enqueue `iters` CG iterations (no host sync).  tol > 0: kernels become
+// no-ops once sqrt(rho) <= tol*||b|| (flags[1]).
+static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, int iters, double tol,
+                                    CgRun* run) {
+  const int64_t n = h->m_loc;
+  double* p = cg_p(h);
+  const void* xg = h->dist ? h->xpad : (const void*)p;
+  const int vg = (int)h->vgrid, sg = (int)h->grid;
+  const int64_t pstride = std::max(h->grid, h->vgrid);
+  for (int c = 0; c < iters; ++c) {
+    const int it = run->it++;
+    ST(gather_p(h, s));
+    ST(run_spmv(h, s, h->vals, xg, h->q, 1.0, 0.0, p, h->part_pq));
+    SumSrc pq;
+    ST(reduce_src(h, s, SumSrc{h->part_pq, sg}, 1, &pq));
+    double* pnew = h->part_rr + ((it + 1) & 1) * pstride;
+    k_cg_zr<<<vg, 256, 0, s>>>(n, pq, run->rr_old, p, h->q, z, h->r, pnew, h->flags);
+    LAUNCHED();
+    SumSrc rr_new;
+    ST(reduce_src(h, s, SumSrc{pnew, vg}, 2 + ((it + 1) & 1), &rr_new));
+    k_cg_p<<<vg, 256, 0, s>>>(n, rr_new, run->rr_old, h->r, p, h->flags, tol, run->rr_b, it);
+    LAUNCHED();
+    run->rr_old = rr_new;
+  }
+  return SPMV_OK;
+}
+
+// Residual SpMV (Fig. 4 verbatim: r = A z) into q and the norm partials.
+template <bool NPB>
+static spmv_status cg_resid(spmv_csr_s* h, cudaStream_t s, const double* b, const double* z) {
+  const void* zg = z;
+  if (h->dist) {
+    double* mine = (double*)h->xpad + h->dist->rank * h->maxlen;
+    if (h->m_loc > 0) CK(cudaMemcpyAsync(mine, z, sizeof(double) * h->m_loc, cudaMemcpyDeviceToDevice, s));
+    ST(gather_p(h, s));
+    zg = h->xpad;
+  }
+  ST(run_spmv(h, s, h->vals, zg, h->q, 1.0, 0.0, nullptr, nullptr));
+  k_cg_resid<NPB><<<(int)h->vgrid, 256, 0, s>>>(h->m_loc, b, h->q, z, h->part_res, h->part_xz,
+                                               h->part_zz);
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+static spmv_status stage_in(spmv_csr_s* h, cudaStream_t s, const void* src, double** dev_stage,
+                            const double** use, bool copy) {
+  const int k = mem_kind(src, h->device);
+  if (k == 1 || (src == nullptr && h->m_loc == 0)) { *use = (const double*)src; return SPMV_OK; }
+  if (k < 0) return arg_fail("vector is device memory of another GPU");
+  ST(ensure_buf((void**)dev_stage, sizeof(double) * std::max<int64_t>(h->m_loc, 1)));
+  if (copy && h->m_loc > 0)
+    CK(cudaMemcpyAsync(*dev_stage, src, sizeof(double) * h->m_loc, cudaMemcpyHostToDevice, s));
+  *use = *dev_stage;
+  return SPMV_OK;
+}
+
+extern "C" spmv_status cg_solve(spmv_csr_t h, const void* b, void* x, int32_t max_iter, double tol,
+                                int32_t* iters_out, double* rnorm_out) {
+  if (!h) return arg_fail("handle is NULL");
+  if (h->dt != SPMV_F64) { g_err = "cg_solve is fp64 only"; return SPMV_ERR_UNSUPPORTED; }
+  if (h->m != h->n) return arg_fail("cg_solve needs a square matrix");
+  if (max_iter < 0 || !(tol >= 0.0)) return arg_fail("max_iter >= 0, tol >= 0");
+  if ((!b || !x) && h->m_loc > 0) return arg_fail("b and x must not be NULL");
+  CK(cudaSetDevice(h->device));
+  ST(cg_alloc(h));
+  cudaStream_t s = h->stream;
+  const double* bd;
+  const double* xd;
+  ST(stage_in(h, s, b, &h->stage_x, &bd, true));
+  ST(stage_in(h, s, x, &h->stage_z, &xd, false));
+  double* xw = const_cast<double*>(xd);
+  CK(cudaMemsetAsync(h->flags, 0, sizeof(int) * 4, s));
+  CgRun run;
+  ST(cg_enqueue_init(h, s, bd, xw, &run));
+  if (tol == 0.0) {
+    ST(cg_enqueue_iters(h, s, xw, max_iter, 0.0, &run));
+  } else {
+    // chunks of iterations; the kernels are no-ops once converged, the host
+    // polls the converged flag between chunks
+    const int chunk = 8;
+    for (int done = 0; done < max_iter; done += chunk) {
+      ST(cg_enqueue_iters(h, s, xw, std::min(chunk, max_iter - done), tol, &run));
+      int hf[4];
+      CK(cudaMemcpyAsync(hf, h->flags, sizeof(int) * 4, cudaMemcpyDeviceToHost, s));
+      CK(cudaStreamSynchronize(s));
+      if (hf[1] || hf[0]) break;
+    }
+  }
+  ST(cg_resid<false>(h, s, bd, xw));
+  SumSrc res;
+  ST(reduce_src(h, s, SumSrc{h->part_res, (int)h->vgrid}, 4, &res));
+  k_finish_norm<<<1, 32, 0, s>>>(res, h->out2 + 1);
+  LAUNCHED();
+  int hf[4];
+  double rn = 0;
+  CK(cudaMemcpyAsync(hf, h->flags, sizeof(int) * 4, cudaMemcpyDeviceToHost, s));
+  CK(cudaMemcpyAsync(&rn, h->out2 + 1, sizeof(double), cudaMemcpyDeviceToHost, s));
+  if (xd != x && h->m_loc > 0)
+    CK(cudaMemcpyAsync(x, xd, sizeof(double) * h->m_loc, cudaMemcpyDeviceToHost, s));
+  CK(cudaStreamSynchronize(s));
+  if (iters_out) *iters_out = hf[0] ? 0 : hf[2];
+  if (rnorm_out) *rnorm_out = rn;
+  if (hf[0]) { g_err = "CG breakdown: p.Ap == 0 or not finite"; return SPMV_ERR_BREAKDOWN; }
+  return SPMV_OK;
+}
+
+// The whole NAS outer iteration enqueued on stream s (used for capture).
+static spmv_status npb_enqueue(spmv_csr_s* h, cudaStream_t s, double* x, double* z, int cgitmax,
+                               double shift, double* out2) {
+  CgRun run;
+  ST(cg_enqueue_init(h, s, x, z, &run));
+  ST(cg_enqueue_iters(h, s, z, cgitmax, 0.0, &run));
+  ST(cg_resid<true>(h, s, x, z));
+  SumSrc res, xz, zz;
+  const int vg = (int)h->vgrid;
+  ST(reduce_src(h, s, SumSrc{h->part_res, vg}, 4, &res));
+  ST(reduce_src(h, s, SumSrc{h->part_xz, vg}, 5, &xz));
+  ST(reduce_src(h, s, SumSrc{h->part_zz, vg}, 6, &zz));
+  k_npb_finish<<<vg, 256, 0, s>>>(h->m_loc, res, xz, zz, z, x, shift, out2);
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+static bool use_graphs() {
+  int v = 1;
+  env_int("SPMV_GRAPH", &v);
+  return v != 0;
+}
+
+extern "C" spmv_status cg_npb_outer(spmv_csr_t h, void* x, void* z, int32_t cgitmax, double shift,
+                                    double* out2) {
+  if (!h) return arg_fail("handle is NULL");
+  if (h->dt != SPMV_F64) { g_err = "cg_npb_outer is fp64 only"; return SPMV_ERR_UNSUPPORTED; }
+  if (h->m != h->n) return arg_fail("needs a square matrix");
+  if (cgitmax < 0) return arg_fail("cgitmax >= 0");
+  if (!out2) return arg_fail("out2 is NULL");
+  if ((!x || !z) && h->m_loc > 0) return arg_fail("x and z must not be NULL");
+  CK(cudaSetDevice(h->device));
+  ST(cg_alloc(h));
+  cudaStream_t s = h->stream;
+  const double *xd, *zd;
+  ST(stage_in(h, s, x, &h->stage_x, &xd, true));
+  ST(stage_in(h, s, z, &h->stage_z, &zd, false));
+  const int ok = mem_kind(out2, h->device);
+  double* o2 = h->out2;  // the graph writes here; copied to out2 after the launch
+  double* xw = const_cast<double*>(xd);
+  double* zw = const_cast<double*>(zd);
+  if (use_graphs()) {
+    Graph& g = h->g_npb;
+    if (!g.exec || g.k0 != xw || g.k1 != zw || g.ki != cgitmax || g.kd != shift) {
+      g.reset();
+      const uint64_t before = g_launches.load();
+      CK(cudaStreamBeginCapture(h->cap, cudaStreamCaptureModeThreadLocal));
+      spmv_status st = npb_enqueue(h, h->cap, xw, zw, cgitmax, shift, o2);
+      cudaGraph_t graph = nullptr;
+      cudaError_t e = cudaStreamEndCapture(h->cap, &graph);
+      if (st != SPMV_OK) { if (graph) cudaGraphDestroy(graph); return st; }
+      if (e != cudaSuccess) return cuda_fail(e, "graph capture", __LINE__);
+      e = cudaGraphInstantiate(&g.exec, graph, 0);
+      cudaGraphDestroy(graph);
+      if (e != cudaSuccess) { g.exec = nullptr; return cuda_fail(e, "graph instantiate", __LINE__); }
+      g.nodes = g_launches.load() - before;
+      g_launches.fetch_sub(g.nodes);  // counted when replayed
+      g.k0 = xw; g.k1 = zw; g.ki = cgitmax; g.kd = shift;
+    }
+    CK(cudaGraphLaunch(g.exec, s));
+    g_launches.fetch_add(g.nodes);
+  } else {
+    ST(npb_enqueue(h, s, xw, zw, cgitmax, shift, o2));
+  }
+  bool sync = false;
+  if (ok == 1) CK(cudaMemcpyAsync(out2, o2, sizeof(double) * 2, cudaMemcpyDeviceToDevice, s));
+  if (xd != x && h->m_loc > 0) {
+    CK(cudaMemcpyAsync(x, xd, sizeof(double) * h->m_loc, cudaMemcpyDeviceToHost, s));
+    sync = true;
+  }
+  if (zd != z && h->m_loc > 0) {
+    CK(cudaMemcpyAsync(z, zd, sizeof(double) * h->m_loc, cudaMemcpyDeviceToHost, s));
+    sync = true;
+  }
+  if (ok != 1) {
+    CK(cudaMemcpyAsync(out2, o2, sizeof(double) * 2, cudaMemcpyDeviceToHost, s));
+    sync = true;
+  }
+  if (sync) {
+    int hf[4];
+    CK(cudaMemcpyAsync(hf, h->flags, sizeof(int) * 4, cudaMemcpyDeviceToHost, s));
+    CK(cudaStreamSynchronize(s));
+    if (hf[0]) { g_err = "CG breakdown"; return SPMV_ERR_BREAKDOWN; }
+  }
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_cg_status(spmv_csr_t h) {
+  if (!h) return arg_fail("handle is NULL");
+  if (!h->flags) return SPMV_OK;
+  CK(cudaSetDevice(h->device));
+  int hf[4];
+  CK(cudaMemcpyAsync(hf, h->flags, sizeof(int) * 4, cudaMemcpyDeviceToHost, h->stream));
+  CK(cudaStreamSynchronize(h->stream));
+  if (hf[0]) { g_err = "CG breakdown"; return SPMV_ERR_BREAKDOWN; }
+  return SPMV_OK;
+}
+
+// ---------------------------------------------------------- introspection
+extern "C" spmv_status spmv_csr_partition(const int32_t* rowptr, int64_t m, int32_t P,
+                                          int64_t* bounds) {
+  if (!rowptr || !bounds || m < 0 || P < 1) return arg_fail("bad partition arguments");
+  const int64_t base = rowptr[0];
+  const int64_t nnz = (int64_t)rowptr[m] - base;
+  bounds[0] = 0;
+  for (int32_t r = 1; r < P; ++r) {
+    const int64_t t = ((int64_t)r * nnz) / P;
+    int64_t lo = 0, hi = m;
+    while (lo < hi) {
+      const int64_t mid = lo + ((hi - lo) >> 1);
+      if ((int64_t)rowptr[mid] - base >= t) hi = mid; else lo = mid + 1;
+    }
+    bounds[r] = lo;
+  }
+  bounds[P] = m;
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_csr_merge_splits(const int32_t* rowptr, int64_t m, int64_t C,
+                                             int64_t* split_row, int64_t* split_nz) {
+  if (!rowptr || !split_row || !split_nz || m < 0 || C < 1) return arg_fail("bad merge-split arguments");
+  const int64_t base = rowptr[0];
+  const int64_t nnz = (int64_t)rowptr[m] - base;
+  for (int64_t c = 0; c <= C; ++c) {
+    const int64_t d = (c * (m + nnz)) / C;
+    // largest i in [max(0,d-nnz), min(d,m)] with row_end(i-1) <= d - i  (i rows consumed)
+    int64_t lo = std::max<int64_t>(0, d - nnz), hi = std::min<int64_t>(d, m);
+    while (lo < hi) {
+      const int64_t i = lo + ((hi - lo + 1) >> 1);
+      // consuming i rows needs row end i-1 (value rowptr[i]-base) <= j = d - i
+      if ((int64_t)rowptr[i] - base <= d - i) lo = i; else hi = i - 1;
+    }
+    split_row[c] = lo;
+    split_nz[c] = d - lo;
+  }
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_dist_plan_host(const int32_t* rowptr, const int32_t* colidx, int64_t m,
+                                           int32_t nranks, int32_t rank, int64_t* bounds,
+                                           int64_t* maxlen, int32_t* colidx_local) {
+  if (!rowptr || !bounds || !maxlen || nranks < 1 || rank < 0 || rank >= nranks)
+    return arg_fail("bad dist plan arguments");
+  ST(spmv_csr_partition(rowptr, m, nranks, bounds));
+  int64_t ml = 1;
+  for (int r = 0; r < nranks; ++r) ml = std::max<int64_t>(ml, bounds[r + 1] - bounds[r]);
+  *maxlen = ml;
+  if (!colidx_local) return SPMV_OK;
+  const int64_t k0 = rowptr[bounds[rank]], k1 = rowptr[bounds[rank + 1]];
+  for (int64_t k = k0; k < k1; ++k) {
+    const int64_t c = colidx[k];
+    // owner: the last rank whose block starts at or before c
+    const int64_t* it = std::upper_bound(bounds, bounds + nranks, c);
+    const int64_t s = (it - bounds) - 1;
+    colidx_local[k - k0] = (int32_t)(s * ml + (c - bounds[s]));
+  }
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_dist_colidx(spmv_csr_t h, int32_t* colidx_local_host) {
+  if (!h || !colidx_local_host) return arg_fail("NULL argument");
+  if (!h->dist) return arg_fail("not a distributed handle");
+  CK(cudaSetDevice(h->device));
+  CK(cudaMemcpy(colidx_local_host, h->ci_own, sizeof(int32_t) * (size_t)(h->k1 - h->k0),
+                cudaMemcpyDeviceToHost));
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_csr_info(spmv_csr_t h, spmv_info_t* info) {
+  if (!h || !info) return arg_fail("NULL argument");
+  memset(info, 0, sizeof *info);
+  info->kernel = h->kernel;
+  info->vec_lanes = h->lanes;
+  info->row_min = h->row_min;
+  info->row_max = h->row_max;
+  info->row_mean = h->row_mean;
+  info->row_cv = h->row_cv;
+  info->m_local = h->m_loc;
+  info->row_begin = h->row0;
+  info->row_end = h->row0 + h->m_loc;
+  info->nnz_local = h->k1 - h->k0;
+  info->rank = h->dist ? h->dist->rank : 0;
+  info->nranks = h->dist ? h->dist->nranks : 1;
+  info->sorted_cols = h->sorted;
+  info->grid = h->grid;
+  return SPMV_OK;
+}
+
+extern "C" uint64_t spmv_launch_count(void) { return g_launches.load(); }
+
+extern "C" const char* spmv_status_string(spmv_status s) {
+  switch (s) {
+    case SPMV_OK: return "SPMV_OK";
+    case SPMV_ERR_ARG: return "SPMV_ERR_ARG";
+    case SPMV_ERR_INDEX: return "SPMV_ERR_INDEX";
+    case SPMV_ERR_ALIAS: return "SPMV_ERR_ALIAS";
+    case SPMV_ERR_CUDA: return "SPMV_ERR_CUDA";
+    case SPMV_ERR_NCCL: return "SPMV_ERR_NCCL";
+    case SPMV_ERR_NOMEM: return "SPMV_ERR_NOMEM";
+    case SPMV_ERR_BREAKDOWN: return "SPMV_ERR_BREAKDOWN";
+    case SPMV_ERR_UNSUPPORTED: return "SPMV_ERR_UNSUPPORTED";
+  }
+  return "unknown spmv_status";
+}
+
+extern "C" const char* spmv_last_error_string(void) { return g_err.c_str(); }
+
+// ------------------------------------------------------------------ dist
+extern "C" spmv_status spmv_dist_get_unique_id(void* id128) {
+  if (!id128) return arg_fail("id128 is NULL");
+  static_assert(sizeof(ncclUniqueId) == 128, "ncclUniqueId is 128 bytes");
+  NK(ncclGetUniqueId((ncclUniqueId*)id128));
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_dist_init(spmv_dist_t* out, int32_t rank, int32_t nranks,
+                                      const void* id128, int32_t device) {
+  if (!out || !id128 || nranks < 1 || rank < 0 || rank >= nranks) return arg_fail("bad dist arguments");
+  *out = nullptr;
+  CK(cudaSetDevice(device));
+  spmv_dist_s* d = new spmv_dist_s();
+  d->rank = rank;
+  d->nranks = nranks;
+  d->device = device;
+  ncclUniqueId id;
+  memcpy(&id, id128, sizeof id);
+  ncclResult_t r = ncclCommInitRank(&d->comm, nranks, id, rank);
+  if (r != ncclSuccess) {
+    g_err = std::string("ncclCommInitRank: ") + ncclGetErrorString(r);
+    delete d;
+    return SPMV_ERR_NCCL;
+  }
+  *out = d;
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_dist_destroy(spmv_dist_t d) {
+  if (!d) return SPMV_OK;
+  spmv_status st = SPMV_OK;
+  if (d->comm) {
+    ncclResult_t r = ncclCommDestroy(d->comm);
+    if (r != ncclSuccess) { g_err = ncclGetErrorString(r); st = SPMV_ERR_NCCL; }
+  }
+  delete d;
+  return st;
+}

@@ -1,0 +1,238 @@
+"""GPU parity of spmv_csr against the CPU oracle (element by element, per-row
+tolerance of BJ.ns: 1e-12 (fp64) / 1e-5 (fp32) of sum_k |a_ik x_k|), through
+the C ABI.  Covers every kernel variant, the adversarial zoo of SURVEY 4.3,
+the alpha/beta conventions, the error paths, and the full-size NAS B/C and
+Parboil-shaped matrices of BASELINE.json."""
+import numpy as np
+import pytest
+
+import gen
+import oracle
+from gpu_util import check_rows, to_dev
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def torch_dev():
+    import torch
+    return torch, torch.device("cuda:0")
+
+
+@pytest.fixture(scope="module")
+def sp():
+    import paper_conf_asplos_ginsbachrsbdo18_b200 as sp
+    return sp
+
+
+def run_case(sp, torch, dev, A, x_h, *, alpha=1.0, beta=0.0, y0=None, kernel="auto", lanes=0,
+             validate=True, what=""):
+    f32 = A.vals.dtype == np.float32
+    tdt = torch.float32 if f32 else torch.float64
+    rp, ci, va = to_dev(A, dev)
+    x = torch.from_numpy(np.ascontiguousarray(x_h)).to(dev)
+    y_old = y0 if y0 is not None else np.full(A.m, np.nan, dtype=A.vals.dtype)
+    y = torch.from_numpy(y_old.copy()).to(dev)
+    with sp.CSRMatrix(rp, ci, va, A.n, kernel=kernel, vec_lanes=lanes, validate=validate) as M:
+        M.spmv(x, y, alpha, beta)
+        torch.cuda.synchronize()
+        info = M.info()
+    y_ref, bound = oracle.spmv(A.rowptr, A.colidx, A.vals, x_h, y_old, alpha, beta)
+    check_rows(y.cpu().numpy(), y_ref, bound, A.vals.dtype, what)
+    return info
+
+
+def zoo():
+    """(name, CSR) adversarial cases; the paper's silent corners."""
+    r = np.random.default_rng(42)
+    cases = []
+    cases.append(("m0", gen.CSR(0, 5, np.zeros(1, np.int32), np.zeros(0, np.int32), np.zeros(0))))
+    cases.append(("nnz0", gen.CSR(7, 3, np.zeros(8, np.int32), np.zeros(0, np.int32), np.zeros(0))))
+    cases.append(("n1", gen.from_dense(r.standard_normal((9, 1)))))
+    rp = np.array([0, 0, 0, 3, 3, 5, 5, 5, 5], np.int32)
+    cases.append(("trailing_empty", gen.CSR(8, 4, rp, r.integers(0, 4, 5).astype(np.int32), r.standard_normal(5))))
+    L = r.integers(0, 6, 3000)
+    L[1234] = 100000
+    rp = np.concatenate([[0], np.cumsum(L)]).astype(np.int32)
+    nnz = int(rp[-1])
+    cases.append(("one_long_row", gen.CSR(3000, 5000, rp, r.integers(0, 5000, nnz).astype(np.int32), r.standard_normal(nnz))))
+    rows = r.integers(0, 50, 2000)
+    cases.append(("dups_unsorted", gen.from_coo(50, 20, rows, r.integers(0, 20, 2000), r.standard_normal(2000))))
+    A = gen.powerlaw(m=20000, lmax=3000.0, beta=0.6, seed=5, f32=False)
+    cases.append(("powerlaw_small", A))
+    cases.append(("laplace1d", gen.laplace1d(100001)))
+    cases.append(("stencil27_9", gen.stencil27(9)))
+    cases.append(("makea_S", gen.makea("S")))
+    return cases
+
+
+ZOO = zoo()
+
+
+@pytest.mark.parametrize("lanes", [0, 1, 2, 4, 8, 16, 32])
+@pytest.mark.parametrize("name,A", ZOO, ids=[c[0] for c in ZOO])
+def test_zoo_fp64(sp, torch_dev, name, A, lanes):
+    torch, dev = torch_dev
+    x = gen.uniform(A.n, seed=11)
+    run_case(sp, torch, dev, A, x, lanes=lanes, what=f"{name} lanes={lanes}")
+
+
+@pytest.mark.parametrize("name,A", ZOO, ids=[c[0] for c in ZOO])
+def test_zoo_fp32(sp, torch_dev, name, A):
+    torch, dev = torch_dev
+    A32 = A.astype(np.float32)
+    x = gen.uniform(A.n, seed=12, f32=True)
+    run_case(sp, torch, dev, A32, x, what=f"{name} fp32")
+
+
+@pytest.mark.parametrize("unroll", ["2", "4", "8"])
+def test_unroll_variants(sp, torch_dev, unroll, monkeypatch):
+    torch, dev = torch_dev
+    monkeypatch.setenv("SPMV_UNROLL", unroll)
+    A = gen.makea("W")
+    for lanes in (4, 32):
+        run_case(sp, torch, dev, A, gen.uniform(A.n, seed=3), lanes=lanes, what=f"unroll {unroll}")
+
+
+@pytest.mark.parametrize("alpha,beta", [(1.0, 0.0), (2.5, 0.0), (1.0, 1.0), (-0.5, 3.0), (0.0, 2.0),
+                                        (0.0, 0.0)])
+@pytest.mark.parametrize("f32", [False, True])
+def test_alpha_beta(sp, torch_dev, alpha, beta, f32):
+    torch, dev = torch_dev
+    A = gen.makea("S")
+    if f32:
+        A = A.astype(np.float32)
+    x = gen.uniform(A.n, seed=4, f32=f32)
+    if alpha == 0.0:
+        x = np.full(A.n, np.nan, dtype=x.dtype)  # A and x must not be read
+    y0 = gen.uniform(A.m, seed=5, f32=f32)
+    if beta == 0.0:
+        y0 = np.full(A.m, np.nan, dtype=y0.dtype)  # y must not be read
+    run_case(sp, torch, dev, A, x, alpha=alpha, beta=beta, y0=y0, what=f"a={alpha} b={beta}")
+
+
+def test_rowptr_offset_and_misaligned_views(sp, torch_dev):
+    """rowptr[0] != 0 (R2) and base pointers misaligned to 16 B (views at offset 1)."""
+    torch, dev = torch_dev
+    A = gen.makea("S")
+    off = 3
+    rp = torch.from_numpy(A.rowptr + off).to(dev)
+    ci_full = torch.from_numpy(np.concatenate([np.full(off, 0, np.int32), A.colidx])).to(dev)
+    va_full = torch.from_numpy(np.concatenate([np.full(off, np.nan), A.vals])).to(dev)
+    # misalign: shift the whole structure by one element inside a bigger buffer
+    ci_buf = torch.zeros(ci_full.numel() + 1, dtype=torch.int32, device=dev)
+    va_buf = torch.zeros(va_full.numel() + 1, dtype=torch.float64, device=dev)
+    ci_buf[1:] = ci_full
+    va_buf[1:] = va_full
+    ci, va = ci_buf[1:], va_buf[1:]
+    x_h = gen.uniform(A.n, seed=8)
+    xb = torch.zeros(A.n + 1, dtype=torch.float64, device=dev)
+    xb[1:] = torch.from_numpy(x_h).to(dev)
+    x = xb[1:]
+    y = torch.full((A.m,), float("nan"), dtype=torch.float64, device=dev)
+    with sp.CSRMatrix(rp, ci, va, A.n, validate=True) as M:
+        M.spmv(x, y)
+        torch.cuda.synchronize()
+    y_ref, bound = oracle.spmv(A.rowptr, A.colidx, A.vals, x_h)
+    check_rows(y.cpu().numpy(), y_ref, bound, np.float64, "offset/misaligned")
+
+
+def test_vals_may_change_per_call(sp, torch_dev):
+    torch, dev = torch_dev
+    A = gen.makea("S")
+    rp, ci, va = to_dev(A, dev)
+    v2_h = gen.uniform(A.nnz, seed=21)
+    v2 = torch.from_numpy(v2_h).to(dev)
+    x_h = gen.uniform(A.n, seed=22)
+    x = torch.from_numpy(x_h).to(dev)
+    y = torch.empty(A.m, dtype=torch.float64, device=dev)
+    with sp.CSRMatrix(rp, ci, va, A.n) as M:
+        M.spmv(x, y, vals=v2)
+        torch.cuda.synchronize()
+    y_ref, bound = oracle.spmv(A.rowptr, A.colidx, v2_h, x_h)
+    check_rows(y.cpu().numpy(), y_ref, bound, np.float64, "vals per call")
+
+
+def test_errors(sp, torch_dev):
+    torch, dev = torch_dev
+    A = gen.makea("S")
+    rp, ci, va = to_dev(A, dev)
+    x = torch.zeros(A.n, dtype=torch.float64, device=dev)
+    y = torch.zeros(A.m, dtype=torch.float64, device=dev)
+    M = sp.CSRMatrix(rp, ci, va, A.n)
+    # aliasing: y == x (R13)
+    with pytest.raises(sp.SpmvError) as e:
+        M.spmv(y[: A.n], y)
+    assert e.value.status == sp.SPMV_ERR_ALIAS
+    with pytest.raises(sp.SpmvError) as e:
+        M.spmv(x, va[: A.m])
+    assert e.value.status == sp.SPMV_ERR_ALIAS
+    # host pointer where a device pointer is needed
+    xh = torch.zeros(A.n, dtype=torch.float64)
+    with pytest.raises(sp.SpmvError) as e:
+        M.spmv(xh, y)
+    assert e.value.status == sp.SPMV_ERR_ARG
+    # structure binding mismatch
+    import ctypes
+    st = sp.spmv_csr_c(M.handle, A.m + 1, A.n, A.nnz, rp.data_ptr(), ci.data_ptr(), va.data_ptr(),
+                       x.data_ptr(), y.data_ptr(), 1.0, 0.0)
+    assert st == sp.SPMV_ERR_ARG
+    M.destroy()
+    # nnz mismatch at create (R1)
+    h = ctypes.c_void_p()
+    st = sp.spmv_csr_create_c(ctypes.byref(h), 0, A.m, A.n, A.nnz + 1, rp.data_ptr(), ci.data_ptr(),
+                              va.data_ptr(), None)
+    assert st == sp.SPMV_ERR_ARG
+    # validate: column out of range, decreasing rowptr
+    bad = ci.clone()
+    bad[5] = A.n
+    with pytest.raises(sp.SpmvError) as e:
+        sp.CSRMatrix(rp, bad, va, A.n, validate=True)
+    assert e.value.status == sp.SPMV_ERR_INDEX
+    rp2 = rp.clone()
+    rp2[10] = rp2[12] + 1
+    rp2[11] = rp2[12] + 1  # keeps rowptr[m] - rowptr[0] == nnz
+    with pytest.raises(sp.SpmvError) as e:
+        sp.CSRMatrix(rp2, ci, va, A.n, validate=True)
+    assert e.value.status == sp.SPMV_ERR_INDEX
+
+
+def test_launch_count_increases(sp, torch_dev):
+    torch, dev = torch_dev
+    A = gen.makea("S")
+    rp, ci, va = to_dev(A, dev)
+    x = torch.ones(A.n, dtype=torch.float64, device=dev)
+    y = torch.empty(A.m, dtype=torch.float64, device=dev)
+    with sp.CSRMatrix(rp, ci, va, A.n) as M:
+        c0 = sp.launch_count()
+        for _ in range(5):
+            M.spmv(x, y)
+        assert sp.launch_count() - c0 == 5
+
+
+@pytest.mark.parametrize("cls", ["B", "C"])
+def test_nas_full_size(sp, torch_dev, cls):
+    """BJ.cfg[1], BJ.cfg[3]: every row of the full-size matrix, in the launch
+    configuration bench.py times (auto kernel)."""
+    torch, dev = torch_dev
+    A = gen.makea(cls)
+    x = gen.uniform(A.n, seed=31)
+    info = run_case(sp, torch, dev, A, x, what=f"NAS {cls}")
+    assert info["kernel_name"] in ("vector", "merge", "xstat", "scalar")
+
+
+def test_parboil_full_size_fp32(sp, torch_dev):
+    """BJ.cfg[2]: 1M rows, power-law row lengths, fp32."""
+    torch, dev = torch_dev
+    A = gen.powerlaw()
+    x = gen.uniform(A.n, seed=41, f32=True)
+    run_case(sp, torch, dev, A, x, what="parboil fp32")
+    # sanity of the tolerance: the plain fp32 sequential loop also passes
+    rp, ci, v = A.rowptr, A.colidx, A.vals
+    rows = np.arange(0, A.m, 997)
+    y_ref, bound = oracle.spmv(rp, ci, v, x)
+    for i in rows:
+        s = np.float32(0)
+        for k in range(rp[i], rp[i + 1]):
+            s = np.float32(s + np.float32(v[k] * x[ci[k]]))
+        assert abs(float(s) - y_ref[i]) <= 1e-5 * bound[i]
