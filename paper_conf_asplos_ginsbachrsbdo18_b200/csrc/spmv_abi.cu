@@ -19,6 +19,7 @@
 #include "analysis_kernels.cuh"
 #include "cg_kernels.cuh"
 #include "spmv_kernels.cuh"
+#include "xstat_kernel.cuh"
 
 using namespace spmv;
 
@@ -103,6 +104,14 @@ struct spmv_csr_s {
   int64_t row_min = 0, row_max = 0;
   double row_mean = 0, row_cv = 0;
   int32_t sorted = 0;
+  // XSTAT (x-stationary cluster kernel)
+  int xB = 0, xW = 0, xR = 1024, xG = 8, nclusters = 0;
+  size_t xsmem = 0;
+  int64_t nx = 0;                     // length of the x the kernels read
+  int* seg = nullptr;
+  long long* crow = nullptr;
+  void (*xk)(XstatArgs) = nullptr;
+  void (*xk_dot)(XstatArgs) = nullptr;
   // dist
   spmv_dist_s* dist = nullptr;
   std::vector<long long> bounds;
@@ -183,6 +192,118 @@ static void launch_vec(int lanes, int unroll, int64_t grid, cudaStream_t s, cons
   }
 }
 
+template <typename T, bool DOT>
+static void (*xstat_fn(int G))(XstatArgs) {
+  switch (G) {
+    case 4: return k_spmv_xstat<T, 4, 4, DOT>;
+    case 16: return k_spmv_xstat<T, 16, 4, DOT>;
+    case 32: return k_spmv_xstat<T, 32, 4, DOT>;
+    default: return k_spmv_xstat<T, 8, 4, DOT>;
+  }
+}
+
+static spmv_status launch_xstat(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
+                                double alpha, double beta, const double* w, double* part) {
+  XstatArgs a;
+  a.m = h->m_loc;
+  a.nx = h->nx;
+  a.W = h->xW;
+  a.R = h->xR;
+  a.rowptr = h->rp_loc;
+  a.colidx = h->ci_loc;
+  a.vals = vals;
+  a.seg = h->seg;
+  a.crow = h->crow;
+  a.x = x;
+  a.y = y;
+  a.alpha = alpha;
+  a.beta = beta;
+  a.w = w;
+  a.part = part;
+  if (h->dt == SPMV_F32) {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+  }
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = dim3((unsigned)(h->nclusters * h->xB), 1, 1);
+  cfg.blockDim = dim3(1024, 1, 1);
+  cfg.dynamicSmemBytes = h->xsmem;
+  cfg.stream = s;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeClusterDimension;
+  at[0].val.clusterDim.x = (unsigned)h->xB;
+  at[0].val.clusterDim.y = 1;
+  at[0].val.clusterDim.z = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  CK(cudaLaunchKernelEx(&cfg, part ? h->xk_dot : h->xk, a));
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+// XSTAT set-up (create): column-block width, cluster size, split points,
+// static nnz-balanced cluster row ranges.  Returns false if not eligible.
+static spmv_status xstat_setup(spmv_csr_s* h, bool* ok) {
+  *ok = false;
+  if (!h->sorted || h->m_loc == 0 || h->nx == 0) return SPMV_OK;
+  const size_t budget = 200 * 1024;  // of the 227 KB a CTA may use
+  const size_t pb = 3 * (size_t)h->xR * sizeof(double) + 16;
+  if (budget <= pb) return SPMV_OK;
+  int B = (int)cdiv((int64_t)h->ts * h->nx, (int64_t)(budget - pb));
+  if (B < 1) B = 1;
+  int forced = 0;
+  if (env_int("SPMV_XSTAT_B", &forced) && forced >= B && forced <= 8) B = forced;
+  if (B > 8) return SPMV_OK;
+  int W = (int)cdiv(h->nx, B);
+  W = (W + 3) & ~3;
+  const size_t xbytes = ((size_t)W * h->ts + 15) & ~size_t(15);
+  const size_t smem = xbytes + 3 * (size_t)h->xR * sizeof(double);
+  const double seg_mean = h->row_mean / B;
+  int G = seg_mean < 12 ? 4 : seg_mean < 24 ? 8 : seg_mean < 48 ? 16 : 32;
+  int g2 = 0;
+  if (env_int("SPMV_XSTAT_G", &g2) && (g2 == 4 || g2 == 8 || g2 == 16 || g2 == 32)) G = g2;
+  void (*fn)(XstatArgs) = h->dt == SPMV_F64 ? xstat_fn<double, false>(G) : xstat_fn<float, false>(G);
+  void (*fnd)(XstatArgs) = h->dt == SPMV_F64 ? xstat_fn<double, true>(G) : nullptr;
+  CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+  if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = dim3((unsigned)B, 1, 1);
+  cfg.blockDim = dim3(1024, 1, 1);
+  cfg.dynamicSmemBytes = smem;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeClusterDimension;
+  at[0].val.clusterDim.x = (unsigned)B;
+  at[0].val.clusterDim.y = 1;
+  at[0].val.clusterDim.z = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  int ncl = 0;
+  cudaError_t e = cudaOccupancyMaxActiveClusters(&ncl, fn, &cfg);
+  if (e != cudaSuccess || ncl < 1) { cudaGetLastError(); return SPMV_OK; }
+  int nc_env = 0;
+  if (env_int("SPMV_XSTAT_CLUSTERS", &nc_env) && nc_env >= 1 && nc_env <= ncl) ncl = nc_env;
+  cudaStream_t s = h->stream;
+  if (B > 1) {
+    CK(cudaMalloc(&h->seg, sizeof(int) * (size_t)(B - 1) * (size_t)h->m_loc));
+    k_xstat_splits<<<std::min<int64_t>(cdiv(h->m_loc, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
+        h->m_loc, h->rp_loc, h->ci_loc, B, W, h->seg);
+    LAUNCHED();
+  }
+  CK(cudaMalloc(&h->crow, sizeof(long long) * (ncl + 1)));
+  k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(h->m_loc, h->rp_loc, ncl, h->crow);
+  LAUNCHED();
+  CK(cudaStreamSynchronize(s));
+  h->xB = B;
+  h->xW = W;
+  h->xG = G;
+  h->xsmem = smem;
+  h->nclusters = ncl;
+  h->xk = fn;
+  h->xk_dot = fnd;
+  *ok = true;
+  return SPMV_OK;
+}
+
 // Local SpMV of the handle: y = alpha*A_loc*x + beta*y (+ partial w.y per CTA).
 static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
                             double alpha, double beta, const double* w, double* part) {
@@ -199,6 +320,7 @@ static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, con
     LAUNCHED();
     return SPMV_OK;
   }
+  if (h->kernel == SPMV_KERNEL_XSTAT) return launch_xstat(h, s, vals, x, y, alpha, beta, w, part);
   SpmvArgs a;
   a.m = h->m_loc;
   a.rowptr = h->rp_loc;
@@ -321,20 +443,22 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
     double* dpart = nullptr;
     if (cudaMalloc(&dpart, sizeof(double) * 5 * g) != cudaSuccess)
       return fail(cuda_fail(cudaErrorMemoryAllocation, "cudaMalloc", __LINE__));
-    k_row_stats<<<g, 256, 0, s>>>(m, rowptr, colidx, 0, dpart);
+    k_row_stats<<<g, 256, 0, s>>>(m, rowptr, colidx, nnz > 0 ? 1 : 0, dpart);
     g_launches.fetch_add(1);
     std::vector<double> hp(5 * g);
     cudaError_t e = cudaMemcpyAsync(hp.data(), dpart, sizeof(double) * 5 * g, cudaMemcpyDeviceToHost, s);
     if (e == cudaSuccess) e = cudaStreamSynchronize(s);
     cudaFree(dpart);
     if (e != cudaSuccess) return fail(cuda_fail(e, "row stats", __LINE__));
-    double mn = 1e300, mx = -1e300, sum = 0, sq = 0;
+    double mn = 1e300, mx = -1e300, sum = 0, sq = 0, uns = 0;
     for (int64_t b = 0; b < g; ++b) {
+      uns += hp[5 * b + 4];
       mn = std::min(mn, hp[5 * b]);
       mx = std::max(mx, hp[5 * b + 1]);
       sum += hp[5 * b + 2];
       sq += hp[5 * b + 3];
     }
+    h->sorted = (uns == 0.0) ? 1 : 0;
     h->row_min = (int64_t)mn;
     h->row_max = (int64_t)mx;
     h->row_mean = sum / (double)m;
@@ -397,7 +521,19 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
   int rk = 0, rl = 0;
   if (!env_int("SPMV_KERNEL", &rk)) rk = o.kernel;
   if (!env_int("SPMV_LANES", &rl)) rl = o.vec_lanes;
+  h->nx = o.dist ? (int64_t)h->maxlen * o.dist->nranks : n;
   choose_kernel(h, rk, rl);
+  if (rk == SPMV_KERNEL_XSTAT || rk == SPMV_KERNEL_AUTO) {
+    bool ok = false;
+    spmv_status st = xstat_setup(h, &ok);
+    if (st != SPMV_OK) return fail(st);
+    // auto: x-stationary whenever x fits a cluster's shared memory and rows are
+    // long enough for the split to pay
+    if (ok && (rk == SPMV_KERNEL_XSTAT || h->row_mean >= 16.0)) {
+      h->kernel = SPMV_KERNEL_XSTAT;
+      h->grid = (int64_t)h->nclusters * h->xB;
+    }
+  }
   CK(cudaStreamCreateWithFlags(&h->cap, cudaStreamNonBlocking));
   CK(cudaEventCreateWithFlags(&h->ev_a, cudaEventDisableTiming));
   CK(cudaEventCreateWithFlags(&h->ev_b, cudaEventDisableTiming));
@@ -412,7 +548,7 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   cudaError_t e = h->stream ? cudaStreamSynchronize(h->stream) : cudaDeviceSynchronize();
   if (e != cudaSuccess) st = cuda_fail(e, "pending asynchronous error", __LINE__);
   h->g_npb.reset();
-  void* bufs[] = {h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
+  void* bufs[] = {h->seg, h->crow, h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
                   h->stage_x, h->stage_z};
   for (void* b : bufs)
@@ -472,7 +608,7 @@ static spmv_status cg_alloc(spmv_csr_s* h) {
   ST(ensure_buf((void**)&h->q, nb));
   if (!h->dist) ST(ensure_buf((void**)&h->p_single, nb));
   ST(ensure_buf((void**)&h->part_pq, pb));
-  ST(ensure_buf((void**)&h->part_rr, 2 * pb));
+  ST(ensure_buf((void**)&h->part_rr, 3 * pb));  // [0],[1]: parity slots; [2]: ||b||^2 (init)
   ST(ensure_buf((void**)&h->part_res, pb));
   ST(ensure_buf((void**)&h->part_xz, pb));
   ST(ensure_buf((void**)&h->part_zz, pb));
@@ -517,9 +653,10 @@ struct CgRun {
 static spmv_status cg_enqueue_init(spmv_csr_s* h, cudaStream_t s, const double* b, double* z,
                                    CgRun* run) {
   const int vg = (int)h->vgrid;
-  k_cg_init<<<vg, 256, 0, s>>>(h->m_loc, b, z, h->r, cg_p(h), h->part_rr);
+  double* prb = h->part_rr + 2 * std::max(h->grid, h->vgrid);
+  k_cg_init<<<vg, 256, 0, s>>>(h->m_loc, b, z, h->r, cg_p(h), prb);
   LAUNCHED();
-  ST(reduce_src(h, s, SumSrc{h->part_rr, vg}, 0, &run->rr_b));
+  ST(reduce_src(h, s, SumSrc{prb, vg}, 0, &run->rr_b));
   run->rr_old = run->rr_b;
   run->it = 0;
   return SPMV_OK;

@@ -33,6 +33,8 @@ def run_case(sp, torch, dev, A, x_h, *, alpha=1.0, beta=0.0, y0=None, kernel="au
     x = torch.from_numpy(np.ascontiguousarray(x_h)).to(dev)
     y_old = y0 if y0 is not None else np.full(A.m, np.nan, dtype=A.vals.dtype)
     y = torch.from_numpy(y_old.copy()).to(dev)
+    if lanes and kernel == "auto":
+        kernel = "vector"
     with sp.CSRMatrix(rp, ci, va, A.n, kernel=kernel, vec_lanes=lanes, validate=validate) as M:
         M.spmv(x, y, alpha, beta)
         torch.cuda.synchronize()
@@ -236,3 +238,32 @@ def test_parboil_full_size_fp32(sp, torch_dev):
         for k in range(rp[i], rp[i + 1]):
             s = np.float32(s + np.float32(v[k] * x[ci[k]]))
         assert abs(float(s) - y_ref[i]) <= 1e-5 * bound[i]
+
+
+@pytest.mark.parametrize("cfg", [{}, {"SPMV_XSTAT_B": "2"}, {"SPMV_XSTAT_B": "8"},
+                                 {"SPMV_XSTAT_G": "4"}, {"SPMV_XSTAT_G": "32", "SPMV_XSTAT_B": "3"},
+                                 {"SPMV_XSTAT_CLUSTERS": "1"}])
+@pytest.mark.parametrize("name,A", ZOO, ids=[c[0] for c in ZOO])
+def test_zoo_xstat(sp, torch_dev, name, A, cfg, monkeypatch):
+    """x-stationary cluster kernel (thread-block clusters + DSMEM reduction):
+    every zoo case with sorted columns, several cluster sizes / lane groups /
+    cluster counts (1 cluster = many row tiles, exercises the triple buffer)."""
+    torch, dev = torch_dev
+    for k, v in cfg.items():
+        monkeypatch.setenv(k, v)
+    x = gen.uniform(A.n, seed=13)
+    info = run_case(sp, torch, dev, A, x, kernel="xstat", what=f"{name} xstat {cfg}")
+    if name not in ("dups_unsorted", "m0", "nnz0"):
+        assert info["kernel_name"] == "xstat", info
+    A32 = A.astype(np.float32)
+    run_case(sp, torch, dev, A32, gen.uniform(A.n, seed=14, f32=True), kernel="xstat",
+             what=f"{name} xstat fp32 {cfg}")
+
+
+def test_xstat_alpha_beta_and_offset(sp, torch_dev):
+    torch, dev = torch_dev
+    A = gen.makea("W")
+    x = gen.uniform(A.n, seed=15)
+    y0 = gen.uniform(A.m, seed=16)
+    for a, b in [(2.0, -1.0), (0.0, 3.0), (1.0, 0.0)]:
+        run_case(sp, torch, dev, A, x, alpha=a, beta=b, y0=y0, kernel="xstat", what=f"xstat a={a} b={b}")

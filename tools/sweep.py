@@ -1,0 +1,79 @@
+#!/usr/bin/env python3
+"""Kernel-selection sweep (the paper's "try every API, keep the fastest",
+P:275-280): times every SpMV kernel variant alone on the BASELINE configs
+(CUDA events, L2 flushed before each launch) and prints one JSON line per
+variant with GB/s against the algorithmic bytes.  GPU only."""
+import json
+import os
+import statistics
+import sys
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+
+import numpy as np
+import torch
+
+import gen
+import paper_conf_asplos_ginsbachrsbdo18_b200 as sp
+
+VARIANTS = [("auto", {}, {})] + [(f"vector{g}", {"kernel": "vector", "vec_lanes": g}, {}) for g in (4, 8, 16, 32)] + \
+    [(f"vector32_u{u}", {"kernel": "vector", "vec_lanes": 32}, {"SPMV_UNROLL": str(u)}) for u in (2, 8)] + \
+    [(f"xstat_B{b}_G{g}", {"kernel": "xstat"}, {"SPMV_XSTAT_B": str(b), "SPMV_XSTAT_G": str(g)})
+     for b in (2, 4, 8) for g in (4, 8, 16, 32)]
+
+
+def time_variant(A, x, y, kw, env, reps=20):
+    for k, v in env.items():
+        os.environ[k] = v
+    try:
+        M = sp.CSRMatrix(*A, **kw)
+    finally:
+        for k in env:
+            os.environ.pop(k, None)
+    info = M.info()
+    flush = torch.empty(256 << 20, dtype=torch.int8, device="cuda")
+    for _ in range(3):
+        M.spmv(x, y)
+    ts = []
+    for _ in range(reps):
+        flush.zero_()
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record()
+        M.spmv(x, y)
+        b.record()
+        b.synchronize()
+        ts.append(a.elapsed_time(b))
+    M.destroy()
+    return statistics.median(ts), info
+
+
+def main():
+    which = sys.argv[1:] or ["B", "C", "parboil"]
+    dev = torch.device("cuda:0")
+    for w in which:
+        if w == "parboil":
+            C = gen.powerlaw()
+        elif w.startswith("stencil"):
+            C = gen.stencil27(int(w[7:]))
+        else:
+            C = gen.makea(w)
+        rp = torch.from_numpy(C.rowptr).to(dev)
+        ci = torch.from_numpy(C.colidx).to(dev)
+        va = torch.from_numpy(C.vals).to(dev)
+        x = torch.from_numpy(gen.uniform(C.n, seed=1, f32=C.vals.dtype == np.float32)).to(dev)
+        y = torch.empty(C.m, dtype=va.dtype, device=dev)
+        nbytes = C.bytes_per_spmv()
+        for name, kw, env in VARIANTS:
+            try:
+                ms, info = time_variant((rp, ci, va, C.n), x, y, kw, env)
+            except Exception as e:  # noqa
+                print(json.dumps({"matrix": w, "variant": name, "error": str(e)[:200]}), flush=True)
+                continue
+            print(json.dumps({"matrix": w, "variant": name, "kernel": info["kernel_name"],
+                              "lanes": info["vec_lanes"], "us": round(ms * 1e3, 2),
+                              "gbs": round(nbytes / (ms / 1e3) / 1e9, 1),
+                              "gflops": round(2 * C.nnz / (ms / 1e3) / 1e9, 1)}), flush=True)
+
+
+if __name__ == "__main__":
+    main()
