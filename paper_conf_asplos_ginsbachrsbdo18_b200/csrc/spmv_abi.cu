@@ -192,14 +192,18 @@ static void launch_vec(int lanes, int unroll, int64_t grid, cudaStream_t s, cons
   }
 }
 
-template <typename T, bool DOT>
-static void (*xstat_fn(int G))(XstatArgs) {
+template <typename T, bool DOT, int U>
+static void (*xstat_fn_u(int G))(XstatArgs) {
   switch (G) {
-    case 4: return k_spmv_xstat<T, 4, 4, DOT>;
-    case 16: return k_spmv_xstat<T, 16, 4, DOT>;
-    case 32: return k_spmv_xstat<T, 32, 4, DOT>;
-    default: return k_spmv_xstat<T, 8, 4, DOT>;
+    case 4: return k_spmv_xstat<T, 4, U, DOT>;
+    case 16: return k_spmv_xstat<T, 16, U, DOT>;
+    case 32: return k_spmv_xstat<T, 32, U, DOT>;
+    default: return k_spmv_xstat<T, 8, U, DOT>;
   }
+}
+template <typename T, bool DOT>
+static void (*xstat_fn(int G, int U))(XstatArgs) {
+  return U == 8 ? xstat_fn_u<T, DOT, 8>(G) : xstat_fn_u<T, DOT, 4>(G);
 }
 
 static spmv_status launch_xstat(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
@@ -247,23 +251,28 @@ static spmv_status xstat_setup(spmv_csr_s* h, bool* ok) {
   *ok = false;
   if (!h->sorted || h->m_loc == 0 || h->nx == 0) return SPMV_OK;
   const size_t budget = 200 * 1024;  // of the 227 KB a CTA may use
-  const size_t pb = 3 * (size_t)h->xR * sizeof(double) + 16;
+  const size_t pb = 3 * (size_t)h->xR * sizeof(double) + 4 * (size_t)h->xR * sizeof(int) + 16;
   if (budget <= pb) return SPMV_OK;
   int B = (int)cdiv((int64_t)h->ts * h->nx, (int64_t)(budget - pb));
   if (B < 1) B = 1;
+  // cluster sizes that tile the GPCs well: 1, 2, 4, 8
+  B = B <= 1 ? 1 : B <= 2 ? 2 : B <= 4 ? 4 : B <= 8 ? 8 : B;
   int forced = 0;
   if (env_int("SPMV_XSTAT_B", &forced) && forced >= B && forced <= 8) B = forced;
   if (B > 8) return SPMV_OK;
   int W = (int)cdiv(h->nx, B);
   W = (W + 3) & ~3;
   const size_t xbytes = ((size_t)W * h->ts + 15) & ~size_t(15);
-  const size_t smem = xbytes + 3 * (size_t)h->xR * sizeof(double);
+  const size_t smem = xbytes + 3 * (size_t)h->xR * sizeof(double) + 4 * (size_t)h->xR * sizeof(int);
   const double seg_mean = h->row_mean / B;
-  int G = seg_mean < 12 ? 4 : seg_mean < 24 ? 8 : seg_mean < 48 ? 16 : 32;
+  // lanes x unroll ~ the mean segment length, unroll 8 for memory-level parallelism
+  int G = seg_mean < 48 ? 4 : seg_mean < 96 ? 8 : seg_mean < 192 ? 16 : 32;
+  int U = 8;
   int g2 = 0;
   if (env_int("SPMV_XSTAT_G", &g2) && (g2 == 4 || g2 == 8 || g2 == 16 || g2 == 32)) G = g2;
-  void (*fn)(XstatArgs) = h->dt == SPMV_F64 ? xstat_fn<double, false>(G) : xstat_fn<float, false>(G);
-  void (*fnd)(XstatArgs) = h->dt == SPMV_F64 ? xstat_fn<double, true>(G) : nullptr;
+  if (env_int("SPMV_XSTAT_U", &g2) && (g2 == 4 || g2 == 8)) U = g2;
+  void (*fn)(XstatArgs) = h->dt == SPMV_F64 ? xstat_fn<double, false>(G, U) : xstat_fn<float, false>(G, U);
+  void (*fnd)(XstatArgs) = h->dt == SPMV_F64 ? xstat_fn<double, true>(G, U) : nullptr;
   CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
   if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
   cudaLaunchConfig_t cfg = {};

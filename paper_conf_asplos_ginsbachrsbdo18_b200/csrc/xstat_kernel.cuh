@@ -89,7 +89,8 @@ __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
   }
 }
 
-// Dynamic shared memory: [xs: W*sizeof(T), 16-B aligned][pbuf: 3*R doubles][mbarrier]
+// Dynamic shared memory: [xs: W*sizeof(T), 16-B aligned][pbuf: 3*R doubles]
+//                        [bnd: 2 x 2 x R ints (double-buffered segment bounds)]
 template <typename T, int G, int U, bool DOT>
 __global__ void __launch_bounds__(1024, 1)
 k_spmv_xstat(XstatArgs a) {
@@ -100,16 +101,17 @@ k_spmv_xstat(XstatArgs a) {
   const int B = (int)cluster.num_blocks();
   const int b = (int)cluster_rank();
   const int c = (int)cluster_id();
+  const int R = a.R;
 
   T* xs = reinterpret_cast<T*>(smem);
   double* pbuf = reinterpret_cast<double*>(smem + ((size_t(a.W) * sizeof(T) + 15) & ~size_t(15)));
+  int* bnd = reinterpret_cast<int*>(pbuf + 3 * R);  // [2][2][R]
   const T* __restrict__ vals = static_cast<const T*>(a.vals);
   const T* __restrict__ xg = static_cast<const T*>(a.x);
   const int* __restrict__ colidx = a.colidx;
   const int* __restrict__ rowptr = a.rowptr;
   const int* __restrict__ seg = a.seg;
   const int64_t m = a.m;
-  const int R = a.R;
 
   // ---- x column block b -> shared memory (one TMA bulk copy + scalar tail)
   const int64_t col0 = int64_t(b) * a.W;
@@ -140,17 +142,38 @@ k_spmv_xstat(XstatArgs a) {
   const int fin_lo = (b * R) / B, fin_hi = ((b + 1) * R) / B;
   double dacc = 0.0;
 
+  // segment bounds of tile t: every thread loads rows j = tid, tid+blockDim ...
+  auto load_bounds = [&](int t, int* dst) {
+    const int64_t rt = r0c + int64_t(t) * R;
+    const int nrows = int(cmin64(R, r1c - rt));
+    for (int j = threadIdx.x; j < nrows; j += blockDim.x) {
+      const int64_t i = rt + j;
+      dst[j] = (b == 0) ? __ldg(rowptr + i) : __ldg(seg + int64_t(b - 1) * m + i);
+      dst[R + j] = (b == B - 1) ? __ldg(rowptr + i + 1) : __ldg(seg + int64_t(b) * m + i);
+    }
+  };
+  if (ntiles > 0) load_bounds(0, bnd);
+
   mbar_wait(&bar, 0);
   __syncthreads();
 
   auto process = [&](int t) {
     double* pb = pbuf + (t % 3) * R;
+    const int* bb = bnd + (t & 1) * 2 * R;
     const int64_t rt = r0c + int64_t(t) * R;
     const int nrows = int(cmin64(R, r1c - rt));
+    // prefetch the bounds of tile t+1 into registers; stored after the tile
+    int pf0 = 0, pf1 = 0;
+    const bool has_next = (t + 1 < ntiles);
+    const int64_t rn = rt + R;
+    const int nnext = has_next ? int(cmin64(R, r1c - rn)) : 0;
+    const int jn = threadIdx.x;  // R <= blockDim.x is not assumed: loop below covers the rest
+    if (jn < nnext) {
+      pf0 = (b == 0) ? __ldg(rowptr + rn + jn) : __ldg(seg + int64_t(b - 1) * m + rn + jn);
+      pf1 = (b == B - 1) ? __ldg(rowptr + rn + jn + 1) : __ldg(seg + int64_t(b) * m + rn + jn);
+    }
     for (int j = group; j < nrows; j += ngroups) {
-      const int64_t i = rt + j;
-      const int k0 = (b == 0) ? __ldg(rowptr + i) : __ldg(seg + int64_t(b - 1) * m + i);
-      const int k1 = (b == B - 1) ? __ldg(rowptr + i + 1) : __ldg(seg + int64_t(b) * m + i);
+      const int k0 = bb[j], k1 = bb[R + j];
       double s = 0.0;
       for (int kb = k0 + lane; kb < k1; kb += G * U) {
         int cc[U];
@@ -166,6 +189,14 @@ k_spmv_xstat(XstatArgs a) {
       }
       if (G > 1) s = group_sum<G>(s, gmask);
       if (lane == 0) pb[j] = s;
+    }
+    if (has_next) {
+      int* nb = bnd + ((t + 1) & 1) * 2 * R;
+      if (jn < nnext) { nb[jn] = pf0; nb[R + jn] = pf1; }
+      for (int j = jn + blockDim.x; j < nnext; j += blockDim.x) {
+        nb[j] = (b == 0) ? __ldg(rowptr + rn + j) : __ldg(seg + int64_t(b - 1) * m + rn + j);
+        nb[R + j] = (b == B - 1) ? __ldg(rowptr + rn + j + 1) : __ldg(seg + int64_t(b) * m + rn + j);
+      }
     }
   };
 

@@ -18,8 +18,9 @@ import paper_conf_asplos_ginsbachrsbdo18_b200 as sp
 
 VARIANTS = [("auto", {}, {})] + [(f"vector{g}", {"kernel": "vector", "vec_lanes": g}, {}) for g in (4, 8, 16, 32)] + \
     [(f"vector32_u{u}", {"kernel": "vector", "vec_lanes": 32}, {"SPMV_UNROLL": str(u)}) for u in (2, 8)] + \
-    [(f"xstat_B{b}_G{g}", {"kernel": "xstat"}, {"SPMV_XSTAT_B": str(b), "SPMV_XSTAT_G": str(g)})
-     for b in (2, 4, 8) for g in (4, 8, 16, 32)]
+    [(f"xstat_B{b}_G{g}_U{u}", {"kernel": "xstat"}, {"SPMV_XSTAT_B": str(b), "SPMV_XSTAT_G": str(g),
+                                                     "SPMV_XSTAT_U": str(u)})
+     for b in (2, 4, 8) for g in (4, 8, 16) for u in (4, 8)]
 
 
 def time_variant(A, x, y, kw, env, reps=20):
