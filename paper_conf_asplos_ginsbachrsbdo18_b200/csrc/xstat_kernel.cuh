@@ -217,11 +217,17 @@ k_spmv_xstat(XstatArgs a) {
     }
   };
 
+  // The bounds of tile t+1 are written during process(t) by every thread, so
+  // all threads of the CTA must finish process(t) before any starts
+  // process(t+1) (__syncthreads); the split cluster barrier alone only orders
+  // tiles t-1 and t+1.
   if (ntiles > 0) {
     process(0);
+    __syncthreads();
     cluster_arrive();
     for (int t = 1; t < ntiles; ++t) {
       process(t);
+      __syncthreads();
       cluster_wait();
       finalize(t - 1);
       cluster_arrive();
