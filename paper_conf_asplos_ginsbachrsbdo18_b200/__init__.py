@@ -32,20 +32,20 @@ _ST = ctypes.c_int
 SPMV_OK, SPMV_ERR_ARG, SPMV_ERR_INDEX, SPMV_ERR_ALIAS, SPMV_ERR_CUDA = 0, 1, 2, 3, 4
 SPMV_ERR_NCCL, SPMV_ERR_NOMEM, SPMV_ERR_BREAKDOWN, SPMV_ERR_UNSUPPORTED = 5, 6, 7, 8
 SPMV_F64, SPMV_F32 = 0, 1
-KERNELS = {"auto": 0, "scalar": 1, "vector": 2, "merge": 3, "xstat": 4}
+KERNELS = {"auto": 0, "scalar": 1, "vector": 2, "merge": 3, "xstat": 4, "xplan": 5}
 KERNEL_NAMES = {v: k for k, v in KERNELS.items()}
 
 
 class SpmvOpts(ctypes.Structure):
     _fields_ = [("stream", _P), ("kernel", _I32), ("vec_lanes", _I32), ("validate", _I32),
-                ("l2_window", _I32), ("dist", _P)]
+                ("plan", _I32), ("dist", _P)]
 
 
 class SpmvInfo(ctypes.Structure):
     _fields_ = [("kernel", _I32), ("vec_lanes", _I32), ("row_min", _I64), ("row_max", _I64),
                 ("row_mean", _D), ("row_cv", _D), ("m_local", _I64), ("row_begin", _I64),
                 ("row_end", _I64), ("nnz_local", _I64), ("rank", _I32), ("nranks", _I32),
-                ("sorted_cols", _I32), ("grid", _I64)]
+                ("sorted_cols", _I32), ("grid", _I64), ("cluster", _I32), ("plan_bytes", _I64)]
 
 
 def _decl(name, args, res=_ST):
@@ -61,6 +61,7 @@ spmv_csr_c = _decl("spmv_csr", [_P, _I64, _I64, _I64, _P, _P, _P, _P, _P, _D, _D
 cg_solve_c = _decl("cg_solve", [_P, _P, _P, _I32, _D, ctypes.POINTER(_I32), ctypes.POINTER(_D)])
 cg_npb_outer_c = _decl("cg_npb_outer", [_P, _P, _P, _I32, _D, _P])
 spmv_cg_status_c = _decl("spmv_cg_status", [_P])
+spmv_csr_update_values_c = _decl("spmv_csr_update_values", [_P, _P])
 spmv_csr_destroy_c = _decl("spmv_csr_destroy", [_P])
 spmv_csr_partition_c = _decl("spmv_csr_partition", [_P, _I64, _I32, _P])
 spmv_csr_merge_splits_c = _decl("spmv_csr_merge_splits", [_P, _I64, _I64, _P, _P])
@@ -76,6 +77,7 @@ spmv_dist_colidx_c = _decl("spmv_dist_colidx", [_P, _P])
 
 # every symbol include/spmv.h declares (checked by tests/test_abi.py)
 EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_status",
+           "spmv_csr_update_values",
            "spmv_csr_destroy", "spmv_csr_partition", "spmv_csr_merge_splits", "spmv_csr_info",
            "spmv_launch_count", "spmv_status_string", "spmv_last_error_string",
            "spmv_dist_get_unique_id", "spmv_dist_init", "spmv_dist_destroy", "spmv_dist_plan_host",
@@ -180,7 +182,8 @@ class CSRMatrix:
     """
 
     def __init__(self, rowptr, colidx, vals, n: int | None = None, *, kernel: str = "auto",
-                 vec_lanes: int = 0, validate: bool = False, stream=None, dist: Dist | None = None):
+                 vec_lanes: int = 0, validate: bool = False, stream=None, dist: Dist | None = None,
+                 plan: bool = True):
         import torch
         assert rowptr.dtype == torch.int32 and colidx.dtype == torch.int32
         assert vals.dtype in (torch.float64, torch.float32)
@@ -197,7 +200,7 @@ class CSRMatrix:
         o.kernel = KERNELS[kernel]
         o.vec_lanes = int(vec_lanes)
         o.validate = int(bool(validate))
-        o.l2_window = 0
+        o.plan = int(bool(plan))
         o.dist = dist.handle if dist is not None else None
         nnz = int(rowptr[-1].item()) - int(rowptr[0].item()) if self.m >= 0 else 0
         self.nnz = nnz
@@ -236,6 +239,11 @@ class CSRMatrix:
         out = np.zeros(self._info["nnz_local"], dtype=np.int32)
         _check(spmv_dist_colidx_c(self.handle, out.ctypes.data), "spmv_dist_colidx")
         return out
+
+    def update_values(self, vals):
+        """Re-bind the values (same structure) and refresh the plan copy."""
+        _check(spmv_csr_update_values_c(self.handle, _ptr(vals)), "spmv_csr_update_values")
+        self.vals = vals
 
     def cg_status(self):
         _check(spmv_cg_status_c(self.handle), "spmv_cg_status")

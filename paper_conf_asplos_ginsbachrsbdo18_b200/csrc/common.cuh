@@ -57,6 +57,19 @@ __device__ __forceinline__ double block_sum(double v, double* red) {
   return t;
 }
 
+// Deterministic sum over the first nw warps of the block only (named barrier
+// 1), for warp-specialised kernels whose other warps do not participate.
+__device__ __forceinline__ double block_sum_n(double v, double* red, int nw) {
+  const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
+  v = warp_sum(v);
+  asm volatile("bar.sync 1, %0;\n" ::"r"(nw * 32) : "memory");
+  if (lane == 0) red[wid] = v;
+  asm volatile("bar.sync 1, %0;\n" ::"r"(nw * 32) : "memory");
+  double t = (lane < nw) ? red[lane] : 0.0;
+  t = warp_sum(t);
+  return t;
+}
+
 // A scalar source for the CG kernels: either `count` per-block partials to be
 // summed (single GPU: every consuming block sums them in the same fixed order,
 // so all blocks see bit-identical scalars), or count == 1 pointing at a

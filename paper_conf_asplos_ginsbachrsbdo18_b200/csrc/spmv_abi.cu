@@ -20,6 +20,7 @@
 #include "cg_kernels.cuh"
 #include "spmv_kernels.cuh"
 #include "xstat_kernel.cuh"
+#include "xplan_kernel.cuh"
 
 using namespace spmv;
 
@@ -100,7 +101,7 @@ struct spmv_csr_s {
   const int32_t* ci_loc = nullptr;   // colidx (single) or renumbered copy - k0 (dist)
   // kernel choice
   int32_t kernel = SPMV_KERNEL_VECTOR, lanes = 32, unroll = 4;
-  int64_t grid = 1, vgrid = 1;
+  int64_t grid = 1, vgrid = 1, grid_vec = 1;
   int64_t row_min = 0, row_max = 0;
   double row_mean = 0, row_cv = 0;
   int32_t sorted = 0;
@@ -112,6 +113,19 @@ struct spmv_csr_s {
   long long* crow = nullptr;
   void (*xk)(XstatArgs) = nullptr;
   void (*xk_dot)(XstatArgs) = nullptr;
+  // XPLAN (column-blocked device plan of A)
+  struct {
+    bool built = false;
+    int B = 0, W = 0, CH = 0, ncl = 0, ntiles = 0;
+    size_t smem = 0;
+    int64_t total = 0;
+    long long *crow = nullptr, *toff = nullptr;
+    int *tile0 = nullptr, *rofs = nullptr, *tlen = nullptr, *seg = nullptr;
+    void* pv = nullptr;
+    uint16_t* pc = nullptr;
+    void (*k)(XplanArgs) = nullptr;
+    void (*kdot)(XplanArgs) = nullptr;
+  } xp;
   // dist
   spmv_dist_s* dist = nullptr;
   std::vector<long long> bounds;
@@ -313,6 +327,181 @@ static spmv_status xstat_setup(spmv_csr_s* h, bool* ok) {
   return SPMV_OK;
 }
 
+template <typename T, bool DOT>
+static void (*xplan_fn(int G))(XplanArgs) {
+  switch (G) {
+    case 4: return k_spmv_xplan<T, 4, DOT>;
+    case 16: return k_spmv_xplan<T, 16, DOT>;
+    default: return k_spmv_xplan<T, 8, DOT>;
+  }
+}
+
+static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha,
+                                double beta, const double* w, double* part) {
+  XplanArgs a;
+  a.nx = h->nx;
+  a.W = h->xp.W;
+  a.CH = h->xp.CH;
+  a.pvals = h->xp.pv;
+  a.pcols = h->xp.pc;
+  a.rofs = h->xp.rofs;
+  a.toff = h->xp.toff;
+  a.tlen = h->xp.tlen;
+  a.crow = h->xp.crow;
+  a.tile0 = h->xp.tile0;
+  a.x = x;
+  a.y = y;
+  a.alpha = alpha;
+  a.beta = beta;
+  a.w = w;
+  a.part = part;
+  if (h->dt == SPMV_F32) {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+  }
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = dim3((unsigned)(h->xp.ncl * h->xp.B), 1, 1);
+  cfg.blockDim = dim3(XP_THREADS, 1, 1);
+  cfg.dynamicSmemBytes = h->xp.smem;
+  cfg.stream = s;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeClusterDimension;
+  at[0].val.clusterDim.x = (unsigned)h->xp.B;
+  at[0].val.clusterDim.y = 1;
+  at[0].val.clusterDim.z = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  CK(cudaLaunchKernelEx(&cfg, part ? h->xp.kdot : h->xp.k, a));
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+// Pack (or re-pack, values_only) the nonzeros into the plan streams.
+static spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only) {
+  cudaStream_t s = h->stream;
+  const int64_t g = std::min<int64_t>(cdiv(h->m_loc * 32, 256), 16LL * num_sms(h->device));
+  if (h->dt == SPMV_F64)
+    k_xplan_pack<double><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const double*)vals, h->xp.seg, h->m_loc,
+                                          h->xp.B, h->xp.W, h->xp.crow, h->xp.tile0, h->xp.ncl, h->xp.rofs,
+                                          h->xp.toff, (double*)h->xp.pv, h->xp.pc, values_only);
+  else
+    k_xplan_pack<float><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const float*)vals, h->xp.seg, h->m_loc,
+                                         h->xp.B, h->xp.W, h->xp.crow, h->xp.tile0, h->xp.ncl, h->xp.rofs,
+                                         h->xp.toff, (float*)h->xp.pv, h->xp.pc, values_only);
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+// Build the column-blocked plan (create).  *ok = false if not eligible.
+static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
+  *ok = false;
+  if (!h->sorted || h->m_loc == 0 || h->nx == 0 || h->k1 - h->k0 == 0) return SPMV_OK;
+  const size_t ts = h->ts;
+  const size_t smem_cap = 227 * 1024 - 1024;  // dynamic smem a CTA may use (static ~0.5 KB)
+  const size_t fixed = 3 * (size_t)(XP_R + 4) * 4 + 3 * (size_t)XP_R * 8;
+  const size_t stage_min = (size_t)XP_S * 1024 * (ts + 2);
+  if (smem_cap <= fixed + stage_min) return SPMV_OK;
+  const size_t xbudget = smem_cap - fixed - stage_min;
+  int B = (int)cdiv((int64_t)(ts * h->nx), (int64_t)xbudget);
+  B = B <= 1 ? 1 : B <= 2 ? 2 : B <= 4 ? 4 : B <= 8 ? 8 : 16;
+  int forced = 0;
+  if (env_int("SPMV_XPLAN_B", &forced) && forced >= B && forced <= 8 && (forced & (forced - 1)) == 0) B = forced;
+  if (B > 8) return SPMV_OK;
+  int W = (int)cdiv(h->nx, B);
+  W = (W + 7) & ~7;
+  if (W > 65535) return SPMV_OK;
+  const size_t xbytes = ((size_t)W * ts + 127) & ~size_t(127);
+  int CH = (int)((smem_cap - fixed - xbytes) / ((size_t)XP_S * (ts + 2)));
+  CH = std::min(CH, 4096) & ~7;
+  int ch_env = 0;
+  if (env_int("SPMV_XPLAN_CH", &ch_env) && ch_env >= 64 && ch_env <= CH) CH = ch_env & ~7;
+  if (CH < 256) return SPMV_OK;
+  const size_t smem = xbytes + (size_t)XP_S * CH * (ts + 2) + fixed;
+  const double seg_mean = h->row_mean / B;
+  int G = seg_mean < 12 ? 4 : seg_mean < 48 ? 8 : 16;
+  int g2 = 0;
+  if (env_int("SPMV_XPLAN_G", &g2) && (g2 == 4 || g2 == 8 || g2 == 16)) G = g2;
+  void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? xplan_fn<double, false>(G) : xplan_fn<float, false>(G);
+  void (*fnd)(XplanArgs) = h->dt == SPMV_F64 ? xplan_fn<double, true>(G) : nullptr;
+  CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+  if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = dim3((unsigned)B, 1, 1);
+  cfg.blockDim = dim3(XP_THREADS, 1, 1);
+  cfg.dynamicSmemBytes = smem;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeClusterDimension;
+  at[0].val.clusterDim.x = (unsigned)B;
+  at[0].val.clusterDim.y = 1;
+  at[0].val.clusterDim.z = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  int ncl = 0;
+  cudaError_t e = cudaOccupancyMaxActiveClusters(&ncl, fn, &cfg);
+  if (e != cudaSuccess || ncl < 1) { cudaGetLastError(); return SPMV_OK; }
+  int nc_env = 0;
+  if (env_int("SPMV_XPLAN_CLUSTERS", &nc_env) && nc_env >= 1 && nc_env <= ncl) ncl = nc_env;
+  cudaStream_t s = h->stream;
+  auto& P = h->xp;
+  P.B = B; P.W = W; P.CH = CH; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd;
+  // cluster row ranges (nnz-balanced)
+  CK(cudaMalloc(&P.crow, sizeof(long long) * (ncl + 1)));
+  k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(h->m_loc, h->rp_loc, ncl, P.crow);
+  LAUNCHED();
+  std::vector<long long> crow(ncl + 1);
+  CK(cudaMemcpyAsync(crow.data(), P.crow, sizeof(long long) * (ncl + 1), cudaMemcpyDeviceToHost, s));
+  CK(cudaStreamSynchronize(s));
+  std::vector<int> tile0(ncl + 1, 0);
+  for (int c = 0; c < ncl; ++c) tile0[c + 1] = tile0[c] + (int)cdiv(crow[c + 1] - crow[c], XP_R);
+  const int ntiles = tile0[ncl];
+  P.ntiles = ntiles;
+  CK(cudaMalloc(&P.tile0, sizeof(int) * (ncl + 1)));
+  CK(cudaMemcpyAsync(P.tile0, tile0.data(), sizeof(int) * (ncl + 1), cudaMemcpyHostToDevice, s));
+  // split points
+  if (B > 1) {
+    CK(cudaMalloc(&P.seg, sizeof(int) * (size_t)(B - 1) * (size_t)h->m_loc));
+    k_xstat_splits<<<std::min<int64_t>(cdiv(h->m_loc, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
+        h->m_loc, h->rp_loc, h->ci_loc, B, W, P.seg);
+    LAUNCHED();
+  }
+  // row offsets + tile lengths
+  const size_t nTB = (size_t)std::max(ntiles, 1) * B;
+  CK(cudaMalloc(&P.rofs, sizeof(int) * nTB * (XP_R + 4)));
+  CK(cudaMalloc(&P.tlen, sizeof(int) * nTB));
+  CK(cudaMalloc(&P.toff, sizeof(long long) * nTB));
+  if (ntiles > 0) {
+    k_xplan_rofs<<<(unsigned)(ntiles * B), XP_R, 0, s>>>(h->rp_loc, P.seg, h->m_loc, B, P.crow, P.tile0, ncl,
+                                                          P.rofs, P.tlen);
+    LAUNCHED();
+  }
+  std::vector<int> tl(nTB, 0);
+  CK(cudaMemcpyAsync(tl.data(), P.tlen, sizeof(int) * nTB, cudaMemcpyDeviceToHost, s));
+  CK(cudaStreamSynchronize(s));
+  // padded lengths and offsets, streams of one CTA contiguous: order [c][b][t]
+  std::vector<long long> toff(nTB, 0);
+  long long pos = 0;
+  for (int c = 0; c < ncl; ++c)
+    for (int bb = 0; bb < B; ++bb)
+      for (int t = tile0[c]; t < tile0[c + 1]; ++t) {
+        const size_t idx = (size_t)t * B + bb;
+        tl[idx] = (tl[idx] + 7) & ~7;
+        toff[idx] = pos;
+        pos += tl[idx];
+      }
+  P.total = pos;
+  CK(cudaMemcpyAsync(P.tlen, tl.data(), sizeof(int) * nTB, cudaMemcpyHostToDevice, s));
+  CK(cudaMemcpyAsync(P.toff, toff.data(), sizeof(long long) * nTB, cudaMemcpyHostToDevice, s));
+  CK(cudaMalloc(&P.pv, ts * (size_t)std::max<int64_t>(pos, 8)));
+  CK(cudaMalloc(&P.pc, 2 * (size_t)std::max<int64_t>(pos, 8)));
+  CK(cudaMemsetAsync(P.pv, 0, ts * (size_t)std::max<int64_t>(pos, 8), s));
+  CK(cudaMemsetAsync(P.pc, 0, 2 * (size_t)std::max<int64_t>(pos, 8), s));
+  ST(xplan_pack(h, h->vals, 0));
+  CK(cudaStreamSynchronize(s));
+  P.built = true;
+  *ok = true;
+  return SPMV_OK;
+}
+
 // Local SpMV of the handle: y = alpha*A_loc*x + beta*y (+ partial w.y per CTA).
 static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
                             double alpha, double beta, const double* w, double* part) {
@@ -329,6 +518,8 @@ static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, con
     LAUNCHED();
     return SPMV_OK;
   }
+  if (h->kernel == SPMV_KERNEL_XPLAN && vals == h->vals) return launch_xplan(h, s, x, y, alpha, beta, w, part);
+  const int64_t vgrid_spmv = h->kernel == SPMV_KERNEL_XPLAN ? h->grid_vec : h->grid;
   if (h->kernel == SPMV_KERNEL_XSTAT) return launch_xstat(h, s, vals, x, y, alpha, beta, w, part);
   SpmvArgs a;
   a.m = h->m_loc;
@@ -342,12 +533,12 @@ static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, con
   a.w = w;
   a.part = part;
   if (h->dt == SPMV_F64) {
-    if (part) launch_vec<double, true>(h->lanes, h->unroll, h->grid, s, a);
-    else launch_vec<double, false>(h->lanes, h->unroll, h->grid, s, a);
+    if (part) launch_vec<double, true>(h->lanes, h->unroll, vgrid_spmv, s, a);
+    else launch_vec<double, false>(h->lanes, h->unroll, vgrid_spmv, s, a);
   } else {
     a.alpha = (double)(float)alpha;
     a.beta = (double)(float)beta;
-    launch_vec<float, false>(h->lanes, h->unroll, h->grid, s, a);
+    launch_vec<float, false>(h->lanes, h->unroll, vgrid_spmv, s, a);
   }
   LAUNCHED();
   return SPMV_OK;
@@ -377,6 +568,7 @@ static void choose_kernel(spmv_csr_s* h, int req_kernel, int req_lanes) {
   // fixed grid-stride grid (deterministic CTA partials): 8 CTAs of 256 per SM
   const int64_t groups_per_cta = 256 / lanes;
   h->grid = std::max<int64_t>(1, std::min<int64_t>(cdiv(h->m_loc, groups_per_cta), 8LL * sms));
+  h->grid_vec = h->grid;
   h->vgrid = std::max<int64_t>(1, std::min<int64_t>(cdiv(h->m_loc, 1024), 4LL * sms));
 }
 
@@ -532,13 +724,25 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
   if (!env_int("SPMV_LANES", &rl)) rl = o.vec_lanes;
   h->nx = o.dist ? (int64_t)h->maxlen * o.dist->nranks : n;
   choose_kernel(h, rk, rl);
-  if (rk == SPMV_KERNEL_XSTAT || rk == SPMV_KERNEL_AUTO) {
+  int plan = o.plan;
+  env_int("SPMV_PLAN", &plan);
+  if (rk == SPMV_KERNEL_XPLAN || (rk == SPMV_KERNEL_AUTO && plan)) {
+    // auto + plan: the column-blocked x-stationary plan whenever x fits the
+    // shared memory of a cluster and rows are long enough
+    if (rk == SPMV_KERNEL_XPLAN || h->row_mean >= 16.0) {
+      bool ok = false;
+      spmv_status st = xplan_build(h, &ok);
+      if (st != SPMV_OK) return fail(st);
+      if (ok) {
+        h->kernel = SPMV_KERNEL_XPLAN;
+        h->grid = (int64_t)h->xp.ncl * h->xp.B;
+      }
+    }
+  } else if (rk == SPMV_KERNEL_XSTAT) {
     bool ok = false;
     spmv_status st = xstat_setup(h, &ok);
     if (st != SPMV_OK) return fail(st);
-    // auto: x-stationary whenever x fits a cluster's shared memory and rows are
-    // long enough for the split to pay
-    if (ok && (rk == SPMV_KERNEL_XSTAT || h->row_mean >= 16.0)) {
+    if (ok) {
       h->kernel = SPMV_KERNEL_XSTAT;
       h->grid = (int64_t)h->nclusters * h->xB;
     }
@@ -557,7 +761,8 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   cudaError_t e = h->stream ? cudaStreamSynchronize(h->stream) : cudaDeviceSynchronize();
   if (e != cudaSuccess) st = cuda_fail(e, "pending asynchronous error", __LINE__);
   h->g_npb.reset();
-  void* bufs[] = {h->seg, h->crow, h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
+  void* bufs[] = {h->xp.crow, h->xp.toff, h->xp.tile0, h->xp.rofs, h->xp.tlen, h->xp.seg, h->xp.pv, h->xp.pc,
+                  h->seg, h->crow, h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
                   h->stage_x, h->stage_z};
   for (void* b : bufs)
@@ -611,7 +816,7 @@ extern "C" spmv_status spmv_csr(spmv_csr_t h, int64_t m, int64_t n, int64_t nnz,
 static spmv_status cg_alloc(spmv_csr_s* h) {
   if (h->z) return SPMV_OK;
   const size_t nb = sizeof(double) * (size_t)std::max<int64_t>(h->m_loc, 1);
-  const size_t pb = sizeof(double) * (size_t)std::max<int64_t>(std::max(h->grid, h->vgrid), 1);
+  const size_t pb = sizeof(double) * (size_t)std::max<int64_t>(std::max(std::max(h->grid, h->grid_vec), h->vgrid), 1);
   ST(ensure_buf((void**)&h->z, nb));
   ST(ensure_buf((void**)&h->r, nb));
   ST(ensure_buf((void**)&h->q, nb));
@@ -662,7 +867,7 @@ struct CgRun {
 static spmv_status cg_enqueue_init(spmv_csr_s* h, cudaStream_t s, const double* b, double* z,
                                    CgRun* run) {
   const int vg = (int)h->vgrid;
-  double* prb = h->part_rr + 2 * std::max(h->grid, h->vgrid);
+  double* prb = h->part_rr + 2 * std::max(std::max(h->grid, h->grid_vec), h->vgrid);
   k_cg_init<<<vg, 256, 0, s>>>(h->m_loc, b, z, h->r, cg_p(h), prb);
   LAUNCHED();
   ST(reduce_src(h, s, SumSrc{prb, vg}, 0, &run->rr_b));
@@ -679,7 +884,7 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
   double* p = cg_p(h);
   const void* xg = h->dist ? h->xpad : (const void*)p;
   const int vg = (int)h->vgrid, sg = (int)h->grid;
-  const int64_t pstride = std::max(h->grid, h->vgrid);
+  const int64_t pstride = std::max(std::max(h->grid, h->grid_vec), h->vgrid);
   for (int c = 0; c < iters; ++c) {
     const int it = run->it++;
     ST(gather_p(h, s));
@@ -864,6 +1069,16 @@ extern "C" spmv_status cg_npb_outer(spmv_csr_t h, void* x, void* z, int32_t cgit
   return SPMV_OK;
 }
 
+extern "C" spmv_status spmv_csr_update_values(spmv_csr_t h, const void* vals) {
+  if (!h) return arg_fail("handle is NULL");
+  CK(cudaSetDevice(h->device));
+  ST(need_device(vals, h->device, "vals must be a device pointer", h->nnz == 0));
+  h->vals = vals;
+  if (h->xp.built) ST(xplan_pack(h, vals, 1));
+  h->g_npb.reset();
+  return SPMV_OK;
+}
+
 extern "C" spmv_status spmv_cg_status(spmv_csr_t h) {
   if (!h) return arg_fail("handle is NULL");
   if (!h->flags) return SPMV_OK;
@@ -962,6 +1177,8 @@ extern "C" spmv_status spmv_csr_info(spmv_csr_t h, spmv_info_t* info) {
   info->nranks = h->dist ? h->dist->nranks : 1;
   info->sorted_cols = h->sorted;
   info->grid = h->grid;
+  info->cluster = h->kernel == SPMV_KERNEL_XPLAN ? h->xp.B : h->kernel == SPMV_KERNEL_XSTAT ? h->xB : 0;
+  info->plan_bytes = h->xp.built ? (int64_t)h->xp.total * (int64_t)(h->ts + 2) : 0;
   return SPMV_OK;
 }
 

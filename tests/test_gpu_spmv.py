@@ -272,3 +272,62 @@ def test_xstat_alpha_beta_and_offset(sp, torch_dev):
     y0 = gen.uniform(A.m, seed=16)
     for a, b in [(2.0, -1.0), (0.0, 3.0), (1.0, 0.0)]:
         run_case(sp, torch, dev, A, x, alpha=a, beta=b, y0=y0, kernel="xstat", what=f"xstat a={a} b={b}")
+
+
+@pytest.mark.parametrize("cfg", [{}, {"SPMV_XPLAN_B": "2"}, {"SPMV_XPLAN_B": "8"}, {"SPMV_XPLAN_G": "4"},
+                                 {"SPMV_XPLAN_G": "16", "SPMV_XPLAN_B": "4"}, {"SPMV_XPLAN_CH": "64"},
+                                 {"SPMV_XPLAN_CLUSTERS": "1", "SPMV_XPLAN_CH": "256"}])
+@pytest.mark.parametrize("name,A", ZOO, ids=[c[0] for c in ZOO])
+def test_zoo_xplan(sp, torch_dev, name, A, cfg, monkeypatch):
+    """x-stationary kernel over the column-blocked plan (TMA bulk pipeline,
+    clusters, DSMEM reduction): cluster sizes, lane groups, tiny chunks (many
+    chunks per tile, rows split across chunks) and a single cluster (many
+    tiles: exercises the triple-buffered partials and the split barrier)."""
+    torch, dev = torch_dev
+    for k, v in cfg.items():
+        monkeypatch.setenv(k, v)
+    x = gen.uniform(A.n, seed=17)
+    info = run_case(sp, torch, dev, A, x, kernel="xplan", what=f"{name} xplan {cfg}")
+    k = np.arange(A.rowptr[0] + 1, A.rowptr[-1])
+    starts = np.zeros(A.colidx.shape[0] + 1, bool)
+    starts[A.rowptr[:-1]] = True
+    inner = ~starts[k]
+    sorted_cols = bool(np.all(A.colidx[k][inner] > A.colidx[k - 1][inner]))
+    if sorted_cols and A.nnz > 0:
+        assert info["kernel_name"] == "xplan", info
+        assert info["plan_bytes"] >= A.nnz * 10
+    A32 = A.astype(np.float32)
+    run_case(sp, torch, dev, A32, gen.uniform(A.n, seed=18, f32=True), kernel="xplan",
+             what=f"{name} xplan fp32 {cfg}")
+
+
+def test_xplan_alpha_beta_update_values(sp, torch_dev):
+    torch, dev = torch_dev
+    A = gen.makea("A")
+    x_h = gen.uniform(A.n, seed=19)
+    y0 = gen.uniform(A.m, seed=20)
+    for a, b in [(2.0, -1.0), (0.0, 3.0), (1.0, 0.0), (-1.5, 1.0)]:
+        info = run_case(sp, torch, dev, A, x_h, alpha=a, beta=b, y0=y0, what=f"xplan a={a} b={b}")
+        assert info["kernel_name"] == "xplan"
+    # in-place value change + update_values (the paper's lazy-copy flag)
+    rp, ci, va = to_dev(A, dev)
+    x = torch.from_numpy(x_h).to(dev)
+    y = torch.empty(A.m, dtype=torch.float64, device=dev)
+    with sp.CSRMatrix(rp, ci, va, A.n) as M:
+        assert M.info()["kernel_name"] == "xplan"
+        v2_h = gen.uniform(A.nnz, seed=23)
+        va.copy_(torch.from_numpy(v2_h))
+        M.update_values(va)
+        M.spmv(x, y)
+        torch.cuda.synchronize()
+    y_ref, bound = oracle.spmv(A.rowptr, A.colidx, v2_h, x_h)
+    check_rows(y.cpu().numpy(), y_ref, bound, np.float64, "xplan update_values")
+
+
+def test_plan_off_uses_zero_copy(sp, torch_dev):
+    torch, dev = torch_dev
+    A = gen.makea("S")
+    rp, ci, va = to_dev(A, dev)
+    with sp.CSRMatrix(rp, ci, va, A.n, plan=False) as M:
+        inf = M.info()
+        assert inf["kernel_name"] == "vector" and inf["plan_bytes"] == 0
