@@ -114,15 +114,14 @@ struct spmv_csr_s {
   void (*xk)(XstatArgs) = nullptr;
   void (*xk_dot)(XstatArgs) = nullptr;
   // XPLAN (column-blocked device plan of A)
-  struct {
+  struct XPlan {
     bool built = false;
-    int B = 0, W = 0, CH = 0, ncl = 0, ntiles = 0;
+    int B = 0, W = 0, SB = 0, ncl = 0, ntiles = 0, nrec = 0;
     size_t smem = 0;
-    int64_t total = 0;
-    long long *crow = nullptr, *toff = nullptr;
-    int *tile0 = nullptr, *rofs = nullptr, *tlen = nullptr, *seg = nullptr;
-    void* pv = nullptr;
-    uint16_t* pc = nullptr;
+    int64_t bytes = 0;
+    long long *crow = nullptr, *rec_off = nullptr;
+    int *cta_rec = nullptr, *rec_tile = nullptr, *seg = nullptr, *row_rec = nullptr, *row_pos = nullptr;
+    unsigned char* plan = nullptr;
     void (*k)(XplanArgs) = nullptr;
     void (*kdot)(XplanArgs) = nullptr;
   } xp;
@@ -341,14 +340,12 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   XplanArgs a;
   a.nx = h->nx;
   a.W = h->xp.W;
-  a.CH = h->xp.CH;
-  a.pvals = h->xp.pv;
-  a.pcols = h->xp.pc;
-  a.rofs = h->xp.rofs;
-  a.toff = h->xp.toff;
-  a.tlen = h->xp.tlen;
+  a.SB = h->xp.SB;
+  a.plan = h->xp.plan;
+  a.rec_off = h->xp.rec_off;
+  a.rec_tile = h->xp.rec_tile;
+  a.cta_rec = h->xp.cta_rec;
   a.crow = h->xp.crow;
-  a.tile0 = h->xp.tile0;
   a.x = x;
   a.y = y;
   a.alpha = alpha;
@@ -376,18 +373,18 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   return SPMV_OK;
 }
 
-// Pack (or re-pack, values_only) the nonzeros into the plan streams.
+// Pack (or re-pack, values_only) the nonzeros into the plan records.
 static spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only) {
   cudaStream_t s = h->stream;
   const int64_t g = std::min<int64_t>(cdiv(h->m_loc * 32, 256), 16LL * num_sms(h->device));
   if (h->dt == SPMV_F64)
     k_xplan_pack<double><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const double*)vals, h->xp.seg, h->m_loc,
-                                          h->xp.B, h->xp.W, h->xp.crow, h->xp.tile0, h->xp.ncl, h->xp.rofs,
-                                          h->xp.toff, (double*)h->xp.pv, h->xp.pc, values_only);
+                                          h->xp.B, h->xp.W, h->xp.rec_off, h->xp.row_rec, h->xp.row_pos,
+                                          h->xp.plan, values_only);
   else
     k_xplan_pack<float><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const float*)vals, h->xp.seg, h->m_loc,
-                                         h->xp.B, h->xp.W, h->xp.crow, h->xp.tile0, h->xp.ncl, h->xp.rofs,
-                                         h->xp.toff, (float*)h->xp.pv, h->xp.pc, values_only);
+                                         h->xp.B, h->xp.W, h->xp.rec_off, h->xp.row_rec, h->xp.row_pos,
+                                         h->xp.plan, values_only);
   LAUNCHED();
   return SPMV_OK;
 }
@@ -396,12 +393,12 @@ static spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only) 
 static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   *ok = false;
   if (!h->sorted || h->m_loc == 0 || h->nx == 0 || h->k1 - h->k0 == 0) return SPMV_OK;
-  const size_t ts = h->ts;
-  const size_t smem_cap = 227 * 1024 - 1024;  // dynamic smem a CTA may use (static ~0.5 KB)
-  const size_t fixed = 3 * (size_t)(XP_R + 4) * 4 + 3 * (size_t)XP_R * 8;
-  const size_t stage_min = (size_t)XP_S * 1024 * (ts + 2);
-  if (smem_cap <= fixed + stage_min) return SPMV_OK;
-  const size_t xbudget = smem_cap - fixed - stage_min;
+  const int ts = (int)h->ts;
+  const size_t smem_cap = 227 * 1024 - 1024;  // dynamic smem a CTA may use (static < 1 KB)
+  const size_t pbuf = 3 * (size_t)XP_R * 8;
+  const size_t sb_min = 16 * 1024;
+  if (smem_cap <= pbuf + XP_S * sb_min) return SPMV_OK;
+  const size_t xbudget = smem_cap - pbuf - XP_S * sb_min;
   int B = (int)cdiv((int64_t)(ts * h->nx), (int64_t)xbudget);
   B = B <= 1 ? 1 : B <= 2 ? 2 : B <= 4 ? 4 : B <= 8 ? 8 : 16;
   int forced = 0;
@@ -411,14 +408,12 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   W = (W + 7) & ~7;
   if (W > 65535) return SPMV_OK;
   const size_t xbytes = ((size_t)W * ts + 127) & ~size_t(127);
-  int CH = (int)((smem_cap - fixed - xbytes) / ((size_t)XP_S * (ts + 2)));
-  CH = std::min(CH, 4096) & ~7;
-  int ch_env = 0;
-  if (env_int("SPMV_XPLAN_CH", &ch_env) && ch_env >= 64 && ch_env <= CH) CH = ch_env & ~7;
-  if (CH < 256) return SPMV_OK;
-  const size_t smem = xbytes + (size_t)XP_S * CH * (ts + 2) + fixed;
+  size_t SB = std::min<size_t>((smem_cap - xbytes - pbuf) / XP_S, 32 * 1024) & ~size_t(15);
+  int sb_env = 0;
+  if (env_int("SPMV_XPLAN_SB", &sb_env) && sb_env >= 1024 && (size_t)sb_env <= SB) SB = (size_t)sb_env & ~size_t(15);
+  const size_t smem = xbytes + XP_S * SB + pbuf;
   const double seg_mean = h->row_mean / B;
-  int G = seg_mean < 12 ? 4 : seg_mean < 48 ? 8 : 16;
+  int G = seg_mean < 12 ? 4 : seg_mean < 40 ? 8 : 16;
   int g2 = 0;
   if (env_int("SPMV_XPLAN_G", &g2) && (g2 == 4 || g2 == 8 || g2 == 16)) G = g2;
   void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? xplan_fn<double, false>(G) : xplan_fn<float, false>(G);
@@ -443,10 +438,17 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   if (env_int("SPMV_XPLAN_CLUSTERS", &nc_env) && nc_env >= 1 && nc_env <= ncl) ncl = nc_env;
   cudaStream_t s = h->stream;
   auto& P = h->xp;
-  P.B = B; P.W = W; P.CH = CH; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd;
-  // cluster row ranges (nnz-balanced)
+  auto cleanup = [&]() {
+    void* bufs[] = {P.crow, P.rec_off, P.cta_rec, P.rec_tile, P.seg, P.row_rec, P.row_pos, P.plan};
+    for (void* q : bufs)
+      if (q) cudaFree(q);
+    P = spmv_csr_s::XPlan();
+  };
+  P.B = B; P.W = W; P.SB = (int)SB; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd;
+  const int64_t m = h->m_loc;
+  // cluster row ranges (nnz-balanced) and tiles
   CK(cudaMalloc(&P.crow, sizeof(long long) * (ncl + 1)));
-  k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(h->m_loc, h->rp_loc, ncl, P.crow);
+  k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(m, h->rp_loc, ncl, P.crow);
   LAUNCHED();
   std::vector<long long> crow(ncl + 1);
   CK(cudaMemcpyAsync(crow.data(), P.crow, sizeof(long long) * (ncl + 1), cudaMemcpyDeviceToHost, s));
@@ -455,48 +457,83 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   for (int c = 0; c < ncl; ++c) tile0[c + 1] = tile0[c] + (int)cdiv(crow[c + 1] - crow[c], XP_R);
   const int ntiles = tile0[ncl];
   P.ntiles = ntiles;
-  CK(cudaMalloc(&P.tile0, sizeof(int) * (ncl + 1)));
-  CK(cudaMemcpyAsync(P.tile0, tile0.data(), sizeof(int) * (ncl + 1), cudaMemcpyHostToDevice, s));
-  // split points
+  int* d_tile0 = nullptr;
+  CK(cudaMalloc(&d_tile0, sizeof(int) * (ncl + 1)));
+  CK(cudaMemcpyAsync(d_tile0, tile0.data(), sizeof(int) * (ncl + 1), cudaMemcpyHostToDevice, s));
   if (B > 1) {
-    CK(cudaMalloc(&P.seg, sizeof(int) * (size_t)(B - 1) * (size_t)h->m_loc));
-    k_xstat_splits<<<std::min<int64_t>(cdiv(h->m_loc, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
-        h->m_loc, h->rp_loc, h->ci_loc, B, W, P.seg);
+    CK(cudaMalloc(&P.seg, sizeof(int) * (size_t)(B - 1) * (size_t)m));
+    k_xstat_splits<<<std::min<int64_t>(cdiv(m, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
+        m, h->rp_loc, h->ci_loc, B, W, P.seg);
     LAUNCHED();
   }
-  // row offsets + tile lengths
-  const size_t nTB = (size_t)std::max(ntiles, 1) * B;
-  CK(cudaMalloc(&P.rofs, sizeof(int) * nTB * (XP_R + 4)));
-  CK(cudaMalloc(&P.tlen, sizeof(int) * nTB));
-  CK(cudaMalloc(&P.toff, sizeof(long long) * nTB));
-  if (ntiles > 0) {
-    k_xplan_rofs<<<(unsigned)(ntiles * B), XP_R, 0, s>>>(h->rp_loc, P.seg, h->m_loc, B, P.crow, P.tile0, ncl,
-                                                          P.rofs, P.tlen);
-    LAUNCHED();
-  }
-  std::vector<int> tl(nTB, 0);
-  CK(cudaMemcpyAsync(tl.data(), P.tlen, sizeof(int) * nTB, cudaMemcpyDeviceToHost, s));
+  // pass 0: records and bytes per (tile, b)
+  const int64_t nTB = (int64_t)ntiles * B;
+  int *d_nrec = nullptr, *d_bad = nullptr, *d_rec_first = nullptr;
+  long long *d_bytes = nullptr, *d_byte_first = nullptr;
+  auto free_tmp = [&]() {
+    void* q[] = {d_tile0, d_nrec, d_bad, d_rec_first, d_bytes, d_byte_first};
+    for (void* x : q)
+      if (x) cudaFree(x);
+  };
+  CK(cudaMalloc(&d_nrec, sizeof(int) * std::max<int64_t>(nTB, 1)));
+  CK(cudaMalloc(&d_bytes, sizeof(long long) * std::max<int64_t>(nTB, 1)));
+  CK(cudaMalloc(&d_rec_first, sizeof(int) * std::max<int64_t>(nTB, 1)));
+  CK(cudaMalloc(&d_byte_first, sizeof(long long) * std::max<int64_t>(nTB, 1)));
+  CK(cudaMalloc(&d_bad, sizeof(int)));
+  CK(cudaMemsetAsync(d_bad, 0, sizeof(int), s));
+  const unsigned rg = (unsigned)cdiv(std::max<int64_t>(nTB, 1), 128);
+  k_xplan_records<<<rg, 128, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, d_tile0, ncl, ntiles, ts, (int)SB, 0, d_nrec,
+                                     d_bytes, nullptr, nullptr, nullptr, nullptr, nullptr, nullptr, nullptr, d_bad);
+  LAUNCHED();
+  std::vector<int> nrec(std::max<int64_t>(nTB, 1));
+  std::vector<long long> nbytes(std::max<int64_t>(nTB, 1));
+  int bad = 0;
+  CK(cudaMemcpyAsync(nrec.data(), d_nrec, sizeof(int) * nTB, cudaMemcpyDeviceToHost, s));
+  CK(cudaMemcpyAsync(nbytes.data(), d_bytes, sizeof(long long) * nTB, cudaMemcpyDeviceToHost, s));
+  CK(cudaMemcpyAsync(&bad, d_bad, sizeof(int), cudaMemcpyDeviceToHost, s));
   CK(cudaStreamSynchronize(s));
-  // padded lengths and offsets, streams of one CTA contiguous: order [c][b][t]
-  std::vector<long long> toff(nTB, 0);
+  if (bad) {  // a row segment does not fit one record: not eligible
+    free_tmp();
+    cleanup();
+    return SPMV_OK;
+  }
+  // stream order [c][b][t]: records of one CTA contiguous
+  std::vector<int> rec_first(std::max<int64_t>(nTB, 1)), cta_rec(ncl * B + 1);
+  std::vector<long long> byte_first(std::max<int64_t>(nTB, 1));
+  int rec = 0;
   long long pos = 0;
   for (int c = 0; c < ncl; ++c)
-    for (int bb = 0; bb < B; ++bb)
+    for (int bb = 0; bb < B; ++bb) {
+      cta_rec[c * B + bb] = rec;
       for (int t = tile0[c]; t < tile0[c + 1]; ++t) {
-        const size_t idx = (size_t)t * B + bb;
-        tl[idx] = (tl[idx] + 7) & ~7;
-        toff[idx] = pos;
-        pos += tl[idx];
+        const size_t id = (size_t)t * B + bb;
+        rec_first[id] = rec;
+        byte_first[id] = pos;
+        rec += nrec[id];
+        pos += nbytes[id];
       }
-  P.total = pos;
-  CK(cudaMemcpyAsync(P.tlen, tl.data(), sizeof(int) * nTB, cudaMemcpyHostToDevice, s));
-  CK(cudaMemcpyAsync(P.toff, toff.data(), sizeof(long long) * nTB, cudaMemcpyHostToDevice, s));
-  CK(cudaMalloc(&P.pv, ts * (size_t)std::max<int64_t>(pos, 8)));
-  CK(cudaMalloc(&P.pc, 2 * (size_t)std::max<int64_t>(pos, 8)));
-  CK(cudaMemsetAsync(P.pv, 0, ts * (size_t)std::max<int64_t>(pos, 8), s));
-  CK(cudaMemsetAsync(P.pc, 0, 2 * (size_t)std::max<int64_t>(pos, 8), s));
+    }
+  cta_rec[ncl * B] = rec;
+  P.nrec = rec;
+  P.bytes = pos;
+  CK(cudaMemcpyAsync(d_rec_first, rec_first.data(), sizeof(int) * nTB, cudaMemcpyHostToDevice, s));
+  CK(cudaMemcpyAsync(d_byte_first, byte_first.data(), sizeof(long long) * nTB, cudaMemcpyHostToDevice, s));
+  CK(cudaMalloc(&P.cta_rec, sizeof(int) * (ncl * B + 1)));
+  CK(cudaMemcpyAsync(P.cta_rec, cta_rec.data(), sizeof(int) * (ncl * B + 1), cudaMemcpyHostToDevice, s));
+  CK(cudaMalloc(&P.rec_off, sizeof(long long) * (rec + 1)));
+  CK(cudaMalloc(&P.rec_tile, sizeof(int) * std::max(rec, 1)));
+  CK(cudaMemcpyAsync(P.rec_off + rec, &pos, sizeof(long long), cudaMemcpyHostToDevice, s));
+  CK(cudaMalloc(&P.plan, (size_t)std::max<long long>(pos, 16)));
+  CK(cudaMemsetAsync(P.plan, 0, (size_t)std::max<long long>(pos, 16), s));
+  CK(cudaMalloc(&P.row_rec, sizeof(int) * (size_t)B * (size_t)m));
+  CK(cudaMalloc(&P.row_pos, sizeof(int) * (size_t)B * (size_t)m));
+  k_xplan_records<<<rg, 128, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, d_tile0, ncl, ntiles, ts, (int)SB, 1, d_nrec,
+                                     d_bytes, d_rec_first, d_byte_first, P.rec_off, P.rec_tile, P.plan, P.row_rec,
+                                     P.row_pos, d_bad);
+  LAUNCHED();
   ST(xplan_pack(h, h->vals, 0));
   CK(cudaStreamSynchronize(s));
+  free_tmp();
   P.built = true;
   *ok = true;
   return SPMV_OK;
@@ -761,7 +798,8 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   cudaError_t e = h->stream ? cudaStreamSynchronize(h->stream) : cudaDeviceSynchronize();
   if (e != cudaSuccess) st = cuda_fail(e, "pending asynchronous error", __LINE__);
   h->g_npb.reset();
-  void* bufs[] = {h->xp.crow, h->xp.toff, h->xp.tile0, h->xp.rofs, h->xp.tlen, h->xp.seg, h->xp.pv, h->xp.pc,
+  void* bufs[] = {h->xp.crow, h->xp.rec_off, h->xp.cta_rec, h->xp.rec_tile, h->xp.seg, h->xp.row_rec,
+                  h->xp.row_pos, h->xp.plan,
                   h->seg, h->crow, h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
                   h->stage_x, h->stage_z};
@@ -1178,7 +1216,7 @@ extern "C" spmv_status spmv_csr_info(spmv_csr_t h, spmv_info_t* info) {
   info->sorted_cols = h->sorted;
   info->grid = h->grid;
   info->cluster = h->kernel == SPMV_KERNEL_XPLAN ? h->xp.B : h->kernel == SPMV_KERNEL_XSTAT ? h->xB : 0;
-  info->plan_bytes = h->xp.built ? (int64_t)h->xp.total * (int64_t)(h->ts + 2) : 0;
+  info->plan_bytes = h->xp.built ? (int64_t)h->xp.bytes : 0;
   return SPMV_OK;
 }
 

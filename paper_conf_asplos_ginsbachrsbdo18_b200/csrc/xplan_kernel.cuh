@@ -1,93 +1,103 @@
 // xplan_kernel.cuh -- x-stationary SpMV over a column-blocked device plan of A.
 //
-// Measured on B200 (tools/microbench): random 8-B gathers run at ~1/clk/SM
-// through L1 (one wavefront per line), ~5/clk/SM from local shared memory and
-// ~0.35/clk/SM through DSMEM; TMA bulk copies sustain only ~1 request per 65
-// clk per SM, so they stream HBM at 6.6-7.2 TB/s only in chunks of >= 4 KB.
+// Measured on B200 (tools/microbench):
+//   * random 8-B gathers: ~1/clk/SM through L1 (one wavefront per line),
+//     ~5/clk/SM from local shared memory, ~0.35/clk/SM through DSMEM;
+//   * TMA bulk copies: ~1 request per 65 clk per SM; a ring of 4 x 16 KB
+//     copies per SM streams HBM at 6.7 TB/s on 120 SMs, 8 KB copies cap at
+//     ~4.5 TB/s.
 // NAS-CG rows (random columns) therefore need x in LOCAL shared memory and
-// the nonzeros in large CONTIGUOUS chunks.  The plan (built once at create --
-// the paper's device-resident "lazy copy" of A) re-lays the
-// nonzeros out so that both hold:
+// the nonzeros in large contiguous records.  The plan (built once at create:
+// the paper's device-resident "lazy copy" of A) re-lays A out:
 //
-//   clusters of B CTAs; CTA rank b holds x[b*W, (b+1)*W) in shared memory;
+//   clusters of B CTAs; CTA rank b keeps x[b*W, (b+1)*W) in shared memory;
 //   cluster c owns rows [crow[c], crow[c+1]) (nnz-balanced), cut into tiles of
-//   R rows; for every (tile, b) the entries of those rows whose column lies in
-//   block b are stored contiguously (row-major inside the tile), values in
-//   the matrix precision and columns as uint16 offsets inside the block; the
-//   streams of one CTA (all its tiles) are contiguous in HBM.
+//   R rows; for every (cluster, b) the entries of its rows whose column lies
+//   in block b form one contiguous stream of RECORDS, each <= SB bytes and
+//   holding whole rows of one tile:
+//       int32 header {tile, j0 (first row in tile), nr (rows), n (entries,
+//       multiple of 8)}, uint16 ofs[nr+1] (row starts, padded to 16 B),
+//       T vals[n], uint16 cols[n] (column offsets inside block b).
 //
-// Kernel: one producer warp streams the CTA's tiles through an S-stage ring
-// with cp.async.bulk (chunks of CH entries, mbarrier full/empty pipeline) plus
-// the per-tile row offsets; 16 consumer warps form groups of G lanes, each
-// group owns R/NG fixed rows of every tile and accumulates their partial sums
-// in registers over the chunks (deterministic order); at the end of a tile
-// the partials go to a triple-buffered shared array and, after a split
-// cluster barrier, CTA b reduces rows [b*R/B, (b+1)*R/B) of the tile over the
-// B CTAs by DSMEM reads in rank order and writes y (+ the fused CG dot).
+// Kernel (one CTA per SM, clusters of B): one producer warp streams the CTA's
+// records through S slots with one cp.async.bulk each (mbarrier full/empty);
+// slot s is consumed by its own WPS warps, which split the record's rows,
+// gather x from shared memory and write each row's block partial into a
+// triple-buffered tile array.  At a tile boundary a split cluster barrier
+// (arrive ... wait one tile later) lets CTA b sum rows [b*R/B, (b+1)*R/B) of
+// the previous tile over the B CTAs through DSMEM in rank order and write y
+// (+ the fused CG dot).  Deterministic: fixed row->lane mapping and reduction
+// order, no atomics.
 #pragma once
 #include <cooperative_groups.h>
 
 #include "common.cuh"
-#include "xstat_kernel.cuh"  // cluster/mbarrier/bulk helpers
+#include "xstat_kernel.cuh"  // cluster / mbarrier / bulk-copy helpers
 
 namespace spmv {
 
-constexpr int XP_R = 256;          // rows per tile
-constexpr int XP_CONSUMERS = 512;  // consumer threads (16 warps)
+constexpr int XP_R = 256;   // rows per tile
+constexpr int XP_S = 4;     // record slots (pipeline stages)
+constexpr int XP_WPS = 4;   // consumer warps per slot
+constexpr int XP_CONSUMERS = XP_S * XP_WPS * 32;
 constexpr int XP_THREADS = XP_CONSUMERS + 32;
-constexpr int XP_S = 4;            // pipeline stages
+constexpr int XP_HDR = 16;  // record header bytes
+
+__host__ __device__ constexpr int xp_ofs_bytes(int nr) { return ((nr + 1) * 2 + 15) & ~15; }
 
 struct XplanArgs {
-  int64_t nx;               // length of x
-  int W;                    // column block width
-  int CH;                   // entries per chunk (multiple of 8)
-  const void* pvals;        // plan values (T)
-  const uint16_t* pcols;    // plan column offsets inside the block
-  const int* rofs;          // [tile][b][R+1] row offsets inside the tile stream
-  const long long* toff;    // [tile][b] entry offset of the tile stream (multiple of 8)
-  const int* tlen;          // [tile][b] padded entry count (multiple of 8)
-  const long long* crow;    // [ncl+1] cluster row ranges
-  const int* tile0;         // [ncl+1] first global tile of each cluster
+  int64_t nx;                  // length of x
+  int W;                       // column block width
+  int SB;                      // slot bytes (max record size)
+  const unsigned char* plan;   // record streams
+  const long long* rec_off;    // [nrec+1] byte offset of every record
+  const int* rec_tile;         // [nrec] tile (within the cluster) of every record
+  const int* cta_rec;          // [ncl*B+1] first record of CTA (c, b)
+  const long long* crow;       // [ncl+1] cluster row ranges
   const void* x;
   void* y;
   double alpha, beta;
-  const void* w;            // DOT: w[i]
-  double* part;             // DOT: one partial per CTA
+  const void* w;               // DOT: w[i]
+  double* part;                // DOT: one partial per CTA
 };
 
 __device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
   asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];\n" ::"r"(smem_u32(bar)) : "memory");
 }
 
-// smem layout (dynamic): xs [W*sizeof(T) rounded to 128] | stage vals [S][CH] T |
-// stage cols [S][CH] u16 | rofs [3][R+1] int | pbuf [3][R] double
+// Cluster barrier without the GPU-scope release fence of the .release form
+// (which waits for this thread's outstanding GLOBAL stores, here the y
+// writes): shared-memory partials are published to the peers by a
+// cluster-scope fence, then a relaxed arrive.
+__device__ __forceinline__ void cluster_arrive_smem() {
+  asm volatile("fence.acq_rel.cluster;\n" ::: "memory");
+  asm volatile("barrier.cluster.arrive.relaxed.aligned;\n" ::: "memory");
+}
+
+// smem (dynamic): xs [W*sizeof(T) rounded to 128] | slots [S][SB] | pbuf [3][R] double
 template <typename T, int G, bool DOT>
 __global__ void __launch_bounds__(XP_THREADS, 1)
 k_spmv_xplan(XplanArgs a) {
   extern __shared__ __align__(128) unsigned char smem[];
-  __shared__ uint64_t full[XP_S], empty[XP_S], rbar[3], xbar;
+  __shared__ uint64_t full[XP_S], empty[XP_S], xbar;
   __shared__ double red[32];
   cgx::cluster_group cluster = cgx::this_cluster();
   const int B = (int)cluster.num_blocks();
   const int b = (int)cluster_rank();
   const int c = (int)cluster_id();
   constexpr int R = XP_R;
-  constexpr int NG = XP_CONSUMERS / G;
-  constexpr int RPG = R / NG;  // rows per group per tile
-  const int CH = a.CH;
+  const int SB = a.SB;
 
   const size_t xbytes = (size_t(a.W) * sizeof(T) + 127) & ~size_t(127);
   T* xs = reinterpret_cast<T*>(smem);
-  T* sv = reinterpret_cast<T*>(smem + xbytes);
-  uint16_t* sc = reinterpret_cast<uint16_t*>(smem + xbytes + size_t(XP_S) * CH * sizeof(T));
-  int* srofs = reinterpret_cast<int*>(smem + xbytes + size_t(XP_S) * CH * (sizeof(T) + 2));
-  double* pbuf = reinterpret_cast<double*>(smem + xbytes + size_t(XP_S) * CH * (sizeof(T) + 2) + 3 * (R + 4) * 4);
+  unsigned char* slots = smem + xbytes;
+  double* pbuf = reinterpret_cast<double*>(slots + size_t(XP_S) * SB);
 
   const int warp = threadIdx.x >> 5;
   const bool producer = warp == XP_CONSUMERS / 32;
   const int64_t r0c = a.crow[c], r1c = a.crow[c + 1];
   const int ntiles = int((r1c - r0c + R - 1) / R);
-  const int tbase = a.tile0[c];
+  const int rb = a.cta_rec[c * B + b], re = a.cta_rec[c * B + b + 1];
 
   const int64_t col0 = int64_t(b) * a.W;
   const int64_t ncols = cmax64(0, cmin64(a.W, a.nx - col0));
@@ -98,9 +108,8 @@ k_spmv_xplan(XplanArgs a) {
   if (threadIdx.x == 0) {
     for (int s = 0; s < XP_S; ++s) {
       mbar_init(&full[s], 1);
-      mbar_init(&empty[s], XP_CONSUMERS / 32);
+      mbar_init(&empty[s], XP_WPS);
     }
-    for (int s = 0; s < 3; ++s) mbar_init(&rbar[s], 1);
     mbar_init(&xbar, 1);
     asm volatile("fence.mbarrier_init.release.cluster;\n" ::: "memory");
   }
@@ -114,125 +123,96 @@ k_spmv_xplan(XplanArgs a) {
       mbar_expect_tx(&xbar, xb);
       if (xb) bulk_g2s(xs, xg + col0, xb, &xbar);
     }
-    const T* __restrict__ pv = static_cast<const T*>(a.pvals);
-    int gc = 0;  // global chunk counter of this CTA
-    for (int t = 0; t < ntiles; ++t) {
-      const int tg = tbase + t;
-      const int64_t off = a.toff[int64_t(tg) * B + b];
-      const int len = a.tlen[int64_t(tg) * B + b];
+    int t = 0;
+    for (int k = rb; k <= re; ++k) {
+      const int tk = (k < re) ? a.rec_tile[k] : ntiles;
+      for (; t < tk; ++t) {  // all records of tile t issued
+        if (t > 0) cluster_wait();
+        cluster_arrive_smem();
+      }
+      if (k == re) break;
+      const int j = k - rb, s = j % XP_S;
+      if (j >= XP_S) mbar_wait(&empty[s], ((j / XP_S) - 1) & 1);
       if (lane == 0) {
-        const int rs = t % 3;
-        // R+1 offsets, stored padded to R+4 ints (1040 B, a 16-B multiple)
-        mbar_expect_tx(&rbar[rs], uint32_t((R + 4) * 4));
-        bulk_g2s(srofs + rs * (R + 4), a.rofs + (int64_t(tg) * B + b) * (R + 4), uint32_t((R + 4) * 4), &rbar[rs]);
+        const uint32_t bytes = uint32_t(a.rec_off[k + 1] - a.rec_off[k]);
+        mbar_expect_tx(&full[s], bytes);
+        bulk_g2s(slots + size_t(s) * SB, a.plan + a.rec_off[k], bytes, &full[s]);
       }
-      for (int e0 = 0; e0 < len; e0 += CH, ++gc) {
-        const int n = min(CH, len - e0);
-        const int s = gc % XP_S;
-        if (gc >= XP_S) mbar_wait(&empty[s], ((gc / XP_S) - 1) & 1);
-        if (lane == 0) {
-          const uint32_t vb = uint32_t(n * sizeof(T)), cb = uint32_t(n * 2);
-          mbar_expect_tx(&full[s], vb + cb);
-          bulk_g2s(sv + size_t(s) * CH, pv + off + e0, vb, &full[s]);
-          bulk_g2s(sc + size_t(s) * CH, a.pcols + off + e0, cb, &full[s]);
-        }
-        __syncwarp();
-      }
-      // tile t issued
-      if (t == 0) {
-        cluster_arrive();
-      } else {
-        cluster_wait();
-        cluster_arrive();
-      }
+      __syncwarp();
     }
     if (ntiles > 0) cluster_wait();
   } else {
     // ----------------------------------------------------------- consumers
+    const int s = warp / XP_WPS, sub = warp % XP_WPS;
     const int lane = threadIdx.x & (G - 1);
     const unsigned wl = threadIdx.x & 31;
     const unsigned gmask = (G == 32) ? 0xffffffffu : (((1u << G) - 1u) << (wl & ~(unsigned)(G - 1)));
-    const int group = threadIdx.x / G;
+    const int gw = (threadIdx.x & 31) / G;  // group inside the warp
+    constexpr int GPW = 32 / G;             // groups per warp
     const double alpha = a.alpha, beta = a.beta;
     const int fin_lo = (b * R) / B, fin_hi = ((b + 1) * R) / B;
     double dacc = 0.0;
-    // tail of the x block not covered by the bulk copy
     for (int64_t j = bulk_elems + threadIdx.x; j < ncols; j += XP_CONSUMERS) xs[j] = xg[col0 + j];
     asm volatile("bar.sync 1, %0;\n" ::"r"(XP_CONSUMERS) : "memory");
     mbar_wait(&xbar, 0);
 
-    int gc = 0;
-    auto process = [&](int t) {
-      const int tg = tbase + t;
-      const int len = a.tlen[int64_t(tg) * B + b];
-      const int64_t rt = r0c + int64_t(t) * R;
-      const int nrows = int(cmin64(R, r1c - rt));
-      const int rs = t % 3;
-      mbar_wait(&rbar[rs], (t / 3) & 1);
-      const int* ro = srofs + rs * (R + 4);
-      int lo[RPG], hi[RPG];
-      double acc[RPG];
-#pragma unroll
-      for (int i = 0; i < RPG; ++i) {
-        const int j = group + i * NG;
-        lo[i] = (j < nrows) ? ro[j] : 0;
-        hi[i] = (j < nrows) ? ro[j + 1] : 0;
-        acc[i] = 0.0;
-      }
-      for (int e0 = 0; e0 < len; e0 += CH, ++gc) {
-        const int s = gc % XP_S;
-        mbar_wait(&full[s], (gc / XP_S) & 1);
-        const T* v = sv + size_t(s) * CH - e0;
-        const uint16_t* cc = sc + size_t(s) * CH - e0;
-        const int e1 = e0 + CH;
-#pragma unroll
-        for (int i = 0; i < RPG; ++i) {
-          const int l0 = max(lo[i], e0), l1 = min(hi[i], e1);
-          int e = l0 + lane;
-          for (; e + G < l1; e += 2 * G) {
-            const uint16_t c0 = cc[e], c1 = cc[e + G];
-            const T v0 = v[e], v1 = v[e + G];
-            acc[i] += double(v0) * double(xs[c0]);
-            acc[i] += double(v1) * double(xs[c1]);
-          }
-          if (e < l1) acc[i] += double(v[e]) * double(xs[cc[e]]);
-        }
-        __syncwarp();
-        if ((threadIdx.x & 31) == 0) mbar_arrive(&empty[s]);
-      }
-      double* pb = pbuf + (t % 3) * R;
-#pragma unroll
-      for (int i = 0; i < RPG; ++i) {
-        double sum = (G > 1) ? group_sum<G>(acc[i], gmask) : acc[i];
-        const int j = group + i * NG;
-        if (lane == 0 && j < nrows) pb[j] = sum;
-      }
-    };
     auto finalize = [&](int t) {
       const double* pb = pbuf + (t % 3) * R;
       const int64_t rt = r0c + int64_t(t) * R;
       const int nrows = int(cmin64(R, r1c - rt));
       for (int j = fin_lo + threadIdx.x; j < min(fin_hi, nrows); j += XP_CONSUMERS) {
-        double s = 0.0;
-        for (int q = 0; q < B; ++q) s += *cluster.map_shared_rank(pb + j, q);
+        double sum = 0.0;
+        for (int q = 0; q < B; ++q) sum += *cluster.map_shared_rank(pb + j, q);
         const int64_t i = rt + j;
         T* y = static_cast<T*>(a.y);
-        double r = alpha * s;
+        double r = alpha * sum;
         if (beta != 0.0) r += beta * double(y[i]);
         const T out = T(r);
         y[i] = out;
         if (DOT) dacc += double(static_cast<const T*>(a.w)[i]) * double(out);
       }
     };
-    if (ntiles > 0) {
-      process(0);
-      cluster_arrive();
-      for (int t = 1; t < ntiles; ++t) {
-        process(t);
-        cluster_wait();
-        finalize(t - 1);
-        cluster_arrive();
+    // every row of a tile lies in exactly one record of this CTA (empty
+    // segments included), so each pbuf entry is written before it is read.
+    int t = 0;
+    for (int k = rb + s; ; k += XP_S) {
+      const int tk = (k < re) ? a.rec_tile[k] : ntiles;
+      for (; t < tk; ++t) {  // tile boundary after tile t
+        if (t > 0) {
+          cluster_wait();
+          finalize(t - 1);
+        }
+        cluster_arrive_smem();
       }
+      if (k >= re) break;
+      const int j = k - rb;
+      mbar_wait(&full[s], (j / XP_S) & 1);
+      const unsigned char* rec = slots + size_t(s) * SB;
+      const int* hdr = reinterpret_cast<const int*>(rec);
+      const int j0 = hdr[1], nr = hdr[2], n = hdr[3];
+      const uint16_t* ofs = reinterpret_cast<const uint16_t*>(rec + XP_HDR);
+      const T* v = reinterpret_cast<const T*>(rec + XP_HDR + xp_ofs_bytes(nr));
+      const uint16_t* cc = reinterpret_cast<const uint16_t*>(rec + XP_HDR + xp_ofs_bytes(nr) + size_t(n) * sizeof(T));
+      double* pb = pbuf + (hdr[0] % 3) * R;
+      // rows r = sub*GPW + gw + m*(WPS*GPW)
+      for (int r = sub * GPW + gw; r < nr; r += XP_WPS * GPW) {
+        const int e0 = ofs[r], e1 = ofs[r + 1];
+        double acc = 0.0;
+        int e = e0 + lane;
+        for (; e + G < e1; e += 2 * G) {
+          const uint16_t c0 = cc[e], c1 = cc[e + G];
+          const T v0 = v[e], v1 = v[e + G];
+          acc += double(v0) * double(xs[c0]);
+          acc += double(v1) * double(xs[c1]);
+        }
+        if (e < e1) acc += double(v[e]) * double(xs[cc[e]]);
+        if (G > 1) acc = group_sum<G>(acc, gmask);
+        if (lane == 0) pb[j0 + r] = acc;
+      }
+      __syncwarp();
+      if ((threadIdx.x & 31) == 0) mbar_arrive(&empty[s]);
+    }
+    if (ntiles > 0) {
       cluster_wait();
       finalize(ntiles - 1);
     }
@@ -247,70 +227,117 @@ k_spmv_xplan(XplanArgs a) {
 }
 
 // ---------------------------------------------------------------- builders
-// Per (tile, b): row lengths inside block b -> row offsets (exclusive scan)
-// and the tile's entry count.  One CTA (R threads) per (global tile, b).
-__global__ void __launch_bounds__(XP_R)
-k_xplan_rofs(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_t m, int B,
-             const long long* __restrict__ crow, const int* __restrict__ tile0, int ncl,
-             int* __restrict__ rofs, int* __restrict__ tlen_raw) {
-  __shared__ int sc[XP_R];
-  const int tg = blockIdx.x / B, b = blockIdx.x % B;
+// Row segment [k0, k1) of row i in column block b.
+__device__ __forceinline__ void xp_seg(const int* rowptr, const int* seg, int64_t m, int B, int b, int64_t i,
+                                       int* k0, int* k1) {
+  *k0 = (b == 0) ? rowptr[i] : seg[int64_t(b - 1) * m + i];
+  *k1 = (b == B - 1) ? rowptr[i + 1] : seg[int64_t(b) * m + i];
+}
+
+__device__ __forceinline__ int xp_rec_bytes(int nr, int n, int ts) {
+  return XP_HDR + xp_ofs_bytes(nr) + n * ts + n * 2;
+}
+
+// Greedy cut of the rows of (tile, b) into records of <= SB bytes, whole rows
+// only.  pass 0: counts records and bytes (too-long row -> *bad = 1);
+// pass 1: writes headers/offsets, the record table and every row's
+// (record, position) for the pack kernel.  One thread per (tile, b).
+__global__ void k_xplan_records(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_t m, int B,
+                                const long long* __restrict__ crow, const int* __restrict__ tile0, int ncl,
+                                int ntiles, int ts, int SB, int pass, int* __restrict__ nrec,
+                                long long* __restrict__ bytes, const int* __restrict__ rec_first,
+                                const long long* __restrict__ byte_first, long long* __restrict__ rec_off,
+                                int* __restrict__ rec_tile, unsigned char* __restrict__ plan,
+                                int* __restrict__ row_rec, int* __restrict__ row_pos, int* __restrict__ bad) {
+  const int64_t id = int64_t(blockIdx.x) * blockDim.x + threadIdx.x;
+  if (id >= int64_t(ntiles) * B) return;
+  const int tg = int(id / B), b = int(id % B);
   int c = 0;
   while (c + 1 < ncl && tile0[c + 1] <= tg) ++c;
   const int t = tg - tile0[c];
   const int64_t rt = crow[c] + int64_t(t) * XP_R;
   const int nrows = int(cmin64(XP_R, crow[c + 1] - rt));
-  const int j = threadIdx.x;
-  int L = 0;
-  if (j < nrows) {
-    const int64_t i = rt + j;
-    const int k0 = (b == 0) ? rowptr[i] : seg[int64_t(b - 1) * m + i];
-    const int k1 = (b == B - 1) ? rowptr[i + 1] : seg[int64_t(b) * m + i];
-    L = k1 - k0;
+  int cnt = 0;
+  long long tot = 0;
+  int r = 0;
+  int rec = pass ? rec_first[id] : 0;
+  long long off = pass ? byte_first[id] : 0;
+  while (r < nrows) {
+    // grow a record from row r
+    int nr = 0, n = 0;
+    while (r + nr < nrows) {
+      int k0, k1;
+      xp_seg(rowptr, seg, m, B, b, rt + r + nr, &k0, &k1);
+      const int L = k1 - k0;
+      const int n2 = (n + L + 7) & ~7;
+      if (xp_rec_bytes(nr + 1, n2, ts) > SB) {
+        if (nr == 0) { atomicExch(bad, 1); return; }
+        break;
+      }
+      n += L;
+      ++nr;
+    }
+    const int np = (n + 7) & ~7;
+    const int nb = xp_rec_bytes(nr, np, ts);
+    if (pass) {
+      unsigned char* p = plan + off;
+      int* hdr = reinterpret_cast<int*>(p);
+      hdr[0] = t;
+      hdr[1] = r;
+      hdr[2] = nr;
+      hdr[3] = np;
+      uint16_t* ofs = reinterpret_cast<uint16_t*>(p + XP_HDR);
+      int e = 0;
+      for (int q = 0; q < nr; ++q) {
+        int k0, k1;
+        xp_seg(rowptr, seg, m, B, b, rt + r + q, &k0, &k1);
+        ofs[q] = uint16_t(e);
+        row_rec[int64_t(b) * m + rt + r + q] = rec;
+        row_pos[int64_t(b) * m + rt + r + q] = e;
+        e += k1 - k0;
+      }
+      ofs[nr] = uint16_t(e);
+      rec_off[rec] = off;
+      rec_tile[rec] = t;
+      ++rec;
+      off += nb;
+    }
+    ++cnt;
+    tot += nb;
+    r += nr;
   }
-  sc[j] = L;
-  __syncthreads();
-  for (int d = 1; d < XP_R; d <<= 1) {  // inclusive Hillis-Steele scan
-    const int v = (j >= d) ? sc[j - d] : 0;
-    __syncthreads();
-    sc[j] += v;
-    __syncthreads();
+  if (!pass) {
+    nrec[id] = cnt;
+    bytes[id] = tot;
   }
-  int* ro = rofs + (int64_t(tg) * B + b) * (XP_R + 4);
-  ro[j + 1] = sc[j];
-  if (j == 0) ro[0] = 0;
-  if (j < 3) ro[XP_R + 1 + j] = sc[XP_R - 1];  // padding of the 16-B copy
-  if (j == XP_R - 1) tlen_raw[int64_t(tg) * B + b] = sc[j];
 }
 
-// Scatter every nonzero into its (tile, block) stream: warp per row.
+// Scatter every nonzero into its record: warp per row.
 template <typename T>
 __global__ void __launch_bounds__(256)
 k_xplan_pack(const int* __restrict__ rowptr, const int* __restrict__ colidx, const T* __restrict__ vals,
-             const int* __restrict__ seg, int64_t m, int B, int W, const long long* __restrict__ crow,
-             const int* __restrict__ tile0, int ncl, const int* __restrict__ rofs,
-             const long long* __restrict__ toff, T* __restrict__ pv, uint16_t* __restrict__ pc, int values_only) {
+             const int* __restrict__ seg, int64_t m, int B, int W, const long long* __restrict__ rec_off,
+             const int* __restrict__ row_rec, const int* __restrict__ row_pos, unsigned char* __restrict__ plan,
+             int values_only) {
   const int lane = threadIdx.x & 31;
   for (int64_t i = (int64_t(blockIdx.x) * blockDim.x + threadIdx.x) / 32; i < m;
        i += int64_t(gridDim.x) * blockDim.x / 32) {
-    // cluster of row i (binary search in crow) and its tile
-    int lo = 0, hi = ncl - 1;
-    while (lo < hi) {
-      const int mid = (lo + hi + 1) >> 1;
-      if (crow[mid] <= i) lo = mid; else hi = mid - 1;
-    }
-    const int c = lo;
-    const int t = int((i - crow[c]) / XP_R);
-    const int j = int((i - crow[c]) % XP_R);
-    const int tg = tile0[c] + t;
     const int k0 = rowptr[i], k1 = rowptr[i + 1];
     for (int k = k0 + lane; k < k1; k += 32) {
       const int col = colidx[k];
       const int bb = col / W;
       const int s0 = (bb == 0) ? k0 : seg[int64_t(bb - 1) * m + i];
-      const int64_t dst = toff[int64_t(tg) * B + bb] + rofs[(int64_t(tg) * B + bb) * (XP_R + 4) + j] + (k - s0);
-      pv[dst] = vals[k];
-      if (!values_only) pc[dst] = uint16_t(col - bb * W);
+      const int rec = row_rec[int64_t(bb) * m + i];
+      unsigned char* p = plan + rec_off[rec];
+      const int* hdr = reinterpret_cast<const int*>(p);
+      const int nr = hdr[2], n = hdr[3];
+      const int pos = row_pos[int64_t(bb) * m + i] + (k - s0);
+      T* v = reinterpret_cast<T*>(p + XP_HDR + xp_ofs_bytes(nr));
+      v[pos] = vals[k];
+      if (!values_only) {
+        uint16_t* cc = reinterpret_cast<uint16_t*>(p + XP_HDR + xp_ofs_bytes(nr) + size_t(n) * sizeof(T));
+        cc[pos] = uint16_t(col - bb * W);
+      }
     }
   }
 }

@@ -220,7 +220,7 @@ def test_nas_full_size(sp, torch_dev, cls):
     A = gen.makea(cls)
     x = gen.uniform(A.n, seed=31)
     info = run_case(sp, torch, dev, A, x, what=f"NAS {cls}")
-    assert info["kernel_name"] in ("vector", "merge", "xstat", "scalar")
+    assert info["kernel_name"] in ("vector", "merge", "xstat", "xplan", "scalar")
 
 
 def test_parboil_full_size_fp32(sp, torch_dev):
@@ -275,14 +275,15 @@ def test_xstat_alpha_beta_and_offset(sp, torch_dev):
 
 
 @pytest.mark.parametrize("cfg", [{}, {"SPMV_XPLAN_B": "2"}, {"SPMV_XPLAN_B": "8"}, {"SPMV_XPLAN_G": "4"},
-                                 {"SPMV_XPLAN_G": "16", "SPMV_XPLAN_B": "4"}, {"SPMV_XPLAN_CH": "64"},
-                                 {"SPMV_XPLAN_CLUSTERS": "1", "SPMV_XPLAN_CH": "256"}])
+                                 {"SPMV_XPLAN_G": "16", "SPMV_XPLAN_B": "4"}, {"SPMV_XPLAN_SB": "2048"},
+                                 {"SPMV_XPLAN_CLUSTERS": "1", "SPMV_XPLAN_SB": "4096"}])
 @pytest.mark.parametrize("name,A", ZOO, ids=[c[0] for c in ZOO])
 def test_zoo_xplan(sp, torch_dev, name, A, cfg, monkeypatch):
     """x-stationary kernel over the column-blocked plan (TMA bulk pipeline,
-    clusters, DSMEM reduction): cluster sizes, lane groups, tiny chunks (many
-    chunks per tile, rows split across chunks) and a single cluster (many
-    tiles: exercises the triple-buffered partials and the split barrier)."""
+    clusters, DSMEM reduction): cluster sizes, lane groups, small records
+    (many records per tile; rows that do not fit a record make the plan
+    ineligible -> zero-copy fallback) and a single cluster (many tiles:
+    exercises the triple-buffered partials and the split barrier)."""
     torch, dev = torch_dev
     for k, v in cfg.items():
         monkeypatch.setenv(k, v)
@@ -293,7 +294,7 @@ def test_zoo_xplan(sp, torch_dev, name, A, cfg, monkeypatch):
     starts[A.rowptr[:-1]] = True
     inner = ~starts[k]
     sorted_cols = bool(np.all(A.colidx[k][inner] > A.colidx[k - 1][inner]))
-    if sorted_cols and A.nnz > 0:
+    if sorted_cols and A.nnz > 0 and "SPMV_XPLAN_SB" not in cfg:
         assert info["kernel_name"] == "xplan", info
         assert info["plan_bytes"] >= A.nnz * 10
     A32 = A.astype(np.float32)
