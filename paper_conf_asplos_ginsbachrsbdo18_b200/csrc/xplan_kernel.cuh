@@ -23,11 +23,14 @@
 // records through S slots with one cp.async.bulk each (mbarrier full/empty);
 // slot s is consumed by its own WPS warps, which split the record's rows,
 // gather x from shared memory and write each row's block partial into a
-// triple-buffered tile array.  At a tile boundary a split cluster barrier
-// (arrive ... wait one tile later) lets CTA b sum rows [b*R/B, (b+1)*R/B) of
-// the previous tile over the B CTAs through DSMEM in rank order and write y
-// (+ the fused CG dot).  Deterministic: fixed row->lane mapping and reduction
-// order, no atomics.
+// triple-buffered receive array of the CTA that owns the row (rows
+// [q*R/B, (q+1)*R/B) of a tile belong to CTA q) with st.async, which completes
+// transaction bytes on the owner's mbarrier of that tile.  The owner waits for
+// all B partials of its rows, sums them in rank order and writes y (+ the
+// fused CG dot).  A relaxed split cluster barrier (arrive after tile t, wait
+// after tile t+1) bounds how far a CTA may run ahead, so a receive buffer is
+// never overwritten before its tile was reduced.  No fences on the steady
+// path, deterministic (fixed row->lane mapping and summation order).
 #pragma once
 #include <cooperative_groups.h>
 
@@ -65,21 +68,33 @@ __device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
   asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];\n" ::"r"(smem_u32(bar)) : "memory");
 }
 
-// Cluster barrier without the GPU-scope release fence of the .release form
-// (which waits for this thread's outstanding GLOBAL stores, here the y
-// writes): shared-memory partials are published to the peers by a
-// cluster-scope fence, then a relaxed arrive.
-__device__ __forceinline__ void cluster_arrive_smem() {
-  asm volatile("fence.acq_rel.cluster;\n" ::: "memory");
+// Relaxed cluster-barrier arrive: no memory ordering (the .release form and
+// fence.acq_rel.cluster both lower to MEMBAR.ALL.GPU, which waits for every
+// outstanding global store).  Used only for buffer back-pressure; the row
+// partials travel by st.async with mbarrier transaction counts.
+__device__ __forceinline__ void cluster_arrive_relaxed() {
   asm volatile("barrier.cluster.arrive.relaxed.aligned;\n" ::: "memory");
 }
+__device__ __forceinline__ uint32_t mapa_u32(uint32_t laddr, uint32_t rank) {
+  uint32_t r;
+  asm volatile("mapa.shared::cluster.u32 %0, %1, %2;\n" : "=r"(r) : "r"(laddr), "r"(rank));
+  return r;
+}
+// 8-byte store into a peer CTA's shared memory that completes `bytes` on the
+// peer's mbarrier (no fence needed, the mbarrier phase orders it).
+__device__ __forceinline__ void st_async_f64(uint32_t raddr, double v, uint32_t rbar) {
+  asm volatile("st.async.shared::cluster.mbarrier::complete_tx::bytes.b64 [%0], %1, [%2];\n" ::"r"(raddr),
+               "l"(__double_as_longlong(v)), "r"(rbar)
+               : "memory");
+}
 
-// smem (dynamic): xs [W*sizeof(T) rounded to 128] | slots [S][SB] | pbuf [3][R] double
+// smem (dynamic): xs [W*sizeof(T) rounded to 128] | slots [S][SB] | recv [3][R] double
+//                 (recv[t%3][b*(R/B) + jl]: partial of CTA b for owned row jl)
 template <typename T, int G, bool DOT>
 __global__ void __launch_bounds__(XP_THREADS, 1)
 k_spmv_xplan(XplanArgs a) {
   extern __shared__ __align__(128) unsigned char smem[];
-  __shared__ uint64_t full[XP_S], empty[XP_S], xbar;
+  __shared__ uint64_t full[XP_S], empty[XP_S], xbar, tbar[3];
   __shared__ double red[32];
   cgx::cluster_group cluster = cgx::this_cluster();
   const int B = (int)cluster.num_blocks();
@@ -91,7 +106,8 @@ k_spmv_xplan(XplanArgs a) {
   const size_t xbytes = (size_t(a.W) * sizeof(T) + 127) & ~size_t(127);
   T* xs = reinterpret_cast<T*>(smem);
   unsigned char* slots = smem + xbytes;
-  double* pbuf = reinterpret_cast<double*>(slots + size_t(XP_S) * SB);
+  double* recv = reinterpret_cast<double*>(slots + size_t(XP_S) * SB);
+  const int RB = R / B;  // rows of a tile owned by each CTA
 
   const int warp = threadIdx.x >> 5;
   const bool producer = warp == XP_CONSUMERS / 32;
@@ -111,9 +127,22 @@ k_spmv_xplan(XplanArgs a) {
       mbar_init(&empty[s], XP_WPS);
     }
     mbar_init(&xbar, 1);
+    for (int q = 0; q < 3; ++q) mbar_init(&tbar[q], 1);
     asm volatile("fence.mbarrier_init.release.cluster;\n" ::: "memory");
   }
   __syncthreads();
+  // bytes of partials this CTA receives for tile t: B per owned existing row
+  auto recv_bytes = [&](int t) -> uint32_t {
+    const int nrows = int(cmin64(R, r1c - (r0c + int64_t(t) * R)));
+    const int own = max(0, min((b + 1) * RB, nrows) - b * RB);
+    return uint32_t(own * B * 8);
+  };
+  if (threadIdx.x == 0)
+    for (int t = 0; t < 3 && t < ntiles; ++t) mbar_expect_tx(&tbar[t], recv_bytes(t));
+  // every CTA of the cluster must have initialised its barriers before peers
+  // send partials to it
+  cluster_arrive();
+  cluster_wait();
 
   if (producer) {
     // ------------------------------------------------------------ producer
@@ -128,7 +157,7 @@ k_spmv_xplan(XplanArgs a) {
       const int tk = (k < re) ? a.rec_tile[k] : ntiles;
       for (; t < tk; ++t) {  // all records of tile t issued
         if (t > 0) cluster_wait();
-        cluster_arrive_smem();
+        cluster_arrive_relaxed();
       }
       if (k == re) break;
       const int j = k - rb, s = j % XP_S;
@@ -157,13 +186,14 @@ k_spmv_xplan(XplanArgs a) {
     mbar_wait(&xbar, 0);
 
     auto finalize = [&](int t) {
-      const double* pb = pbuf + (t % 3) * R;
+      const double* rv = recv + (t % 3) * R;
       const int64_t rt = r0c + int64_t(t) * R;
       const int nrows = int(cmin64(R, r1c - rt));
-      for (int j = fin_lo + threadIdx.x; j < min(fin_hi, nrows); j += XP_CONSUMERS) {
+      mbar_wait(&tbar[t % 3], (t / 3) & 1);
+      for (int jl = threadIdx.x; jl < RB && b * RB + jl < nrows; jl += XP_CONSUMERS) {
         double sum = 0.0;
-        for (int q = 0; q < B; ++q) sum += *cluster.map_shared_rank(pb + j, q);
-        const int64_t i = rt + j;
+        for (int q = 0; q < B; ++q) sum += rv[q * RB + jl];
+        const int64_t i = rt + b * RB + jl;
         T* y = static_cast<T*>(a.y);
         double r = alpha * sum;
         if (beta != 0.0) r += beta * double(y[i]);
@@ -171,20 +201,25 @@ k_spmv_xplan(XplanArgs a) {
         y[i] = out;
         if (DOT) dacc += double(static_cast<const T*>(a.w)[i]) * double(out);
       }
+      // re-arm the buffer for tile t+3 (its partials can only arrive after
+      // this CTA's next arrive, see the barrier argument above)
+      asm volatile("bar.sync 1, %0;\n" ::"r"(XP_CONSUMERS) : "memory");
+      if (threadIdx.x == 0 && t + 3 < ntiles) mbar_expect_tx(&tbar[t % 3], recv_bytes(t + 3));
     };
     // every row of a tile lies in exactly one record of this CTA (empty
     // segments included), so each pbuf entry is written before it is read.
     int t = 0;
+    int tk = (rb + s < re) ? a.rec_tile[rb + s] : ntiles;
     for (int k = rb + s; ; k += XP_S) {
-      const int tk = (k < re) ? a.rec_tile[k] : ntiles;
       for (; t < tk; ++t) {  // tile boundary after tile t
         if (t > 0) {
           cluster_wait();
           finalize(t - 1);
         }
-        cluster_arrive_smem();
+        cluster_arrive_relaxed();
       }
       if (k >= re) break;
+      const int tk_next = (k + XP_S < re) ? a.rec_tile[k + XP_S] : ntiles;  // prefetch
       const int j = k - rb;
       mbar_wait(&full[s], (j / XP_S) & 1);
       const unsigned char* rec = slots + size_t(s) * SB;
@@ -193,7 +228,8 @@ k_spmv_xplan(XplanArgs a) {
       const uint16_t* ofs = reinterpret_cast<const uint16_t*>(rec + XP_HDR);
       const T* v = reinterpret_cast<const T*>(rec + XP_HDR + xp_ofs_bytes(nr));
       const uint16_t* cc = reinterpret_cast<const uint16_t*>(rec + XP_HDR + xp_ofs_bytes(nr) + size_t(n) * sizeof(T));
-      double* pb = pbuf + (hdr[0] % 3) * R;
+      const uint32_t rbase = smem_u32(recv + (hdr[0] % 3) * R + b * RB);
+      const uint32_t rbar_l = smem_u32(&tbar[hdr[0] % 3]);
       // rows r = sub*GPW + gw + m*(WPS*GPW)
       for (int r = sub * GPW + gw; r < nr; r += XP_WPS * GPW) {
         const int e0 = ofs[r], e1 = ofs[r + 1];
@@ -207,10 +243,15 @@ k_spmv_xplan(XplanArgs a) {
         }
         if (e < e1) acc += double(v[e]) * double(xs[cc[e]]);
         if (G > 1) acc = group_sum<G>(acc, gmask);
-        if (lane == 0) pb[j0 + r] = acc;
+        if (lane == 0) {
+          const int j = j0 + r, q = j / RB, jl = j - q * RB;
+          // same layout in every CTA: slot [t%3][b*RB + jl] of the owner q
+          st_async_f64(mapa_u32(rbase + uint32_t(jl * 8), q), acc, mapa_u32(rbar_l, q));
+        }
       }
       __syncwarp();
       if ((threadIdx.x & 31) == 0) mbar_arrive(&empty[s]);
+      tk = tk_next;
     }
     if (ntiles > 0) {
       cluster_wait();
