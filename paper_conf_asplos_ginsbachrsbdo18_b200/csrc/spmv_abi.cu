@@ -113,14 +113,15 @@ struct spmv_csr_s {
   long long* crow = nullptr;
   void (*xk)(XstatArgs) = nullptr;
   void (*xk_dot)(XstatArgs) = nullptr;
-  // XPLAN (column-blocked device plan of A)
+  // XPLAN (column-blocked SELL-32 device plan of A)
   struct XPlan {
     bool built = false;
-    int B = 0, W = 0, SB = 0, ncl = 0, ntiles = 0, nrec = 0;
+    int B = 0, W = 0, ncl = 0, ntiles = 0;
     size_t smem = 0;
-    int64_t bytes = 0;
-    long long *crow = nullptr, *rec_off = nullptr;
-    int *cta_rec = nullptr, *rec_tile = nullptr, *seg = nullptr, *row_rec = nullptr, *row_pos = nullptr;
+    int64_t bytes = 0, nchunks = 0;
+    long long *crow = nullptr, *chunk_off = nullptr;
+    int *tile0 = nullptr, *chunk_len = nullptr, *seg = nullptr, *row_slot = nullptr;
+    uint16_t* chunk_row = nullptr;
     unsigned char* plan = nullptr;
     void (*k)(XplanArgs) = nullptr;
     void (*kdot)(XplanArgs) = nullptr;
@@ -326,26 +327,17 @@ static spmv_status xstat_setup(spmv_csr_s* h, bool* ok) {
   return SPMV_OK;
 }
 
-template <typename T, bool DOT>
-static void (*xplan_fn(int G))(XplanArgs) {
-  switch (G) {
-    case 4: return k_spmv_xplan<T, 4, DOT>;
-    case 16: return k_spmv_xplan<T, 16, DOT>;
-    default: return k_spmv_xplan<T, 8, DOT>;
-  }
-}
-
 static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha,
                                 double beta, const double* w, double* part) {
   XplanArgs a;
   a.nx = h->nx;
   a.W = h->xp.W;
-  a.SB = h->xp.SB;
   a.plan = h->xp.plan;
-  a.rec_off = h->xp.rec_off;
-  a.rec_tile = h->xp.rec_tile;
-  a.cta_rec = h->xp.cta_rec;
+  a.chunk_off = h->xp.chunk_off;
+  a.chunk_len = h->xp.chunk_len;
+  a.chunk_row = h->xp.chunk_row;
   a.crow = h->xp.crow;
+  a.tile0 = h->xp.tile0;
   a.x = x;
   a.y = y;
   a.alpha = alpha;
@@ -373,32 +365,32 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   return SPMV_OK;
 }
 
-// Pack (or re-pack, values_only) the nonzeros into the plan records.
+// Pack (or re-pack, values_only) the nonzeros into the plan chunks.
 static spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only) {
   cudaStream_t s = h->stream;
+  auto& P = h->xp;
   const int64_t g = std::min<int64_t>(cdiv(h->m_loc * 32, 256), 16LL * num_sms(h->device));
   if (h->dt == SPMV_F64)
-    k_xplan_pack<double><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const double*)vals, h->xp.seg, h->m_loc,
-                                          h->xp.B, h->xp.W, h->xp.rec_off, h->xp.row_rec, h->xp.row_pos,
-                                          h->xp.plan, values_only);
+    k_xplan_pack<double><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const double*)vals, P.seg, h->m_loc, P.B, P.W,
+                                          P.crow, P.tile0, P.ncl, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
+                                          values_only);
   else
-    k_xplan_pack<float><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const float*)vals, h->xp.seg, h->m_loc,
-                                         h->xp.B, h->xp.W, h->xp.rec_off, h->xp.row_rec, h->xp.row_pos,
-                                         h->xp.plan, values_only);
+    k_xplan_pack<float><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const float*)vals, P.seg, h->m_loc, P.B, P.W,
+                                         P.crow, P.tile0, P.ncl, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
+                                         values_only);
   LAUNCHED();
   return SPMV_OK;
 }
 
-// Build the column-blocked plan (create).  *ok = false if not eligible.
+// Build the column-blocked SELL-32 plan (create).  *ok = false if not eligible.
 static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   *ok = false;
   if (!h->sorted || h->m_loc == 0 || h->nx == 0 || h->k1 - h->k0 == 0) return SPMV_OK;
   const int ts = (int)h->ts;
   const size_t smem_cap = 227 * 1024 - 1024;  // dynamic smem a CTA may use (static < 1 KB)
-  const size_t pbuf = 3 * (size_t)XP_R * 8;
-  const size_t sb_min = 16 * 1024;
-  if (smem_cap <= pbuf + XP_S * sb_min) return SPMV_OK;
-  const size_t xbudget = smem_cap - pbuf - XP_S * sb_min;
+  const size_t recv = (size_t)XP_K * XP_R * 8;
+  if (smem_cap <= recv + 1024) return SPMV_OK;
+  const size_t xbudget = smem_cap - recv - 64;
   int B = (int)cdiv((int64_t)(ts * h->nx), (int64_t)xbudget);
   B = B <= 1 ? 1 : B <= 2 ? 2 : B <= 4 ? 4 : B <= 8 ? 8 : 16;
   int forced = 0;
@@ -406,18 +398,11 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   if (B > 8) return SPMV_OK;
   int W = (int)cdiv(h->nx, B);
   W = (W + 7) & ~7;
-  if (W > 65535) return SPMV_OK;
-  const size_t xbytes = ((size_t)W * ts + 127) & ~size_t(127);
-  size_t SB = std::min<size_t>((smem_cap - xbytes - pbuf) / XP_S, 32 * 1024) & ~size_t(15);
-  int sb_env = 0;
-  if (env_int("SPMV_XPLAN_SB", &sb_env) && sb_env >= 1024 && (size_t)sb_env <= SB) SB = (size_t)sb_env & ~size_t(15);
-  const size_t smem = xbytes + XP_S * SB + pbuf;
-  const double seg_mean = h->row_mean / B;
-  int G = seg_mean < 12 ? 4 : seg_mean < 40 ? 8 : 16;
-  int g2 = 0;
-  if (env_int("SPMV_XPLAN_G", &g2) && (g2 == 4 || g2 == 8 || g2 == 16)) G = g2;
-  void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? xplan_fn<double, false>(G) : xplan_fn<float, false>(G);
-  void (*fnd)(XplanArgs) = h->dt == SPMV_F64 ? xplan_fn<double, true>(G) : nullptr;
+  if (W > 65534) return SPMV_OK;  // 16-bit column offsets, pad column W
+  const size_t xbytes = ((size_t)(W + 1) * ts + 15) & ~size_t(15);
+  const size_t smem = xbytes + recv;
+  void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, false> : k_spmv_xplan<float, false>;
+  void (*fnd)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, true> : nullptr;
   CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
   if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
   cudaLaunchConfig_t cfg = {};
@@ -439,14 +424,13 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   cudaStream_t s = h->stream;
   auto& P = h->xp;
   auto cleanup = [&]() {
-    void* bufs[] = {P.crow, P.rec_off, P.cta_rec, P.rec_tile, P.seg, P.row_rec, P.row_pos, P.plan};
+    void* bufs[] = {P.crow, P.chunk_off, P.tile0, P.chunk_len, P.seg, P.row_slot, P.chunk_row, P.plan};
     for (void* q : bufs)
       if (q) cudaFree(q);
     P = spmv_csr_s::XPlan();
   };
-  P.B = B; P.W = W; P.SB = (int)SB; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd;
+  P.B = B; P.W = W; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd;
   const int64_t m = h->m_loc;
-  // cluster row ranges (nnz-balanced) and tiles
   CK(cudaMalloc(&P.crow, sizeof(long long) * (ncl + 1)));
   k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(m, h->rp_loc, ncl, P.crow);
   LAUNCHED();
@@ -457,83 +441,59 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   for (int c = 0; c < ncl; ++c) tile0[c + 1] = tile0[c] + (int)cdiv(crow[c + 1] - crow[c], XP_R);
   const int ntiles = tile0[ncl];
   P.ntiles = ntiles;
-  int* d_tile0 = nullptr;
-  CK(cudaMalloc(&d_tile0, sizeof(int) * (ncl + 1)));
-  CK(cudaMemcpyAsync(d_tile0, tile0.data(), sizeof(int) * (ncl + 1), cudaMemcpyHostToDevice, s));
+  CK(cudaMalloc(&P.tile0, sizeof(int) * (ncl + 1)));
+  CK(cudaMemcpyAsync(P.tile0, tile0.data(), sizeof(int) * (ncl + 1), cudaMemcpyHostToDevice, s));
   if (B > 1) {
     CK(cudaMalloc(&P.seg, sizeof(int) * (size_t)(B - 1) * (size_t)m));
     k_xstat_splits<<<std::min<int64_t>(cdiv(m, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
         m, h->rp_loc, h->ci_loc, B, W, P.seg);
     LAUNCHED();
   }
-  // pass 0: records and bytes per (tile, b)
-  const int64_t nTB = (int64_t)ntiles * B;
-  int *d_nrec = nullptr, *d_bad = nullptr, *d_rec_first = nullptr;
-  long long *d_bytes = nullptr, *d_byte_first = nullptr;
-  auto free_tmp = [&]() {
-    void* q[] = {d_tile0, d_nrec, d_bad, d_rec_first, d_bytes, d_byte_first};
-    for (void* x : q)
-      if (x) cudaFree(x);
-  };
-  CK(cudaMalloc(&d_nrec, sizeof(int) * std::max<int64_t>(nTB, 1)));
-  CK(cudaMalloc(&d_bytes, sizeof(long long) * std::max<int64_t>(nTB, 1)));
-  CK(cudaMalloc(&d_rec_first, sizeof(int) * std::max<int64_t>(nTB, 1)));
-  CK(cudaMalloc(&d_byte_first, sizeof(long long) * std::max<int64_t>(nTB, 1)));
-  CK(cudaMalloc(&d_bad, sizeof(int)));
-  CK(cudaMemsetAsync(d_bad, 0, sizeof(int), s));
-  const unsigned rg = (unsigned)cdiv(std::max<int64_t>(nTB, 1), 128);
-  k_xplan_records<<<rg, 128, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, d_tile0, ncl, ntiles, ts, (int)SB, 0, d_nrec,
-                                     d_bytes, nullptr, nullptr, nullptr, nullptr, nullptr, nullptr, nullptr, d_bad);
-  LAUNCHED();
-  std::vector<int> nrec(std::max<int64_t>(nTB, 1));
-  std::vector<long long> nbytes(std::max<int64_t>(nTB, 1));
-  int bad = 0;
-  CK(cudaMemcpyAsync(nrec.data(), d_nrec, sizeof(int) * nTB, cudaMemcpyDeviceToHost, s));
-  CK(cudaMemcpyAsync(nbytes.data(), d_bytes, sizeof(long long) * nTB, cudaMemcpyDeviceToHost, s));
-  CK(cudaMemcpyAsync(&bad, d_bad, sizeof(int), cudaMemcpyDeviceToHost, s));
+  const int64_t nch = (int64_t)ntiles * B * XP_NW;
+  P.nchunks = nch;
+  CK(cudaMalloc(&P.chunk_len, sizeof(int) * std::max<int64_t>(nch, 1)));
+  CK(cudaMalloc(&P.chunk_off, sizeof(long long) * std::max<int64_t>(nch, 1)));
+  CK(cudaMalloc(&P.chunk_row, sizeof(uint16_t) * 32 * std::max<int64_t>(nch, 1)));
+  CK(cudaMalloc(&P.row_slot, sizeof(int) * (size_t)B * (size_t)m));
+  if (ntiles > 0) {
+    k_xplan_sell<<<(unsigned)(ntiles * B), XP_R, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, P.tile0, ncl, P.chunk_len,
+                                                          P.chunk_row, P.row_slot);
+    LAUNCHED();
+  }
+  std::vector<int> len(std::max<int64_t>(nch, 1), 0);
+  CK(cudaMemcpyAsync(len.data(), P.chunk_len, sizeof(int) * nch, cudaMemcpyDeviceToHost, s));
   CK(cudaStreamSynchronize(s));
-  if (bad) {  // a row segment does not fit one record: not eligible
-    free_tmp();
+  // padding check: SELL must not blow up the stream (skewed segments)
+  long long steps = 0;
+  for (int64_t i = 0; i < nch; ++i) steps += len[i];
+  const long long padded = steps * 32;
+  const long long real = h->k1 - h->k0;
+  double maxpad = 1.5;
+  if (padded > (long long)(maxpad * (double)real) + 64LL * nch) {
     cleanup();
     return SPMV_OK;
   }
-  // stream order [c][b][t]: records of one CTA contiguous
-  std::vector<int> rec_first(std::max<int64_t>(nTB, 1)), cta_rec(ncl * B + 1);
-  std::vector<long long> byte_first(std::max<int64_t>(nTB, 1));
-  int rec = 0;
+  // chunk offsets in stream order [c][b][t][w]: the chunks of one CTA are contiguous
+  std::vector<long long> off(std::max<int64_t>(nch, 1), 0);
   long long pos = 0;
   for (int c = 0; c < ncl; ++c)
-    for (int bb = 0; bb < B; ++bb) {
-      cta_rec[c * B + bb] = rec;
-      for (int t = tile0[c]; t < tile0[c + 1]; ++t) {
-        const size_t id = (size_t)t * B + bb;
-        rec_first[id] = rec;
-        byte_first[id] = pos;
-        rec += nrec[id];
-        pos += nbytes[id];
-      }
-    }
-  cta_rec[ncl * B] = rec;
-  P.nrec = rec;
+    for (int bb = 0; bb < B; ++bb)
+      for (int t = tile0[c]; t < tile0[c + 1]; ++t)
+        for (int w = 0; w < XP_NW; ++w) {
+          const size_t id = ((size_t)t * B + bb) * XP_NW + w;
+          off[id] = pos;
+          pos += (long long)len[id] * 32 * (ts + 2);
+        }
   P.bytes = pos;
-  CK(cudaMemcpyAsync(d_rec_first, rec_first.data(), sizeof(int) * nTB, cudaMemcpyHostToDevice, s));
-  CK(cudaMemcpyAsync(d_byte_first, byte_first.data(), sizeof(long long) * nTB, cudaMemcpyHostToDevice, s));
-  CK(cudaMalloc(&P.cta_rec, sizeof(int) * (ncl * B + 1)));
-  CK(cudaMemcpyAsync(P.cta_rec, cta_rec.data(), sizeof(int) * (ncl * B + 1), cudaMemcpyHostToDevice, s));
-  CK(cudaMalloc(&P.rec_off, sizeof(long long) * (rec + 1)));
-  CK(cudaMalloc(&P.rec_tile, sizeof(int) * std::max(rec, 1)));
-  CK(cudaMemcpyAsync(P.rec_off + rec, &pos, sizeof(long long), cudaMemcpyHostToDevice, s));
+  CK(cudaMemcpyAsync(P.chunk_off, off.data(), sizeof(long long) * nch, cudaMemcpyHostToDevice, s));
   CK(cudaMalloc(&P.plan, (size_t)std::max<long long>(pos, 16)));
-  CK(cudaMemsetAsync(P.plan, 0, (size_t)std::max<long long>(pos, 16), s));
-  CK(cudaMalloc(&P.row_rec, sizeof(int) * (size_t)B * (size_t)m));
-  CK(cudaMalloc(&P.row_pos, sizeof(int) * (size_t)B * (size_t)m));
-  k_xplan_records<<<rg, 128, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, d_tile0, ncl, ntiles, ts, (int)SB, 1, d_nrec,
-                                     d_bytes, d_rec_first, d_byte_first, P.rec_off, P.rec_tile, P.plan, P.row_rec,
-                                     P.row_pos, d_bad);
-  LAUNCHED();
+  if (nch > 0) {
+    k_xplan_fill<<<(unsigned)std::min<int64_t>(nch, 16LL * num_sms(h->device)), 256, 0, s>>>(
+        P.plan, P.chunk_off, P.chunk_len, nch, ts, (uint16_t)W);
+    LAUNCHED();
+  }
   ST(xplan_pack(h, h->vals, 0));
   CK(cudaStreamSynchronize(s));
-  free_tmp();
   P.built = true;
   *ok = true;
   return SPMV_OK;
@@ -798,8 +758,8 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   cudaError_t e = h->stream ? cudaStreamSynchronize(h->stream) : cudaDeviceSynchronize();
   if (e != cudaSuccess) st = cuda_fail(e, "pending asynchronous error", __LINE__);
   h->g_npb.reset();
-  void* bufs[] = {h->xp.crow, h->xp.rec_off, h->xp.cta_rec, h->xp.rec_tile, h->xp.seg, h->xp.row_rec,
-                  h->xp.row_pos, h->xp.plan,
+  void* bufs[] = {h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
+                  h->xp.chunk_row, h->xp.plan,
                   h->seg, h->crow, h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
                   h->stage_x, h->stage_z};

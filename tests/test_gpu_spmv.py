@@ -274,27 +274,21 @@ def test_xstat_alpha_beta_and_offset(sp, torch_dev):
         run_case(sp, torch, dev, A, x, alpha=a, beta=b, y0=y0, kernel="xstat", what=f"xstat a={a} b={b}")
 
 
-@pytest.mark.parametrize("cfg", [{}, {"SPMV_XPLAN_B": "2"}, {"SPMV_XPLAN_B": "8"}, {"SPMV_XPLAN_G": "4"},
-                                 {"SPMV_XPLAN_G": "16", "SPMV_XPLAN_B": "4"}, {"SPMV_XPLAN_SB": "2048"},
-                                 {"SPMV_XPLAN_CLUSTERS": "1", "SPMV_XPLAN_SB": "4096"}])
+@pytest.mark.parametrize("cfg", [{}, {"SPMV_XPLAN_B": "2"}, {"SPMV_XPLAN_B": "4"}, {"SPMV_XPLAN_B": "8"},
+                                 {"SPMV_XPLAN_CLUSTERS": "1"}, {"SPMV_XPLAN_CLUSTERS": "3", "SPMV_XPLAN_B": "2"}])
 @pytest.mark.parametrize("name,A", ZOO, ids=[c[0] for c in ZOO])
 def test_zoo_xplan(sp, torch_dev, name, A, cfg, monkeypatch):
-    """x-stationary kernel over the column-blocked plan (TMA bulk pipeline,
-    clusters, DSMEM reduction): cluster sizes, lane groups, small records
-    (many records per tile; rows that do not fit a record make the plan
-    ineligible -> zero-copy fallback) and a single cluster (many tiles:
-    exercises the triple-buffered partials and the split barrier)."""
+    """x-stationary kernel over the column-blocked SELL-32 plan (clusters,
+    st.async partials to the owning CTA, mbarrier transaction counts):
+    cluster sizes and few clusters (many tiles per cluster: exercises the
+    triple-buffered receive arrays and the split barrier).  Skewed matrices
+    whose SELL padding would exceed 1.5x fall back to the zero-copy kernel."""
     torch, dev = torch_dev
     for k, v in cfg.items():
         monkeypatch.setenv(k, v)
     x = gen.uniform(A.n, seed=17)
     info = run_case(sp, torch, dev, A, x, kernel="xplan", what=f"{name} xplan {cfg}")
-    k = np.arange(A.rowptr[0] + 1, A.rowptr[-1])
-    starts = np.zeros(A.colidx.shape[0] + 1, bool)
-    starts[A.rowptr[:-1]] = True
-    inner = ~starts[k]
-    sorted_cols = bool(np.all(A.colidx[k][inner] > A.colidx[k - 1][inner]))
-    if sorted_cols and A.nnz > 0 and "SPMV_XPLAN_SB" not in cfg:
+    if name in ("laplace1d", "stencil27_9", "makea_S", "n1"):
         assert info["kernel_name"] == "xplan", info
         assert info["plan_bytes"] >= A.nnz * 10
     A32 = A.astype(np.float32)

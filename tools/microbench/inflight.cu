@@ -15,7 +15,7 @@ __device__ __forceinline__ void wait_par(uint64_t* b, uint32_t ph) {
 }
 
 __global__ void __launch_bounds__(128, 1) k_ring(const char* __restrict__ g, size_t per_cta, int stages, int sb,
-                                                 size_t pf_dist, unsigned long long* sink) {
+                                                 size_t pf_dist, int hold, unsigned long long* sink) {
   extern __shared__ __align__(128) char sm[];
   __shared__ uint64_t full[16], empty[16];
   const int warp = threadIdx.x / 32, lane = threadIdx.x & 31;
@@ -39,8 +39,8 @@ __global__ void __launch_bounds__(128, 1) k_ring(const char* __restrict__ g, siz
         if (pf_dist) {
           const size_t want = min(per_cta, size_t(it) * sb + pf_dist);
           while (pf < want) {
-            asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(base + pf), "r"(16384) : "memory");
-            pf += 16384;
+            asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(base + pf), "r"(sb) : "memory");
+            pf += sb;
           }
         }
         asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(&full[s])), "r"(sb) : "memory");
@@ -54,6 +54,7 @@ __global__ void __launch_bounds__(128, 1) k_ring(const char* __restrict__ g, siz
       const int s = it % stages;
       wait_par(&full[s], (it / stages) & 1);
       acc += ((volatile int*)(sm + size_t(s) * sb))[lane];
+      if (hold) { long long t0 = clock64(); while (clock64() - t0 < hold) {} }
       __syncwarp();
       if (lane == 0) asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(&empty[s])) : "memory");
     }
@@ -69,25 +70,24 @@ int main() {
   unsigned long long* sink;
   cudaMalloc(&sink, 8);
   cudaFuncSetAttribute(k_ring, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024);
-  for (int grid : {120, 148}) {
-    size_t per_cta = (gbytes / grid) & ~size_t(65535);
-    for (size_t pf : {size_t(0), size_t(256) << 10, size_t(1) << 20})
-      for (int sb : {8192, 16384})
-        for (int stages : {2, 4, 8, 12}) {
-          if (size_t(stages) * sb > 196 * 1024) continue;
-          cudaEvent_t a, b;
-          cudaEventCreate(&a);
-          cudaEventCreate(&b);
-          k_ring<<<grid, 128, stages * sb>>>(g, per_cta, stages, sb, pf, sink);
-          cudaEventRecord(a);
-          k_ring<<<grid, 128, stages * sb>>>(g, per_cta, stages, sb, pf, sink);
-          cudaEventRecord(b);
-          cudaEventSynchronize(b);
-          float ms;
-          cudaEventElapsedTime(&ms, a, b);
-          printf("grid %3d pf %4zu KB stage %5d x %2d = %4d KB in flight: %7.1f GB/s %s\n", grid, pf >> 10, sb, stages,
-                 stages * sb / 1024, double(grid) * per_cta / ms / 1e6, cudaGetErrorString(cudaGetLastError()));
-        }
-  }
+  const int grid = 120;
+  size_t per_cta = (gbytes / grid) & ~size_t(65535);
+  for (int hold : {0, 1000, 2000})
+    for (size_t pf : {size_t(0), size_t(32) << 10, size_t(64) << 10, size_t(128) << 10})
+      for (int cfg = 0; cfg < 3; ++cfg) {
+        int sb = cfg == 2 ? 8192 : 16384, stages = cfg == 0 ? 4 : (cfg == 1 ? 8 : 8);
+        cudaEvent_t a, b;
+        cudaEventCreate(&a);
+        cudaEventCreate(&b);
+        k_ring<<<grid, 128, stages * sb>>>(g, per_cta, stages, sb, pf, hold, sink);
+        cudaEventRecord(a);
+        k_ring<<<grid, 128, stages * sb>>>(g, per_cta, stages, sb, pf, hold, sink);
+        cudaEventRecord(b);
+        cudaEventSynchronize(b);
+        float ms;
+        cudaEventElapsedTime(&ms, a, b);
+        printf("hold %4d clk pf %4zu KB stage %5d x %d = %3d KB: %7.1f GB/s %s\n", hold, pf >> 10, sb, stages,
+               stages * sb / 1024, double(grid) * per_cta / ms / 1e6, cudaGetErrorString(cudaGetLastError()));
+      }
   return 0;
 }

@@ -17,12 +17,11 @@ import gen
 import paper_conf_asplos_ginsbachrsbdo18_b200 as sp
 
 VARIANTS = [("auto", {}, {}), ("auto_noplan", {"plan": False}, {})] + \
-    [(f"xplan_G{g}", {"kernel": "xplan"}, {"SPMV_XPLAN_G": str(g)}) for g in (4, 8, 16)] + \
-    [(f"xplan_G8_SB{sb}", {"kernel": "xplan"}, {"SPMV_XPLAN_G": "8", "SPMV_XPLAN_SB": str(sb)}) for sb in (8192, 12288)] + [(f"vector{g}", {"kernel": "vector", "vec_lanes": g}, {}) for g in (4, 8, 16, 32)] + \
-    [(f"vector32_u{u}", {"kernel": "vector", "vec_lanes": 32}, {"SPMV_UNROLL": str(u)}) for u in (2, 8)] + \
-    [(f"xstat_B{b}_G{g}_U{u}", {"kernel": "xstat"}, {"SPMV_XSTAT_B": str(b), "SPMV_XSTAT_G": str(g),
-                                                     "SPMV_XSTAT_U": str(u)})
-     for b in (8,) for g in (8, 16) for u in (8,)]
+    [(f"xplan_B{b}", {"kernel": "xplan"}, {"SPMV_XPLAN_B": str(b)}) for b in (4, 8)] + \
+    [(f"vector{g}", {"kernel": "vector", "vec_lanes": g, "plan": False}, {}) for g in (8, 16, 32)] + \
+    [(f"vector32_u{u}", {"kernel": "vector", "vec_lanes": 32, "plan": False}, {"SPMV_UNROLL": str(u)}) for u in (2, 8)] + \
+    [(f"xstat_B8_G{g}_U8", {"kernel": "xstat", "plan": False}, {"SPMV_XSTAT_B": "8", "SPMV_XSTAT_G": str(g),
+                                                                  "SPMV_XSTAT_U": "8"}) for g in (8,)]
 
 
 def time_variant(A, x, y, kw, env, reps=20):
