@@ -36,7 +36,10 @@
 
 namespace spmv {
 
-constexpr int XP_NW = 16;            // warps per CTA
+#ifndef XP_NW_DEF
+#define XP_NW_DEF 32
+#endif
+constexpr int XP_NW = XP_NW_DEF;     // warps per CTA
 constexpr int XP_R = 32 * XP_NW;     // rows per tile
 constexpr int XP_THREADS = 32 * XP_NW;
 constexpr int XP_K = 3;              // receive buffers
@@ -162,7 +165,10 @@ k_spmv_xplan(XplanArgs a) {
   double dacc = 0.0;
 
   auto process = [&](int t) {
-    const int64_t cid = (int64_t(tbase + t) * B + b) * XP_NW + warp;
+    // chunks are sorted longest first: alternate the order every tile so each
+    // warp's work over two consecutive tiles (one barrier interval) balances
+    const int wc = (t & 1) ? (XP_NW - 1 - warp) : warp;
+    const int64_t cid = (int64_t(tbase + t) * B + b) * XP_NW + wc;
     const int len = a.chunk_len[cid];
     const int row = a.chunk_row[cid * 32 + lane];
     const unsigned char* V = a.plan + a.chunk_off[cid] + size_t(lane) * 2 * sizeof(T);
@@ -214,8 +220,12 @@ k_spmv_xplan(XplanArgs a) {
       y[i] = out;
       if (DOT) dacc += double(static_cast<const T*>(a.w)[i]) * double(out);
     }
-    __syncthreads();  // all reads of recv[t%K] done before it is re-armed
-    if (threadIdx.x == 0 && t + XP_K < ntiles) mbar_expect_tx(&tbar[t % XP_K], recv_bytes(t + XP_K));
+    // all reads of recv[t%K] (threads < RB) done before thread 0 re-arms it
+    const int nfin = (RB + 31) & ~31;
+    if (int(threadIdx.x) < nfin) {
+      asm volatile("bar.sync 2, %0;\n" ::"r"(nfin) : "memory");
+      if (threadIdx.x == 0 && t + XP_K < ntiles) mbar_expect_tx(&tbar[t % XP_K], recv_bytes(t + XP_K));
+    }
   };
 
   // Buffer reuse: partials of tile t+K (K = 3) are sent only after the sender
