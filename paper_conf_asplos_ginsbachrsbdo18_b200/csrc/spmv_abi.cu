@@ -178,6 +178,22 @@ static bool overlap(const void* a, size_t na, const void* b, size_t nb) {
 
 static int64_t cdiv(int64_t a, int64_t b) { return (a + b - 1) / b; }
 
+// SPMV_DEBUG=1: trace the create-time plan build on stderr (synchronising).
+static bool dbg() {
+  static int v = -1;
+  if (v < 0) { v = 0; env_int("SPMV_DEBUG", &v); }
+  return v != 0;
+}
+#define DBG(...)                                                                    \
+  do {                                                                              \
+    if (dbg()) {                                                                    \
+      cudaError_t e__ = cudaDeviceSynchronize();                                    \
+      fprintf(stderr, "[spmv] %s:%d (%s) ", __func__, __LINE__, cudaGetErrorString(e__)); \
+      fprintf(stderr, __VA_ARGS__);                                                 \
+      fprintf(stderr, "\n");                                                        \
+    }                                                                               \
+  } while (0)
+
 static spmv_status ensure_buf(void** p, size_t bytes) {
   if (*p) return SPMV_OK;
   CK(cudaMalloc(p, bytes > 0 ? bytes : 8));
@@ -336,6 +352,7 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   a.chunk_off = h->xp.chunk_off;
   a.chunk_len = h->xp.chunk_len;
   a.chunk_row = h->xp.chunk_row;
+  a.dbg = dbg() ? 1 : 0;
   a.crow = h->xp.crow;
   a.tile0 = h->xp.tile0;
   a.x = x;
@@ -430,6 +447,7 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
     P = spmv_csr_s::XPlan();
   };
   P.B = B; P.W = W; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd;
+  DBG("B=%d W=%d ncl=%d smem=%zu", B, W, ncl, smem);
   const int64_t m = h->m_loc;
   CK(cudaMalloc(&P.crow, sizeof(long long) * (ncl + 1)));
   k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(m, h->rp_loc, ncl, P.crow);
@@ -441,6 +459,7 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   for (int c = 0; c < ncl; ++c) tile0[c + 1] = tile0[c] + (int)cdiv(crow[c + 1] - crow[c], XP_R);
   const int ntiles = tile0[ncl];
   P.ntiles = ntiles;
+  DBG("ntiles=%d", ntiles);
   CK(cudaMalloc(&P.tile0, sizeof(int) * (ncl + 1)));
   CK(cudaMemcpyAsync(P.tile0, tile0.data(), sizeof(int) * (ncl + 1), cudaMemcpyHostToDevice, s));
   if (B > 1) {
@@ -449,6 +468,7 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
         m, h->rp_loc, h->ci_loc, B, W, P.seg);
     LAUNCHED();
   }
+  DBG("splits done");
   const int64_t nch = (int64_t)ntiles * B * XP_NW;
   P.nchunks = nch;
   CK(cudaMalloc(&P.chunk_len, sizeof(int) * std::max<int64_t>(nch, 1)));
@@ -460,6 +480,7 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
                                                           P.chunk_row, P.row_slot);
     LAUNCHED();
   }
+  DBG("sell done nch=%lld", (long long)nch);
   std::vector<int> len(std::max<int64_t>(nch, 1), 0);
   CK(cudaMemcpyAsync(len.data(), P.chunk_len, sizeof(int) * nch, cudaMemcpyDeviceToHost, s));
   CK(cudaStreamSynchronize(s));
@@ -492,7 +513,9 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
         P.plan, P.chunk_off, P.chunk_len, nch, ts, (uint16_t)W);
     LAUNCHED();
   }
+  DBG("fill done bytes=%lld", (long long)pos);
   ST(xplan_pack(h, h->vals, 0));
+  DBG("pack done");
   CK(cudaStreamSynchronize(s));
   P.built = true;
   *ok = true;

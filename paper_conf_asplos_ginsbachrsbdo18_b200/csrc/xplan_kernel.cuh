@@ -58,10 +58,16 @@ struct XplanArgs {
   double alpha, beta;
   const void* w;               // DOT: w[i]
   double* part;                // DOT: one partial per CTA
+  int dbg;
 };
 
 __device__ __forceinline__ void cluster_arrive_relaxed() {
-  asm volatile("barrier.cluster.arrive.relaxed.aligned;\n" ::: "memory");
+  __syncwarp();
+#ifdef XP_RELEASE_ARRIVE
+  asm volatile("barrier.cluster.arrive.release;\n" ::: "memory");
+#else
+  asm volatile("barrier.cluster.arrive.relaxed;\n" ::: "memory");
+#endif
 }
 __device__ __forceinline__ uint32_t mapa_u32(uint32_t laddr, uint32_t rank) {
   uint32_t r;
@@ -159,7 +165,7 @@ k_spmv_xplan(XplanArgs a) {
   // peers must have initialised their barriers before partials are sent
   cluster_arrive();
   cluster_wait();
-  mbar_wait(&xbar, 0);
+  mbar_wait(&xbar, 0, 1);
 
   const double alpha = a.alpha, beta = a.beta;
   double dacc = 0.0;
@@ -204,12 +210,20 @@ k_spmv_xplan(XplanArgs a) {
     }
   };
 
+  // Only the RB finalizer threads (rounded up to whole warps) wait on the
+  // tile's mbarrier; all of them pass the wait before thread 0 re-arms it for
+  // tile t+K.  (If every thread waited, a late warp could miss the phase: a
+  // re-arm that expects 0 bytes completes the next phase at once and flips
+  // the parity back -- an ABA deadlock seen on CTAs owning no rows of a
+  // cluster's last tile.)
+  const int nfin = (RB + 31) & ~31;
   auto finalize = [&](int t) {
+    if (int(threadIdx.x) >= nfin) return;
     const double* rv = recv + (t % XP_K) * R;
     const int64_t rt = r0c + int64_t(t) * R;
     const int nrows = int(cmin64(R, r1c - rt));
-    mbar_wait(&tbar[t % XP_K], (t / XP_K) & 1);
-    for (int jl = threadIdx.x; jl < RB && b * RB + jl < nrows; jl += blockDim.x) {
+    mbar_wait(&tbar[t % XP_K], (t / XP_K) & 1, 1000000 * ntiles + 1000 * t + int(recv_bytes(t) / 8));
+    for (int jl = threadIdx.x; jl < RB && b * RB + jl < nrows; jl += nfin) {
       double sum = 0.0;
       for (int q = 0; q < B; ++q) sum += rv[q * RB + jl];
       const int64_t i = rt + b * RB + jl;
@@ -220,12 +234,8 @@ k_spmv_xplan(XplanArgs a) {
       y[i] = out;
       if (DOT) dacc += double(static_cast<const T*>(a.w)[i]) * double(out);
     }
-    // all reads of recv[t%K] (threads < RB) done before thread 0 re-arms it
-    const int nfin = (RB + 31) & ~31;
-    if (int(threadIdx.x) < nfin) {
-      asm volatile("bar.sync 2, %0;\n" ::"r"(nfin) : "memory");
-      if (threadIdx.x == 0 && t + XP_K < ntiles) mbar_expect_tx(&tbar[t % XP_K], recv_bytes(t + XP_K));
-    }
+    asm volatile("bar.sync 2, %0;\n" ::"r"(nfin) : "memory");
+    if (threadIdx.x == 0 && t + XP_K < ntiles) mbar_expect_tx(&tbar[t % XP_K], recv_bytes(t + XP_K));
   };
 
   // Buffer reuse: partials of tile t+K (K = 3) are sent only after the sender

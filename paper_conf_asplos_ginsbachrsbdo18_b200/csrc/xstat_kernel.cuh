@@ -46,11 +46,16 @@ __device__ __forceinline__ int64_t cmax64(int64_t a, int64_t b) { return a > b ?
 __device__ __forceinline__ uint32_t smem_u32(const void* p) {
   return static_cast<uint32_t>(__cvta_generic_to_shared(p));
 }
+// Cluster barrier halves.  The non-.aligned forms plus __syncwarp(): the
+// callers reach them from divergent code, and inline asm gives the compiler
+// no reason to reconverge the warp before an .aligned barrier.
 __device__ __forceinline__ void cluster_arrive() {
-  asm volatile("barrier.cluster.arrive.release.aligned;\n" ::: "memory");
+  __syncwarp();
+  asm volatile("barrier.cluster.arrive.release;\n" ::: "memory");
 }
 __device__ __forceinline__ void cluster_wait() {
-  asm volatile("barrier.cluster.wait.acquire.aligned;\n" ::: "memory");
+  __syncwarp();
+  asm volatile("barrier.cluster.wait.acquire;\n" ::: "memory");
 }
 __device__ __forceinline__ uint32_t cluster_rank() {
   uint32_t r;
@@ -78,14 +83,27 @@ __device__ __forceinline__ void mbar_expect_tx(uint64_t* bar, uint32_t bytes) {
   asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;\n" ::"r"(smem_u32(bar)), "r"(bytes)
                : "memory");
 }
-__device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
+// Wait for the phase of `parity` to complete.  Watchdog: a wait that spins for
+// more than ~4e9 cycles (~2 s) reports the barrier and traps, turning a
+// deadlock into a launch error instead of a hung GPU.
+__device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity, int tag = -1) {
   uint32_t ok = 0;
-  while (!ok) {
+  long long t0 = 0;
+  for (uint32_t spin = 0; !ok; ++spin) {
     asm volatile(
         "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n selp.u32 %0, 1, 0, p;\n}\n"
         : "=r"(ok)
         : "r"(smem_u32(bar)), "r"(parity)
         : "memory");
+    if (!ok && (spin & 1023) == 1023) {
+      const long long now = clock64();
+      if (t0 == 0) t0 = now;
+      else if (now - t0 > 4000000000LL) {
+        printf("spmv: mbarrier wait timeout block %d thread %d bar smem 0x%x parity %u tag %d\n", blockIdx.x,
+               threadIdx.x, smem_u32(bar), parity, tag);
+        __trap();
+      }
+    }
   }
 }
 

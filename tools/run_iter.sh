@@ -1,2 +1,2 @@
-PYTEST_ARGS="-k xplan or nas or npb" SWEEP="C B" bash tools/gpu_quick.sh
+SWEEP="C B" bash tools/gpu_quick.sh
 bash tools/gpu_prof.sh xplanC C xplan
