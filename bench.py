@@ -85,7 +85,7 @@ class ClockSampler:
         try:
             self.proc = subprocess.Popen(
                 ["nvidia-smi", "-i", str(self.gpu), f"--query-gpu={self.FIELDS}", "--format=csv,noheader,nounits",
-                 "-lms", "200"], stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+                 "-lms", "50"], stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
             self.t = threading.Thread(target=self._read, daemon=True)
             self.t.start()
         except Exception:
@@ -176,12 +176,12 @@ def run_ours(args):
     x = torch.ones(nl, dtype=torch.float64, device=dev)
     z = torch.empty(nl, dtype=torch.float64, device=dev)
     out2 = torch.zeros(2, dtype=torch.float64, device=dev)
+    clocks = ClockSampler(local)
+    clocks.start()
     for _ in range(args.warmup):
         M.npb_outer(x, z, 25, shift, out2)
     barrier()
     x.fill_(1.0)
-    clocks = ClockSampler(local)
-    clocks.start()
     ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
     launches0 = sp.launch_count()
     zetas = []
@@ -196,7 +196,6 @@ def run_ours(args):
     M.cg_status()
     step_ms = [a.elapsed_time(b) for a, b in ev]
     t_ms = max_over_ranks(sum(step_ms))
-    clk = clocks.stop()
     zeta_last = float(out2[0].item())
     value = 25.0 * args.steps / (t_ms / 1e3)
 
@@ -236,6 +235,7 @@ def run_ours(args):
         b.record(stream)
         b.synchronize()
         sp_ms.append(a.elapsed_time(b))
+    clk = clocks.stop()
     # algorithmic bytes of this rank's launch: local nnz*(8+4) + 4*(m_loc+1) + 8*n (x) + 8*m_loc (y)
     nnz_loc = info["nnz_local"]
     spmv_bytes = nnz_loc * 12 + 4 * (nl + 1) + 8 * A.n + 8 * nl
@@ -248,8 +248,7 @@ def run_ours(args):
     if os.path.exists(tf) and world == 1:
         try:
             tj = json.load(open(tf))
-            key = f"class{CLS}:{info['kernel_name']}:lanes{info['vec_lanes']}"
-            traffic = tj.get(key)
+            traffic = tj.get(f"class{CLS}:{info['kernel_name']}")
         except Exception:
             traffic = None
 
@@ -277,7 +276,8 @@ def run_ours(args):
             "cg_gbs_effective": round(value * (spmv_bytes + 10 * 8 * nl) / 1e9 * world, 1),
             "roofline": {"bound": "hbm", "achieved": round(achieved, 1), "peak": peak, "unit": "GB/s",
                          "frac": round(achieved / peak, 4), "traffic": traffic,
-                         "peak_source": peak_src, "kernel": f"k_spmv_vector<double,{info['vec_lanes']}>"},
+                         "peak_source": peak_src, "kernel": f"k_spmv_{info['kernel_name']}<double>",
+                         "traffic_source": "profiles/spmv_traffic.json (ncu --set full, dram__bytes_read+write per launch)"},
             "e2e": {"value": round(e2e_val, 2), "unit": UNIT, "h2d_bytes_per_step": 8 * nl,
                     "d2h_bytes_per_step": 2 * 8 * nl + 16},
             "gpu_launches": int(launches),

@@ -11,7 +11,7 @@ timeout 600 python bench.py --steps 10 --warmup 3 > gpurun_out/bench.json 2> gpu
 if [ -n "$NCU" ]; then
   timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none -c 400 --csv \
      --log-file gpurun_out/ncu_launches.csv python bench.py --steps 2 --warmup 3 --no-cpu > gpurun_out/ncu_bench.log 2>&1
-  timeout 900 ncu --set full --clock-control none --import-source on -k regex:k_spmv -s 30 -c 2 \
+  timeout 900 ncu --set full --clock-control none --import-source on -k regex:k_spmv -s 30 -c 1 \
      -o gpurun_out/prof_spmv -f python bench.py --steps 2 --warmup 3 --no-cpu > gpurun_out/ncu_full.log 2>&1
 fi
 tail -3 gpurun_out/pytest_gpu.log
