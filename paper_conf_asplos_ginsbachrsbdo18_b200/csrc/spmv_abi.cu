@@ -353,6 +353,8 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   a.chunk_len = h->xp.chunk_len;
   a.chunk_row = h->xp.chunk_row;
   a.dbg = dbg() ? 1 : 0;
+  a.prefetch = 0;
+  env_int("SPMV_XPLAN_PF", &a.prefetch);
   a.crow = h->xp.crow;
   a.tile0 = h->xp.tile0;
   a.x = x;
@@ -469,14 +471,14 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
     LAUNCHED();
   }
   DBG("splits done");
-  const int64_t nch = (int64_t)ntiles * B * XP_NW;
+  const int64_t nch = (int64_t)ntiles * B * XP_CPT;
   P.nchunks = nch;
   CK(cudaMalloc(&P.chunk_len, sizeof(int) * std::max<int64_t>(nch, 1)));
   CK(cudaMalloc(&P.chunk_off, sizeof(long long) * std::max<int64_t>(nch, 1)));
   CK(cudaMalloc(&P.chunk_row, sizeof(uint16_t) * 32 * std::max<int64_t>(nch, 1)));
   CK(cudaMalloc(&P.row_slot, sizeof(int) * (size_t)B * (size_t)m));
   if (ntiles > 0) {
-    k_xplan_sell<<<(unsigned)(ntiles * B), XP_R, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, P.tile0, ncl, P.chunk_len,
+    k_xplan_sell<<<(unsigned)(ntiles * B), XP_THREADS, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, P.tile0, ncl, P.chunk_len,
                                                           P.chunk_row, P.row_slot);
     LAUNCHED();
   }
@@ -500,8 +502,8 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   for (int c = 0; c < ncl; ++c)
     for (int bb = 0; bb < B; ++bb)
       for (int t = tile0[c]; t < tile0[c + 1]; ++t)
-        for (int w = 0; w < XP_NW; ++w) {
-          const size_t id = ((size_t)t * B + bb) * XP_NW + w;
+        for (int w = 0; w < XP_CPT; ++w) {
+          const size_t id = ((size_t)t * B + bb) * XP_CPT + w;
           off[id] = pos;
           pos += (long long)len[id] * 32 * (ts + 2);
         }

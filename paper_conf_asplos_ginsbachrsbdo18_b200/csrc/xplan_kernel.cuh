@@ -40,7 +40,9 @@ namespace spmv {
 #define XP_NW_DEF 32
 #endif
 constexpr int XP_NW = XP_NW_DEF;     // warps per CTA
-constexpr int XP_R = 32 * XP_NW;     // rows per tile
+constexpr int XP_CPW = 2;            // chunks per warp per tile (paired longest + shortest)
+constexpr int XP_CPT = XP_NW * XP_CPW;  // chunks per tile
+constexpr int XP_R = 32 * XP_CPT;    // rows per tile
 constexpr int XP_THREADS = 32 * XP_NW;
 constexpr int XP_K = 3;              // receive buffers
 
@@ -48,9 +50,9 @@ struct XplanArgs {
   int64_t nx;                  // length of x
   int W;                       // column block width (pad column = W)
   const unsigned char* plan;   // chunk data
-  const long long* chunk_off;  // [tile][b][w] byte offset of chunk data
-  const int* chunk_len;        // [tile][b][w] steps (even)
-  const uint16_t* chunk_row;   // [tile][b][w][32] tile-local row of each lane (0xffff = none)
+  const long long* chunk_off;  // [tile][b][chunk] byte offset of chunk data
+  const int* chunk_len;        // [tile][b][chunk] steps (even)
+  const uint16_t* chunk_row;   // [tile][b][chunk][32] tile-local row of each lane (0xffff = none)
   const long long* crow;       // [ncl+1] cluster row ranges
   const int* tile0;            // [ncl+1] first global tile of each cluster
   const void* x;
@@ -59,6 +61,7 @@ struct XplanArgs {
   const void* w;               // DOT: w[i]
   double* part;                // DOT: one partial per CTA
   int dbg;
+  int prefetch;                // 1: L2-prefetch the warp's chunk of the next tile
 };
 
 __device__ __forceinline__ void cluster_arrive_relaxed() {
@@ -170,15 +173,19 @@ k_spmv_xplan(XplanArgs a) {
   const double alpha = a.alpha, beta = a.beta;
   double dacc = 0.0;
 
-  auto process = [&](int t) {
-    // chunks are sorted longest first: alternate the order every tile so each
-    // warp's work over two consecutive tiles (one barrier interval) balances
-    const int wc = (t & 1) ? (XP_NW - 1 - warp) : warp;
-    const int64_t cid = (int64_t(tbase + t) * B + b) * XP_NW + wc;
+  auto process_chunk = [&](int t, int ch) {
+    const int64_t cid = (int64_t(tbase + t) * B + b) * XP_CPT + ch;
     const int len = a.chunk_len[cid];
     const int row = a.chunk_row[cid * 32 + lane];
-    const unsigned char* V = a.plan + a.chunk_off[cid] + size_t(lane) * 2 * sizeof(T);
-    const unsigned char* C = a.plan + a.chunk_off[cid] + size_t(len) * 32 * sizeof(T) + size_t(lane) * 4;
+    const unsigned char* base = a.plan + a.chunk_off[cid];
+    if (a.prefetch && lane == 0 && t + 1 < ntiles) {
+      const int64_t nid = cid + int64_t(B) * XP_CPT;
+      const uint32_t nb = uint32_t(a.chunk_len[nid]) * 32u * uint32_t(sizeof(T) + 2);
+      if (nb) asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a.plan + a.chunk_off[nid]), "r"(nb)
+                           : "memory");
+    }
+    const unsigned char* V = base + size_t(lane) * 2 * sizeof(T);
+    const unsigned char* C = base + size_t(len) * 32 * sizeof(T) + size_t(lane) * 4;
     constexpr size_t VS = 32 * 2 * sizeof(T);  // bytes per step pair (vals)
     double acc = 0.0;
     int p = 0;
@@ -208,6 +215,11 @@ k_spmv_xplan(XplanArgs a) {
       const uint32_t laddr = smem_u32(recv + (t % XP_K) * R + b * RB + jl);
       st_async_f64(mapa_u32(laddr, q), acc, mapa_u32(smem_u32(&tbar[t % XP_K]), q));
     }
+  };
+  // chunks are sorted longest first: warp w takes chunk w and chunk CPT-1-w
+  auto process = [&](int t) {
+    process_chunk(t, warp);
+    if (XP_CPW == 2) process_chunk(t, XP_CPT - 1 - warp);
   };
 
   // Only the RB finalizer threads (rounded up to whole warps) wait on the
@@ -269,50 +281,59 @@ __device__ __forceinline__ void xp_seg(const int* rowptr, const int* seg, int64_
   *k1 = (b == B - 1) ? rowptr[i + 1] : seg[int64_t(b) * m + i];
 }
 
-// One CTA (R threads) per (global tile, b): sort the tile's rows by segment
-// length (descending, ties by row: bitonic sort of (len, row) keys), cut into
-// NW chunks of 32 lanes, record each chunk's even step count and each row's
-// (chunk, lane) slot.
-__global__ void __launch_bounds__(XP_R)
+// One CTA (XP_THREADS threads, R/XP_THREADS rows each) per (global tile, b):
+// sort the tile's rows by segment length (descending, ties by row: bitonic
+// sort of (len, row) keys), cut into CPT chunks of 32 lanes, record each
+// chunk's even step count and each row's slot (chunk = slot/32, lane = slot%32).
+__global__ void __launch_bounds__(XP_THREADS)
 k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_t m, int B,
              const long long* __restrict__ crow, const int* __restrict__ tile0, int ncl, int* __restrict__ chunk_len,
              uint16_t* __restrict__ chunk_row, int* __restrict__ row_slot) {
   __shared__ unsigned long long key[XP_R];
+  constexpr int PER = XP_R / XP_THREADS;
   const int tg = blockIdx.x / B, b = blockIdx.x % B;
   int c = 0;
   while (c + 1 < ncl && tile0[c + 1] <= tg) ++c;
   const int t = tg - tile0[c];
   const int64_t rt = crow[c] + int64_t(t) * XP_R;
   const int nrows = int(cmin64(XP_R, crow[c + 1] - rt));
-  const int j = threadIdx.x;
-  int L = -1;  // absent rows sort last
-  if (j < nrows) {
-    int k0, k1;
-    xp_seg(rowptr, seg, m, B, b, rt + j, &k0, &k1);
-    L = k1 - k0;
+  for (int e = 0; e < PER; ++e) {
+    const int j = threadIdx.x + e * XP_THREADS;
+    int L = -1;  // absent rows sort last
+    if (j < nrows) {
+      int k0, k1;
+      xp_seg(rowptr, seg, m, B, b, rt + j, &k0, &k1);
+      L = k1 - k0;
+    }
+    // descending by L, then ascending by row: key = (~(L+1)) << 32 | j, ascending
+    key[j] = (static_cast<unsigned long long>(~static_cast<uint32_t>(L + 1)) << 32) | uint32_t(j);
   }
-  // descending by L, then ascending by row: key = (~(L+1)) << 32 | j, ascending
-  key[j] = (static_cast<unsigned long long>(~static_cast<uint32_t>(L + 1)) << 32) | uint32_t(j);
   __syncthreads();
   for (int k = 2; k <= XP_R; k <<= 1)
     for (int s = k >> 1; s > 0; s >>= 1) {
-      const int p = j ^ s;
-      if (p > j) {
-        const bool up = (j & k) == 0;
-        const unsigned long long a0 = key[j], a1 = key[p];
-        if ((a0 > a1) == up) { key[j] = a1; key[p] = a0; }
+      for (int e = 0; e < PER; ++e) {
+        const int j = threadIdx.x + e * XP_THREADS;
+        const int p = j ^ s;
+        if (p > j) {
+          const bool up = (j & k) == 0;
+          const unsigned long long a0 = key[j], a1 = key[p];
+          if ((a0 > a1) == up) { key[j] = a1; key[p] = a0; }
+        }
       }
       __syncthreads();
     }
-  const unsigned long long kk = key[j];
-  const int row = int(kk & 0xffffffffu);
-  const int Ls = int(~uint32_t(kk >> 32)) - 1;
-  const int w = j / 32, ln = j % 32;
-  const int64_t cid = (int64_t(tg) * B + b) * XP_NW + w;
-  chunk_row[cid * 32 + ln] = (Ls >= 0) ? uint16_t(row) : uint16_t(0xffff);
-  if (Ls >= 0) row_slot[int64_t(b) * m + rt + row] = j;  // chunk w = j/32, lane = j%32
-  // chunk length = the first (longest) lane's length, rounded up to even
-  if (ln == 0) chunk_len[cid] = (max(Ls, 0) + 1) & ~1;
+  for (int e = 0; e < PER; ++e) {
+    const int j = threadIdx.x + e * XP_THREADS;
+    const unsigned long long kk = key[j];
+    const int row = int(kk & 0xffffffffu);
+    const int Ls = int(~uint32_t(kk >> 32)) - 1;
+    const int w = j / 32, ln = j % 32;
+    const int64_t cid = (int64_t(tg) * B + b) * XP_CPT + w;
+    chunk_row[cid * 32 + ln] = (Ls >= 0) ? uint16_t(row) : uint16_t(0xffff);
+    if (Ls >= 0) row_slot[int64_t(b) * m + rt + row] = j;
+    // chunk length = the first (longest) lane's length, rounded up to even
+    if (ln == 0) chunk_len[cid] = (max(Ls, 0) + 1) & ~1;
+  }
 }
 
 // Scatter every nonzero into its chunk slot: warp per row.
@@ -338,7 +359,7 @@ k_xplan_pack(const int* __restrict__ rowptr, const int* __restrict__ colidx, con
       const int bb = col / W;
       const int s0 = (bb == 0) ? k0 : seg[int64_t(bb - 1) * m + i];
       const int slot = row_slot[int64_t(bb) * m + i];
-      const int64_t cid = (int64_t(tg) * B + bb) * XP_NW + slot / 32;
+      const int64_t cid = (int64_t(tg) * B + bb) * XP_CPT + slot / 32;
       const int ln = slot % 32, len = chunk_len[cid];
       const int s = k - s0;  // step
       unsigned char* base = plan + chunk_off[cid];
