@@ -40,11 +40,18 @@ namespace spmv {
 #define XP_NW_DEF 32
 #endif
 constexpr int XP_NW = XP_NW_DEF;     // warps per CTA
-constexpr int XP_CPW = 2;            // chunks per warp per tile (paired longest + shortest)
+#ifndef XP_CPW_DEF
+#define XP_CPW_DEF 2
+#endif
+constexpr int XP_CPW = XP_CPW_DEF;   // chunks per warp per tile (paired longest + shortest)
 constexpr int XP_CPT = XP_NW * XP_CPW;  // chunks per tile
 constexpr int XP_R = 32 * XP_CPT;    // rows per tile
 constexpr int XP_THREADS = 32 * XP_NW;
 constexpr int XP_K = 3;              // receive buffers
+#ifndef XP_U_DEF
+#define XP_U_DEF 8
+#endif
+constexpr int XP_U = XP_U_DEF;       // step pairs (16-B loads) in flight per lane
 
 struct XplanArgs {
   int64_t nx;                  // length of x
@@ -188,27 +195,29 @@ k_spmv_xplan(XplanArgs a) {
     const unsigned char* C = base + size_t(len) * 32 * sizeof(T) + size_t(lane) * 4;
     constexpr size_t VS = 32 * 2 * sizeof(T);  // bytes per step pair (vals)
     double acc = 0.0;
-    int p = 0;
     const int np = len >> 1;  // step pairs
-    for (; p + 4 <= np; p += 4) {
-      Pair<T> v[4];
-      uint32_t cc[4];
+    const uint32_t padcc = uint32_t(W) | (uint32_t(W) << 16);  // both steps -> x pad 0.0
+    // every batch issues up to XP_U independent 16-B loads (the tail batch is
+    // predicated: masked pairs contribute 0 * x[W] = 0), so a chunk costs
+    // ceil(np / XP_U) memory round trips
+    for (int p = 0; p < np; p += XP_U) {
+      Pair<T> v[XP_U];
+      uint32_t cc[XP_U];
 #pragma unroll
-      for (int u = 0; u < 4; ++u) {
-        v[u] = Pair<T>::load(V + size_t(p + u) * VS);
-        cc[u] = ldg_stream4(C + size_t(p + u) * 128);
+      for (int u = 0; u < XP_U; ++u) {
+        if (p + u < np) {
+          v[u] = Pair<T>::load(V + size_t(p + u) * VS);
+          cc[u] = ldg_stream4(C + size_t(p + u) * 128);
+        } else {
+          v[u] = Pair<T>{T(0), T(0)};
+          cc[u] = padcc;
+        }
       }
 #pragma unroll
-      for (int u = 0; u < 4; ++u) {
+      for (int u = 0; u < XP_U; ++u) {
         acc += double(v[u].a) * double(xs[cc[u] & 0xffffu]);
         acc += double(v[u].b) * double(xs[cc[u] >> 16]);
       }
-    }
-    for (; p < np; ++p) {
-      const Pair<T> v = Pair<T>::load(V + size_t(p) * VS);
-      const uint32_t cc = ldg_stream4(C + size_t(p) * 128);
-      acc += double(v.a) * double(xs[cc & 0xffffu]);
-      acc += double(v.b) * double(xs[cc >> 16]);
     }
     if (row != 0xffff) {
       const int q = row / RB, jl = row - q * RB;
@@ -218,8 +227,11 @@ k_spmv_xplan(XplanArgs a) {
   };
   // chunks are sorted longest first: warp w takes chunk w and chunk CPT-1-w
   auto process = [&](int t) {
-    process_chunk(t, warp);
-    if (XP_CPW == 2) process_chunk(t, XP_CPT - 1 - warp);
+#pragma unroll 1
+    for (int h = 0; h < XP_CPW; h += 2) {
+      process_chunk(t, h * XP_NW / 2 + warp);
+      if (h + 1 < XP_CPW) process_chunk(t, XP_CPT - 1 - (h * XP_NW / 2 + warp));
+    }
   };
 
   // Only the RB finalizer threads (rounded up to whole warps) wait on the
@@ -228,7 +240,7 @@ k_spmv_xplan(XplanArgs a) {
   // re-arm that expects 0 bytes completes the next phase at once and flips
   // the parity back -- an ABA deadlock seen on CTAs owning no rows of a
   // cluster's last tile.)
-  const int nfin = (RB + 31) & ~31;
+  const int nfin = min((RB + 31) & ~31, XP_THREADS);
   auto finalize = [&](int t) {
     if (int(threadIdx.x) >= nfin) return;
     const double* rv = recv + (t % XP_K) * R;
