@@ -119,8 +119,8 @@ struct spmv_csr_s {
     int B = 0, W = 0, ncl = 0, ntiles = 0;
     size_t smem = 0;
     int64_t bytes = 0, nchunks = 0;
-    long long* chunk_off = nullptr;
-    int *counter = nullptr, *chunk_len = nullptr, *seg = nullptr, *row_slot = nullptr;
+    long long *crow = nullptr, *chunk_off = nullptr;
+    int *tile0 = nullptr, *chunk_len = nullptr, *seg = nullptr, *row_slot = nullptr;
     uint16_t* chunk_row = nullptr;
     unsigned char* plan = nullptr;
     void (*k)(XplanArgs) = nullptr;
@@ -353,9 +353,10 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   a.chunk_len = h->xp.chunk_len;
   a.chunk_row = h->xp.chunk_row;
   a.dbg = dbg() ? 1 : 0;
-  a.m = h->m_loc;
-  a.ntiles = h->xp.ntiles;
-  a.counter = h->xp.counter;
+  a.prefetch = 0;
+  env_int("SPMV_XPLAN_PF", &a.prefetch);
+  a.crow = h->xp.crow;
+  a.tile0 = h->xp.tile0;
   a.x = x;
   a.y = y;
   a.alpha = alpha;
@@ -378,7 +379,6 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   at[0].val.clusterDim.z = 1;
   cfg.attrs = at;
   cfg.numAttrs = 1;
-  CK(cudaMemsetAsync(h->xp.counter, 0, sizeof(int), s));  // dynamic tile counter
   CK(cudaLaunchKernelEx(&cfg, part ? h->xp.kdot : h->xp.k, a));
   LAUNCHED();
   return SPMV_OK;
@@ -391,10 +391,12 @@ static spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only) 
   const int64_t g = std::min<int64_t>(cdiv(h->m_loc * 32, 256), 16LL * num_sms(h->device));
   if (h->dt == SPMV_F64)
     k_xplan_pack<double><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const double*)vals, P.seg, h->m_loc, P.B, P.W,
-                                          P.chunk_off, P.chunk_len, P.row_slot, P.plan, values_only);
+                                          P.crow, P.tile0, P.ncl, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
+                                          values_only);
   else
     k_xplan_pack<float><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const float*)vals, P.seg, h->m_loc, P.B, P.W,
-                                         P.chunk_off, P.chunk_len, P.row_slot, P.plan, values_only);
+                                         P.crow, P.tile0, P.ncl, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
+                                         values_only);
   LAUNCHED();
   return SPMV_OK;
 }
@@ -441,7 +443,7 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   cudaStream_t s = h->stream;
   auto& P = h->xp;
   auto cleanup = [&]() {
-    void* bufs[] = {P.counter, P.chunk_off, P.chunk_len, P.seg, P.row_slot, P.chunk_row, P.plan};
+    void* bufs[] = {P.crow, P.chunk_off, P.tile0, P.chunk_len, P.seg, P.row_slot, P.chunk_row, P.plan};
     for (void* q : bufs)
       if (q) cudaFree(q);
     P = spmv_csr_s::XPlan();
@@ -449,10 +451,19 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   P.B = B; P.W = W; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd;
   DBG("B=%d W=%d ncl=%d smem=%zu", B, W, ncl, smem);
   const int64_t m = h->m_loc;
-  const int ntiles = (int)cdiv(m, XP_R);
+  CK(cudaMalloc(&P.crow, sizeof(long long) * (ncl + 1)));
+  k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(m, h->rp_loc, ncl, P.crow);
+  LAUNCHED();
+  std::vector<long long> crow(ncl + 1);
+  CK(cudaMemcpyAsync(crow.data(), P.crow, sizeof(long long) * (ncl + 1), cudaMemcpyDeviceToHost, s));
+  CK(cudaStreamSynchronize(s));
+  std::vector<int> tile0(ncl + 1, 0);
+  for (int c = 0; c < ncl; ++c) tile0[c + 1] = tile0[c] + (int)cdiv(crow[c + 1] - crow[c], XP_R);
+  const int ntiles = tile0[ncl];
   P.ntiles = ntiles;
   DBG("ntiles=%d", ntiles);
-  CK(cudaMalloc(&P.counter, sizeof(int)));
+  CK(cudaMalloc(&P.tile0, sizeof(int) * (ncl + 1)));
+  CK(cudaMemcpyAsync(P.tile0, tile0.data(), sizeof(int) * (ncl + 1), cudaMemcpyHostToDevice, s));
   if (B > 1) {
     CK(cudaMalloc(&P.seg, sizeof(int) * (size_t)(B - 1) * (size_t)m));
     k_xstat_splits<<<std::min<int64_t>(cdiv(m, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
@@ -467,8 +478,8 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   CK(cudaMalloc(&P.chunk_row, sizeof(uint16_t) * 32 * std::max<int64_t>(nch, 1)));
   CK(cudaMalloc(&P.row_slot, sizeof(int) * (size_t)B * (size_t)m));
   if (ntiles > 0) {
-    k_xplan_sell<<<(unsigned)(ntiles * B), XP_THREADS, 0, s>>>(h->rp_loc, P.seg, m, B, P.chunk_len, P.chunk_row,
-                                                                P.row_slot);
+    k_xplan_sell<<<(unsigned)(ntiles * B), XP_THREADS, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, P.tile0, ncl, P.chunk_len,
+                                                          P.chunk_row, P.row_slot);
     LAUNCHED();
   }
   DBG("sell done nch=%lld", (long long)nch);
@@ -485,13 +496,17 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
     cleanup();
     return SPMV_OK;
   }
-  // chunk offsets in tile-major order [tile][b][chunk]
+  // chunk offsets in stream order [c][b][t][w]: the chunks of one CTA are contiguous
   std::vector<long long> off(std::max<int64_t>(nch, 1), 0);
   long long pos = 0;
-  for (int64_t id = 0; id < nch; ++id) {
-    off[id] = pos;
-    pos += (long long)len[id] * 32 * (ts + 2);
-  }
+  for (int c = 0; c < ncl; ++c)
+    for (int bb = 0; bb < B; ++bb)
+      for (int t = tile0[c]; t < tile0[c + 1]; ++t)
+        for (int w = 0; w < XP_CPT; ++w) {
+          const size_t id = ((size_t)t * B + bb) * XP_CPT + w;
+          off[id] = pos;
+          pos += (long long)len[id] * 32 * (ts + 2);
+        }
   P.bytes = pos;
   CK(cudaMemcpyAsync(P.chunk_off, off.data(), sizeof(long long) * nch, cudaMemcpyHostToDevice, s));
   CK(cudaMalloc(&P.plan, (size_t)std::max<long long>(pos, 16)));
@@ -742,8 +757,7 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
       if (st != SPMV_OK) return fail(st);
       if (ok) {
         h->kernel = SPMV_KERNEL_XPLAN;
-        // dot partials: one per (tile, cluster rank), see k_spmv_xplan
-        h->grid = std::max<int64_t>(1, (int64_t)h->xp.ntiles * h->xp.B);
+        h->grid = (int64_t)h->xp.ncl * h->xp.B;
       }
     }
   } else if (rk == SPMV_KERNEL_XSTAT) {
@@ -769,7 +783,7 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   cudaError_t e = h->stream ? cudaStreamSynchronize(h->stream) : cudaDeviceSynchronize();
   if (e != cudaSuccess) st = cuda_fail(e, "pending asynchronous error", __LINE__);
   h->g_npb.reset();
-  void* bufs[] = {h->xp.counter, h->xp.chunk_off, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
+  void* bufs[] = {h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
                   h->xp.chunk_row, h->xp.plan,
                   h->seg, h->crow, h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,

@@ -11,8 +11,8 @@
 // device-resident "lazy copy" of A) re-lays A out as
 //
 //   clusters of B CTAs; CTA rank b keeps x[b*W, (b+1)*W) (+ a zero pad at W)
-//   in shared memory; the rows are cut into tiles of R = 32*CPT rows, claimed
-//   dynamically by the clusters (see below); inside a tile the rows are sorted by the
+//   in shared memory; cluster c owns rows [crow[c], crow[c+1]) (nnz-balanced),
+//   cut into tiles of R = 32*NW rows; inside a tile the rows are sorted by the
 //   length of their segment in block b (SELL-C-sigma with C = 32, sigma = R)
 //   and cut into NW chunks of 32 rows.  Chunk (tile, b, w) stores len (even)
 //   steps column-major: vals as [len/2][32 lanes][2] (2 values per lane per
@@ -60,15 +60,15 @@ struct XplanArgs {
   const long long* chunk_off;  // [tile][b][chunk] byte offset of chunk data
   const int* chunk_len;        // [tile][b][chunk] steps (even)
   const uint16_t* chunk_row;   // [tile][b][chunk][32] tile-local row of each lane (0xffff = none)
-  int64_t m;                   // rows
-  int ntiles;                  // ceil(m / R)
-  int* counter;                // tile counter (zeroed before every launch)
+  const long long* crow;       // [ncl+1] cluster row ranges
+  const int* tile0;            // [ncl+1] first global tile of each cluster
   const void* x;
   void* y;
   double alpha, beta;
   const void* w;               // DOT: w[i]
-  double* part;                // DOT: one partial per (tile, b): part[tile*B + b]
+  double* part;                // DOT: one partial per CTA
   int dbg;
+  int prefetch;                // 1: L2-prefetch the warp's chunk of the next tile
 };
 
 __device__ __forceinline__ void cluster_arrive_relaxed() {
@@ -129,94 +129,68 @@ struct Pair<float> {
   }
 };
 
-// st.async of a 4-byte value into a peer CTA, completing 4 transaction bytes.
-__device__ __forceinline__ void st_async_u32(uint32_t raddr, uint32_t v, uint32_t rbar) {
-  asm volatile("st.async.shared::cluster.mbarrier::complete_tx::bytes.b32 [%0], %1, [%2];\n" ::"r"(raddr), "r"(v),
-               "r"(rbar)
-               : "memory");
-}
-
 // smem (dynamic): xs [(W+1)*sizeof(T) rounded to 16] | recv [K][R] double
-//   recv[s%K][b*(R/B) + jl]: partial of CTA b for owned row jl of the tile of step s
-//
-// Scheduling: tiles (R consecutive rows) are claimed dynamically: the leader
-// thread of every cluster (rank 0, thread 0) takes the next tile with an
-// atomicAdd one step ahead and sends its id to the B CTAs with st.async into
-// a ring of 4 slots (mbarrier transaction bytes), so fast clusters take more
-// tiles and the kernel ends together.  Protocol (s = step):
-//   init: every CTA arms slots 0..3; after the first cluster barrier the
-//         leader sends the tiles of steps 0 and 1;
-//   step s: all threads wait slot s%4 (tile of step s; >= ntiles ends the
-//         loop), process it, and in the finalize section (after the cluster
-//         barrier wait of step s-1) thread 0 re-arms slot (s+2)%4 for step s+2
-//         (its last reader, step s-2, is over for every thread) and the leader
-//         sends the tile of step s+1 into slot (s+1)%4 (armed at step s-1 or at
-//         init, i.e. before every CTA's arrive that the leader waited for).
-// Every tile row is sent exactly B partials (absent rows of the last tile send
-// 0.0), so the receive byte count of a step is constant.
+//   recv[t%K][b*(R/B) + jl]: partial of CTA b for owned row jl
 template <typename T, bool DOT>
 __global__ void __launch_bounds__(XP_THREADS, 1)
 k_spmv_xplan(XplanArgs a) {
   extern __shared__ __align__(128) unsigned char smem[];
-  __shared__ uint64_t xbar, tbar[XP_K], sbar[4];
-  __shared__ int stile[4];
+  __shared__ uint64_t xbar, tbar[XP_K];
   __shared__ double red[32];
   const int B = (int)cgx::this_cluster().num_blocks();
   const int b = (int)cluster_rank();
+  const int c = (int)cluster_id();
   constexpr int R = XP_R;
   const int RB = R / B;
   const int W = a.W;
-  const int ntiles = a.ntiles;
-  const int64_t m = a.m;
 
   T* xs = reinterpret_cast<T*>(smem);
   double* recv = reinterpret_cast<double*>(smem + ((size_t(W + 1) * sizeof(T) + 15) & ~size_t(15)));
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-  const bool leader = (b == 0 && threadIdx.x == 0);
+  const int64_t r0c = a.crow[c], r1c = a.crow[c + 1];
+  const int ntiles = int((r1c - r0c + R - 1) / R);
+  const int tbase = a.tile0[c];
 
   const int64_t col0 = int64_t(b) * W;
   const int64_t ncols = cmax64(0, cmin64(W, a.nx - col0));
   const T* __restrict__ xg = static_cast<const T*>(a.x);
   const bool x_aligned = (reinterpret_cast<uintptr_t>(xg + col0) & 15) == 0;
   const int64_t bulk_elems = x_aligned ? ((ncols * int64_t(sizeof(T))) & ~int64_t(15)) / int64_t(sizeof(T)) : 0;
-  const uint32_t recv_bytes = uint32_t(RB * B * 8);
 
+  auto recv_bytes = [&](int t) -> uint32_t {
+    const int nrows = int(cmin64(R, r1c - (r0c + int64_t(t) * R)));
+    const int own = max(0, min((b + 1) * RB, nrows) - b * RB);
+    return uint32_t(own * B * 8);
+  };
   if (threadIdx.x == 0) {
     mbar_init(&xbar, 1);
     for (int q = 0; q < XP_K; ++q) mbar_init(&tbar[q], 1);
-    for (int q = 0; q < 4; ++q) mbar_init(&sbar[q], 1);
     asm volatile("fence.mbarrier_init.release.cluster;\n" ::: "memory");
     const uint32_t xb = uint32_t(bulk_elems * sizeof(T));
     mbar_expect_tx(&xbar, xb);
     if (xb) bulk_g2s(xs, xg + col0, xb, &xbar);
-    for (int q = 0; q < XP_K; ++q) mbar_expect_tx(&tbar[q], recv_bytes);
-    for (int q = 0; q < 4; ++q) mbar_expect_tx(&sbar[q], 4);
+    for (int t = 0; t < XP_K && t < ntiles; ++t) mbar_expect_tx(&tbar[t], recv_bytes(t));
   }
   for (int64_t j = bulk_elems + threadIdx.x; j <= W; j += blockDim.x) xs[j] = (j < ncols) ? xg[col0 + j] : T(0);
-  int next_tile = 0;
-  if (leader) next_tile = atomicAdd(a.counter, 1);
-  // peers must have initialised their barriers before anything is sent
+  // peers must have initialised their barriers before partials are sent
   cluster_arrive();
   cluster_wait();
-  auto send_tile = [&](int step, int tile) {
-    const uint32_t slot = smem_u32(&stile[step & 3]), bar = smem_u32(&sbar[step & 3]);
-    for (int q = 0; q < B; ++q) st_async_u32(mapa_u32(slot, q), uint32_t(tile), mapa_u32(bar, q));
-  };
-  if (leader) {
-    send_tile(0, next_tile);
-    send_tile(1, atomicAdd(a.counter, 1));
-    next_tile = atomicAdd(a.counter, 1);  // tile of step 2
-  }
   mbar_wait(&xbar, 0, 1);
 
   const double alpha = a.alpha, beta = a.beta;
   double dacc = 0.0;
 
-  auto process_chunk = [&](int s, int tile, int ch) {
-    const int64_t cid = (int64_t(tile) * B + b) * XP_CPT + ch;
+  auto process_chunk = [&](int t, int ch) {
+    const int64_t cid = (int64_t(tbase + t) * B + b) * XP_CPT + ch;
     const int len = a.chunk_len[cid];
     const int row = a.chunk_row[cid * 32 + lane];
     const unsigned char* base = a.plan + a.chunk_off[cid];
+    if (a.prefetch && lane == 0 && t + 1 < ntiles) {
+      const int64_t nid = cid + int64_t(B) * XP_CPT;
+      const uint32_t nb = uint32_t(a.chunk_len[nid]) * 32u * uint32_t(sizeof(T) + 2);
+      if (nb) asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a.plan + a.chunk_off[nid]), "r"(nb)
+                           : "memory");
+    }
     const unsigned char* V = base + size_t(lane) * 2 * sizeof(T);
     const unsigned char* C = base + size_t(len) * 32 * sizeof(T) + size_t(lane) * 4;
     constexpr size_t VS = 32 * 2 * sizeof(T);  // bytes per step pair (vals)
@@ -245,90 +219,67 @@ k_spmv_xplan(XplanArgs a) {
         acc += double(v[u].b) * double(xs[cc[u] >> 16]);
       }
     }
-    // every row slot of the tile gets B partials (absent rows: 0.0)
-    const int j = row & 0x7fff, q = j / RB, jl = j - q * RB;
-    const uint32_t laddr = smem_u32(recv + (s % XP_K) * R + b * RB + jl);
-    st_async_f64(mapa_u32(laddr, q), (row & 0x8000) ? 0.0 : acc, mapa_u32(smem_u32(&tbar[s % XP_K]), q));
+    if (row != 0xffff) {
+      const int q = row / RB, jl = row - q * RB;
+      const uint32_t laddr = smem_u32(recv + (t % XP_K) * R + b * RB + jl);
+      st_async_f64(mapa_u32(laddr, q), acc, mapa_u32(smem_u32(&tbar[t % XP_K]), q));
+    }
   };
   // chunks are sorted longest first: warp w takes chunk w and chunk CPT-1-w
-  auto process = [&](int s, int tile) {
+  auto process = [&](int t) {
 #pragma unroll 1
     for (int h = 0; h < XP_CPW; h += 2) {
-      process_chunk(s, tile, h * XP_NW / 2 + warp);
-      if (h + 1 < XP_CPW) process_chunk(s, tile, XP_CPT - 1 - (h * XP_NW / 2 + warp));
+      process_chunk(t, h * XP_NW / 2 + warp);
+      if (h + 1 < XP_CPW) process_chunk(t, XP_CPT - 1 - (h * XP_NW / 2 + warp));
     }
   };
 
-  // Only the RB finalizer threads (whole warps) wait on the step's receive
-  // mbarrier, and all of them pass it before thread 0 re-arms it (a late
-  // waiter could otherwise miss the phase: parity ABA).  The dot partial of
-  // (tile, b) goes to part[tile*B + b]: deterministic whichever cluster ran it.
+  // Only the RB finalizer threads (rounded up to whole warps) wait on the
+  // tile's mbarrier; all of them pass the wait before thread 0 re-arms it for
+  // tile t+K.  (If every thread waited, a late warp could miss the phase: a
+  // re-arm that expects 0 bytes completes the next phase at once and flips
+  // the parity back -- an ABA deadlock seen on CTAs owning no rows of a
+  // cluster's last tile.)
   const int nfin = min((RB + 31) & ~31, XP_THREADS);
-  auto finalize = [&](int s, int tile) {
-    if (int(threadIdx.x) < nfin) {
-      const double* rv = recv + (s % XP_K) * R;
-      const int64_t rt = int64_t(tile) * R;
-      const int nrows = int(cmin64(R, m - rt));
-      mbar_wait(&tbar[s % XP_K], (s / XP_K) & 1, 1000000 + 1000 * tile + s);
-      double dt = 0.0;
-      for (int jl = threadIdx.x; jl < RB && b * RB + jl < nrows; jl += nfin) {
-        double sum = 0.0;
-        for (int q = 0; q < B; ++q) sum += rv[q * RB + jl];
-        const int64_t i = rt + b * RB + jl;
-        T* y = static_cast<T*>(a.y);
-        double r = alpha * sum;
-        if (beta != 0.0) r += beta * double(y[i]);
-        const T out = T(r);
-        y[i] = out;
-        if (DOT) dt += double(static_cast<const T*>(a.w)[i]) * double(out);
-      }
-      if (DOT) {
-        dt = warp_sum(dt);
-        if (lane == 0) red[warp] = dt;
-      }
-      asm volatile("bar.sync 2, %0;\n" ::"r"(nfin) : "memory");
-      if (threadIdx.x == 0) {
-        mbar_expect_tx(&tbar[s % XP_K], recv_bytes);  // re-arm for step s+K
-        if (DOT) {
-          double tot = 0.0;
-          for (int w = 0; w < nfin / 32; ++w) tot += red[w];
-          a.part[int64_t(tile) * B + b] = tot;
-        }
-      }
+  auto finalize = [&](int t) {
+    if (int(threadIdx.x) >= nfin) return;
+    const double* rv = recv + (t % XP_K) * R;
+    const int64_t rt = r0c + int64_t(t) * R;
+    const int nrows = int(cmin64(R, r1c - rt));
+    mbar_wait(&tbar[t % XP_K], (t / XP_K) & 1, 1000000 * ntiles + 1000 * t + int(recv_bytes(t) / 8));
+    for (int jl = threadIdx.x; jl < RB && b * RB + jl < nrows; jl += nfin) {
+      double sum = 0.0;
+      for (int q = 0; q < B; ++q) sum += rv[q * RB + jl];
+      const int64_t i = rt + b * RB + jl;
+      T* y = static_cast<T*>(a.y);
+      double r = alpha * sum;
+      if (beta != 0.0) r += beta * double(y[i]);
+      const T out = T(r);
+      y[i] = out;
+      if (DOT) dacc += double(static_cast<const T*>(a.w)[i]) * double(out);
     }
-  };
-  auto next_step_tile = [&](int s) -> int {  // tile of step s (waits for the leader's id)
-    mbar_wait(&sbar[s & 3], (s >> 2) & 1, 2000000 + s);
-    return stile[s & 3];
-  };
-  auto boundary = [&](int s) {  // after the cluster-barrier wait of step s-1
-    if (threadIdx.x == 0 && s >= 2) mbar_expect_tx(&sbar[(s + 2) & 3], 4);  // slot for step s+2
-    if (leader) {
-      send_tile(s + 1, next_tile);
-      next_tile = atomicAdd(a.counter, 1);
-    }
+    asm volatile("bar.sync 2, %0;\n" ::"r"(nfin) : "memory");
+    if (threadIdx.x == 0 && t + XP_K < ntiles) mbar_expect_tx(&tbar[t % XP_K], recv_bytes(t + XP_K));
   };
 
-  int s = 0;
-  int tile = next_step_tile(0);
-  int prev = -1;
-  if (tile < ntiles) {
-    process(0, tile);
+  // Buffer reuse: partials of tile t+K (K = 3) are sent only after the sender
+  // passed wait(t+1), i.e. after every CTA arrived(t+1), which each does after
+  // finalize(t) (reads of recv[t%K] + re-arm of tbar[t%K]).
+  if (ntiles > 0) {
+    process(0);
     cluster_arrive_relaxed();
-    prev = tile;
-    for (s = 1;; ++s) {
-      // the tile of step s was sent during step s-1 (or at init for s = 1)
-      tile = next_step_tile(s);
-      if (tile >= ntiles) break;
-      process(s, tile);
+    for (int t = 1; t < ntiles; ++t) {
+      process(t);
       cluster_wait();
-      finalize(s - 1, prev);
-      boundary(s);
+      finalize(t - 1);
       cluster_arrive_relaxed();
-      prev = tile;
     }
     cluster_wait();
-    finalize(s - 1, prev);
+    finalize(ntiles - 1);
+  }
+  if (DOT) {
+    const double tsum = block_sum(dacc, red);
+    if (threadIdx.x == 0) a.part[blockIdx.x] = tsum;
   }
   // leave together (peers may still be sending to / reading this CTA)
   cluster_arrive();
@@ -342,19 +293,22 @@ __device__ __forceinline__ void xp_seg(const int* rowptr, const int* seg, int64_
   *k1 = (b == B - 1) ? rowptr[i + 1] : seg[int64_t(b) * m + i];
 }
 
-// One CTA (XP_THREADS threads, R/XP_THREADS rows each) per (tile, b), tile g =
-// rows [g*R, (g+1)*R): sort the tile's rows by segment length (descending, ties
-// by row: bitonic sort of (len, row) keys), cut into CPT chunks of 32 lanes,
-// record each chunk's even step count, each lane's tile row (bit 15 set for
-// rows beyond m, which send 0.0) and each row's slot (chunk slot/32, lane slot%32).
+// One CTA (XP_THREADS threads, R/XP_THREADS rows each) per (global tile, b):
+// sort the tile's rows by segment length (descending, ties by row: bitonic
+// sort of (len, row) keys), cut into CPT chunks of 32 lanes, record each
+// chunk's even step count and each row's slot (chunk = slot/32, lane = slot%32).
 __global__ void __launch_bounds__(XP_THREADS)
 k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_t m, int B,
-             int* __restrict__ chunk_len, uint16_t* __restrict__ chunk_row, int* __restrict__ row_slot) {
+             const long long* __restrict__ crow, const int* __restrict__ tile0, int ncl, int* __restrict__ chunk_len,
+             uint16_t* __restrict__ chunk_row, int* __restrict__ row_slot) {
   __shared__ unsigned long long key[XP_R];
   constexpr int PER = XP_R / XP_THREADS;
   const int tg = blockIdx.x / B, b = blockIdx.x % B;
-  const int64_t rt = int64_t(tg) * XP_R;
-  const int nrows = int(cmin64(XP_R, m - rt));
+  int c = 0;
+  while (c + 1 < ncl && tile0[c + 1] <= tg) ++c;
+  const int t = tg - tile0[c];
+  const int64_t rt = crow[c] + int64_t(t) * XP_R;
+  const int nrows = int(cmin64(XP_R, crow[c + 1] - rt));
   for (int e = 0; e < PER; ++e) {
     const int j = threadIdx.x + e * XP_THREADS;
     int L = -1;  // absent rows sort last
@@ -387,7 +341,7 @@ k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_
     const int Ls = int(~uint32_t(kk >> 32)) - 1;
     const int w = j / 32, ln = j % 32;
     const int64_t cid = (int64_t(tg) * B + b) * XP_CPT + w;
-    chunk_row[cid * 32 + ln] = uint16_t(row) | ((Ls >= 0) ? uint16_t(0) : uint16_t(0x8000));
+    chunk_row[cid * 32 + ln] = (Ls >= 0) ? uint16_t(row) : uint16_t(0xffff);
     if (Ls >= 0) row_slot[int64_t(b) * m + rt + row] = j;
     // chunk length = the first (longest) lane's length, rounded up to even
     if (ln == 0) chunk_len[cid] = (max(Ls, 0) + 1) & ~1;
@@ -398,13 +352,19 @@ k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_
 template <typename T>
 __global__ void __launch_bounds__(256)
 k_xplan_pack(const int* __restrict__ rowptr, const int* __restrict__ colidx, const T* __restrict__ vals,
-             const int* __restrict__ seg, int64_t m, int B, int W, const long long* __restrict__ chunk_off,
+             const int* __restrict__ seg, int64_t m, int B, int W, const long long* __restrict__ crow,
+             const int* __restrict__ tile0, int ncl, const long long* __restrict__ chunk_off,
              const int* __restrict__ chunk_len, const int* __restrict__ row_slot, unsigned char* __restrict__ plan,
              int values_only) {
   const int lane = threadIdx.x & 31;
   for (int64_t i = (int64_t(blockIdx.x) * blockDim.x + threadIdx.x) / 32; i < m;
        i += int64_t(gridDim.x) * blockDim.x / 32) {
-    const int tg = int(i / XP_R);
+    int lo = 0, hi = ncl - 1;
+    while (lo < hi) {
+      const int mid = (lo + hi + 1) >> 1;
+      if (crow[mid] <= i) lo = mid; else hi = mid - 1;
+    }
+    const int tg = tile0[lo] + int((i - crow[lo]) / XP_R);
     const int k0 = rowptr[i], k1 = rowptr[i + 1];
     for (int k = k0 + lane; k < k1; k += 32) {
       const int col = colidx[k];
