@@ -141,8 +141,11 @@ def run_ours(args):
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
     d = None
-    if world > 1:
-        dist.init_process_group("nccl", device_id=dev)
+    # SPMV_BENCH_FORCE_DIST=1 runs the row-sharded NCCL path even with one rank
+    # (how the multi-GPU code is exercised on the 1-GPU development box)
+    use_dist = world > 1 or os.environ.get("SPMV_BENCH_FORCE_DIST") == "1"
+    if use_dist:
+        dist.init_process_group("nccl", device_id=dev, rank=rank, world_size=world)
         d = sp.Dist(rank, world, local)
 
     na, nonzer, niter, shift = gen.NPB_CLASSES[CLS]
@@ -161,12 +164,12 @@ def run_ours(args):
 
     def barrier():
         torch.cuda.synchronize(dev)
-        if world > 1:
+        if use_dist:
             dist.barrier(device_ids=[local])
         torch.cuda.synchronize(dev)
 
     def max_over_ranks(v: float) -> float:
-        if world == 1:
+        if not use_dist:
             return v
         t = torch.tensor([v], dtype=torch.float64, device=dev)
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
@@ -265,6 +268,7 @@ def run_ours(args):
             "data": "synthetic (exact NPB makea class C generator, seeded)",
             "config": workload_config(A, world),
             "impl": "ours",
+            "distributed_path": bool(use_dist),
             "kernel": {"name": info["kernel_name"], "vec_lanes": info["vec_lanes"], "grid": info["grid"]},
             "spmv": {
                 "gbs": round(achieved, 1), "gflops": round(2 * nnz_loc / (sp_avg / 1e3) / 1e9, 1),
@@ -289,7 +293,7 @@ def run_ours(args):
     M.destroy()
     if d is not None:
         d.close()
-    if world > 1:
+    if use_dist:
         dist.destroy_process_group()
 
 
