@@ -48,6 +48,22 @@ def log(*a):
     print(*a, file=sys.stderr, flush=True)
 
 
+class stdout_to_stderr:
+    """Route fd 1 to fd 2 while NCCL initialises: NCCL may print its version
+    banner on stdout, and the bench contract is one JSON line on stdout."""
+
+    def __enter__(self):
+        sys.stdout.flush()
+        self.saved = os.dup(1)
+        os.dup2(2, 1)
+        return self
+
+    def __exit__(self, *a):
+        sys.stdout.flush()
+        os.dup2(self.saved, 1)
+        os.close(self.saved)
+
+
 def measured_peaks():
     p = os.path.join(ROOT, "MEASURED_PEAKS.json")
     try:
@@ -145,8 +161,10 @@ def run_ours(args):
     # (how the multi-GPU code is exercised on the 1-GPU development box)
     use_dist = world > 1 or os.environ.get("SPMV_BENCH_FORCE_DIST") == "1"
     if use_dist:
-        dist.init_process_group("nccl", device_id=dev, rank=rank, world_size=world)
-        d = sp.Dist(rank, world, local)
+        with stdout_to_stderr():
+            dist.init_process_group("nccl", device_id=dev, rank=rank, world_size=world)
+            d = sp.Dist(rank, world, local)
+            dist.barrier(device_ids=[local])
 
     na, nonzer, niter, shift = gen.NPB_CLASSES[CLS]
     t0 = time.time()
