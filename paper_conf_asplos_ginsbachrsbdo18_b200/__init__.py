@@ -62,6 +62,7 @@ cg_solve_c = _decl("cg_solve", [_P, _P, _P, _I32, _D, ctypes.POINTER(_I32), ctyp
 cg_npb_outer_c = _decl("cg_npb_outer", [_P, _P, _P, _I32, _D, _P])
 spmv_cg_status_c = _decl("spmv_cg_status", [_P])
 spmv_csr_update_values_c = _decl("spmv_csr_update_values", [_P, _P])
+spmv_csr_merge_splits_device_c = _decl("spmv_csr_merge_splits_device", [_P, _P, _P, _I64, ctypes.POINTER(_I64)])
 spmv_csr_destroy_c = _decl("spmv_csr_destroy", [_P])
 spmv_csr_partition_c = _decl("spmv_csr_partition", [_P, _I64, _I32, _P])
 spmv_csr_merge_splits_c = _decl("spmv_csr_merge_splits", [_P, _I64, _I64, _P, _P])
@@ -77,7 +78,7 @@ spmv_dist_colidx_c = _decl("spmv_dist_colidx", [_P, _P])
 
 # every symbol include/spmv.h declares (checked by tests/test_abi.py)
 EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_status",
-           "spmv_csr_update_values",
+           "spmv_csr_update_values", "spmv_csr_merge_splits_device",
            "spmv_csr_destroy", "spmv_csr_partition", "spmv_csr_merge_splits", "spmv_csr_info",
            "spmv_launch_count", "spmv_status_string", "spmv_last_error_string",
            "spmv_dist_get_unique_id", "spmv_dist_init", "spmv_dist_destroy", "spmv_dist_plan_host",
@@ -239,6 +240,19 @@ class CSRMatrix:
         out = np.zeros(self._info["nnz_local"], dtype=np.int32)
         _check(spmv_dist_colidx_c(self.handle, out.ctypes.data), "spmv_dist_colidx")
         return out
+
+    def merge_splits_device(self):
+        """(split_row, split_nz) the MERGE kernel uses, or None."""
+        import numpy as np
+        cnt = _I64(0)
+        _check(spmv_csr_merge_splits_device_c(self.handle, None, None, 0, ctypes.byref(cnt)), "merge_splits_device")
+        if cnt.value == 0:
+            return None
+        sr = np.zeros(cnt.value, np.int64)
+        sn = np.zeros(cnt.value, np.int64)
+        _check(spmv_csr_merge_splits_device_c(self.handle, sr.ctypes.data, sn.ctypes.data, cnt.value,
+                                              ctypes.byref(cnt)), "merge_splits_device")
+        return sr, sn
 
     def update_values(self, vals):
         """Re-bind the values (same structure) and refresh the plan copy."""

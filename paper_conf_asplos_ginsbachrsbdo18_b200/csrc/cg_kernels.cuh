@@ -141,6 +141,17 @@ __global__ void k_finish_norm(SumSrc res, double* out) {
   if (threadIdx.x == 0) *out = sqrt(rr);
 }
 
+// Per-CTA partials of w.y (used after SpMV kernels without a fused dot).
+__global__ void __launch_bounds__(256)
+k_dot_partials(int64_t n, const double* __restrict__ w, const double* __restrict__ y, double* __restrict__ part) {
+  __shared__ double red[8];
+  double acc = 0.0;
+  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n; j += int64_t(gridDim.x) * blockDim.x)
+    acc += w[j] * y[j];
+  const double t = block_sum(acc, red);
+  if (threadIdx.x == 0) part[blockIdx.x] = t;
+}
+
 // Distributed mode: sum `count` partials into one value (then all-reduced).
 __global__ void k_finalize(SumSrc s, double* out) {
   __shared__ double s0;

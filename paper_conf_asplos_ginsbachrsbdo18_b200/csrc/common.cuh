@@ -8,6 +8,9 @@ namespace spmv {
 
 constexpr int kNumSMs = 148;  // B200: 2 dies x 74 SMs (queried at run time too)
 
+__device__ __forceinline__ int64_t cmin64(int64_t a, int64_t b) { return a < b ? a : b; }
+__device__ __forceinline__ int64_t cmax64(int64_t a, int64_t b) { return a > b ? a : b; }
+
 // ---------------------------------------------------------------- loads
 // Streamed operands (vals, colidx) are read exactly once per SpMV: bypass L1
 // so the L1 capacity is left to the x gathers (ld.global.nc.L1::no_allocate).

@@ -21,6 +21,7 @@
 #include "spmv_kernels.cuh"
 #include "xstat_kernel.cuh"
 #include "xplan_kernel.cuh"
+#include "merge_kernel.cuh"
 
 using namespace spmv;
 
@@ -126,6 +127,13 @@ struct spmv_csr_s {
     void (*k)(XplanArgs) = nullptr;
     void (*kdot)(XplanArgs) = nullptr;
   } xp;
+  // MERGE (merge-path tiles)
+  struct {
+    int ntiles = 0;
+    long long *split_row = nullptr, *split_nz = nullptr;
+    double *head = nullptr, *carry = nullptr;
+    int* head_flag = nullptr;
+  } mg;
   // dist
   spmv_dist_s* dist = nullptr;
   std::vector<long long> bounds;
@@ -524,6 +532,56 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   return SPMV_OK;
 }
 
+static spmv_status merge_setup(spmv_csr_s* h) {
+  const int64_t items = h->m_loc + (h->k1 - h->k0);
+  const int64_t C = std::max<int64_t>(1, cdiv(items, MG_D));
+  if (C > 2147483647LL) return arg_fail("matrix too large for the merge kernel");
+  auto& G = h->mg;
+  G.ntiles = (int)C;
+  CK(cudaMalloc(&G.split_row, sizeof(long long) * (C + 1)));
+  CK(cudaMalloc(&G.split_nz, sizeof(long long) * (C + 1)));
+  CK(cudaMalloc(&G.head, sizeof(double) * C));
+  CK(cudaMalloc(&G.carry, sizeof(double) * C));
+  CK(cudaMalloc(&G.head_flag, sizeof(int) * C));
+  k_merge_splits<<<(unsigned)cdiv(C + 1, 256), 256, 0, h->stream>>>(h->m_loc, h->rp_loc, C, G.split_row, G.split_nz);
+  LAUNCHED();
+  CK(cudaStreamSynchronize(h->stream));
+  return SPMV_OK;
+}
+
+static spmv_status launch_merge(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
+                                double alpha, double beta) {
+  MergeArgs a;
+  a.m = h->m_loc;
+  a.ntiles = h->mg.ntiles;
+  a.rowptr = h->rp_loc;
+  a.colidx = h->ci_loc;
+  a.vals = vals;
+  a.split_row = h->mg.split_row;
+  a.split_nz = h->mg.split_nz;
+  a.x = x;
+  a.y = y;
+  a.alpha = alpha;
+  a.beta = beta;
+  a.head = h->mg.head;
+  a.carry = h->mg.carry;
+  a.head_flag = h->mg.head_flag;
+  if (h->dt == SPMV_F64) {
+    k_spmv_merge<double><<<a.ntiles, MG_NT, 0, s>>>(a);
+    LAUNCHED();
+    k_merge_fixup<double><<<(unsigned)cdiv(a.ntiles, 256), 256, 0, s>>>(a);
+    LAUNCHED();
+  } else {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+    k_spmv_merge<float><<<a.ntiles, MG_NT, 0, s>>>(a);
+    LAUNCHED();
+    k_merge_fixup<float><<<(unsigned)cdiv(a.ntiles, 256), 256, 0, s>>>(a);
+    LAUNCHED();
+  }
+  return SPMV_OK;
+}
+
 // Local SpMV of the handle: y = alpha*A_loc*x + beta*y (+ partial w.y per CTA).
 static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
                             double alpha, double beta, const double* w, double* part) {
@@ -543,6 +601,14 @@ static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, con
   if (h->kernel == SPMV_KERNEL_XPLAN && vals == h->vals) return launch_xplan(h, s, x, y, alpha, beta, w, part);
   const int64_t vgrid_spmv = h->kernel == SPMV_KERNEL_XPLAN ? h->grid_vec : h->grid;
   if (h->kernel == SPMV_KERNEL_XSTAT) return launch_xstat(h, s, vals, x, y, alpha, beta, w, part);
+  if (h->kernel == SPMV_KERNEL_MERGE) {
+    ST(launch_merge(h, s, vals, x, y, alpha, beta));
+    if (part) {  // no fused dot in the merge kernel: one pass over w, y
+      k_dot_partials<<<(int)h->vgrid, 256, 0, s>>>(h->m_loc, w, (const double*)y, part);
+      LAUNCHED();
+    }
+    return SPMV_OK;
+  }
   SpmvArgs a;
   a.m = h->m_loc;
   a.rowptr = h->rp_loc;
@@ -760,6 +826,17 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
         h->grid = (int64_t)h->xp.ncl * h->xp.B;
       }
     }
+  }
+  if (h->kernel != SPMV_KERNEL_XPLAN && rk != SPMV_KERNEL_VECTOR && rk != SPMV_KERNEL_SCALAR && rk != SPMV_KERNEL_XSTAT &&
+      h->m_loc > 0 &&
+      (rk == SPMV_KERNEL_MERGE || (double)h->row_max > 32.0 * std::max(h->row_mean, 1.0))) {
+    // skewed rows (a long row would pin one warp of the vector kernel): merge path
+    spmv_status st = merge_setup(h);
+    if (st != SPMV_OK) return fail(st);
+    h->kernel = SPMV_KERNEL_MERGE;
+    h->grid = h->vgrid;  // dot partials come from k_dot_partials
+  }
+  if (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_MERGE) {
   } else if (rk == SPMV_KERNEL_XSTAT) {
     bool ok = false;
     spmv_status st = xstat_setup(h, &ok);
@@ -783,7 +860,7 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   cudaError_t e = h->stream ? cudaStreamSynchronize(h->stream) : cudaDeviceSynchronize();
   if (e != cudaSuccess) st = cuda_fail(e, "pending asynchronous error", __LINE__);
   h->g_npb.reset();
-  void* bufs[] = {h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
+  void* bufs[] = {h->mg.split_row, h->mg.split_nz, h->mg.head, h->mg.carry, h->mg.head_flag, h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
                   h->xp.chunk_row, h->xp.plan,
                   h->seg, h->crow, h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
@@ -1180,6 +1257,18 @@ extern "C" spmv_status spmv_dist_colidx(spmv_csr_t h, int32_t* colidx_local_host
   CK(cudaSetDevice(h->device));
   CK(cudaMemcpy(colidx_local_host, h->ci_own, sizeof(int32_t) * (size_t)(h->k1 - h->k0),
                 cudaMemcpyDeviceToHost));
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_csr_merge_splits_device(spmv_csr_t h, int64_t* split_row, int64_t* split_nz,
+                                                    int64_t cap, int64_t* count) {
+  if (!h || !count) return arg_fail("NULL argument");
+  *count = h->kernel == SPMV_KERNEL_MERGE ? (int64_t)h->mg.ntiles + 1 : 0;
+  if (*count == 0 || !split_row || !split_nz) return SPMV_OK;
+  if (cap < *count) return arg_fail("cap too small");
+  CK(cudaSetDevice(h->device));
+  CK(cudaMemcpy(split_row, h->mg.split_row, sizeof(long long) * (size_t)*count, cudaMemcpyDeviceToHost));
+  CK(cudaMemcpy(split_nz, h->mg.split_nz, sizeof(long long) * (size_t)*count, cudaMemcpyDeviceToHost));
   return SPMV_OK;
 }
 

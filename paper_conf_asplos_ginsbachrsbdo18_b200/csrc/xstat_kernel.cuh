@@ -41,8 +41,6 @@ struct XstatArgs {
   double* part;           // DOT: one partial per CTA
 };
 
-__device__ __forceinline__ int64_t cmin64(int64_t a, int64_t b) { return a < b ? a : b; }
-__device__ __forceinline__ int64_t cmax64(int64_t a, int64_t b) { return a > b ? a : b; }
 __device__ __forceinline__ uint32_t smem_u32(const void* p) {
   return static_cast<uint32_t>(__cvta_generic_to_shared(p));
 }

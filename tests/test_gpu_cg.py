@@ -152,3 +152,21 @@ def test_npb_graph_vs_eager_bitexact(sp, torch_dev, monkeypatch):
     monkeypatch.setenv("SPMV_GRAPH", "0")
     _, z2, r2 = _npb(sp, torch, dev, "S", niter=3)
     assert np.array_equal(z1, z2) and np.array_equal(r1, r2)
+
+
+@pytest.mark.parametrize("kernel", ["merge", "vector", "xstat", "xplan"])
+def test_npb_s_every_kernel(sp, torch_dev, kernel):
+    """NPB class S zeta with every SpMV kernel inside CG (fused or separate dot)."""
+    torch, dev = torch_dev
+    na, nonzer, niter, shift = gen.NPB_CLASSES["S"]
+    A = gen.makea("S")
+    rp, ci, va = to_dev(A, dev)
+    with sp.CSRMatrix(rp, ci, va, A.n, kernel=kernel) as M:
+        assert M.info()["kernel_name"] == kernel
+        x = torch.ones(A.n, dtype=torch.float64, device=dev)
+        z = torch.empty_like(x)
+        out = torch.zeros(2, dtype=torch.float64, device=dev)
+        for _ in range(niter):
+            M.npb_outer(x, z, 25, shift, out)
+        zeta = float(out[0].item())
+    assert abs(zeta - gen.NPB_ZETA["S"]) / gen.NPB_ZETA["S"] <= 1e-10

@@ -326,3 +326,33 @@ def test_plan_off_uses_zero_copy(sp, torch_dev):
     with sp.CSRMatrix(rp, ci, va, A.n, plan=False) as M:
         inf = M.info()
         assert inf["kernel_name"] == "vector" and inf["plan_bytes"] == 0
+
+
+@pytest.mark.parametrize("name,A", ZOO, ids=[c[0] for c in ZOO])
+def test_zoo_merge(sp, torch_dev, name, A):
+    """Merge-path kernel (equal rows+nnz tiles, segmented-scan carries,
+    tile-order fix-up of rows spanning tiles) on every zoo case, fp64 and fp32,
+    and its device splits equal the host/oracle splits bit for bit (R21)."""
+    torch, dev = torch_dev
+    x = gen.uniform(A.n, seed=19)
+    info = run_case(sp, torch, dev, A, x, kernel="merge", what=f"{name} merge")
+    if A.m > 0:
+        assert info["kernel_name"] == "merge"
+        rp, ci, va = to_dev(A, dev)
+        with sp.CSRMatrix(rp, ci, va, A.n, kernel="merge") as M:
+            sr, sn = M.merge_splits_device()
+        C = len(sr) - 1
+        orr, onz = oracle.merge_path(A.rowptr, C)
+        assert np.array_equal(sr, orr) and np.array_equal(sn, onz)
+    A32 = A.astype(np.float32)
+    run_case(sp, torch, dev, A32, gen.uniform(A.n, seed=20, f32=True), kernel="merge", what=f"{name} merge fp32")
+    y0 = gen.uniform(A.m, seed=21)
+    run_case(sp, torch, dev, A, x, alpha=-2.0, beta=0.5, y0=y0, kernel="merge", what=f"{name} merge a/b")
+
+
+def test_parboil_auto_is_merge(sp, torch_dev):
+    torch, dev = torch_dev
+    A = gen.powerlaw()
+    x = gen.uniform(A.n, seed=42, f32=True)
+    info = run_case(sp, torch, dev, A, x, what="parboil auto")
+    assert info["kernel_name"] == "merge"

@@ -1,3 +1,2 @@
-SPMV_BENCH_FORCE_DIST=1 timeout 300 python -m torch.distributed.run --nnodes=1 --nproc-per-node 1 --master-addr 127.0.0.1 --master-port 29511 bench.py --gpus 1 --steps 5 --warmup 3 --no-cpu > gpurun_out/bench_dist1.json 2> gpurun_out/bench_dist1.err; echo "rc $?"; cut -c1-600 gpurun_out/bench_dist1.json; tail -5 gpurun_out/bench_dist1.err
-timeout 300 python -m torch.distributed.run --nnodes=1 --nproc-per-node 1 --master-addr 127.0.0.1 --master-port 29512 bench.py --gpus 1 --steps 5 --warmup 3 --no-cpu > gpurun_out/bench_tr1.json 2> gpurun_out/bench_tr1.err; echo "rc $?"; cut -c1-300 gpurun_out/bench_tr1.json
-timeout 300 python bench.py --impl reference --steps 2 --warmup 3 > gpurun_out/bench_ref.json 2> gpurun_out/bench_ref.err; echo "rc $?"; cut -c1-400 gpurun_out/bench_ref.json
+timeout 600 python -m pytest tests -m gpu -x -q > gpurun_out/pytest_gpu.log 2>&1; echo "pytest exit $?" >> gpurun_out/pytest_gpu.log; tail -3 gpurun_out/pytest_gpu.log; grep -E "^E |FAILED" gpurun_out/pytest_gpu.log | head -8
+for k in merge vector; do timeout 60 python tools/time_one.py $k parboil $k; done
