@@ -69,11 +69,27 @@ k_spmv_merge(MergeArgs a) {
   const int nr = int(r1 - r0), nn = int(k1 - k0);
 
   // 1. stage row ends (relative nz index) and products
+  // all IPT colidx/vals loads of a thread are issued before the x gathers,
+  // and all gathers before any use (IPT independent chains in flight)
   for (int i = tid; i < nr; i += MG_NT) s_end[i] = __ldg(rowptr + r0 + 1 + i) - base;
-  for (int j = tid; j < nn; j += MG_NT) {
-    const int64_t k = base + k0 + j;
-    const int c = ld_stream(a.colidx + k);
-    s_prod[j] = double(ld_stream(vals + k)) * double(__ldg(x + c));
+  {
+    int c[MG_IPT];
+    T v[MG_IPT];
+#pragma unroll
+    for (int u = 0; u < MG_IPT; ++u) {
+      const int j = tid + u * MG_NT;
+      const int64_t k = base + k0 + j;
+      c[u] = (j < nn) ? ld_stream(a.colidx + k) : -1;
+      v[u] = (j < nn) ? ld_stream(vals + k) : T(0);
+    }
+    T xv[MG_IPT];
+#pragma unroll
+    for (int u = 0; u < MG_IPT; ++u) xv[u] = (c[u] >= 0) ? __ldg(x + c[u]) : T(0);
+#pragma unroll
+    for (int u = 0; u < MG_IPT; ++u) {
+      const int j = tid + u * MG_NT;
+      if (j < nn) s_prod[j] = double(v[u]) * double(xv[u]);
+    }
   }
   __syncthreads();
 
@@ -88,18 +104,27 @@ k_spmv_merge(MergeArgs a) {
   const int i_start = lo, j_start = d - lo;
   const int dend = min(d + MG_IPT, nr + nn);
 
-  // walk: carry-out of the row open at the end of this thread's items
+  // walk (fully unrolled, so the emitted partials stay in registers):
+  // item `it` closes row i_start+ (number of earlier closes) when it is a row end
   int i = i_start, j = j_start;
   double run = 0.0;
   int closed = 0;
-  for (int it = d; it < dend; ++it) {
-    if (i < nr && int64_t(s_end[i]) <= k0 + j) {
-      ++i;
-      run = 0.0;
-      closed = 1;
-    } else {
-      run += s_prod[j];
-      ++j;
+  double emit[MG_IPT];
+  uint32_t cmask = 0;  // bit it: item it closed a row
+#pragma unroll
+  for (int it = 0; it < MG_IPT; ++it) {
+    emit[it] = 0.0;
+    if (d + it < dend) {
+      if (i < nr && int64_t(s_end[i]) <= k0 + j) {
+        emit[it] = run;
+        cmask |= 1u << it;
+        ++i;
+        run = 0.0;
+        closed = 1;
+      } else {
+        run += s_prod[j];
+        ++j;
+      }
     }
   }
 
@@ -123,27 +148,27 @@ k_spmv_merge(MergeArgs a) {
   if (lane == 0) exc = SegPair{0, 0.0};
   exc = seg_op(wpre, exc);  // carry-in of this thread (partial of row i_start)
 
-  // 4. emit closed rows
+  // 4. emit closed rows (the first one receives the carry-in)
   T* __restrict__ y = static_cast<T*>(a.y);
   const bool head_deferred = (int64_t(__ldg(rowptr + r0)) - base) < k0;  // row r0 began earlier
-  i = i_start;
-  j = j_start;
-  run = exc.v;
-  for (int it = d; it < dend; ++it) {
-    if (i < nr && int64_t(s_end[i]) <= k0 + j) {
-      const int64_t row = r0 + i;
-      if (i == 0 && head_deferred) {
-        a.head[t] = run;
-      } else {
-        double r = a.alpha * run;
-        if (a.beta != 0.0) r += a.beta * double(y[row]);
-        y[row] = T(r);
+  {
+    int row_i = i_start;
+    bool first = true;
+#pragma unroll
+    for (int it = 0; it < MG_IPT; ++it) {
+      if (cmask & (1u << it)) {
+        const double val = first ? emit[it] + exc.v : emit[it];
+        first = false;
+        const int64_t row = r0 + row_i;
+        if (row_i == 0 && head_deferred) {
+          a.head[t] = val;
+        } else {
+          double r = a.alpha * val;
+          if (a.beta != 0.0) r += a.beta * double(y[row]);
+          y[row] = T(r);
+        }
+        ++row_i;
       }
-      ++i;
-      run = 0.0;
-    } else {
-      run += s_prod[j];
-      ++j;
     }
   }
   if (tid == MG_NT - 1) {
