@@ -45,7 +45,8 @@ class SpmvInfo(ctypes.Structure):
     _fields_ = [("kernel", _I32), ("vec_lanes", _I32), ("row_min", _I64), ("row_max", _I64),
                 ("row_mean", _D), ("row_cv", _D), ("m_local", _I64), ("row_begin", _I64),
                 ("row_end", _I64), ("nnz_local", _I64), ("rank", _I32), ("nranks", _I32),
-                ("sorted_cols", _I32), ("grid", _I64), ("cluster", _I32), ("plan_bytes", _I64)]
+                ("sorted_cols", _I32), ("grid", _I64), ("cluster", _I32), ("plan_bytes", _I64),
+                ("transport", _I32)]
 
 
 def _decl(name, args, res=_ST):
@@ -73,6 +74,9 @@ spmv_last_error_string = _decl("spmv_last_error_string", [], ctypes.c_char_p)
 spmv_dist_get_unique_id_c = _decl("spmv_dist_get_unique_id", [_P])
 spmv_dist_init_c = _decl("spmv_dist_init", [ctypes.POINTER(_P), _I32, _I32, _P, _I32])
 spmv_dist_destroy_c = _decl("spmv_dist_destroy", [_P])
+spmv_dist_init_p2p_c = _decl("spmv_dist_init_p2p", [ctypes.POINTER(_P), _I32, _I32, _I32])
+spmv_csr_p2p_handle_c = _decl("spmv_csr_p2p_handle", [_P, _P])
+spmv_csr_p2p_connect_c = _decl("spmv_csr_p2p_connect", [_P, _P])
 spmv_dist_plan_host_c = _decl("spmv_dist_plan_host", [_P, _P, _I64, _I32, _I32, _P, _P, _P])
 spmv_dist_colidx_c = _decl("spmv_dist_colidx", [_P, _P])
 
@@ -82,7 +86,7 @@ EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_s
            "spmv_csr_destroy", "spmv_csr_partition", "spmv_csr_merge_splits", "spmv_csr_info",
            "spmv_launch_count", "spmv_status_string", "spmv_last_error_string",
            "spmv_dist_get_unique_id", "spmv_dist_init", "spmv_dist_destroy", "spmv_dist_plan_host",
-           "spmv_dist_colidx"]
+           "spmv_dist_colidx", "spmv_dist_init_p2p", "spmv_csr_p2p_handle", "spmv_csr_p2p_connect"]
 
 
 class SpmvError(RuntimeError):
@@ -149,12 +153,26 @@ def spmv_dist_plan_host(rowptr_host, colidx_host, nranks: int, rank: int):
 
 # ------------------------------------------------------------- distributed
 class Dist:
-    """NCCL context of the library, bootstrapped through a torch process group
-    (torch.distributed is used only to broadcast the 128-byte unique id)."""
+    """Distributed context of the library.
 
-    def __init__(self, rank: int, nranks: int, device: int, group=None):
+    transport="nccl": an NCCL communicator bootstrapped through a torch process
+    group (torch.distributed only broadcasts the 128-byte unique id).
+    transport="p2p": no NCCL; exchanges run in the library's kernels over
+    CUDA-IPC peer memory; IPC handles are all-gathered through the torch
+    process group when a CSRMatrix is created.
+    """
+
+    def __init__(self, rank: int, nranks: int, device: int, group=None, transport: str = "nccl"):
         import torch
         import torch.distributed as dist
+        self.group = group
+        self.transport = transport
+        self.rank, self.nranks, self.device = rank, nranks, device
+        if transport == "p2p":
+            h = _P()
+            _check(spmv_dist_init_p2p_c(ctypes.byref(h), rank, nranks, device), "spmv_dist_init_p2p")
+            self.handle = h
+            return
         uid = (ctypes.c_char * 128)()
         if rank == 0:
             _check(spmv_dist_get_unique_id_c(ctypes.addressof(uid)), "spmv_dist_get_unique_id")
@@ -210,6 +228,17 @@ class CSRMatrix:
                                  self.m, self.n, nnz, _ptr(rowptr), _ptr(colidx), _ptr(vals),
                                  ctypes.byref(o)), "spmv_csr_create")
         self.handle = h
+        if dist is not None and dist.transport == "p2p":
+            import torch.distributed as tdist
+            mine = (ctypes.c_char * 64)()
+            _check(spmv_csr_p2p_handle_c(h, ctypes.addressof(mine)), "spmv_csr_p2p_handle")
+            allh = [None] * dist.nranks
+            tdist.all_gather_object(allh, bytes(mine), group=dist.group)
+            buf = (ctypes.c_char * (64 * dist.nranks))()
+            for q, hb in enumerate(allh):
+                ctypes.memmove(ctypes.addressof(buf) + 64 * q, hb, 64)
+            _check(spmv_csr_p2p_connect_c(h, ctypes.addressof(buf)), "spmv_csr_p2p_connect")
+            tdist.barrier(group=dist.group)
         self._info = self.info()
 
     # -- calls ------------------------------------------------------------

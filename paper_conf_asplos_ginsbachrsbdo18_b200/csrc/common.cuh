@@ -73,21 +73,66 @@ __device__ __forceinline__ double block_sum_n(double v, double* red, int nw) {
   return t;
 }
 
-// A scalar source for the CG kernels: either `count` per-block partials to be
-// summed (single GPU: every consuming block sums them in the same fixed order,
-// so all blocks see bit-identical scalars), or count == 1 pointing at a
-// finalized (and, in distributed mode, NCCL-all-reduced) value.
+__device__ __forceinline__ void st_release_sys_u64(unsigned long long* p, unsigned long long v) {
+  asm volatile("st.release.sys.global.u64 [%0], %1;\n" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ unsigned long long ld_acquire_sys_u64(const unsigned long long* p) {
+  unsigned long long v;
+  asm volatile("ld.acquire.sys.global.u64 %0, [%1];\n" : "=l"(v) : "l"(p) : "memory");
+  return v;
+}
+
+// Wait until every peer completed exchange epoch `e` (watchdog: trap after ~2 s).
+__device__ __forceinline__ void p2p_wait_flags(const unsigned long long* flags, int me, int P,
+                                               unsigned long long e) {
+  for (int q = 0; q < P; ++q) {
+    if (q == me) continue;
+    long long t0 = 0;
+    for (uint32_t spin = 0; ld_acquire_sys_u64(flags + q) < e; ++spin) {
+      if ((spin & 1023) == 1023) {
+        const long long now = clock64();
+        if (t0 == 0) t0 = now;
+        else if (now - t0 > 4000000000LL) {
+          printf("spmv: p2p wait timeout rank %d waits rank %d for epoch %llu (has %llu)\n", me, q, e,
+                 ld_acquire_sys_u64(flags + q));
+          __trap();
+        }
+      }
+    }
+  }
+}
+
+// A scalar source for the CG kernels: either `count` > 0 per-block partials to
+// be summed (single GPU: every consuming block sums them in the same fixed
+// order, so all blocks see bit-identical scalars), count == 1 pointing at a
+// finalized (NCCL-all-reduced) value, or count == -P: the P values pushed by
+// the ranks over peer memory (p2p_kernels.cuh), read once flags[q] >= *epoch
+// for every other rank q and summed in rank order (identical on all ranks).
 struct SumSrc {
   const double* p;
   int count;
+  const unsigned long long* flags = nullptr;
+  const unsigned long long* epoch = nullptr;
+  int me = 0;
 };
 
 // Sum of a SumSrc by warp 0 of the block; returns the value in every thread.
 __device__ __forceinline__ double read_sum(SumSrc s, double* slot) {
   if (threadIdx.x < 32) {
+    int n = s.count;
+    if (n < 0) {
+      n = -n;
+      if (threadIdx.x == 0) p2p_wait_flags(s.flags, s.me, n, *s.epoch);
+      __syncwarp();
+    }
     double a = 0.0;
-    for (int i = threadIdx.x; i < s.count; i += 32) a += s.p[i];
-    a = warp_sum(a);
+    if (s.count < 0) {
+      if (threadIdx.x == 0)
+        for (int i = 0; i < n; ++i) a += s.p[i];  // rank order
+    } else {
+      for (int i = threadIdx.x; i < n; i += 32) a += s.p[i];
+      a = warp_sum(a);
+    }
     if (threadIdx.x == 0) *slot = a;
   }
   __syncthreads();

@@ -22,6 +22,7 @@
 #include "xstat_kernel.cuh"
 #include "xplan_kernel.cuh"
 #include "merge_kernel.cuh"
+#include "p2p_kernels.cuh"
 
 using namespace spmv;
 
@@ -67,8 +68,9 @@ static spmv_status arg_fail(const char* why) {
 
 // ------------------------------------------------------------------ types
 struct spmv_dist_s {
-  ncclComm_t comm = nullptr;
+  ncclComm_t comm = nullptr;  // NCCL transport (nullptr for p2p)
   int rank = 0, nranks = 1, device = 0;
+  int p2p = 0;                // 1: exchanges over CUDA-IPC peer memory (p2p_kernels.cuh)
 };
 
 struct Graph {
@@ -140,6 +142,13 @@ struct spmv_csr_s {
   long long maxlen = 0;
   int32_t* ci_own = nullptr;
   void* xpad = nullptr;               // nranks*maxlen, the gathered x / p
+  // p2p transport: the IPC-exported fabric (xpad | exch | flags) and local counters
+  unsigned char* fabric = nullptr;
+  size_t fab_bytes = 0, off_exch = 0, off_flags = 0;
+  unsigned long long* p2p_local = nullptr;  // [0] epoch, [1..NSLOT+1] slot_epoch, then ticket
+  unsigned char** peer_table = nullptr;     // device [P]
+  std::vector<unsigned char*> peers;        // host copy (opened IPC mappings)
+  bool p2p_connected = false;
   // CG workspace (lazy)
   double *z = nullptr, *r = nullptr, *q = nullptr, *p_single = nullptr;
   double *part_pq = nullptr, *part_rr = nullptr, *part_res = nullptr, *part_xz = nullptr,
@@ -789,12 +798,31 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
     h->k0 = kk[0];
     h->k1 = kk[1];
     const int64_t nloc = h->k1 - h->k0;
-    if (cudaMalloc(&h->ci_own, sizeof(int32_t) * std::max<int64_t>(nloc, 1)) != cudaSuccess ||
-        cudaMalloc(&h->xpad, h->ts * (size_t)(maxlen * P)) != cudaSuccess) {
+    bool okm = cudaMalloc(&h->ci_own, sizeof(int32_t) * std::max<int64_t>(nloc, 1)) == cudaSuccess;
+    if (okm && !d->p2p) {
+      okm = cudaMalloc(&h->xpad, h->ts * (size_t)(maxlen * P)) == cudaSuccess;
+      if (okm) cudaMemsetAsync(h->xpad, 0, h->ts * (size_t)(maxlen * P), s);
+    } else if (okm) {
+      // fabric: xpad | exch [NSLOT][P] double | flags [P] u64, one IPC-exportable allocation
+      const size_t xb = (h->ts * (size_t)(maxlen * P) + 255) & ~size_t(255);
+      h->off_exch = xb;
+      h->off_flags = xb + ((sizeof(double) * P2P_NSLOT * P + 255) & ~size_t(255));
+      h->fab_bytes = h->off_flags + ((sizeof(unsigned long long) * P + 255) & ~size_t(255));
+      okm = cudaMalloc(&h->fabric, h->fab_bytes) == cudaSuccess &&
+            cudaMalloc(&h->p2p_local, sizeof(unsigned long long) * (P2P_NSLOT + 4)) == cudaSuccess &&
+            cudaMalloc(&h->peer_table, sizeof(unsigned char*) * P) == cudaSuccess;
+      if (okm) {
+        cudaMemsetAsync(h->fabric, 0, h->fab_bytes, s);
+        cudaMemsetAsync(h->p2p_local, 0, sizeof(unsigned long long) * (P2P_NSLOT + 4), s);
+        h->xpad = h->fabric;
+        h->peers.assign(P, nullptr);
+        h->peers[d->rank] = h->fabric;
+      }
+    }
+    if (!okm) {
       cudaFree(dbounds);
       return fail(cuda_fail(cudaErrorMemoryAllocation, "cudaMalloc", __LINE__));
     }
-    cudaMemsetAsync(h->xpad, 0, h->ts * (size_t)(maxlen * P), s);
     if (nloc > 0) {
       k_renumber<<<std::min<int64_t>(cdiv(nloc, 256), 8LL * sms), 256, sizeof(long long) * (P + 1), s>>>(
           h->k0, h->k1, colidx, dbounds, P, maxlen, h->ci_own);
@@ -860,7 +888,13 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   cudaError_t e = h->stream ? cudaStreamSynchronize(h->stream) : cudaDeviceSynchronize();
   if (e != cudaSuccess) st = cuda_fail(e, "pending asynchronous error", __LINE__);
   h->g_npb.reset();
-  void* bufs[] = {h->mg.split_row, h->mg.split_nz, h->mg.head, h->mg.carry, h->mg.head_flag, h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
+  for (size_t q = 0; q < h->peers.size(); ++q)
+    if (h->peers[q] && h->peers[q] != h->fabric) cudaIpcCloseMemHandle(h->peers[q]);
+  if (h->fabric) {
+    cudaFree(h->fabric);
+    if (h->xpad == h->fabric) h->xpad = nullptr;
+  }
+  void* bufs[] = {h->p2p_local, h->peer_table, h->mg.split_row, h->mg.split_nz, h->mg.head, h->mg.carry, h->mg.head_flag, h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
                   h->xp.chunk_row, h->xp.plan,
                   h->seg, h->crow, h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
@@ -875,6 +909,8 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
 }
 
 // ------------------------------------------------------------------ spmv
+static spmv_status exchange_x(spmv_csr_s* h, cudaStream_t s);
+
 extern "C" spmv_status spmv_csr(spmv_csr_t h, int64_t m, int64_t n, int64_t nnz,
                                 const int32_t* rowptr, const int32_t* colidx, const void* vals,
                                 const void* x, void* y, double alpha, double beta) {
@@ -905,8 +941,7 @@ extern "C" spmv_status spmv_csr(spmv_csr_t h, int64_t m, int64_t n, int64_t nnz,
     spmv_dist_s* d = h->dist;
     char* mine = (char*)h->xpad + ts * (size_t)(d->rank * h->maxlen);
     if (ml > 0 && x != mine) CK(cudaMemcpyAsync(mine, x, ts * (size_t)ml, cudaMemcpyDeviceToDevice, s));
-    NK(ncclAllGather(mine, h->xpad, (size_t)h->maxlen, h->dt == SPMV_F64 ? ncclDouble : ncclFloat,
-                     d->comm, s));
+    ST(exchange_x(h, s));
     xin = h->xpad;
   }
   return run_spmv(h, s, vals, xin, y, alpha, beta, nullptr, nullptr);
@@ -933,6 +968,39 @@ static spmv_status cg_alloc(spmv_csr_s* h) {
   return SPMV_OK;
 }
 
+static P2PCtx p2p_ctx(spmv_csr_s* h) {
+  P2PCtx c;
+  c.peer = h->peer_table;
+  c.off_exch = h->off_exch;
+  c.off_flags = h->off_flags;
+  c.epoch = h->p2p_local;
+  c.slot_epoch = h->p2p_local + 1;
+  c.ticket = reinterpret_cast<int*>(h->p2p_local + 2 + P2P_NSLOT);
+  c.me = h->dist->rank;
+  c.P = h->dist->nranks;
+  return c;
+}
+
+static bool use_p2p(const spmv_csr_s* h) { return h->dist && h->dist->p2p; }
+
+// All-gather of this rank's slice (already at xpad + rank*maxlen) and wait.
+static spmv_status exchange_x(spmv_csr_s* h, cudaStream_t s) {
+  if (use_p2p(h)) {
+    if (!h->p2p_connected) return arg_fail("p2p handle not connected (spmv_csr_p2p_connect)");
+    const P2PCtx c = p2p_ctx(h);
+    const int g = (int)std::max<int64_t>(1, std::min<int64_t>(cdiv(h->m_loc, 256), 2LL * num_sms(h->device)));
+    if (h->dt == SPMV_F64) k_p2p_push_x<double><<<g, 256, 0, s>>>(h->m_loc, h->maxlen, c);
+    else k_p2p_push_x<float><<<g, 256, 0, s>>>(h->m_loc, h->maxlen, c);
+    LAUNCHED();
+    k_p2p_wait_x<<<1, 1, 0, s>>>(c);
+    LAUNCHED();
+    return SPMV_OK;
+  }
+  NK(ncclAllGather((char*)h->xpad + h->ts * (size_t)(h->dist->rank * h->maxlen), h->xpad, (size_t)h->maxlen,
+                   h->dt == SPMV_F64 ? ncclDouble : ncclFloat, h->dist->comm, s));
+  return SPMV_OK;
+}
+
 static double* cg_p(spmv_csr_s* h) {
   if (!h->dist) return h->p_single;
   return (double*)h->xpad + h->dist->rank * h->maxlen;
@@ -942,6 +1010,20 @@ static double* cg_p(spmv_csr_s* h) {
 // and all-reduced over the ranks; single GPU returns the partials unchanged.
 static spmv_status reduce_src(spmv_csr_s* h, cudaStream_t s, SumSrc in, int slot, SumSrc* out) {
   if (!h->dist) { *out = in; return SPMV_OK; }
+  if (use_p2p(h)) {
+    if (!h->p2p_connected) return arg_fail("p2p handle not connected (spmv_csr_p2p_connect)");
+    const P2PCtx c = p2p_ctx(h);
+    k_p2p_push_sum<<<1, 32, 0, s>>>(in, slot, c);
+    LAUNCHED();
+    SumSrc o;
+    o.p = reinterpret_cast<const double*>(h->fabric + h->off_exch) + slot * c.P;
+    o.count = -c.P;
+    o.flags = reinterpret_cast<const unsigned long long*>(h->fabric + h->off_flags);
+    o.epoch = c.slot_epoch + slot;
+    o.me = c.me;
+    *out = o;
+    return SPMV_OK;
+  }
   double* dst = h->scal + slot;
   k_finalize<<<1, 32, 0, s>>>(in, dst);
   LAUNCHED();
@@ -952,9 +1034,7 @@ static spmv_status reduce_src(spmv_csr_s* h, cudaStream_t s, SumSrc in, int slot
 
 static spmv_status gather_p(spmv_csr_s* h, cudaStream_t s) {
   if (!h->dist) return SPMV_OK;
-  NK(ncclAllGather((double*)h->xpad + h->dist->rank * h->maxlen, h->xpad, (size_t)h->maxlen,
-                   ncclDouble, h->dist->comm, s));
-  return SPMV_OK;
+  return exchange_x(h, s);
 }
 
 // CG enqueue state: the scalar sources carried between iterations.
@@ -1286,6 +1366,7 @@ extern "C" spmv_status spmv_csr_info(spmv_csr_t h, spmv_info_t* info) {
   info->row_end = h->row0 + h->m_loc;
   info->nnz_local = h->k1 - h->k0;
   info->rank = h->dist ? h->dist->rank : 0;
+  info->transport = h->dist ? (h->dist->p2p ? 2 : 1) : 0;
   info->nranks = h->dist ? h->dist->nranks : 1;
   info->sorted_cols = h->sorted;
   info->grid = h->grid;
@@ -1339,6 +1420,49 @@ extern "C" spmv_status spmv_dist_init(spmv_dist_t* out, int32_t rank, int32_t nr
     return SPMV_ERR_NCCL;
   }
   *out = d;
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_dist_init_p2p(spmv_dist_t* out, int32_t rank, int32_t nranks, int32_t device) {
+  if (!out || nranks < 1 || rank < 0 || rank >= nranks) return arg_fail("bad dist arguments");
+  *out = nullptr;
+  CK(cudaSetDevice(device));
+  spmv_dist_s* d = new spmv_dist_s();
+  d->rank = rank;
+  d->nranks = nranks;
+  d->device = device;
+  d->p2p = 1;
+  *out = d;
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_csr_p2p_handle(spmv_csr_t h, void* handle64) {
+  if (!h || !handle64) return arg_fail("NULL argument");
+  if (!use_p2p(h)) return arg_fail("not a p2p distributed handle");
+  static_assert(sizeof(cudaIpcMemHandle_t) == 64, "cudaIpcMemHandle_t is 64 bytes");
+  CK(cudaSetDevice(h->device));
+  cudaIpcMemHandle_t m;
+  CK(cudaIpcGetMemHandle(&m, h->fabric));
+  memcpy(handle64, &m, 64);
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_csr_p2p_connect(spmv_csr_t h, const void* handles) {
+  if (!h || !handles) return arg_fail("NULL argument");
+  if (!use_p2p(h)) return arg_fail("not a p2p distributed handle");
+  CK(cudaSetDevice(h->device));
+  const int P = h->dist->nranks, me = h->dist->rank;
+  for (int q = 0; q < P; ++q) {
+    if (q == me || h->peers[q]) continue;
+    cudaIpcMemHandle_t m;
+    memcpy(&m, (const char*)handles + 64 * q, 64);
+    void* ptr = nullptr;
+    CK(cudaIpcOpenMemHandle(&ptr, m, cudaIpcMemLazyEnablePeerAccess));
+    h->peers[q] = (unsigned char*)ptr;
+  }
+  CK(cudaMemcpy(h->peer_table, h->peers.data(), sizeof(unsigned char*) * P, cudaMemcpyHostToDevice));
+  CK(cudaDeviceSynchronize());
+  h->p2p_connected = true;
   return SPMV_OK;
 }
 

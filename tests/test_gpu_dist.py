@@ -77,3 +77,37 @@ def test_dist1_cg_solve(env):
         its, rn = M.cg_solve(b, x, 50, tol=1e-13)
     j = np.arange(50)
     assert np.allclose(x.cpu().numpy(), (j + 1) * (50 - j) / 2.0, rtol=1e-10)
+
+
+@pytest.fixture(scope="module")
+def p2p1(env):
+    torch, dev, sp, d = env
+    dp = sp.Dist(0, 1, 0, transport="p2p")
+    yield dp
+    dp.close()
+
+
+def test_p2p1_spmv_and_npb_bitexact(env, p2p1):
+    """1-rank p2p transport (push/wait kernels, exchange-mode scalar sources)
+    reproduces the single-GPU results bit for bit."""
+    torch, dev, sp, d = env
+    A = gen.makea("S")
+    rp, ci, va = to_dev(A, dev)
+    x = torch.from_numpy(gen.uniform(A.n, seed=5)).to(dev)
+    y1 = torch.empty(A.m, dtype=torch.float64, device=dev)
+    y2 = torch.empty_like(y1)
+    res = []
+    for dd in (None, p2p1):
+        with sp.CSRMatrix(rp, ci, va, A.n, dist=dd) as M:
+            M.spmv(x, y1 if dd is None else y2)
+            xs = torch.ones(A.n, dtype=torch.float64, device=dev)
+            z = torch.empty_like(xs)
+            out = torch.zeros((3, 2), dtype=torch.float64, device=dev)
+            for it in range(3):
+                M.npb_outer(xs, z, 25, 10.0, out[it])
+            torch.cuda.synchronize()
+            res.append(out.cpu().numpy())
+            if dd is not None:
+                assert M.info()["transport"] == 2
+    assert torch.equal(y1, y2)
+    assert np.array_equal(res[0], res[1])
