@@ -82,7 +82,8 @@ def workload_config(A, n_gpus):
         "n": int(A.n), "nnz": int(A.nnz), "cgitmax": 25,
         "bytes_per_spmv": int(A.bytes_per_spmv()),
         "l2": "flushed between timed steps (256 MiB write); A = 436 MB > 126 MB L2",
-        "parallelism": f"row-shard x{n_gpus} (nnz-balanced), NCCL allgather x + allreduce dots",
+        "parallelism": f"row-shard x{n_gpus} (nnz-balanced); x all-gather + dot all-reduces over peer memory "
+                       f"(p2p kernels) or NCCL",
     }
 
 
@@ -160,10 +161,13 @@ def run_ours(args):
     # SPMV_BENCH_FORCE_DIST=1 runs the row-sharded NCCL path even with one rank
     # (how the multi-GPU code is exercised on the 1-GPU development box)
     use_dist = world > 1 or os.environ.get("SPMV_BENCH_FORCE_DIST") == "1"
+    # transport of the row-sharded exchange: "p2p" (our kernels over CUDA-IPC
+    # peer memory / NVLink, default) or "nccl"
+    transport = os.environ.get("SPMV_TRANSPORT", "p2p")
     if use_dist:
         with stdout_to_stderr():
             dist.init_process_group("nccl", device_id=dev, rank=rank, world_size=world)
-            d = sp.Dist(rank, world, local)
+            d = sp.Dist(rank, world, local, transport=transport)
             dist.barrier(device_ids=[local])
 
     na, nonzer, niter, shift = gen.NPB_CLASSES[CLS]
@@ -173,7 +177,18 @@ def run_ours(args):
     rp = torch.from_numpy(A.rowptr).to(dev)
     ci = torch.from_numpy(A.colidx).to(dev)
     va = torch.from_numpy(A.vals).to(dev)
-    M = sp.CSRMatrix(rp, ci, va, A.n, dist=d)
+    try:
+        M = sp.CSRMatrix(rp, ci, va, A.n, dist=d)
+    except sp.SpmvError as e:
+        if d is None or transport != "p2p":
+            raise
+        # peer mappings unavailable on this node: the NCCL transport (all ranks agree)
+        log(f"[rank {rank}] p2p transport unavailable ({e}); using NCCL")
+        d.close()
+        transport = "nccl"
+        with stdout_to_stderr():
+            d = sp.Dist(rank, world, local, transport="nccl")
+        M = sp.CSRMatrix(rp, ci, va, A.n, dist=d)
     info = M.info()
     b0, b1 = info["row_begin"], info["row_end"]
     nl = b1 - b0
@@ -287,6 +302,7 @@ def run_ours(args):
             "config": workload_config(A, world),
             "impl": "ours",
             "distributed_path": bool(use_dist),
+            "transport": transport if use_dist else None,
             "kernel": {"name": info["kernel_name"], "vec_lanes": info["vec_lanes"], "grid": info["grid"]},
             "spmv": {
                 "gbs": round(achieved, 1), "gflops": round(2 * nnz_loc / (sp_avg / 1e3) / 1e9, 1),

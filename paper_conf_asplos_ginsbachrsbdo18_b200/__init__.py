@@ -237,7 +237,15 @@ class CSRMatrix:
             buf = (ctypes.c_char * (64 * dist.nranks))()
             for q, hb in enumerate(allh):
                 ctypes.memmove(ctypes.addressof(buf) + 64 * q, hb, 64)
-            _check(spmv_csr_p2p_connect_c(h, ctypes.addressof(buf)), "spmv_csr_p2p_connect")
+            st = spmv_csr_p2p_connect_c(h, ctypes.addressof(buf))
+            # every rank must agree before anyone uses the peer mappings
+            oks = [None] * dist.nranks
+            tdist.all_gather_object(oks, st == SPMV_OK, group=dist.group)
+            if not all(oks):
+                err = SpmvError(st if st != SPMV_OK else SPMV_ERR_CUDA, "spmv_csr_p2p_connect (some rank failed)")
+                spmv_csr_destroy_c(h)
+                self.handle = None
+                raise err
             tdist.barrier(group=dist.group)
         self._info = self.info()
 

@@ -39,7 +39,7 @@ k_cg_init(int64_t n, const double* __restrict__ b, double* __restrict__ z,
 __global__ void __launch_bounds__(256)
 k_cg_zr(int64_t n, SumSrc pq, SumSrc rr_old, const double* __restrict__ p,
         const double* __restrict__ q, double* __restrict__ z, double* __restrict__ r,
-        double* __restrict__ part_rr_new, int* __restrict__ flags) {
+        double* __restrict__ part_rr_new, int* __restrict__ flags, P2PHook hk) {
   __shared__ double red[8];
   __shared__ double s_pq, s_rr;
   if (flags[1]) return;  // converged (tol mode): no-op
@@ -60,21 +60,36 @@ k_cg_zr(int64_t n, SumSrc pq, SumSrc rr_old, const double* __restrict__ p,
   }
   const double t = block_sum(acc, red);
   if (threadIdx.x == 0) part_rr_new[blockIdx.x] = t;
+  p2p_push_partials_last(hk, part_rr_new, gridDim.x);
 }
 
 // K3.  rr_new: rho', rr_old: rho.  tol > 0: after the update, mark converged
 // once sqrt(rho') <= tol * ||b|| (rr_b: ||b||^2 source), recording `it`+1.
 __global__ void __launch_bounds__(256)
 k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
-       double* __restrict__ p, int* __restrict__ flags, double tol, SumSrc rr_b, int it) {
+       double* __restrict__ p, int* __restrict__ flags, double tol, SumSrc rr_b, int it, P2PHook hk,
+       int64_t xoff) {
   __shared__ double s_new, s_old, s_b;
   if (flags[1]) return;
   const double rho1 = read_sum(rr_new, &s_new);
   const double rho0 = read_sum(rr_old, &s_old);
   const double beta = rho1 / rho0;
   for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n;
-       j += int64_t(gridDim.x) * blockDim.x)
-    p[j] = r[j] + beta * p[j];
+       j += int64_t(gridDim.x) * blockDim.x) {
+    const double pj = r[j] + beta * p[j];
+    p[j] = pj;
+    if (hk.enabled)  // fused all-gather: the slice goes straight into every peer's xpad
+      for (int q = 0; q < hk.c.P; ++q)
+        if (q != hk.c.me) reinterpret_cast<double*>(hk.c.peer[q])[xoff + j] = pj;
+  }
+  if (hk.enabled) {
+    __threadfence_system();
+    __syncthreads();
+    if (threadIdx.x == 0 && atomicAdd(hk.c.ticket, 1) == int(gridDim.x) - 1) {
+      *hk.c.ticket = 0;
+      p2p_signal(hk.c, P2P_XSLOT);
+    }
+  }
   if (tol > 0.0) {
     const double bb = read_sum(rr_b, &s_b);
     if (blockIdx.x == 0 && threadIdx.x == 0) {
@@ -143,13 +158,15 @@ __global__ void k_finish_norm(SumSrc res, double* out) {
 
 // Per-CTA partials of w.y (used after SpMV kernels without a fused dot).
 __global__ void __launch_bounds__(256)
-k_dot_partials(int64_t n, const double* __restrict__ w, const double* __restrict__ y, double* __restrict__ part) {
+k_dot_partials(int64_t n, const double* __restrict__ w, const double* __restrict__ y, double* __restrict__ part,
+               P2PHook hk) {
   __shared__ double red[8];
   double acc = 0.0;
   for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n; j += int64_t(gridDim.x) * blockDim.x)
     acc += w[j] * y[j];
   const double t = block_sum(acc, red);
   if (threadIdx.x == 0) part[blockIdx.x] = t;
+  p2p_push_partials_last(hk, part, gridDim.x);
 }
 
 // Distributed mode: sum `count` partials into one value (then all-reduced).

@@ -102,6 +102,80 @@ __device__ __forceinline__ void p2p_wait_flags(const unsigned long long* flags, 
   }
 }
 
+constexpr int P2P_NSLOT = 8;       // scalar slots (same ids as reduce_src slots)
+constexpr int P2P_XSLOT = P2P_NSLOT;  // slot_epoch index of the x exchange
+
+struct P2PCtx {
+  unsigned char* const* peer;      // device array [P]: fabric base of every rank (own included)
+  size_t off_exch, off_flags;      // byte offsets inside a fabric
+  unsigned long long* epoch;       // local exchange counter
+  unsigned long long* slot_epoch;  // local [P2P_NSLOT + 1]
+  int* ticket;                     // local last-CTA ticket
+  int me, P;
+};
+
+// Publish: bump the local epoch, record it for `slot`, flag every peer.
+__device__ __forceinline__ void p2p_signal(const P2PCtx& c, int slot) {
+  __threadfence_system();
+  const unsigned long long e = *c.epoch + 1;
+  *c.epoch = e;
+  c.slot_epoch[slot] = e;
+  for (int q = 0; q < c.P; ++q) {
+    if (q == c.me) continue;
+    unsigned long long* f = reinterpret_cast<unsigned long long*>(c.peer[q] + c.off_flags);
+    st_release_sys_u64(f + c.me, e);
+  }
+}
+
+// Exchange hook carried by the compute kernels in the p2p transport (all
+// zero / disabled otherwise):
+//   wait_x    -- the kernel reads x from xpad: thread 0 of every CTA first
+//                waits until every peer published the latest x exchange;
+//   push_slot -- the kernel writes one dot partial per CTA into part[]: the
+//                last CTA to finish sums them (read_sum order) and pushes the
+//                value into `push_slot` of every rank (fused all-reduce half).
+struct P2PHook {
+  P2PCtx c;
+  int enabled = 0;
+  int wait_x = 0;
+  int push_slot = -1;
+};
+
+__device__ __forceinline__ void p2p_prologue_wait(const P2PHook& h) {
+  if (h.enabled && h.wait_x) {
+    if (threadIdx.x == 0) {
+      const unsigned long long* flags =
+          reinterpret_cast<const unsigned long long*>(h.c.peer[h.c.me] + h.c.off_flags);
+      p2p_wait_flags(flags, h.c.me, h.c.P, h.c.slot_epoch[P2P_XSLOT]);
+    }
+    __syncthreads();
+  }
+}
+
+// Call from every thread of every CTA after part[blockIdx.x] was written.
+__device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const double* part, int count) {
+  if (!h.enabled || h.push_slot < 0) return;
+  __shared__ int s_last;
+  __threadfence();
+  __syncthreads();
+  if (threadIdx.x == 0) s_last = (atomicAdd(h.c.ticket, 1) == int(gridDim.x) - 1);
+  __syncthreads();
+  if (!s_last) return;
+  if (threadIdx.x < 32) {
+    double a = 0.0;
+    for (int i = threadIdx.x; i < count; i += 32) a += __ldcg(part + i);  // L2: other CTAs' stores
+    a = warp_sum(a);
+    if (threadIdx.x == 0) {
+      *h.c.ticket = 0;
+      for (int q = 0; q < h.c.P; ++q) {
+        double* ex = reinterpret_cast<double*>(h.c.peer[q] + h.c.off_exch);
+        ex[h.push_slot * h.c.P + h.c.me] = a;
+      }
+      p2p_signal(h.c, h.push_slot);
+    }
+  }
+}
+
 // A scalar source for the CG kernels: either `count` > 0 per-block partials to
 // be summed (single GPU: every consuming block sums them in the same fixed
 // order, so all blocks see bit-identical scalars), count == 1 pointing at a

@@ -42,6 +42,7 @@ struct MergeArgs {
   double* head;              // [ntiles] in-tile partial of a deferred first row
   double* carry;             // [ntiles] partial of the row open at the tile end
   int* head_flag;            // [ntiles] 1 if the tile's first closed row is deferred
+  P2PHook hk;                // p2p transport: wait for x
 };
 
 struct SegPair {
@@ -67,6 +68,7 @@ k_spmv_merge(MergeArgs a) {
   const int64_t r0 = a.split_row[t], r1 = a.split_row[t + 1];
   const int64_t k0 = a.split_nz[t], k1 = a.split_nz[t + 1];
   const int nr = int(r1 - r0), nn = int(k1 - k0);
+  p2p_prologue_wait(a.hk);
 
   // 1. stage row ends (relative nz index) and products
   // all IPT colidx/vals loads of a thread are issued before the x gathers,

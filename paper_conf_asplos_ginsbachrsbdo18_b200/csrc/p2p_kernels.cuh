@@ -22,31 +22,6 @@
 
 namespace spmv {
 
-constexpr int P2P_NSLOT = 8;       // scalar slots (same ids as reduce_src slots)
-constexpr int P2P_XSLOT = P2P_NSLOT;  // slot_epoch index of the x exchange
-
-struct P2PCtx {
-  unsigned char* const* peer;      // device array [P]: fabric base of every rank (own included)
-  size_t off_exch, off_flags;      // byte offsets inside a fabric
-  unsigned long long* epoch;       // local exchange counter
-  unsigned long long* slot_epoch;  // local [P2P_NSLOT + 1]
-  int* ticket;                     // local last-CTA ticket
-  int me, P;
-};
-
-// Publish: bump the local epoch, record it for `slot`, flag every peer.
-__device__ __forceinline__ void p2p_signal(const P2PCtx& c, int slot) {
-  __threadfence_system();
-  const unsigned long long e = *c.epoch + 1;
-  *c.epoch = e;
-  c.slot_epoch[slot] = e;
-  for (int q = 0; q < c.P; ++q) {
-    if (q == c.me) continue;
-    unsigned long long* f = reinterpret_cast<unsigned long long*>(c.peer[q] + c.off_flags);
-    st_release_sys_u64(f + c.me, e);
-  }
-}
-
 // All-reduce, push half: sum `in` (fixed order) and push it into slot `slot`
 // of every rank.  One CTA.
 __global__ void k_p2p_push_sum(SumSrc in, int slot, P2PCtx c) {

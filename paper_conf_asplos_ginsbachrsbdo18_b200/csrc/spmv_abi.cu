@@ -254,7 +254,7 @@ static void (*xstat_fn(int G, int U))(XstatArgs) {
 }
 
 static spmv_status launch_xstat(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
-                                double alpha, double beta, const double* w, double* part) {
+                                double alpha, double beta, const double* w, double* part, const P2PHook& hook) {
   XstatArgs a;
   a.m = h->m_loc;
   a.nx = h->nx;
@@ -271,6 +271,7 @@ static spmv_status launch_xstat(spmv_csr_s* h, cudaStream_t s, const void* vals,
   a.beta = beta;
   a.w = w;
   a.part = part;
+  a.hk = hook;
   if (h->dt == SPMV_F32) {
     a.alpha = (double)(float)alpha;
     a.beta = (double)(float)beta;
@@ -361,7 +362,7 @@ static spmv_status xstat_setup(spmv_csr_s* h, bool* ok) {
 }
 
 static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha,
-                                double beta, const double* w, double* part) {
+                                double beta, const double* w, double* part, const P2PHook& hook) {
   XplanArgs a;
   a.nx = h->nx;
   a.W = h->xp.W;
@@ -559,7 +560,7 @@ static spmv_status merge_setup(spmv_csr_s* h) {
 }
 
 static spmv_status launch_merge(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
-                                double alpha, double beta) {
+                                double alpha, double beta, const P2PHook& hook) {
   MergeArgs a;
   a.m = h->m_loc;
   a.ntiles = h->mg.ntiles;
@@ -575,6 +576,7 @@ static spmv_status launch_merge(spmv_csr_s* h, cudaStream_t s, const void* vals,
   a.head = h->mg.head;
   a.carry = h->mg.carry;
   a.head_flag = h->mg.head_flag;
+  a.hk = hook;
   if (h->dt == SPMV_F64) {
     k_spmv_merge<double><<<a.ntiles, MG_NT, 0, s>>>(a);
     LAUNCHED();
@@ -593,7 +595,9 @@ static spmv_status launch_merge(spmv_csr_s* h, cudaStream_t s, const void* vals,
 
 // Local SpMV of the handle: y = alpha*A_loc*x + beta*y (+ partial w.y per CTA).
 static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
-                            double alpha, double beta, const double* w, double* part) {
+                            double alpha, double beta, const double* w, double* part,
+                            const P2PHook* hk = nullptr) {
+  const P2PHook hook = hk ? *hk : P2PHook();
   if (h->m_loc == 0) {
     if (part) {
       CK(cudaMemsetAsync(part, 0, sizeof(double) * h->grid, s));
@@ -607,13 +611,17 @@ static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, con
     LAUNCHED();
     return SPMV_OK;
   }
-  if (h->kernel == SPMV_KERNEL_XPLAN && vals == h->vals) return launch_xplan(h, s, x, y, alpha, beta, w, part);
+  if (h->kernel == SPMV_KERNEL_XPLAN && vals == h->vals) return launch_xplan(h, s, x, y, alpha, beta, w, part, hook);
   const int64_t vgrid_spmv = h->kernel == SPMV_KERNEL_XPLAN ? h->grid_vec : h->grid;
-  if (h->kernel == SPMV_KERNEL_XSTAT) return launch_xstat(h, s, vals, x, y, alpha, beta, w, part);
+  if (h->kernel == SPMV_KERNEL_XSTAT) return launch_xstat(h, s, vals, x, y, alpha, beta, w, part, hook);
   if (h->kernel == SPMV_KERNEL_MERGE) {
-    ST(launch_merge(h, s, vals, x, y, alpha, beta));
+    P2PHook wait_only = hook;
+    wait_only.push_slot = -1;
+    ST(launch_merge(h, s, vals, x, y, alpha, beta, wait_only));
     if (part) {  // no fused dot in the merge kernel: one pass over w, y
-      k_dot_partials<<<(int)h->vgrid, 256, 0, s>>>(h->m_loc, w, (const double*)y, part);
+      P2PHook push_only = hook;
+      push_only.wait_x = 0;
+      k_dot_partials<<<(int)h->vgrid, 256, 0, s>>>(h->m_loc, w, (const double*)y, part, push_only);
       LAUNCHED();
     }
     return SPMV_OK;
@@ -629,6 +637,7 @@ static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, con
   a.beta = beta;
   a.w = w;
   a.part = part;
+  a.hk = hook;
   if (h->dt == SPMV_F64) {
     if (part) launch_vec<double, true>(h->lanes, h->unroll, vgrid_spmv, s, a);
     else launch_vec<double, false>(h->lanes, h->unroll, vgrid_spmv, s, a);
@@ -1008,6 +1017,18 @@ static double* cg_p(spmv_csr_s* h) {
 
 // In distributed mode a SumSrc of per-CTA partials is finalized into scal[slot]
 // and all-reduced over the ranks; single GPU returns the partials unchanged.
+// The exchange-mode scalar source of `slot` (values pushed by every rank).
+static SumSrc p2p_src(spmv_csr_s* h, int slot) {
+  const P2PCtx c = p2p_ctx(h);
+  SumSrc o;
+  o.p = reinterpret_cast<const double*>(h->fabric + h->off_exch) + slot * c.P;
+  o.count = -c.P;
+  o.flags = reinterpret_cast<const unsigned long long*>(h->fabric + h->off_flags);
+  o.epoch = c.slot_epoch + slot;
+  o.me = c.me;
+  return o;
+}
+
 static spmv_status reduce_src(spmv_csr_s* h, cudaStream_t s, SumSrc in, int slot, SumSrc* out) {
   if (!h->dist) { *out = in; return SPMV_OK; }
   if (use_p2p(h)) {
@@ -1015,13 +1036,7 @@ static spmv_status reduce_src(spmv_csr_s* h, cudaStream_t s, SumSrc in, int slot
     const P2PCtx c = p2p_ctx(h);
     k_p2p_push_sum<<<1, 32, 0, s>>>(in, slot, c);
     LAUNCHED();
-    SumSrc o;
-    o.p = reinterpret_cast<const double*>(h->fabric + h->off_exch) + slot * c.P;
-    o.count = -c.P;
-    o.flags = reinterpret_cast<const unsigned long long*>(h->fabric + h->off_flags);
-    o.epoch = c.slot_epoch + slot;
-    o.me = c.me;
-    *out = o;
+    *out = p2p_src(h, slot);
     return SPMV_OK;
   }
   double* dst = h->scal + slot;
@@ -1053,6 +1068,7 @@ static spmv_status cg_enqueue_init(spmv_csr_s* h, cudaStream_t s, const double* 
   ST(reduce_src(h, s, SumSrc{prb, vg}, 0, &run->rr_b));
   run->rr_old = run->rr_b;
   run->it = 0;
+  if (use_p2p(h)) ST(exchange_x(h, s));  // p = b to every peer; later rounds are fused into k_cg_p
   return SPMV_OK;
 }
 
@@ -1065,18 +1081,40 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
   const void* xg = h->dist ? h->xpad : (const void*)p;
   const int vg = (int)h->vgrid, sg = (int)h->grid;
   const int64_t pstride = std::max(std::max(h->grid, h->grid_vec), h->vgrid);
+  const bool p2p = use_p2p(h);
+  P2PHook base;
+  if (p2p) {
+    base.c = p2p_ctx(h);
+    base.enabled = 1;
+  }
   for (int c = 0; c < iters; ++c) {
     const int it = run->it++;
-    ST(gather_p(h, s));
-    ST(run_spmv(h, s, h->vals, xg, h->q, 1.0, 0.0, p, h->part_pq));
     SumSrc pq;
-    ST(reduce_src(h, s, SumSrc{h->part_pq, sg}, 1, &pq));
+    if (p2p) {
+      // fused exchange: the SpMV waits for the peers' p slices (pushed by
+      // k_cg_p / the init exchange) and its last CTA pushes p.q (slot 1)
+      P2PHook hs = base;
+      hs.wait_x = 1;
+      hs.push_slot = 1;
+      ST(run_spmv(h, s, h->vals, xg, h->q, 1.0, 0.0, p, h->part_pq, &hs));
+      pq = p2p_src(h, 1);
+    } else {
+      ST(gather_p(h, s));
+      ST(run_spmv(h, s, h->vals, xg, h->q, 1.0, 0.0, p, h->part_pq));
+      ST(reduce_src(h, s, SumSrc{h->part_pq, sg}, 1, &pq));
+    }
     double* pnew = h->part_rr + ((it + 1) & 1) * pstride;
-    k_cg_zr<<<vg, 256, 0, s>>>(n, pq, run->rr_old, p, h->q, z, h->r, pnew, h->flags);
+    const int rslot = 2 + ((it + 1) & 1);
+    P2PHook hz = base;
+    hz.push_slot = p2p ? rslot : -1;
+    k_cg_zr<<<vg, 256, 0, s>>>(n, pq, run->rr_old, p, h->q, z, h->r, pnew, h->flags, hz);
     LAUNCHED();
     SumSrc rr_new;
-    ST(reduce_src(h, s, SumSrc{pnew, vg}, 2 + ((it + 1) & 1), &rr_new));
-    k_cg_p<<<vg, 256, 0, s>>>(n, rr_new, run->rr_old, h->r, p, h->flags, tol, run->rr_b, it);
+    if (p2p) rr_new = p2p_src(h, rslot);
+    else ST(reduce_src(h, s, SumSrc{pnew, vg}, rslot, &rr_new));
+    // p2p: the p update stores its slice into every peer's x buffer and publishes it
+    const int64_t xoff = h->dist ? (int64_t)h->dist->rank * h->maxlen : 0;
+    k_cg_p<<<vg, 256, 0, s>>>(n, rr_new, run->rr_old, h->r, p, h->flags, tol, run->rr_b, it, base, xoff);
     LAUNCHED();
     run->rr_old = rr_new;
   }

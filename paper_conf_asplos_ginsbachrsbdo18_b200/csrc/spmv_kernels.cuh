@@ -26,6 +26,7 @@ struct SpmvArgs {
   double alpha, beta;
   const void* w;          // DOT: w[i] for local row i
   double* part;           // DOT: one partial per CTA
+  P2PHook hk;             // p2p transport: wait for x / push the dot (common.cuh)
 };
 
 // ----------------------------------------------------------------------------
@@ -38,6 +39,7 @@ template <typename T, int G, int U, bool DOT>
 __global__ void __launch_bounds__(256)
 k_spmv_vector(SpmvArgs a) {
   __shared__ double red[8];
+  p2p_prologue_wait(a.hk);
   const T* __restrict__ vals = static_cast<const T*>(a.vals);
   const T* __restrict__ x = static_cast<const T*>(a.x);
   T* __restrict__ y = static_cast<T*>(a.y);
@@ -83,6 +85,7 @@ k_spmv_vector(SpmvArgs a) {
   if (DOT) {
     const double t = block_sum(dacc, red);
     if (threadIdx.x == 0) a.part[blockIdx.x] = t;
+    p2p_push_partials_last(a.hk, a.part, gridDim.x);
   }
 }
 

@@ -67,6 +67,7 @@ struct XplanArgs {
   double alpha, beta;
   const void* w;               // DOT: w[i]
   double* part;                // DOT: one partial per CTA
+  P2PHook hk;                  // p2p transport: wait for x / push the dot
   int dbg;
   int prefetch;                // 1: L2-prefetch the warp's chunk of the next tile
 };
@@ -157,6 +158,7 @@ k_spmv_xplan(XplanArgs a) {
   const bool x_aligned = (reinterpret_cast<uintptr_t>(xg + col0) & 15) == 0;
   const int64_t bulk_elems = x_aligned ? ((ncols * int64_t(sizeof(T))) & ~int64_t(15)) / int64_t(sizeof(T)) : 0;
 
+  p2p_prologue_wait(a.hk);  // x slices of the peers (p2p transport)
   auto recv_bytes = [&](int t) -> uint32_t {
     const int nrows = int(cmin64(R, r1c - (r0c + int64_t(t) * R)));
     const int own = max(0, min((b + 1) * RB, nrows) - b * RB);
@@ -284,6 +286,7 @@ k_spmv_xplan(XplanArgs a) {
   // leave together (peers may still be sending to / reading this CTA)
   cluster_arrive();
   cluster_wait();
+  if (DOT) p2p_push_partials_last(a.hk, a.part, gridDim.x);
 }
 
 // ---------------------------------------------------------------- builders

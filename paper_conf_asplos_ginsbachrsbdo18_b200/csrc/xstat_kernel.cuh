@@ -39,6 +39,7 @@ struct XstatArgs {
   double alpha, beta;
   const void* w;          // DOT
   double* part;           // DOT: one partial per CTA
+  P2PHook hk;
 };
 
 __device__ __forceinline__ uint32_t smem_u32(const void* p) {
@@ -118,6 +119,7 @@ k_spmv_xstat(XstatArgs a) {
   const int b = (int)cluster_rank();
   const int c = (int)cluster_id();
   const int R = a.R;
+  p2p_prologue_wait(a.hk);
 
   T* xs = reinterpret_cast<T*>(smem);
   double* pbuf = reinterpret_cast<double*>(smem + ((size_t(a.W) * sizeof(T) + 15) & ~size_t(15)));
@@ -257,6 +259,7 @@ k_spmv_xstat(XstatArgs a) {
   if (DOT) {
     const double tsum = block_sum(dacc, red);
     if (threadIdx.x == 0) a.part[blockIdx.x] = tsum;
+    p2p_push_partials_last(a.hk, a.part, gridDim.x);
   }
 }
 
