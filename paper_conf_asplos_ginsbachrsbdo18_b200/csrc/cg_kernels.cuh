@@ -13,6 +13,8 @@
 
 namespace spmv {
 
+constexpr int CG_U = 4;  // elements per thread issued together in the vector kernels
+
 struct CgState {
   int* flags;   // [0] breakdown (sticky), [1] converged, [2] iterations done
 };
@@ -50,13 +52,26 @@ k_cg_zr(int64_t n, SumSrc pq, SumSrc rr_old, const double* __restrict__ p,
   }
   const double alpha = rho / d;
   double acc = 0.0;
-  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n;
-       j += int64_t(gridDim.x) * blockDim.x) {
-    const double zj = z[j] + alpha * p[j];
-    const double rj = r[j] - alpha * q[j];
-    z[j] = zj;
-    r[j] = rj;
-    acc += rj * rj;
+  // CG_U consecutive-stride elements per thread with all loads issued first
+  const int64_t stride = int64_t(gridDim.x) * blockDim.x;
+  for (int64_t j0 = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j0 < n; j0 += CG_U * stride) {
+    double pz[CG_U], pp[CG_U], pr[CG_U], pq_[CG_U];
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) { pz[u] = z[j]; pp[u] = p[j]; pr[u] = r[j]; pq_[u] = q[j]; }
+    }
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) {
+        const double zj = pz[u] + alpha * pp[u];
+        const double rj = pr[u] - alpha * pq_[u];
+        z[j] = zj;
+        r[j] = rj;
+        acc += rj * rj;
+      }
+    }
   }
   const double t = block_sum(acc, red);
   if (threadIdx.x == 0) part_rr_new[blockIdx.x] = t;
@@ -74,20 +89,37 @@ k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
   const double rho1 = read_sum(rr_new, &s_new);
   const double rho0 = read_sum(rr_old, &s_old);
   const double beta = rho1 / rho0;
-  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n;
-       j += int64_t(gridDim.x) * blockDim.x) {
-    const double pj = r[j] + beta * p[j];
-    p[j] = pj;
-    if (hk.enabled)  // fused all-gather: the slice goes straight into every peer's xpad
-      for (int q = 0; q < hk.c.P; ++q)
-        if (q != hk.c.me) reinterpret_cast<double*>(hk.c.peer[q])[xoff + j] = pj;
+  const int64_t stride = int64_t(gridDim.x) * blockDim.x;
+  for (int64_t j0 = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j0 < n; j0 += CG_U * stride) {
+    double pr[CG_U], pp[CG_U];
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) { pr[u] = r[j]; pp[u] = p[j]; }
+    }
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) {
+        const double pj = pr[u] + beta * pp[u];
+        p[j] = pj;
+        if (hk.enabled)  // fused all-gather: the slice goes straight into every peer's xpad
+          for (int q = 0; q < hk.c.P; ++q)
+            if (q != hk.c.me) reinterpret_cast<double*>(hk.c.peer[q])[xoff + j] = pj;
+      }
+    }
   }
   if (hk.enabled) {
-    __threadfence_system();
+    // all peer stores of the CTA happen-before thread 0's system-scope fence
+    // (bar.sync + cumulative fence), which precedes the ticket; the last CTA
+    // publishes with release stores
     __syncthreads();
-    if (threadIdx.x == 0 && atomicAdd(hk.c.ticket, 1) == int(gridDim.x) - 1) {
-      *hk.c.ticket = 0;
-      p2p_signal(hk.c, P2P_XSLOT);
+    if (threadIdx.x == 0) {
+      __threadfence_system();
+      if (atomicAdd(hk.c.ticket, 1) == int(gridDim.x) - 1) {
+        *hk.c.ticket = 0;
+        p2p_signal(hk.c, P2P_XSLOT);
+      }
     }
   }
   if (tol > 0.0) {

@@ -156,9 +156,17 @@ __device__ __forceinline__ void p2p_prologue_wait(const P2PHook& h) {
 __device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const double* part, int count) {
   if (!h.enabled || h.push_slot < 0) return;
   __shared__ int s_last;
-  __threadfence();
+  // part[blockIdx.x] was stored by thread 0: one fence by that thread orders
+  // it before the ticket (threadFenceReduction pattern)
   __syncthreads();
-  if (threadIdx.x == 0) s_last = (atomicAdd(h.c.ticket, 1) == int(gridDim.x) - 1);
+  if (threadIdx.x == 0) {
+    __threadfence();
+    const int tk = atomicAdd(h.c.ticket, 1);
+    s_last = (tk == int(gridDim.x) - 1);
+#ifdef SPMV_P2P_TRACE
+    if (blockIdx.x == 0 || s_last) printf("push_last blk %d ticket %d grid %d slot %d\n", blockIdx.x, tk, gridDim.x, h.push_slot);
+#endif
+  }
   __syncthreads();
   if (!s_last) return;
   if (threadIdx.x < 32) {
@@ -166,6 +174,9 @@ __device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const d
     for (int i = threadIdx.x; i < count; i += 32) a += __ldcg(part + i);  // L2: other CTAs' stores
     a = warp_sum(a);
     if (threadIdx.x == 0) {
+#ifdef SPMV_P2P_TRACE
+      printf("push value %g count %d\n", a, count);
+#endif
       *h.c.ticket = 0;
       for (int q = 0; q < h.c.P; ++q) {
         double* ex = reinterpret_cast<double*>(h.c.peer[q] + h.c.off_exch);
@@ -204,6 +215,7 @@ __device__ __forceinline__ double read_sum(SumSrc s, double* slot) {
       if (threadIdx.x == 0)
         for (int i = 0; i < n; ++i) a += s.p[i];  // rank order
     } else {
+#pragma unroll 4
       for (int i = threadIdx.x; i < n; i += 32) a += s.p[i];
       a = warp_sum(a);
     }

@@ -49,9 +49,9 @@ k_p2p_push_x(int64_t n, int64_t maxlen, P2PCtx c) {
       reinterpret_cast<T*>(c.peer[q])[int64_t(c.me) * maxlen + j] = v;
     }
   }
-  __threadfence_system();
   __syncthreads();
   if (threadIdx.x == 0) {
+    __threadfence_system();  // cumulative: orders the whole CTA's peer stores
     const int t = atomicAdd(c.ticket, 1);
     if (t == int(gridDim.x) - 1) {  // last CTA: every slice store is fenced
       *c.ticket = 0;

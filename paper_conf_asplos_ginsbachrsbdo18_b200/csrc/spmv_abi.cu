@@ -373,6 +373,7 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   a.dbg = dbg() ? 1 : 0;
   a.prefetch = 0;
   env_int("SPMV_XPLAN_PF", &a.prefetch);
+  a.hk = hook;
   a.crow = h->xp.crow;
   a.tile0 = h->xp.tile0;
   a.x = x;
