@@ -432,8 +432,8 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   int B = (int)cdiv((int64_t)(ts * h->nx), (int64_t)xbudget);
   B = B <= 1 ? 1 : B <= 2 ? 2 : B <= 4 ? 4 : B <= 8 ? 8 : 16;
   int forced = 0;
-  if (env_int("SPMV_XPLAN_B", &forced) && forced >= B && forced <= 8 && (forced & (forced - 1)) == 0) B = forced;
-  if (B > 8) return SPMV_OK;
+  if (env_int("SPMV_XPLAN_B", &forced) && forced >= B && forced <= 16 && (forced & (forced - 1)) == 0) B = forced;
+  if (B > 16) return SPMV_OK;
   int W = (int)cdiv(h->nx, B);
   W = (W + 7) & ~7;
   if (W > 65534) return SPMV_OK;  // 16-bit column offsets, pad column W
@@ -443,6 +443,10 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   void (*fnd)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, true> : nullptr;
   CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
   if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+  if (B > 8) {  // clusters of 16 need the non-portable size
+    CK(cudaFuncSetAttribute(fn, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
+    if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
+  }
   cudaLaunchConfig_t cfg = {};
   cfg.gridDim = dim3((unsigned)B, 1, 1);
   cfg.blockDim = dim3(XP_THREADS, 1, 1);

@@ -1,5 +1,1 @@
-timeout 900 python -m pytest tests -m gpu -x -q > gpurun_out/pytest_gpu.log 2>&1; echo "pytest exit $?" >> gpurun_out/pytest_gpu.log; tail -2 gpurun_out/pytest_gpu.log; grep -E "^E |Error|timeout" gpurun_out/pytest_gpu.log | head -12
-for tr in p2p nccl; do SPMV_TRANSPORT=$tr SPMV_BENCH_FORCE_DIST=1 timeout 300 python -m torch.distributed.run --nnodes=1 --nproc-per-node 1 --master-addr 127.0.0.1 --master-port $((29500 + RANDOM % 400)) bench.py --gpus 1 --steps 10 --warmup 3 --no-cpu > gpurun_out/bench_$tr.json 2> gpurun_out/bench_$tr.err; echo "$tr rc $?"; python -c "
-import json; d=json.load(open('gpurun_out/bench_$tr.json')); print(d['transport'], d['value'], d['ms_per_step'], d['zeta_last'], d['gpu_launches'])"; done
-timeout 300 python bench.py --steps 10 --warmup 3 --no-cpu > gpurun_out/bench.json 2> gpurun_out/bench.err; python -c "
-import json; d=json.load(open('gpurun_out/bench.json')); print('single', d['value'], d['ms_per_step'], d['zeta_last'], d['gpu_launches'], d['spmv']['us_avg'])"
+for m in C B; do timeout 60 python tools/time_one.py b16 $m xplan SPMV_XPLAN_B=16; timeout 60 python tools/one.py $m xplan SPMV_XPLAN_B=16 2>&1 | grep -o "'grid': [0-9]*"; done
