@@ -1,0 +1,122 @@
+// Microbenchmark: HBM read bandwidth of plain 16-B LDG streaming (no TMA) by
+// access pattern, the question behind the XPLAN chunk layout:
+//   warp  : each warp streams its own contiguous chunk of CH bytes (the plan's
+//           chunk-per-warp layout), U 16-B loads per lane per round trip;
+//   cta   : the warps of a CTA interleave at U*512-B granularity, so a CTA's
+//           request stream is one sequential sweep of its range;
+//   grid  : classic grid-stride, every load instruction of the grid adjacent.
+// grid = CTAs (1 per SM, NW warps each).  Each CTA reads total/grid bytes.
+#include <cstdint>
+#include <cstdio>
+#include <cstdlib>
+
+__device__ __forceinline__ int4 ldg16(const void* p) {
+  int4 r;
+  asm volatile("ld.global.nc.L1::no_allocate.v4.s32 {%0, %1, %2, %3}, [%4];"
+               : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w)
+               : "l"(p));
+  return r;
+}
+
+template <int U>
+__global__ void __launch_bounds__(1024, 1) k_stream(const char* __restrict__ g, size_t per_cta, int mode, size_t ch,
+                                                    unsigned long long* sink) {
+  const int nw = blockDim.x / 32, warp = threadIdx.x / 32, lane = threadIdx.x & 31;
+  const char* base = g + blockIdx.x * per_cta;
+  unsigned acc = 0;
+  constexpr size_t RT = size_t(U) * 512;  // bytes per warp round trip
+  if (mode == 0) {  // warp-private chunks: chunk (t, w) at (t*nw + w)*ch
+    const size_t nch = per_cta / ch;
+    for (size_t c = warp; c < nch; c += nw) {
+      const char* p = base + c * ch;
+      for (size_t o = 0; o < ch; o += RT) {
+        int4 v[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) v[u] = ldg16(p + o + u * 512 + lane * 16);
+#pragma unroll
+        for (int u = 0; u < U; ++u) acc ^= v[u].x ^ v[u].y ^ v[u].z ^ v[u].w;
+      }
+    }
+  } else if (mode == 1) {  // CTA-sequential sweep
+    const size_t nrt = per_cta / RT;
+    for (size_t r = warp; r < nrt; r += nw) {
+      const char* p = base + r * RT;
+      int4 v[U];
+#pragma unroll
+      for (int u = 0; u < U; ++u) v[u] = ldg16(p + u * 512 + lane * 16);
+#pragma unroll
+      for (int u = 0; u < U; ++u) acc ^= v[u].x ^ v[u].y ^ v[u].z ^ v[u].w;
+    }
+  } else {  // grid-stride over the whole buffer
+    const size_t total = per_cta * gridDim.x;
+    const size_t stride = size_t(gridDim.x) * blockDim.x * 16;
+    for (size_t o = (size_t(blockIdx.x) * blockDim.x + threadIdx.x) * 16; o < total; o += stride * U) {
+      int4 v[U];
+#pragma unroll
+      for (int u = 0; u < U; ++u) {
+        const size_t q = o + u * stride;
+        v[u] = q < total ? ldg16(g + q) : int4{0, 0, 0, 0};
+      }
+#pragma unroll
+      for (int u = 0; u < U; ++u) acc ^= v[u].x ^ v[u].y ^ v[u].z ^ v[u].w;
+    }
+  }
+  if (acc == 0x12345678u) sink[0] = acc;
+}
+
+template <int U>
+static float run(const char* g, int grid, int threads, size_t per_cta, int mode, size_t ch, unsigned long long* sink,
+                 char* flush, size_t fbytes) {
+  cudaEvent_t a, b;
+  cudaEventCreate(&a);
+  cudaEventCreate(&b);
+  float best = 1e30f;
+  for (int rep = 0; rep < 6; ++rep) {
+    cudaMemset(flush, rep, fbytes);
+    cudaEventRecord(a);
+    k_stream<U><<<grid, threads>>>(g, per_cta, mode, ch, sink);
+    cudaEventRecord(b);
+    cudaEventSynchronize(b);
+    float ms;
+    cudaEventElapsedTime(&ms, a, b);
+    if (rep > 0 && ms < best) best = ms;
+  }
+  return best;
+}
+
+int main() {
+  const size_t total = size_t(480) << 20;
+  char *g, *flush;
+  unsigned long long* sink;
+  const size_t fbytes = size_t(256) << 20;
+  cudaMalloc(&g, total + (64 << 20));
+  cudaMalloc(&flush, fbytes);
+  cudaMalloc(&sink, 8);
+  cudaMemset(g, 1, total);
+  const char* names[3] = {"warp-chunk", "cta-seq", "grid-stride"};
+  for (int grid : {120, 148}) {
+    for (int threads : {512, 1024}) {
+      for (int mode = 0; mode < 3; ++mode) {
+        for (int U : {4, 8, 16}) {
+          for (size_t ch : {size_t(8192), size_t(16384)}) {
+            if (mode != 0 && ch != 8192) continue;
+            const size_t RT = size_t(U) * 512;
+            size_t per = total / grid;
+            const size_t q = (mode == 0) ? ch : RT;
+            per = per / q * q;
+            float ms = 0;
+            if (U == 4) ms = run<4>(g, grid, threads, per, mode, ch, sink, flush, fbytes);
+            if (U == 8) ms = run<8>(g, grid, threads, per, mode, ch, sink, flush, fbytes);
+            if (U == 16) ms = run<16>(g, grid, threads, per, mode, ch, sink, flush, fbytes);
+            const double bytes = double(per) * grid;
+            printf("grid %3d thr %4d %-11s U=%2d ch=%5zu  %8.1f GB/s  (%.1f us)\n", grid, threads, names[mode], U,
+                   mode == 0 ? ch : 0, bytes / (ms * 1e-3) / 1e9, ms * 1e3);
+          }
+        }
+      }
+    }
+  }
+  cudaError_t e = cudaDeviceSynchronize();
+  if (e != cudaSuccess) printf("error %s\n", cudaGetErrorString(e));
+  return 0;
+}
