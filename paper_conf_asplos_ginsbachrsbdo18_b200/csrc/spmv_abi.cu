@@ -22,6 +22,7 @@
 #include "xstat_kernel.cuh"
 #include "xplan_kernel.cuh"
 #include "merge_kernel.cuh"
+#include "sell_kernel.cuh"
 #include "p2p_kernels.cuh"
 
 using namespace spmv;
@@ -129,6 +130,14 @@ struct spmv_csr_s {
     void (*k)(XplanArgs) = nullptr;
     void (*kdot)(XplanArgs) = nullptr;
   } xp;
+  // SELL (SELL-32 device plan, x gathered from global memory)
+  struct Sell {
+    bool built = false;
+    int64_t nchunks = 0, pairs = 0, grid = 0;
+    long long* pair_off = nullptr;
+    unsigned char* vals = nullptr;
+    int* cols = nullptr;
+  } sl;
   // MERGE (merge-path tiles)
   struct {
     int ntiles = 0;
@@ -429,8 +438,9 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   const size_t recv = (size_t)XP_K * XP_R * 8;
   if (smem_cap <= recv + 1024) return SPMV_OK;
   const size_t xbudget = smem_cap - recv - 64;
-  int B = (int)cdiv((int64_t)(ts * h->nx), (int64_t)xbudget);
-  B = B <= 1 ? 1 : B <= 2 ? 2 : B <= 4 ? 4 : B <= 8 ? 8 : 16;
+  const int64_t Bneed = cdiv((int64_t)(ts * h->nx), (int64_t)xbudget);
+  if (Bneed > 16) return SPMV_OK;  // x does not fit the shared memory of a 16-CTA cluster
+  int B = Bneed <= 1 ? 1 : Bneed <= 2 ? 2 : Bneed <= 4 ? 4 : Bneed <= 8 ? 8 : 16;
   int forced = 0;
   if (env_int("SPMV_XPLAN_B", &forced) && forced >= B && forced <= 16 && (forced & (forced - 1)) == 0) B = forced;
   if (B > 16) return SPMV_OK;
@@ -439,6 +449,7 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   if (W > 65534) return SPMV_OK;  // 16-bit column offsets, pad column W
   const size_t xbytes = ((size_t)(W + 1) * ts + 15) & ~size_t(15);
   const size_t smem = xbytes + recv;
+  if (smem > smem_cap) return SPMV_OK;
   void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, false> : k_spmv_xplan<float, false>;
   void (*fnd)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, true> : nullptr;
   CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
@@ -547,6 +558,93 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   return SPMV_OK;
 }
 
+// ------------------------------------------------------------------ SELL
+static spmv_status sell_pack(spmv_csr_s* h, const void* vals, int values_only) {
+  cudaStream_t s = h->stream;
+  const int64_t g = std::min<int64_t>(cdiv(h->m_loc, 256), 16LL * num_sms(h->device));
+  if (h->dt == SPMV_F64)
+    k_sell_pack<double><<<g, 256, 0, s>>>(h->m_loc, h->rp_loc, h->ci_loc, (const double*)vals, h->sl.pair_off,
+                                          (double*)h->sl.vals, h->sl.cols, values_only);
+  else
+    k_sell_pack<float><<<g, 256, 0, s>>>(h->m_loc, h->rp_loc, h->ci_loc, (const float*)vals, h->sl.pair_off,
+                                         (float*)h->sl.vals, h->sl.cols, values_only);
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+// Build the SELL-32 plan (create).  Not eligible (*ok = false) when the
+// padding exceeds max_pad x nnz (skewed rows: merge path / vector instead).
+static spmv_status sell_build(spmv_csr_s* h, double max_pad, bool* ok) {
+  *ok = false;
+  const int64_t m = h->m_loc, nnz = h->k1 - h->k0;
+  if (m == 0 || nnz == 0) return SPMV_OK;
+  cudaStream_t s = h->stream;
+  auto& S = h->sl;
+  const int64_t nch = cdiv(m, 32);
+  CK(cudaMalloc(&S.pair_off, sizeof(long long) * (nch + 1)));
+  k_sell_pairs<<<(unsigned)std::min<int64_t>(cdiv(nch, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
+      m, h->rp_loc, nch, S.pair_off);
+  LAUNCHED();
+  std::vector<long long> off(nch + 1);
+  CK(cudaMemcpyAsync(off.data(), S.pair_off, sizeof(long long) * nch, cudaMemcpyDeviceToHost, s));
+  CK(cudaStreamSynchronize(s));
+  long long pos = 0;
+  for (int64_t c = 0; c < nch; ++c) {
+    const long long np = off[c];
+    off[c] = pos;
+    pos += np;
+  }
+  off[nch] = pos;
+  if ((double)pos * 64.0 > max_pad * (double)nnz + 64.0) {
+    cudaFree(S.pair_off);
+    S = spmv_csr_s::Sell();
+    return SPMV_OK;
+  }
+  S.nchunks = nch;
+  S.pairs = pos;
+  const size_t slots = (size_t)std::max<long long>(pos, 1) * 64;  // 32 lanes x 2 steps
+  CK(cudaMemcpyAsync(S.pair_off, off.data(), sizeof(long long) * (nch + 1), cudaMemcpyHostToDevice, s));
+  CK(cudaMalloc(&S.vals, slots * h->ts));
+  CK(cudaMalloc(&S.cols, slots * sizeof(int)));
+  CK(cudaMemsetAsync(S.vals, 0, slots * h->ts, s));
+  CK(cudaMemsetAsync(S.cols, 0xff, slots * sizeof(int), s));  // -1: padding
+  ST(sell_pack(h, h->vals, 0));
+  CK(cudaStreamSynchronize(s));
+  // grid: 8 CTAs of SELL_NT per SM, never more warps than chunks
+  S.grid = std::max<int64_t>(1, std::min<int64_t>(cdiv(nch, SELL_NT / 32), 8LL * num_sms(h->device)));
+  S.built = true;
+  *ok = true;
+  return SPMV_OK;
+}
+
+static spmv_status launch_sell(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha, double beta,
+                               const double* w, double* part, const P2PHook& hook) {
+  SellArgs a;
+  a.m = h->m_loc;
+  a.nchunks = h->sl.nchunks;
+  a.vals = h->sl.vals;
+  a.cols = reinterpret_cast<const int2*>(h->sl.cols);
+  a.pair_off = h->sl.pair_off;
+  a.x = x;
+  a.y = y;
+  a.alpha = alpha;
+  a.beta = beta;
+  a.w = w;
+  a.part = part;
+  a.hk = hook;
+  const unsigned g = (unsigned)h->sl.grid;
+  if (h->dt == SPMV_F64) {
+    if (part) k_spmv_sell<double, true><<<g, SELL_NT, 0, s>>>(a);
+    else k_spmv_sell<double, false><<<g, SELL_NT, 0, s>>>(a);
+  } else {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+    k_spmv_sell<float, false><<<g, SELL_NT, 0, s>>>(a);
+  }
+  LAUNCHED();
+  return SPMV_OK;
+}
+
 static spmv_status merge_setup(spmv_csr_s* h) {
   const int64_t items = h->m_loc + (h->k1 - h->k0);
   const int64_t C = std::max<int64_t>(1, cdiv(items, MG_D));
@@ -617,7 +715,9 @@ static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, con
     return SPMV_OK;
   }
   if (h->kernel == SPMV_KERNEL_XPLAN && vals == h->vals) return launch_xplan(h, s, x, y, alpha, beta, w, part, hook);
-  const int64_t vgrid_spmv = h->kernel == SPMV_KERNEL_XPLAN ? h->grid_vec : h->grid;
+  if (h->kernel == SPMV_KERNEL_SELL && vals == h->vals) return launch_sell(h, s, x, y, alpha, beta, w, part, hook);
+  const int64_t vgrid_spmv =
+      (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_SELL) ? h->grid_vec : h->grid;
   if (h->kernel == SPMV_KERNEL_XSTAT) return launch_xstat(h, s, vals, x, y, alpha, beta, w, part, hook);
   if (h->kernel == SPMV_KERNEL_MERGE) {
     P2PHook wait_only = hook;
@@ -869,7 +969,20 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
       }
     }
   }
-  if (h->kernel != SPMV_KERNEL_XPLAN && rk != SPMV_KERNEL_VECTOR && rk != SPMV_KERNEL_SCALAR && rk != SPMV_KERNEL_XSTAT &&
+  if (h->kernel != SPMV_KERNEL_XPLAN && (rk == SPMV_KERNEL_SELL || (rk == SPMV_KERNEL_AUTO && plan))) {
+    // auto + plan, x too large for the clusters (or short rows): the SELL-32
+    // plan with global x gathers when the rows are regular enough that the
+    // 32-row chunks pad little (the 27-point stencil); forced: any padding
+    bool ok = false;
+    spmv_status st = sell_build(h, rk == SPMV_KERNEL_SELL ? 1e30 : 1.2, &ok);
+    if (st != SPMV_OK) return fail(st);
+    if (ok) {
+      h->kernel = SPMV_KERNEL_SELL;
+      h->grid = h->sl.grid;
+    }
+  }
+  if (h->kernel != SPMV_KERNEL_XPLAN && h->kernel != SPMV_KERNEL_SELL && rk != SPMV_KERNEL_VECTOR &&
+      rk != SPMV_KERNEL_SCALAR && rk != SPMV_KERNEL_XSTAT &&
       h->m_loc > 0 &&
       (rk == SPMV_KERNEL_MERGE || (double)h->row_max > 32.0 * std::max(h->row_mean, 1.0))) {
     // skewed rows (a long row would pin one warp of the vector kernel): merge path
@@ -878,7 +991,7 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
     h->kernel = SPMV_KERNEL_MERGE;
     h->grid = h->vgrid;  // dot partials come from k_dot_partials
   }
-  if (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_MERGE) {
+  if (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_MERGE || h->kernel == SPMV_KERNEL_SELL) {
   } else if (rk == SPMV_KERNEL_XSTAT) {
     bool ok = false;
     spmv_status st = xstat_setup(h, &ok);
@@ -909,7 +1022,7 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
     if (h->xpad == h->fabric) h->xpad = nullptr;
   }
   void* bufs[] = {h->p2p_local, h->peer_table, h->mg.split_row, h->mg.split_nz, h->mg.head, h->mg.carry, h->mg.head_flag, h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
-                  h->xp.chunk_row, h->xp.plan,
+                  h->xp.chunk_row, h->xp.plan, h->sl.pair_off, h->sl.vals, h->sl.cols,
                   h->seg, h->crow, h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
                   h->stage_x, h->stage_z};
@@ -1298,6 +1411,7 @@ extern "C" spmv_status spmv_csr_update_values(spmv_csr_t h, const void* vals) {
   ST(need_device(vals, h->device, "vals must be a device pointer", h->nnz == 0));
   h->vals = vals;
   if (h->xp.built) ST(xplan_pack(h, vals, 1));
+  if (h->sl.built) ST(sell_pack(h, vals, 1));
   h->g_npb.reset();
   return SPMV_OK;
 }
@@ -1414,7 +1528,9 @@ extern "C" spmv_status spmv_csr_info(spmv_csr_t h, spmv_info_t* info) {
   info->sorted_cols = h->sorted;
   info->grid = h->grid;
   info->cluster = h->kernel == SPMV_KERNEL_XPLAN ? h->xp.B : h->kernel == SPMV_KERNEL_XSTAT ? h->xB : 0;
-  info->plan_bytes = h->xp.built ? (int64_t)h->xp.bytes : 0;
+  info->plan_bytes = h->xp.built ? (int64_t)h->xp.bytes
+                   : h->sl.built  ? (int64_t)h->sl.pairs * 64 * (int64_t)(h->ts + 4)
+                                  : 0;
   return SPMV_OK;
 }
 

@@ -217,11 +217,20 @@ k_spmv_xplan(XplanArgs a) {
       }
 #pragma unroll
       for (int u = 0; u < XP_U; ++u) {
+#ifdef XP_DBG_NOX  // timing experiment: no x gathers (wrong results)
+        acc += double(v[u].a) * double(cc[u] & 0xffffu) + double(v[u].b);
+#else
         acc += double(v[u].a) * double(xs[cc[u] & 0xffffu]);
         acc += double(v[u].b) * double(xs[cc[u] >> 16]);
+#endif
       }
     }
+#ifdef XP_DBG_NOSYNC  // timing experiment: no partial exchange / tile barriers (wrong results)
+    if (acc == 1.2345) static_cast<T*>(a.y)[0] = T(acc);
+    if (false) {
+#else
     if (row != 0xffff) {
+#endif
       const int q = row / RB, jl = row - q * RB;
       const uint32_t laddr = smem_u32(recv + (t % XP_K) * R + b * RB + jl);
       st_async_f64(mapa_u32(laddr, q), acc, mapa_u32(smem_u32(&tbar[t % XP_K]), q));
@@ -267,7 +276,12 @@ k_spmv_xplan(XplanArgs a) {
   // Buffer reuse: partials of tile t+K (K = 3) are sent only after the sender
   // passed wait(t+1), i.e. after every CTA arrived(t+1), which each does after
   // finalize(t) (reads of recv[t%K] + re-arm of tbar[t%K]).
+#ifdef XP_DBG_NOSYNC
+  for (int t = 0; t < ntiles; ++t) process(t);
+  if (false) {
+#else
   if (ntiles > 0) {
+#endif
     process(0);
     cluster_arrive_relaxed();
     for (int t = 1; t < ntiles; ++t) {

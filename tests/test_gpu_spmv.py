@@ -240,6 +240,56 @@ def test_parboil_full_size_fp32(sp, torch_dev):
         assert abs(float(s) - y_ref[i]) <= 1e-5 * bound[i]
 
 
+def _sample_rows(A, rows):
+    """Sub-CSR of the given rows (same columns) for per-row oracle checks."""
+    lens = (A.rowptr[rows + 1] - A.rowptr[rows]).astype(np.int64)
+    rp = np.concatenate([[0], np.cumsum(lens)]).astype(np.int32)
+    idx = np.concatenate([np.arange(A.rowptr[i], A.rowptr[i + 1]) for i in rows])
+    return gen.CSR(len(rows), A.n, rp, A.colidx[idx], A.vals[idx])
+
+
+@pytest.fixture(scope="module")
+def stencil256():
+    return gen.stencil27(256)
+
+
+@pytest.mark.parametrize("kernel", ["auto", "vector"])
+def test_stencil256_full_size(sp, torch_dev, stencil256, kernel):  # auto = the SELL plan
+    """BJ.cfg[4] at full size (16.8M rows, 449,455,096 nnz, fp64), in the launch
+    configuration bench/sweep time: (1) A*1 = 27 - cnt_i on EVERY row, exact
+    (R19: centre 26, neighbours -1; all partial sums are small integers);
+    (2) a random x on 4096 sampled rows (every boundary class included) vs the
+    oracle, per-row tolerance."""
+    torch, dev = torch_dev
+    A = stencil256
+    N = 256
+    assert A.nnz == (3 * N - 2) ** 3
+    rp, ci, va = to_dev(A, dev)
+    y = torch.empty(A.m, dtype=torch.float64, device=dev)
+    ones = torch.ones(A.n, dtype=torch.float64, device=dev)
+    with sp.CSRMatrix(rp, ci, va, A.n, kernel=kernel) as M:
+        if kernel == "auto":
+            assert M.info()["kernel_name"] == "sell"
+        M.spmv(ones, y)
+        torch.cuda.synchronize()
+        yo = y.cpu().numpy()
+        i = np.arange(A.m)
+        xx, yy, zz = i % N, (i // N) % N, i // (N * N)
+        cnt = 1
+        for c in (xx, yy, zz):
+            cnt = cnt * (3 - (c == 0) - (c == N - 1))
+        assert np.array_equal(yo, (27 - cnt).astype(np.float64)), "A*1 closed form"
+        x_h = gen.uniform(A.n, seed=77)
+        M.spmv(torch.from_numpy(x_h).to(dev), y)
+        torch.cuda.synchronize()
+        rng = np.random.default_rng(5)
+        rows = np.unique(np.concatenate([rng.integers(0, A.m, 4000), [0, N - 1, N * N - 1, A.m - 1,
+                                                                       N * N * (N // 2) + N * (N // 2) + N // 2]]))
+        S = _sample_rows(A, rows)
+        y_ref, bound = oracle.spmv(S.rowptr, S.colidx, S.vals, x_h)
+        check_rows(y[torch.from_numpy(rows).to(dev)].cpu().numpy(), y_ref, bound, np.float64, f"stencil256 {kernel}")
+
+
 @pytest.mark.parametrize("cfg", [{}, {"SPMV_XSTAT_B": "2"}, {"SPMV_XSTAT_B": "8"},
                                  {"SPMV_XSTAT_G": "4"}, {"SPMV_XSTAT_G": "32", "SPMV_XSTAT_B": "3"},
                                  {"SPMV_XSTAT_CLUSTERS": "1"}])
@@ -348,6 +398,50 @@ def test_zoo_merge(sp, torch_dev, name, A):
     run_case(sp, torch, dev, A32, gen.uniform(A.n, seed=20, f32=True), kernel="merge", what=f"{name} merge fp32")
     y0 = gen.uniform(A.m, seed=21)
     run_case(sp, torch, dev, A, x, alpha=-2.0, beta=0.5, y0=y0, kernel="merge", what=f"{name} merge a/b")
+
+
+@pytest.mark.parametrize("name,A", ZOO, ids=[c[0] for c in ZOO])
+def test_zoo_sell(sp, torch_dev, name, A):
+    """SELL-32 plan with global x gathers (forced: any padding), fp64 and fp32,
+    alpha/beta with NaN in y_old, and the zero-copy fallback for a per-call
+    vals pointer."""
+    torch, dev = torch_dev
+    x = gen.uniform(A.n, seed=25)
+    info = run_case(sp, torch, dev, A, x, kernel="sell", what=f"{name} sell")
+    if A.m > 0 and A.nnz > 0:
+        assert info["kernel_name"] == "sell" and info["plan_bytes"] >= A.nnz * 12
+    A32 = A.astype(np.float32)
+    run_case(sp, torch, dev, A32, gen.uniform(A.n, seed=26, f32=True), kernel="sell", what=f"{name} sell fp32")
+    y0 = gen.uniform(A.m, seed=27)
+    run_case(sp, torch, dev, A, x, alpha=-2.0, beta=0.5, y0=y0, kernel="sell", what=f"{name} sell a/b")
+    run_case(sp, torch, dev, A, x, alpha=0.0, beta=2.0, y0=y0, kernel="sell", what=f"{name} sell a=0")
+
+
+def test_sell_auto_update_values_and_vals_override(sp, torch_dev):
+    """auto + plan picks SELL for the 27-point stencil at N=96 (x = 7 MB,
+    beyond the shared memory of a 16-CTA cluster); then in-place values +
+    update_values, and a different vals pointer (zero-copy path)."""
+    torch, dev = torch_dev
+    A = gen.stencil27(96)
+    x_h = gen.uniform(A.n, seed=28)
+    info = run_case(sp, torch, dev, A, x_h, what="stencil64 auto")
+    assert info["kernel_name"] == "sell", info
+    rp, ci, va = to_dev(A, dev)
+    x = torch.from_numpy(x_h).to(dev)
+    y = torch.empty(A.m, dtype=torch.float64, device=dev)
+    v2_h = gen.uniform(A.nnz, seed=29)
+    with sp.CSRMatrix(rp, ci, va, A.n) as M:
+        va.copy_(torch.from_numpy(v2_h))
+        M.update_values(va)
+        M.spmv(x, y)
+        torch.cuda.synchronize()
+        y_ref, bound = oracle.spmv(A.rowptr, A.colidx, v2_h, x_h)
+        check_rows(y.cpu().numpy(), y_ref, bound, np.float64, "sell update_values")
+        v3 = torch.from_numpy(gen.uniform(A.nnz, seed=30)).to(dev)
+        M.spmv(x, y, vals=v3)
+        torch.cuda.synchronize()
+        y_ref, bound = oracle.spmv(A.rowptr, A.colidx, v3.cpu().numpy(), x_h)
+        check_rows(y.cpu().numpy(), y_ref, bound, np.float64, "sell vals override")
 
 
 def test_parboil_auto_is_merge(sp, torch_dev):

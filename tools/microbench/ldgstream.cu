@@ -18,6 +18,12 @@ __device__ __forceinline__ int4 ldg16(const void* p) {
   return r;
 }
 
+__device__ __forceinline__ unsigned ldg4(const void* p) {
+  unsigned r;
+  asm volatile("ld.global.nc.L1::no_allocate.u32 %0, [%1];" : "=r"(r) : "l"(p));
+  return r;
+}
+
 template <int U>
 __global__ void __launch_bounds__(1024, 1) k_stream(const char* __restrict__ g, size_t per_cta, int mode, size_t ch,
                                                     unsigned long long* sink) {
@@ -46,6 +52,34 @@ __global__ void __launch_bounds__(1024, 1) k_stream(const char* __restrict__ g, 
       for (int u = 0; u < U; ++u) v[u] = ldg16(p + u * 512 + lane * 16);
 #pragma unroll
       for (int u = 0; u < U; ++u) acc ^= v[u].x ^ v[u].y ^ v[u].z ^ v[u].w;
+    }
+  } else if (mode == 3 || mode == 4) {
+    // XPLAN-like chunks of CH bytes: 4/5 values (16-B loads), 1/5 columns
+    // (4-B loads), one pair = 512 B of values + 128 B of columns per warp.
+    // mode 3: two regions per chunk (values then columns: two streams per warp)
+    // mode 4: interleaved groups [U x 512 B values][U x 128 B columns]
+    const size_t nch = per_cta / ch;
+    const size_t npairs = ch / 640;
+    for (size_t c = warp; c < nch; c += nw) {
+      const char* p = base + c * ch;
+      for (size_t q = 0; q < npairs; q += U) {
+        int4 v[U];
+        unsigned w[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) {
+          const size_t pr = q + u;
+          if (mode == 3) {
+            v[u] = ldg16(p + pr * 512 + lane * 16);
+            w[u] = ldg4(p + npairs * 512 + pr * 128 + lane * 4);
+          } else {
+            const size_t g = pr / U, r = pr % U;
+            v[u] = ldg16(p + g * U * 640 + r * 512 + lane * 16);
+            w[u] = ldg4(p + g * U * 640 + U * 512 + r * 128 + lane * 4);
+          }
+        }
+#pragma unroll
+        for (int u = 0; u < U; ++u) acc ^= v[u].x ^ v[u].y ^ v[u].z ^ v[u].w ^ w[u];
+      }
     }
   } else {  // grid-stride over the whole buffer
     const size_t total = per_cta * gridDim.x;
@@ -93,16 +127,18 @@ int main() {
   cudaMalloc(&flush, fbytes);
   cudaMalloc(&sink, 8);
   cudaMemset(g, 1, total);
-  const char* names[3] = {"warp-chunk", "cta-seq", "grid-stride"};
-  for (int grid : {120, 148}) {
-    for (int threads : {512, 1024}) {
-      for (int mode = 0; mode < 3; ++mode) {
-        for (int U : {4, 8, 16}) {
-          for (size_t ch : {size_t(8192), size_t(16384)}) {
-            if (mode != 0 && ch != 8192) continue;
+  const char* names[5] = {"warp-chunk", "cta-seq", "grid-stride", "xplan-2str", "xplan-intl"};
+  for (int grid : {120}) {
+    for (int threads : {1024}) {
+      for (int mode = 0; mode < 5; ++mode) {
+        for (int U : {4, 8}) {
+          for (size_t ch : {size_t(8192), size_t(10240), size_t(20480)}) {
+            if (mode == 0 && ch == 10240) continue;
+            if ((mode == 1 || mode == 2) && ch != 8192) continue;
+            if (mode >= 3 && ch == 8192) continue;
             const size_t RT = size_t(U) * 512;
             size_t per = total / grid;
-            const size_t q = (mode == 0) ? ch : RT;
+            const size_t q = (mode == 0 || mode >= 3) ? ch : RT;
             per = per / q * q;
             float ms = 0;
             if (U == 4) ms = run<4>(g, grid, threads, per, mode, ch, sink, flush, fbytes);
@@ -110,7 +146,7 @@ int main() {
             if (U == 16) ms = run<16>(g, grid, threads, per, mode, ch, sink, flush, fbytes);
             const double bytes = double(per) * grid;
             printf("grid %3d thr %4d %-11s U=%2d ch=%5zu  %8.1f GB/s  (%.1f us)\n", grid, threads, names[mode], U,
-                   mode == 0 ? ch : 0, bytes / (ms * 1e-3) / 1e9, ms * 1e3);
+                   (mode == 0 || mode >= 3) ? ch : 0, bytes / (ms * 1e-3) / 1e9, ms * 1e3);
           }
         }
       }

@@ -15,7 +15,7 @@ import gen
 import paper_conf_asplos_ginsbachrsbdo18_b200 as sp
 
 w, kern = sys.argv[1], sys.argv[2]
-C = gen.powerlaw() if w == "parboil" else gen.makea(w)
+C = gen.powerlaw() if w == "parboil" else gen.stencil27(int(w[7:])) if w.startswith("stencil") else gen.makea(w)
 dev = torch.device("cuda:0")
 rp, ci, va = (torch.from_numpy(a).to(dev) for a in (C.rowptr, C.colidx, C.vals))
 x = torch.from_numpy(gen.uniform(C.n, seed=1, f32=C.vals.dtype == np.float32)).to(dev)
