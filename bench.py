@@ -12,14 +12,15 @@ tail (a4), row-sharded over N GPUs with the NCCL exchange (a5); the handle is
 created once (a1, device-resident A, the paper's lazy copying P:1175-1184).
 
 value  = CG iterations per second of the whole job (25 per step; the residual
-         SpMV is timed but not counted, reading R23), device-timed with CUDA
-         events per step, L2 flushed between steps, max over ranks.
+         SpMV is timed but not counted, reading R23): K steps back to back
+         between two CUDA events on the launching stream (A is larger than
+         L2, so no flush is needed between steps), max over ranks.
 e2e    = the same metric through the public API with HOST buffers: x copied in
          from pinned memory and x, z, {zeta, rnorm} copied back every step.
 roofline = the SpMV kernel (the dominant kernel, ~97% of the step's bytes),
-         timed alone with CUDA events on the launching stream (L2 flushed
-         before each launch): algorithmic bytes / duration vs the measured
-         HBM copy bandwidth of MEASURED_PEAKS.json.
+         timed alone with CUDA events on the launching stream (an L2 flush
+         queued ahead of the start event): algorithmic bytes / duration vs
+         the measured HBM copy bandwidth of MEASURED_PEAKS.json.
 cpu_baseline = the CPU oracle (oracle/, plain C, 1 thread) on a bounded sample.
 `--impl reference` times the oracle itself as the reference arm.
 """
@@ -81,7 +82,8 @@ def workload_config(A, n_gpus):
                     f"1 step = 1 NPB outer iteration (25 CG its + residual SpMV)",
         "n": int(A.n), "nnz": int(A.nnz), "cgitmax": 25,
         "bytes_per_spmv": int(A.bytes_per_spmv()),
-        "l2": "flushed between timed steps (256 MiB write); A = 436 MB > 126 MB L2",
+        "l2": "inputs larger than L2: A = 436 MB as CSR (382 MB as the plan) > 126 MB L2; the K steps run back "
+              "to back (no flush); the roofline leg flushes L2 (256 MiB write) before each SpMV",
         "parallelism": f"row-shard x{n_gpus} (nnz-balanced); x all-gather + dot all-reduces over peer memory "
                        f"(p2p kernels) or NCCL",
     }
@@ -218,20 +220,20 @@ def run_ours(args):
         M.npb_outer(x, z, 25, shift, out2)
     barrier()
     x.fill_(1.0)
-    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
+    # A (436 MB as CSR, 382 MB as the plan) is larger than the 126 MB L2, so
+    # the K steps run back to back in one event-bracketed region (no flush:
+    # the timing rules' "inputs larger than L2" option)
+    ev0, ev1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     launches0 = sp.launch_count()
-    zetas = []
+    barrier()
+    ev0.record(stream)
     for k in range(args.steps):
-        flush.zero_()  # L2 flush, outside the timed events
-        barrier()
-        ev[k][0].record(stream)
         M.npb_outer(x, z, 25, shift, out2)
-        ev[k][1].record(stream)
+    ev1.record(stream)
     barrier()
     launches = sp.launch_count() - launches0
     M.cg_status()
-    step_ms = [a.elapsed_time(b) for a, b in ev]
-    t_ms = max_over_ranks(sum(step_ms))
+    t_ms = max_over_ranks(ev0.elapsed_time(ev1))
     zeta_last = float(out2[0].item())
     value = 25.0 * args.steps / (t_ms / 1e3)
 
@@ -263,8 +265,10 @@ def run_ours(args):
         M.spmv(p, q)
     sp_ms = []
     for _ in range(reps):
-        flush.zero_()
         barrier()
+        # L2 flush queued ahead of the start event on the same stream: the
+        # kernel starts cold, and the timed region holds no host launch gap
+        flush.zero_()
         a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         a.record(stream)
         M.spmv(p, q)

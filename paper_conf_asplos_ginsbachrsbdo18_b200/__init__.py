@@ -79,6 +79,8 @@ spmv_csr_p2p_handle_c = _decl("spmv_csr_p2p_handle", [_P, _P])
 spmv_csr_p2p_connect_c = _decl("spmv_csr_p2p_connect", [_P, _P])
 spmv_dist_plan_host_c = _decl("spmv_dist_plan_host", [_P, _P, _I64, _I32, _I32, _P, _P, _P])
 spmv_dist_colidx_c = _decl("spmv_dist_colidx", [_P, _P])
+spmv_dist_halo_host_c = _decl("spmv_dist_halo_host", [_P, _P, _I64, _I32, _P])
+spmv_dist_halo_c = _decl("spmv_dist_halo", [_P, _P, _P])
 
 # every symbol include/spmv.h declares (checked by tests/test_abi.py)
 EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_status",
@@ -86,7 +88,8 @@ EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_s
            "spmv_csr_destroy", "spmv_csr_partition", "spmv_csr_merge_splits", "spmv_csr_info",
            "spmv_launch_count", "spmv_status_string", "spmv_last_error_string",
            "spmv_dist_get_unique_id", "spmv_dist_init", "spmv_dist_destroy", "spmv_dist_plan_host",
-           "spmv_dist_colidx", "spmv_dist_init_p2p", "spmv_csr_p2p_handle", "spmv_csr_p2p_connect"]
+           "spmv_dist_colidx", "spmv_dist_init_p2p", "spmv_csr_p2p_handle", "spmv_csr_p2p_connect",
+           "spmv_dist_halo_host", "spmv_dist_halo"]
 
 
 class SpmvError(RuntimeError):
@@ -149,6 +152,18 @@ def spmv_dist_plan_host(rowptr_host, colidx_host, nranks: int, rank: int):
     _check(spmv_dist_plan_host_c(rp.ctypes.data, ci.ctypes.data, m, nranks, rank, b.ctypes.data,
                                  ctypes.byref(ml), loc.ctypes.data), "spmv_dist_plan_host")
     return b, ml.value, loc
+
+
+def spmv_dist_halo_host(rowptr_host, colidx_host, nranks: int):
+    """Halo intervals int64[nranks, nranks, 2]: [r, s] = [lo, hi) of rank s's
+    slice that rank r reads (reading R27)."""
+    import numpy as np
+    rp = np.ascontiguousarray(rowptr_host, dtype=np.int32)
+    ci = np.ascontiguousarray(colidx_host, dtype=np.int32)
+    out = np.zeros((nranks, nranks, 2), dtype=np.int64)
+    _check(spmv_dist_halo_host_c(rp.ctypes.data, ci.ctypes.data, rp.shape[0] - 1, nranks, out.ctypes.data),
+           "spmv_dist_halo_host")
+    return out
 
 
 # ------------------------------------------------------------- distributed
@@ -277,6 +292,15 @@ class CSRMatrix:
         out = np.zeros(self._info["nnz_local"], dtype=np.int32)
         _check(spmv_dist_colidx_c(self.handle, out.ctypes.data), "spmv_dist_colidx")
         return out
+
+    def dist_halo(self):
+        """(device-computed halo table int64[P, P, 2], used-by-the-exchange flag)."""
+        import numpy as np
+        P = self._info["nranks"]
+        out = np.zeros((P, P, 2), dtype=np.int64)
+        used = _I32(0)
+        _check(spmv_dist_halo_c(self.handle, out.ctypes.data, ctypes.byref(used)), "spmv_dist_halo")
+        return out, bool(used.value)
 
     def merge_splits_device(self):
         """(split_row, split_nz) the MERGE kernel uses, or None."""

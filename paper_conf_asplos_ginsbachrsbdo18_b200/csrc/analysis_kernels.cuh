@@ -108,4 +108,53 @@ k_renumber(int64_t k0, int64_t k1, const int* __restrict__ colidx, const long lo
   }
 }
 
+// Halo intervals (NEXT-2, reading R27): for destination rank r and source rank
+// s != r, tab[(r*P+s)*2 .. +1] = min / max local index (c - bounds[s]) over the
+// columns c of rank r's rows owned by s (INT_MAX / -1 when there are none).
+// Warp per row over the GLOBAL matrix (every rank computes the whole table,
+// identically: min/max do not depend on the order).  Smem table per CTA,
+// updates only when they change it, then global atomics.
+__global__ void __launch_bounds__(256)
+k_halo_bounds(int64_t m, const int* __restrict__ rowptr, const int* __restrict__ colidx,
+              const long long* __restrict__ bounds, int P, int* __restrict__ tab) {
+  extern __shared__ long long sb[];  // [P+1] bounds, then int [P*P*2]
+  int* st = reinterpret_cast<int*>(sb + P + 1);
+  for (int i = threadIdx.x; i <= P; i += blockDim.x) sb[i] = bounds[i];
+  for (int i = threadIdx.x; i < P * P; i += blockDim.x) {
+    st[2 * i] = 0x7fffffff;
+    st[2 * i + 1] = -1;
+  }
+  __syncthreads();
+  auto owner = [&](long long c) {
+    int lo = 0, hi = P - 1;  // largest s with sb[s] <= c
+    while (lo < hi) {
+      const int mid = (lo + hi + 1) >> 1;
+      if (sb[mid] <= c) lo = mid; else hi = mid - 1;
+    }
+    return lo;
+  };
+  const int lane = threadIdx.x & 31;
+  const int64_t w0 = (int64_t(blockIdx.x) * blockDim.x + threadIdx.x) >> 5;
+  const int64_t nw = (int64_t(gridDim.x) * blockDim.x) >> 5;
+  for (int64_t i = w0; i < m; i += nw) {
+    const int r = owner(i);
+    const int k0 = rowptr[i], k1 = rowptr[i + 1];
+    for (int k = k0 + lane; k < k1; k += 32) {
+      const long long c = colidx[k];
+      const int sidx = owner(c);
+      if (sidx == r) continue;
+      const int li = int(c - sb[sidx]);
+      int* e = st + 2 * (r * P + sidx);
+      if (li < e[0]) atomicMin(e, li);
+      if (li > e[1]) atomicMax(e + 1, li);
+    }
+  }
+  __syncthreads();
+  for (int i = threadIdx.x; i < P * P; i += blockDim.x)
+    if (st[2 * i + 1] >= 0) {
+      atomicMin(tab + 2 * i, st[2 * i]);
+      atomicMax(tab + 2 * i + 1, st[2 * i + 1]);
+    }
+}
+
 }  // namespace spmv

@@ -105,7 +105,7 @@ k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
         p[j] = pj;
         if (hk.enabled)  // fused all-gather: the slice goes straight into every peer's xpad
           for (int q = 0; q < hk.c.P; ++q)
-            if (q != hk.c.me) reinterpret_cast<double*>(hk.c.peer[q])[xoff + j] = pj;
+            if (q != hk.c.me && p2p_sends(hk.c, q, j)) reinterpret_cast<double*>(hk.c.peer[q])[xoff + j] = pj;
       }
     }
   }

@@ -111,8 +111,16 @@ struct P2PCtx {
   unsigned long long* epoch;       // local exchange counter
   unsigned long long* slot_epoch;  // local [P2P_NSLOT + 1]
   int* ticket;                     // local last-CTA ticket
+  const int2* send_iv;             // [P] halo: elements [x, y) of this rank's slice go to rank q (NULL = all)
   int me, P;
 };
+
+// Does element j of this rank's x slice go to rank q (halo interval, NEXT-2)?
+__device__ __forceinline__ bool p2p_sends(const P2PCtx& c, int q, int64_t j) {
+  if (!c.send_iv) return true;
+  const int2 iv = c.send_iv[q];
+  return j >= iv.x && j < iv.y;
+}
 
 // Publish: bump the local epoch, record it for `slot`, flag every peer.
 __device__ __forceinline__ void p2p_signal(const P2PCtx& c, int slot) {

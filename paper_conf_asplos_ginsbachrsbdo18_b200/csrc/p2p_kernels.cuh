@@ -45,7 +45,7 @@ k_p2p_push_x(int64_t n, int64_t maxlen, P2PCtx c) {
   for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n; j += int64_t(gridDim.x) * blockDim.x) {
     const T v = src[j];
     for (int q = 0; q < c.P; ++q) {
-      if (q == c.me) continue;
+      if (q == c.me || !p2p_sends(c, q, j)) continue;
       reinterpret_cast<T*>(c.peer[q])[int64_t(c.me) * maxlen + j] = v;
     }
   }

@@ -149,6 +149,10 @@ struct spmv_csr_s {
   spmv_dist_s* dist = nullptr;
   std::vector<long long> bounds;
   long long maxlen = 0;
+  // halo intervals (NEXT-2, R27): halo[(r*P+s)*2 .. +1] = [lo, hi) of rank s's slice that rank r reads
+  std::vector<long long> halo;
+  int2* send_iv = nullptr;            // device [P]: what this rank sends to each rank
+  bool use_halo = false;              // exchange only the halo intervals (else the whole slices)
   int32_t* ci_own = nullptr;
   void* xpad = nullptr;               // nranks*maxlen, the gathered x / p
   // p2p transport: the IPC-exported fabric (xpad | exch | flags) and local counters
@@ -407,8 +411,29 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   at[0].val.clusterDim.z = 1;
   cfg.attrs = at;
   cfg.numAttrs = 1;
+  a.tstamp = nullptr;
+  int times = 0;
+  if (env_int("SPMV_XPLAN_TIMES", &times) && times) {
+    // diagnostics: per-CTA {start, x ready, streaming done, end} (globaltimer, ns), summarised on stderr
+    const size_t nb = sizeof(unsigned long long) * 4 * cfg.gridDim.x;
+    CK(cudaMalloc(&a.tstamp, nb));
+    CK(cudaMemsetAsync(a.tstamp, 0, nb, s));
+  }
   CK(cudaLaunchKernelEx(&cfg, part ? h->xp.kdot : h->xp.k, a));
   LAUNCHED();
+  if (a.tstamp) {
+    std::vector<unsigned long long> t(4 * cfg.gridDim.x);
+    CK(cudaMemcpyAsync(t.data(), a.tstamp, sizeof(unsigned long long) * t.size(), cudaMemcpyDeviceToHost, s));
+    CK(cudaStreamSynchronize(s));
+    cudaFree(a.tstamp);
+    unsigned long long t0 = ~0ull, tend = 0;
+    for (unsigned i = 0; i < cfg.gridDim.x; ++i) { t0 = std::min(t0, t[4 * i]); tend = std::max(tend, t[4 * i + 3]); }
+    fprintf(stderr, "[xplan times] kernel span %.2f us; per CTA (us from first start): start/xready/streamed/end\n",
+            (tend - t0) / 1e3);
+    for (unsigned i = 0; i < cfg.gridDim.x; ++i)
+      fprintf(stderr, "  cta %3u cl %2u  %6.2f %6.2f %6.2f %6.2f\n", i, i / (unsigned)h->xp.B, (t[4 * i] - t0) / 1e3,
+              (t[4 * i + 1] - t0) / 1e3, (t[4 * i + 2] - t0) / 1e3, (t[4 * i + 3] - t0) / 1e3);
+  }
   return SPMV_OK;
 }
 
@@ -942,9 +967,50 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
           h->k0, h->k1, colidx, dbounds, P, maxlen, h->ci_own);
       g_launches.fetch_add(1);
     }
+    // halo intervals of every (reader, owner) pair from the GLOBAL matrix (identical on all ranks)
+    int* dtab = nullptr;
+    if (P > 1 && m > 0) {
+      const size_t tb = sizeof(int) * 2 * (size_t)P * P;
+      okm = cudaMalloc(&dtab, tb) == cudaSuccess;
+      if (!okm) { cudaFree(dbounds); return fail(cuda_fail(cudaErrorMemoryAllocation, "cudaMalloc", __LINE__)); }
+      std::vector<int> init(2 * (size_t)P * P);
+      for (size_t i = 0; i < init.size(); i += 2) { init[i] = 0x7fffffff; init[i + 1] = -1; }
+      cudaMemcpyAsync(dtab, init.data(), tb, cudaMemcpyHostToDevice, s);
+      const size_t sm = sizeof(long long) * (P + 1) + tb;
+      k_halo_bounds<<<(unsigned)std::min<int64_t>(cdiv(m * 32, 256), 8LL * sms), 256, sm, s>>>(m, rowptr, colidx,
+                                                                                                 dbounds, P, dtab);
+      g_launches.fetch_add(1);
+    }
     e = cudaStreamSynchronize(s);
     cudaFree(dbounds);
-    if (e != cudaSuccess) return fail(cuda_fail(e, "renumber", __LINE__));
+    if (e != cudaSuccess) { cudaFree(dtab); return fail(cuda_fail(e, "renumber", __LINE__)); }
+    h->halo.assign(2 * (size_t)P * P, 0);
+    if (dtab) {
+      std::vector<int> tab(2 * (size_t)P * P);
+      e = cudaMemcpy(tab.data(), dtab, sizeof(int) * tab.size(), cudaMemcpyDeviceToHost);
+      cudaFree(dtab);
+      if (e != cudaSuccess) return fail(cuda_fail(e, "halo", __LINE__));
+      long long vol = 0;
+      for (size_t i = 0; i < tab.size(); i += 2)
+        if (tab[i + 1] >= 0) {
+          h->halo[i] = tab[i];
+          h->halo[i + 1] = (long long)tab[i + 1] + 1;
+          vol += h->halo[i + 1] - h->halo[i];
+        }
+      // exchange only the intervals when they move less than half of the padded all-gather
+      // (a decision every rank takes from the same global table)
+      int hv = 1;
+      env_int("SPMV_HALO", &hv);
+      h->use_halo = hv != 0 && 2 * vol < (long long)P * (P - 1) * maxlen;
+      std::vector<int2> siv(P);
+      for (int q = 0; q < P; ++q) {
+        const size_t i = 2 * ((size_t)q * P + r);  // reader q, owner r (this rank)
+        siv[q] = make_int2((int)h->halo[i], (int)h->halo[i + 1]);
+      }
+      if (cudaMalloc(&h->send_iv, sizeof(int2) * P) != cudaSuccess)
+        return fail(cuda_fail(cudaErrorMemoryAllocation, "cudaMalloc", __LINE__));
+      CK(cudaMemcpy(h->send_iv, siv.data(), sizeof(int2) * P, cudaMemcpyHostToDevice));
+    }
     h->rp_loc = rowptr + h->row0;
     h->ci_loc = h->ci_own - h->k0;  // absolute k addressing
   }
@@ -1023,7 +1089,7 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   }
   void* bufs[] = {h->p2p_local, h->peer_table, h->mg.split_row, h->mg.split_nz, h->mg.head, h->mg.carry, h->mg.head_flag, h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
                   h->xp.chunk_row, h->xp.plan, h->sl.pair_off, h->sl.vals, h->sl.cols,
-                  h->seg, h->crow, h->ci_own, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
+                  h->seg, h->crow, h->ci_own, h->send_iv, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
                   h->stage_x, h->stage_z};
   for (void* b : bufs)
@@ -1105,6 +1171,7 @@ static P2PCtx p2p_ctx(spmv_csr_s* h) {
   c.ticket = reinterpret_cast<int*>(h->p2p_local + 2 + P2P_NSLOT);
   c.me = h->dist->rank;
   c.P = h->dist->nranks;
+  c.send_iv = h->use_halo ? h->send_iv : nullptr;
   return c;
 }
 
@@ -1123,8 +1190,26 @@ static spmv_status exchange_x(spmv_csr_s* h, cudaStream_t s) {
     LAUNCHED();
     return SPMV_OK;
   }
-  NK(ncclAllGather((char*)h->xpad + h->ts * (size_t)(h->dist->rank * h->maxlen), h->xpad, (size_t)h->maxlen,
-                   h->dt == SPMV_F64 ? ncclDouble : ncclFloat, h->dist->comm, s));
+  const ncclDataType_t nt = h->dt == SPMV_F64 ? ncclDouble : ncclFloat;
+  if (h->use_halo) {
+    // halo exchange: send rank q the interval of my slice it reads, receive mine from every owner
+    const int P = h->dist->nranks, me = h->dist->rank;
+    char* xp = (char*)h->xpad;
+    NK(ncclGroupStart());
+    for (int q = 0; q < P; ++q) {
+      if (q == me) continue;
+      const long long* so = &h->halo[2 * ((size_t)q * P + me)];
+      const long long* ro = &h->halo[2 * ((size_t)me * P + q)];
+      if (so[1] > so[0])
+        NK(ncclSend(xp + h->ts * (size_t)(me * h->maxlen + so[0]), (size_t)(so[1] - so[0]), nt, q, h->dist->comm, s));
+      if (ro[1] > ro[0])
+        NK(ncclRecv(xp + h->ts * (size_t)(q * h->maxlen + ro[0]), (size_t)(ro[1] - ro[0]), nt, q, h->dist->comm, s));
+    }
+    NK(ncclGroupEnd());
+    return SPMV_OK;
+  }
+  NK(ncclAllGather((char*)h->xpad + h->ts * (size_t)(h->dist->rank * h->maxlen), h->xpad, (size_t)h->maxlen, nt,
+                   h->dist->comm, s));
   return SPMV_OK;
 }
 
@@ -1485,6 +1570,38 @@ extern "C" spmv_status spmv_dist_plan_host(const int32_t* rowptr, const int32_t*
     const int64_t s = (it - bounds) - 1;
     colidx_local[k - k0] = (int32_t)(s * ml + (c - bounds[s]));
   }
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_dist_halo_host(const int32_t* rowptr, const int32_t* colidx, int64_t m,
+                                           int32_t nranks, int64_t* halo) {
+  if (!rowptr || !halo || nranks < 1) return arg_fail("bad halo arguments");
+  const int P = nranks;
+  std::vector<int64_t> b(P + 1);
+  ST(spmv_csr_partition(rowptr, m, P, b.data()));
+  std::vector<int64_t> lo((size_t)P * P, INT64_MAX), hi((size_t)P * P, -1);
+  for (int r = 0; r < P; ++r)
+    for (int64_t i = b[r]; i < b[r + 1]; ++i)
+      for (int64_t k = rowptr[i]; k < rowptr[i + 1]; ++k) {
+        const int64_t c = colidx[k];
+        const int64_t sidx = (std::upper_bound(b.begin(), b.begin() + P, c) - b.begin()) - 1;
+        if (sidx == r) continue;
+        const size_t e = (size_t)r * P + sidx;
+        lo[e] = std::min(lo[e], c - b[sidx]);
+        hi[e] = std::max(hi[e], c - b[sidx]);
+      }
+  for (size_t e = 0; e < (size_t)P * P; ++e) {
+    halo[2 * e] = hi[e] >= 0 ? lo[e] : 0;
+    halo[2 * e + 1] = hi[e] >= 0 ? hi[e] + 1 : 0;
+  }
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_dist_halo(spmv_csr_t h, int64_t* halo, int32_t* used) {
+  if (!h || !halo) return arg_fail("NULL argument");
+  if (!h->dist) return arg_fail("not a distributed handle");
+  for (size_t i = 0; i < h->halo.size(); ++i) halo[i] = h->halo[i];
+  if (used) *used = h->use_halo ? 1 : 0;
   return SPMV_OK;
 }
 

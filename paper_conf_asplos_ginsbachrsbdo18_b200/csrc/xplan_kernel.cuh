@@ -70,7 +70,14 @@ struct XplanArgs {
   P2PHook hk;                  // p2p transport: wait for x / push the dot
   int dbg;
   int prefetch;                // 1: L2-prefetch the warp's chunk of the next tile
+  unsigned long long* tstamp;  // diagnostics (nullable): per CTA {start, x ready, streaming done, end} globaltimer
 };
+
+__device__ __forceinline__ unsigned long long gtimer() {
+  unsigned long long t;
+  asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
+  return t;
+}
 
 __device__ __forceinline__ void cluster_arrive_relaxed() {
   __syncwarp();
@@ -158,6 +165,7 @@ k_spmv_xplan(XplanArgs a) {
   const bool x_aligned = (reinterpret_cast<uintptr_t>(xg + col0) & 15) == 0;
   const int64_t bulk_elems = x_aligned ? ((ncols * int64_t(sizeof(T))) & ~int64_t(15)) / int64_t(sizeof(T)) : 0;
 
+  if (a.tstamp && threadIdx.x == 0) a.tstamp[4 * blockIdx.x] = gtimer();
   p2p_prologue_wait(a.hk);  // x slices of the peers (p2p transport)
   auto recv_bytes = [&](int t) -> uint32_t {
     const int nrows = int(cmin64(R, r1c - (r0c + int64_t(t) * R)));
@@ -178,6 +186,7 @@ k_spmv_xplan(XplanArgs a) {
   cluster_arrive();
   cluster_wait();
   mbar_wait(&xbar, 0, 1);
+  if (a.tstamp && threadIdx.x == 0) a.tstamp[4 * blockIdx.x + 1] = gtimer();
 
   const double alpha = a.alpha, beta = a.beta;
   double dacc = 0.0;
@@ -290,6 +299,7 @@ k_spmv_xplan(XplanArgs a) {
       finalize(t - 1);
       cluster_arrive_relaxed();
     }
+    if (a.tstamp && lane == 0) atomicMax(a.tstamp + 4 * blockIdx.x + 2, gtimer());  // last warp done streaming
     cluster_wait();
     finalize(ntiles - 1);
   }
@@ -300,6 +310,7 @@ k_spmv_xplan(XplanArgs a) {
   // leave together (peers may still be sending to / reading this CTA)
   cluster_arrive();
   cluster_wait();
+  if (a.tstamp && threadIdx.x == 0) a.tstamp[4 * blockIdx.x + 3] = gtimer();
   if (DOT) p2p_push_partials_last(a.hk, a.part, gridDim.x);
 }
 

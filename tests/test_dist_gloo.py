@@ -25,6 +25,23 @@ def _free_port():
     return p
 
 
+def _halo_brute(A, bounds, world):
+    """Reading R27 written out: per (reader r, owner s != r), min and max of
+    c - b_s over the columns c of r's rows owned by s; [0, 0) if none."""
+    import numpy as np
+    out = np.zeros((world, world, 2), dtype=np.int64)
+    rows = np.repeat(np.arange(A.m), np.diff(A.rowptr))
+    reader = np.searchsorted(bounds, rows, side="right") - 1
+    owner = np.searchsorted(bounds, A.colidx, side="right") - 1
+    for r in range(world):
+        for s_ in range(world):
+            sel = (reader == r) & (owner == s_)
+            if r != s_ and sel.any():
+                li = A.colidx[sel].astype(np.int64) - bounds[s_]
+                out[r, s_] = (li.min(), li.max() + 1)
+    return out
+
+
 def _worker(rank, world, port, cls, q):
     import sys
     sys.path.insert(0, ROOT)
@@ -37,7 +54,12 @@ def _worker(rank, world, port, cls, q):
     try:
         dist.init_process_group("gloo", init_method=f"tcp://127.0.0.1:{port}", rank=rank,
                                 world_size=world)
-        A = gen.makea(cls) if cls != "powerlaw" else gen.powerlaw(m=5000, lmax=800.0, seed=2, f32=False)
+        if cls == "powerlaw":
+            A = gen.powerlaw(m=5000, lmax=800.0, seed=2, f32=False)
+        elif cls == "stencil":
+            A = gen.stencil27(12)
+        else:
+            A = gen.makea(cls)
         bounds, maxlen, ci_loc = sp.spmv_dist_plan_host(A.rowptr, A.colidx, world, rank)
         assert np.array_equal(bounds, oracle.partition(A.rowptr, world))
         x = gen.uniform(A.n, seed=77)
@@ -48,6 +70,24 @@ def _worker(rank, world, port, cls, q):
         parts = [torch.zeros(maxlen, dtype=torch.float64) for _ in range(world)]
         dist.all_gather(parts, mine)
         xpad = torch.cat(parts).numpy()
+        # halo intervals (NEXT-2, R27): keep only what each owner would send
+        # this rank; everything else becomes NaN, so a missed column shows
+        halo = sp.spmv_dist_halo_host(A.rowptr, A.colidx, world)
+        assert np.array_equal(halo, _halo_brute(A, bounds, world))
+        for s_ in range(world):
+            if s_ == rank:
+                continue
+            lo, hi = halo[rank, s_]
+            seg = xpad[s_ * maxlen:(s_ + 1) * maxlen]
+            seg[:lo] = np.nan
+            seg[hi:] = np.nan
+        if cls == "stencil":  # at most one plane + one line + 1 from a neighbour, nothing from others
+            for s_ in range(world):
+                ln = halo[rank, s_, 1] - halo[rank, s_, 0]
+                if s_ != rank and abs(s_ - rank) == 1:
+                    assert 12 * 12 <= ln <= 12 * 12 + 12 + 1, ln
+                elif s_ != rank:
+                    assert ln == 0
         # local block, rebased rowptr, renumbered columns
         rp_loc = (A.rowptr[b0:b1 + 1] - A.rowptr[b0]).astype(np.int32)
         v_loc = A.vals[A.rowptr[b0]:A.rowptr[b1]]
@@ -70,7 +110,7 @@ def _worker(rank, world, port, cls, q):
 
 
 @pytest.mark.parametrize("world", [2, 3])
-@pytest.mark.parametrize("cls", ["S", "powerlaw"])
+@pytest.mark.parametrize("cls", ["S", "powerlaw", "stencil"])
 def test_dist_plan_gloo(world, cls):
     from paper_conf_asplos_ginsbachrsbdo18_b200 import build
     build.build()
