@@ -57,6 +57,8 @@ def lib():
         L.oracle_partition.argtypes = [_P, _I64, _I32, _P]
         L.oracle_partition.restype = None
         L.oracle_merge_path.argtypes = [_P, _I64, _I64, _P, _P]
+        L.oracle_stencil27.argtypes = [_I64, _I64, _I64, _P, _P, _P, _D, _D, _P, _P]
+        L.oracle_stencil27.restype = None
         L.oracle_merge_path.restype = None
         _lib = L
     return _lib
@@ -158,3 +160,19 @@ def merge_path(rowptr, pieces):
     sn = np.zeros(pieces + 1, dtype=np.int64)
     lib().oracle_merge_path(_ptr(rowptr), m, int(pieces), _ptr(sr), _ptr(sn))
     return sr, sn
+
+
+LAPLACE27 = np.array([-1.0] * 13 + [26.0] + [-1.0] * 13)  # reading R19 weights, w[(dz+1)*9+(dy+1)*3+(dx+1)]
+
+
+def stencil27(nx, ny, nz, x, w=None, y_old=None, alpha=1.0, beta=0.0):
+    """Matrix-free 27-point stencil (Fig. 13 Stencil idiom, R19): (y_ref, bound)."""
+    w = LAPLACE27 if w is None else np.ascontiguousarray(w, dtype=np.float64)
+    assert w.shape == (27,)
+    n = nx * ny * nz
+    x = _c(x, np.float64)
+    yo = _c(y_old if y_old is not None else np.zeros(n), np.float64)
+    y = np.empty(n)
+    b = np.empty(n)
+    lib().oracle_stencil27(nx, ny, nz, _ptr(w), _ptr(x), _ptr(yo), alpha, beta, _ptr(y), _ptr(b))
+    return y, b

@@ -81,6 +81,7 @@ spmv_dist_plan_host_c = _decl("spmv_dist_plan_host", [_P, _P, _I64, _I32, _I32, 
 spmv_dist_colidx_c = _decl("spmv_dist_colidx", [_P, _P])
 spmv_dist_halo_host_c = _decl("spmv_dist_halo_host", [_P, _P, _I64, _I32, _P])
 spmv_dist_halo_c = _decl("spmv_dist_halo", [_P, _P, _P])
+stencil27_apply_c = _decl("stencil27_apply", [_ST, _I64, _I64, _I64, _P, _P, _P, _D, _D, _P])
 
 # every symbol include/spmv.h declares (checked by tests/test_abi.py)
 EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_status",
@@ -89,7 +90,7 @@ EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_s
            "spmv_launch_count", "spmv_status_string", "spmv_last_error_string",
            "spmv_dist_get_unique_id", "spmv_dist_init", "spmv_dist_destroy", "spmv_dist_plan_host",
            "spmv_dist_colidx", "spmv_dist_init_p2p", "spmv_csr_p2p_handle", "spmv_csr_p2p_connect",
-           "spmv_dist_halo_host", "spmv_dist_halo"]
+           "spmv_dist_halo_host", "spmv_dist_halo", "stencil27_apply"]
 
 
 class SpmvError(RuntimeError):
@@ -164,6 +165,24 @@ def spmv_dist_halo_host(rowptr_host, colidx_host, nranks: int):
     _check(spmv_dist_halo_host_c(rp.ctypes.data, ci.ctypes.data, rp.shape[0] - 1, nranks, out.ctypes.data),
            "spmv_dist_halo_host")
     return out
+
+
+def stencil27_apply(nx: int, ny: int, nz: int, x, y, alpha: float = 1.0, beta: float = 0.0, w27=None,
+                    stream=None):
+    """Matrix-free 27-point stencil y <- alpha*A27 x + beta*y on an nx*ny*nz grid
+    (the paper's Stencil idiom, Fig. 13; reading R19 weights unless w27 gives
+    27 weights indexed (dz+1)*9+(dy+1)*3+(dx+1)).  Asynchronous."""
+    import numpy as np
+    import torch
+    dt = SPMV_F64 if y.dtype == torch.float64 else SPMV_F32
+    w = None if w27 is None else np.ascontiguousarray(w27, dtype=np.float64)
+    if w is not None and w.shape != (27,):
+        raise ValueError("w27 must hold 27 weights")
+    if stream is None:
+        stream = torch.cuda.current_stream(y.device).cuda_stream if y.is_cuda else 0
+    _check(stencil27_apply_c(dt, nx, ny, nz, None if w is None else w.ctypes.data, _ptr(x), _ptr(y),
+                             float(alpha), float(beta), stream), "stencil27_apply")
+    return y
 
 
 # ------------------------------------------------------------- distributed

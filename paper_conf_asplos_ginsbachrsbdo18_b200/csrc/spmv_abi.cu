@@ -23,6 +23,7 @@
 #include "xplan_kernel.cuh"
 #include "merge_kernel.cuh"
 #include "sell_kernel.cuh"
+#include "stencil_kernel.cuh"
 #include "p2p_kernels.cuh"
 
 using namespace spmv;
@@ -1570,6 +1571,60 @@ extern "C" spmv_status spmv_dist_plan_host(const int32_t* rowptr, const int32_t*
     const int64_t s = (it - bounds) - 1;
     colidx_local[k - k0] = (int32_t)(s * ml + (c - bounds[s]));
   }
+  return SPMV_OK;
+}
+
+// ------------------------------------------------------ matrix-free stencil
+extern "C" spmv_status stencil27_apply(spmv_dtype dt, int64_t nx, int64_t ny, int64_t nz, const double* w27,
+                                       const void* x, void* y, double alpha, double beta, void* stream) {
+  if (dt != SPMV_F64 && dt != SPMV_F32) return arg_fail("dtype must be SPMV_F64 or SPMV_F32");
+  if (nx < 0 || ny < 0 || nz < 0) return arg_fail("grid dimensions must be >= 0");
+  if (nx > 0 && ny > 0 && nz > 0 && (nx > INT64_MAX / ny || nx * ny > INT64_MAX / nz))
+    return arg_fail("grid too large");
+  const int64_t n = nx * ny * nz;
+  if (n == 0) return SPMV_OK;
+  if (nx > 2147483647LL / ST_TX || ny > 2147483647LL) return arg_fail("grid too large");
+  int dev = 0;
+  CK(cudaGetDevice(&dev));
+  const size_t ts = dt == SPMV_F64 ? 8 : 4;
+  ST(need_device(y, dev, "y must be a device pointer on the current device", false));
+  if (alpha != 0.0) ST(need_device(x, dev, "x must be a device pointer on the current device", false));
+  if (alpha != 0.0 && overlap(y, ts * (size_t)n, x, ts * (size_t)n)) {
+    g_err = "y overlaps x";
+    return SPMV_ERR_ALIAS;
+  }
+  cudaStream_t s = (cudaStream_t)stream;
+  const int sms = num_sms(dev);
+  if (alpha == 0.0) {  // A and x are not read (R6)
+    const int64_t g = std::min<int64_t>(cdiv(n, 256), 4LL * sms);
+    if (dt == SPMV_F64) k_scale<double><<<g, 256, 0, s>>>(n, (double*)y, beta);
+    else k_scale<float><<<g, 256, 0, s>>>(n, (float*)y, (double)(float)beta);
+    LAUNCHED();
+    return SPMV_OK;
+  }
+  StencilArgs a;
+  a.nx = nx; a.ny = ny; a.nz = nz;
+  for (int i = 0; i < 27; ++i) a.w[i] = w27 ? w27[i] : (i == 13 ? 26.0 : -1.0);  // R19 Laplacian by default
+  a.x = x; a.y = y;
+  a.alpha = alpha; a.beta = beta;
+  if (dt == SPMV_F32) {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+    for (int i = 0; i < 27; ++i) a.w[i] = (double)(float)a.w[i];
+  }
+  // z ranges: enough CTAs for ~8 per SM, each marching >= 16 planes (2 halo planes per range)
+  const int64_t bx = cdiv(nx, ST_TX), by = cdiv(ny, ST_TY);
+  int64_t zs = std::max<int64_t>(1, std::min<int64_t>(cdiv(8LL * sms, bx * by), cdiv(nz, 16)));
+  int zc = (int)cdiv(nz, zs);
+  int env = 0;
+  if (env_int("SPMV_STENCIL_ZCHUNK", &env) && env > 0) zc = env;
+  zs = cdiv(nz, zc);
+  a.zchunk = zc;
+  if (by > 65535 || zs > 65535) return arg_fail("grid too large for the stencil launch");
+  const dim3 grid((unsigned)bx, (unsigned)by, (unsigned)zs);
+  if (dt == SPMV_F64) k_stencil27<double><<<grid, ST_NT, 0, s>>>(a);
+  else k_stencil27<float><<<grid, ST_NT, 0, s>>>(a);
+  LAUNCHED();
   return SPMV_OK;
 }
 

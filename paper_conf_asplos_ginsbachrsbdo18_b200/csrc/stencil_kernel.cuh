@@ -1,0 +1,156 @@
+// stencil_kernel.cuh -- matrix-free 27-point stencil:
+// the paper's Stencil idiom (Fig. 13: a loop nest whose
+// store is a kernel function of reads at constant offsets), with the kernel
+// function a weighted sum over the 3x3x3 neighbourhood and Dirichlet
+// truncation (reading R19): for every grid point p = x + nx*(y + ny*z)
+//     y[p] = alpha * sum_{d in {-1,0,1}^3, p+d inside} w[d] * x[p+d] + beta * y[p]
+// It is the operator whose CSR form is BJ.cfg[4]; with R19's weights (26, -1)
+// the result equals spmv_csr on gen.stencil27 (same terms, same order).
+//
+// 2.5-D blocking: a CTA owns a TX x TY tile of (x, y) and marches a range of
+// z planes.  Each plane (+ a one-point halo) is staged once in shared memory
+// (double-buffered, the next plane's loads in flight while the current one is
+// consumed); a plane zp contributes its 3x3 in-plane neighbourhood to three
+// outputs held in registers: z = zp+1 (weights of dz = -1), z = zp (dz = 0)
+// and z = zp-1 (dz = +1), after which output zp-1 is complete and stored.
+// Every output therefore receives its 27 terms in ascending linear index
+// (dz, dy, dx), exactly the CSR row order (points outside the grid are staged
+// as 0 and add an exact zero), accumulated with FMA like the CSR kernels
+// (reading R11).  A bit-exact variant (separate round-to-nearest mul and add,
+// as the oracle's -ffp-contract=off loop) measured 108 us on 256^3: 54 fp64
+// operations per point make it fp64-ALU-bound (~49 us of DMUL/DADD issue at
+// 64 per clock per SM) before memory; the FMA form halves that.  HBM traffic:
+// x once (+2 halo planes per z range, mostly L2 hits) and y once:
+// 2*sizeof(T) bytes per point.
+// Measured on 256^3 fp64 (tools/run_stencil_variants.sh): 1 point per thread
+// 86 us whatever the prefetch depth (1-4 planes in flight: not latency-bound;
+// ncu: issue-bound, ~130 instructions per point incl. the 27 weights held in
+// uniform registers); 2 rows per thread 76-78 us (shared loads and loop
+// overhead amortised), 4 rows 80 us (register-limited occupancy).
+#pragma once
+#include "common.cuh"
+
+namespace spmv {
+
+#ifndef ST_RY_DEF
+#define ST_RY_DEF 2
+#endif
+constexpr int ST_RY = ST_RY_DEF;  // outputs per thread along y (register blocking: shared loads and
+                                  // loop overhead amortised over ST_RY points)
+constexpr int ST_TX = 32, ST_NT = 256, ST_TY = (ST_NT / ST_TX) * ST_RY;
+constexpr int ST_PX = ST_TX + 2, ST_PY = ST_TY + 2, ST_PN = ST_PX * ST_PY;
+constexpr int ST_LPT = (ST_PN + ST_NT - 1) / ST_NT;  // plane elements staged per thread
+#ifndef ST_PF_DEF
+#define ST_PF_DEF 1
+#endif
+constexpr int ST_PF = ST_PF_DEF;  // planes whose loads are in flight (register ring)
+
+struct StencilArgs {
+  int64_t nx, ny, nz;
+  int zchunk;          // planes per CTA (blockIdx.z)
+  double w[27];        // w[(dz+1)*9 + (dy+1)*3 + (dx+1)]
+  const void* x;
+  void* y;
+  double alpha, beta;
+};
+
+template <typename T>
+__global__ void __launch_bounds__(ST_NT)
+k_stencil27(StencilArgs a) {
+  __shared__ T pl[2][ST_PN];
+  const T* __restrict__ x = static_cast<const T*>(a.x);
+  T* __restrict__ y = static_cast<T*>(a.y);
+  const int tx = threadIdx.x % ST_TX, ty = (threadIdx.x / ST_TX) * ST_RY;  // first of ST_RY rows
+  const int64_t nx = a.nx, ny = a.ny, nz = a.nz, nxy = nx * ny;
+  const int64_t x0 = int64_t(blockIdx.x) * ST_TX, y0 = int64_t(blockIdx.y) * ST_TY;
+  const int64_t z0 = int64_t(blockIdx.z) * a.zchunk;
+  const int64_t z1 = cmin64(nz, z0 + a.zchunk);
+  const int64_t gx = x0 + tx, gy = y0 + ty;
+
+  // staging: element e of the haloed plane -> (lx, ly); global offset inside a plane or -1
+  int64_t off[ST_LPT];
+#pragma unroll
+  for (int u = 0; u < ST_LPT; ++u) {
+    const int e = threadIdx.x + u * ST_NT;
+    off[u] = -1;
+    if (e < ST_PN) {
+      const int64_t X = x0 + (e % ST_PX) - 1, Y = y0 + (e / ST_PX) - 1;
+      if (X >= 0 && X < nx && Y >= 0 && Y < ny) off[u] = X + nx * Y;
+    }
+  }
+  // register ring: v[k] holds plane zp+1+k while plane zp is consumed
+  T v[ST_PF][ST_LPT];
+  auto fetch = [&](int64_t zp, T* dst) {
+    const bool zin = zp >= 0 && zp < nz && zp <= z1;
+#pragma unroll
+    for (int u = 0; u < ST_LPT; ++u) dst[u] = (zin && off[u] >= 0) ? __ldg(x + zp * nxy + off[u]) : T(0);
+  };
+  auto stash = [&](int buf, const T* src) {
+#pragma unroll
+    for (int u = 0; u < ST_LPT; ++u) {
+      const int e = threadIdx.x + u * ST_NT;
+      if (e < ST_PN) pl[buf][e] = src[u];
+    }
+  };
+
+  const double alpha = a.alpha, beta = a.beta;
+  double acc_m[ST_RY], acc_c[ST_RY], acc_p[ST_RY];  // outputs zp-1, zp, zp+1 of each row
+#pragma unroll
+  for (int r = 0; r < ST_RY; ++r) acc_m[r] = acc_c[r] = acc_p[r] = 0.0;
+  {
+    T v0[ST_LPT];
+    fetch(z0 - 1, v0);
+    stash(0, v0);
+  }
+#pragma unroll
+  for (int k = 0; k < ST_PF; ++k) fetch(z0 + k, v[k]);
+  __syncthreads();
+  int cur = 0;
+  for (int64_t zp = z0 - 1; zp <= z1; ++zp) {
+    T vf[ST_LPT];
+    fetch(zp + 1 + ST_PF, vf);  // ST_PF planes ahead (zeros past z1: never stashed)
+    const T* P = pl[cur];
+#pragma unroll
+    for (int sy = 0; sy < ST_RY + 2; ++sy)  // plane rows ty-1 .. ty+ST_RY
+#pragma unroll
+      for (int dx = 0; dx < 3; ++dx) {
+        const double xv = double(P[(ty + sy) * ST_PX + tx + dx]);
+#pragma unroll
+        for (int r = 0; r < ST_RY; ++r) {
+          const int dy = sy - r;  // row offset + 1 of this value for output row r
+          if (dy < 0 || dy > 2) continue;
+          acc_p[r] = fma(a.w[0 * 9 + dy * 3 + dx], xv, acc_p[r]);  // output zp+1, dz = -1
+          acc_c[r] = fma(a.w[1 * 9 + dy * 3 + dx], xv, acc_c[r]);  // output zp,   dz =  0
+          acc_m[r] = fma(a.w[2 * 9 + dy * 3 + dx], xv, acc_m[r]);  // output zp-1, dz = +1
+        }
+      }
+    const int64_t zo = zp - 1;  // complete now
+    if (gx < nx && zo >= z0 && zo < z1) {
+#pragma unroll
+      for (int r = 0; r < ST_RY; ++r) {
+        if (gy + r >= ny) continue;
+        const int64_t p = gx + nx * (gy + r) + nxy * zo;
+        double res = alpha * acc_m[r];
+        if (beta != 0.0) res += beta * double(y[p]);
+        y[p] = T(res);
+      }
+    }
+#pragma unroll
+    for (int r = 0; r < ST_RY; ++r) {
+      acc_m[r] = acc_c[r];
+      acc_c[r] = acc_p[r];
+      acc_p[r] = 0.0;
+    }
+    if (zp + 1 <= z1) stash(cur ^ 1, v[0]);
+    __syncthreads();
+    cur ^= 1;
+#pragma unroll
+    for (int k = 0; k + 1 < ST_PF; ++k)
+#pragma unroll
+      for (int u = 0; u < ST_LPT; ++u) v[k][u] = v[k + 1][u];
+#pragma unroll
+    for (int u = 0; u < ST_LPT; ++u) v[ST_PF - 1][u] = vf[u];
+  }
+}
+
+}  // namespace spmv

@@ -244,3 +244,56 @@ def test_merge_path_characterisation(C):
                      and (i == 0 or A[i - 1] <= d - i)
                      and (i == m or d - i == 0 or A[i] > d - i - 1)]
             assert cands == [(sr[c], sn[c])], (rp, c, cands, sr[c], sn[c])
+
+
+# ---------------------------------------------------------------- stencil27
+# oracle_stencil27 (Fig. 13 Stencil idiom, reading R19), pinned to closed
+# forms, exact shifts, and the CSR oracle on the generator's matrix.
+
+@pytest.mark.parametrize("dims", [(1, 1, 1), (2, 3, 5), (7, 4, 3), (9, 9, 9)])
+def test_stencil27_laplace_closed_forms(dims):
+    nx, ny, nz = dims
+    n = nx * ny * nz
+    i = np.arange(n)
+    xx, yy, zz = i % nx, (i // nx) % ny, i // (nx * ny)
+    cnt = np.ones(n, dtype=np.int64)
+    for c, N in ((xx, nx), (yy, ny), (zz, nz)):
+        cnt *= (np.minimum(c + 1, N - 1) - np.maximum(c - 1, 0) + 1)
+    y, b = oracle.stencil27(nx, ny, nz, np.ones(n))
+    assert np.array_equal(y, (27 - cnt).astype(np.float64))  # A*1 = 26 - (cnt - 1)
+    # affine fields vanish on interior points (weights sum to 0, symmetric offsets)
+    f = 3.0 + 2.0 * xx - 5.0 * yy + 7.0 * zz
+    y, _ = oracle.stencil27(nx, ny, nz, f)
+    inner = (xx > 0) & (xx < nx - 1) & (yy > 0) & (yy < ny - 1) & (zz > 0) & (zz < nz - 1)
+    assert np.all(y[inner] == 0.0)
+
+
+@pytest.mark.parametrize("d", [(0, 0, 0), (1, 0, 0), (-1, 1, 0), (1, -1, -1), (0, 0, 1)])
+def test_stencil27_one_hot_weight_is_a_shift(d):
+    """w = e_d: y[p] = x[p + d] when p + d is inside the grid, else 0 (exact)."""
+    nx, ny, nz = 6, 5, 4
+    dx, dy, dz = d
+    w = np.zeros(27)
+    w[(dz + 1) * 9 + (dy + 1) * 3 + (dx + 1)] = 1.0
+    x = gen.uniform(nx * ny * nz, seed=3)
+    y, _ = oracle.stencil27(nx, ny, nz, x, w=w)
+    for z in range(nz):
+        for yy in range(ny):
+            for xx in range(nx):
+                p = xx + nx * (yy + ny * z)
+                q = (xx + dx, yy + dy, z + dz)
+                inside = 0 <= q[0] < nx and 0 <= q[1] < ny and 0 <= q[2] < nz
+                assert y[p] == (x[q[0] + nx * (q[1] + ny * q[2])] if inside else 0.0)
+
+
+@pytest.mark.parametrize("N", [2, 5, 12])
+def test_stencil27_equals_csr_oracle_bitwise(N):
+    """R19 weights on an N^3 grid == oracle_spmv_f64 on gen.stencil27(N): same
+    terms in the same (ascending column) order, so bit for bit; alpha/beta too."""
+    A = gen.stencil27(N)
+    x = gen.uniform(A.n, seed=4)
+    y0 = gen.uniform(A.m, seed=5)
+    for a, b in [(1.0, 0.0), (-2.5, 0.5), (0.0, 3.0)]:
+        ys, bs = oracle.stencil27(N, N, N, x, y_old=y0, alpha=a, beta=b)
+        yc, bc = oracle.spmv(A.rowptr, A.colidx, A.vals, x, y0, a, b)
+        assert np.array_equal(ys, yc) and np.array_equal(bs, bc)

@@ -67,6 +67,27 @@ def main():
         x = torch.from_numpy(gen.uniform(C.n, seed=1, f32=C.vals.dtype == np.float32)).to(dev)
         y = torch.empty(C.m, dtype=va.dtype, device=dev)
         nbytes = C.bytes_per_spmv()
+        if w.startswith("stencil"):
+            # the matrix-free operator of the same matrix (NEXT-3): algorithmic bytes of the CSR
+            # form reported for comparison, and its own 2*8 B per point
+            N = int(w[7:])
+            flush = torch.empty(256 << 20, dtype=torch.int8, device=dev)
+            for _ in range(3):
+                sp.stencil27_apply(N, N, N, x, y)
+            ts = []
+            for _ in range(20):
+                flush.zero_()
+                a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                a.record()
+                sp.stencil27_apply(N, N, N, x, y)
+                b.record()
+                b.synchronize()
+                ts.append(a.elapsed_time(b))
+            ms = statistics.median(ts)
+            print(json.dumps({"matrix": w, "variant": "matrix_free", "kernel": "stencil27", "us": round(ms * 1e3, 2),
+                              "gbs": round(nbytes / (ms / 1e3) / 1e9, 1),
+                              "own_gbs": round(16 * C.m / (ms / 1e3) / 1e9, 1),
+                              "gflops": round(2 * C.nnz / (ms / 1e3) / 1e9, 1)}), flush=True)
         for name, kw, env in VARIANTS:
             try:
                 ms, info = time_variant((rp, ci, va, C.n), x, y, kw, env)
