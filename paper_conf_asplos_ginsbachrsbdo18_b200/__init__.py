@@ -32,7 +32,7 @@ _ST = ctypes.c_int
 SPMV_OK, SPMV_ERR_ARG, SPMV_ERR_INDEX, SPMV_ERR_ALIAS, SPMV_ERR_CUDA = 0, 1, 2, 3, 4
 SPMV_ERR_NCCL, SPMV_ERR_NOMEM, SPMV_ERR_BREAKDOWN, SPMV_ERR_UNSUPPORTED = 5, 6, 7, 8
 SPMV_F64, SPMV_F32 = 0, 1
-KERNELS = {"auto": 0, "scalar": 1, "vector": 2, "merge": 3, "xstat": 4, "xplan": 5, "sell": 6}
+KERNELS = {"auto": 0, "scalar": 1, "vector": 2, "merge": 3, "xstat": 4, "xplan": 5, "sell": 6, "sellsort": 7}
 KERNEL_NAMES = {v: k for k, v in KERNELS.items()}
 
 

@@ -12,8 +12,10 @@
 #include <string>
 #include <vector>
 
+#include <cub/device/device_radix_sort.cuh>
 #include <cuda_runtime.h>
 #include <nccl.h>
+#include <functional>
 
 #include "../../include/spmv.h"
 #include "analysis_kernels.cuh"
@@ -134,7 +136,12 @@ struct spmv_csr_s {
   // SELL (SELL-32 device plan, x gathered from global memory)
   struct Sell {
     bool built = false;
-    int64_t nchunks = 0, pairs = 0, grid = 0;
+    int sorted = 0;
+    int64_t nchunks = 0, pairs = 0, grid = 0, nlong = 0, nseg = 0, nmulti = 0;
+    int* perm = nullptr;
+    SellSeg* seg = nullptr;     // long-row segments
+    double* seg_part = nullptr;
+    int* seg_cnt = nullptr;
     long long* pair_off = nullptr;
     unsigned char* vals = nullptr;
     int* cols = nullptr;
@@ -587,30 +594,97 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
 // ------------------------------------------------------------------ SELL
 static spmv_status sell_pack(spmv_csr_s* h, const void* vals, int values_only) {
   cudaStream_t s = h->stream;
-  const int64_t g = std::min<int64_t>(cdiv(h->m_loc, 256), 16LL * num_sms(h->device));
+  const auto& S = h->sl;
+  const int64_t g = std::max<int64_t>(1, std::min<int64_t>(cdiv(h->m_loc - S.nlong, 256), 16LL * num_sms(h->device)));
   if (h->dt == SPMV_F64)
-    k_sell_pack<double><<<g, 256, 0, s>>>(h->m_loc, h->rp_loc, h->ci_loc, (const double*)vals, h->sl.pair_off,
-                                          (double*)h->sl.vals, h->sl.cols, values_only);
+    k_sell_pack<double><<<g, 256, 0, s>>>(h->m_loc, h->rp_loc, h->ci_loc, (const double*)vals, S.pair_off, S.perm,
+                                          S.nlong, (double*)S.vals, S.cols, values_only);
   else
-    k_sell_pack<float><<<g, 256, 0, s>>>(h->m_loc, h->rp_loc, h->ci_loc, (const float*)vals, h->sl.pair_off,
-                                         (float*)h->sl.vals, h->sl.cols, values_only);
+    k_sell_pack<float><<<g, 256, 0, s>>>(h->m_loc, h->rp_loc, h->ci_loc, (const float*)vals, S.pair_off, S.perm,
+                                         S.nlong, (float*)S.vals, S.cols, values_only);
   LAUNCHED();
   return SPMV_OK;
 }
 
-// Build the SELL-32 plan (create).  Not eligible (*ok = false) when the
-// padding exceeds max_pad x nnz (skewed rows: merge path / vector instead).
-static spmv_status sell_build(spmv_csr_s* h, double max_pad, bool* ok) {
+// Build the SELL-32 plan (create).  sorted = 0: chunks of consecutive rows;
+// sorted = 1: rows ordered by length (descending, stable device radix sort),
+// rows longer than SELL_LONG kept in the CSR and processed warp-per-row.
+// Not eligible (*ok = false) when the padding exceeds max_pad x nnz.
+static spmv_status sell_build(spmv_csr_s* h, double max_pad, int sorted, bool* ok) {
   *ok = false;
   const int64_t m = h->m_loc, nnz = h->k1 - h->k0;
   if (m == 0 || nnz == 0) return SPMV_OK;
+  if (sorted && m > 2147483647LL) return SPMV_OK;
   cudaStream_t s = h->stream;
   auto& S = h->sl;
-  const int64_t nch = cdiv(m, 32);
+  auto cleanup = [&]() {
+    void* bufs[] = {S.pair_off, S.vals, S.cols, S.perm, S.seg, S.seg_part, S.seg_cnt};
+    for (void* q : bufs)
+      if (q) cudaFree(q);
+    S = spmv_csr_s::Sell();
+  };
+  const int sms = num_sms(h->device);
+  if (sorted) {
+    int *keys = nullptr, *keys_out = nullptr, *ids = nullptr;
+    void* tmp = nullptr;
+    size_t tmp_bytes = 0;
+    CK(cudaMalloc(&keys, sizeof(int) * m));
+    CK(cudaMalloc(&keys_out, sizeof(int) * m));
+    CK(cudaMalloc(&ids, sizeof(int) * m));
+    CK(cudaMalloc(&S.perm, sizeof(int) * m));
+    k_row_len_ids<<<(unsigned)std::min<int64_t>(cdiv(m, 256), 8LL * sms), 256, 0, s>>>(m, h->rp_loc, keys, ids);
+    LAUNCHED();
+    CK(cub::DeviceRadixSort::SortPairsDescending(nullptr, tmp_bytes, keys, keys_out, ids, S.perm, (int)m, 0, 32, s));
+    CK(cudaMalloc(&tmp, tmp_bytes));
+    CK(cub::DeviceRadixSort::SortPairsDescending(tmp, tmp_bytes, keys, keys_out, ids, S.perm, (int)m, 0, 32, s));
+    std::vector<int> sk(m);
+    CK(cudaMemcpyAsync(sk.data(), keys_out, sizeof(int) * m, cudaMemcpyDeviceToHost, s));
+    CK(cudaStreamSynchronize(s));
+    cudaFree(tmp);
+    cudaFree(keys);
+    cudaFree(keys_out);
+    cudaFree(ids);
+    // long rows: the prefix with length > SELL_LONG, cut into segments of <= SELL_SEG entries
+    S.nlong = std::lower_bound(sk.begin(), sk.end(), SELL_LONG, std::greater<int>()) - sk.begin();
+    if (S.nlong > 0) {
+      std::vector<int> lp(S.nlong), rp(m + 1);
+      CK(cudaMemcpy(lp.data(), S.perm, sizeof(int) * S.nlong, cudaMemcpyDeviceToHost));
+      CK(cudaMemcpy(rp.data(), h->rp_loc, sizeof(int) * (m + 1), cudaMemcpyDeviceToHost));
+      std::vector<SellSeg> segs;
+      int npart = 0, ncnt = 0;
+      for (int64_t j = 0; j < S.nlong; ++j) {
+        const int i = lp[j], k0 = rp[i], k1 = rp[i + 1];
+        const int ns = (int)cdiv(k1 - k0, SELL_SEG);
+        for (int q = 0; q < ns; ++q) {
+          SellSeg g{};
+          g.row = i;
+          g.k0 = k0 + q * SELL_SEG;
+          g.k1 = std::min(k1, g.k0 + SELL_SEG);
+          g.pbase = ns > 1 ? npart : -1;
+          g.sidx = q;
+          g.nseg = ns;
+          g.cslot = ns > 1 ? ncnt : -1;
+          segs.push_back(g);
+        }
+        if (ns > 1) { npart += ns; ++ncnt; }
+      }
+      S.nseg = (int64_t)segs.size();
+      S.nmulti = ncnt;
+      CK(cudaMalloc(&S.seg, sizeof(SellSeg) * segs.size()));
+      CK(cudaMemcpy(S.seg, segs.data(), sizeof(SellSeg) * segs.size(), cudaMemcpyHostToDevice));
+      CK(cudaMalloc(&S.seg_part, sizeof(double) * std::max(npart, 1)));
+      CK(cudaMalloc(&S.seg_cnt, sizeof(int) * std::max(ncnt, 1)));
+      CK(cudaMemset(S.seg_cnt, 0, sizeof(int) * std::max(ncnt, 1)));
+    }
+  }
+  const int64_t nch = cdiv(m - S.nlong, 32);
   CK(cudaMalloc(&S.pair_off, sizeof(long long) * (nch + 1)));
-  k_sell_pairs<<<(unsigned)std::min<int64_t>(cdiv(nch, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
-      m, h->rp_loc, nch, S.pair_off);
-  LAUNCHED();
+  if (nch > 0) {
+    const unsigned g = (unsigned)std::max<int64_t>(1, std::min<int64_t>(cdiv(nch, 256), 8LL * sms));
+    if (sorted) k_sell_pairs_sorted<<<g, 256, 0, s>>>(m, h->rp_loc, S.perm, S.nlong, nch, S.pair_off);
+    else k_sell_pairs<<<g, 256, 0, s>>>(m, h->rp_loc, nch, S.pair_off);
+    LAUNCHED();
+  }
   std::vector<long long> off(nch + 1);
   CK(cudaMemcpyAsync(off.data(), S.pair_off, sizeof(long long) * nch, cudaMemcpyDeviceToHost, s));
   CK(cudaStreamSynchronize(s));
@@ -622,8 +696,7 @@ static spmv_status sell_build(spmv_csr_s* h, double max_pad, bool* ok) {
   }
   off[nch] = pos;
   if ((double)pos * 64.0 > max_pad * (double)nnz + 64.0) {
-    cudaFree(S.pair_off);
-    S = spmv_csr_s::Sell();
+    cleanup();
     return SPMV_OK;
   }
   S.nchunks = nch;
@@ -636,8 +709,9 @@ static spmv_status sell_build(spmv_csr_s* h, double max_pad, bool* ok) {
   CK(cudaMemsetAsync(S.cols, 0xff, slots * sizeof(int), s));  // -1: padding
   ST(sell_pack(h, h->vals, 0));
   CK(cudaStreamSynchronize(s));
-  // grid: 8 CTAs of SELL_NT per SM, never more warps than chunks
-  S.grid = std::max<int64_t>(1, std::min<int64_t>(cdiv(nch, SELL_NT / 32), 8LL * num_sms(h->device)));
+  // grid: 8 CTAs of SELL_NT per SM, never more warps than work items
+  S.grid = std::max<int64_t>(1, std::min<int64_t>(cdiv(nch + S.nseg, SELL_NT / 32), 8LL * sms));
+  S.sorted = sorted;
   S.built = true;
   *ok = true;
   return SPMV_OK;
@@ -648,6 +722,14 @@ static spmv_status launch_sell(spmv_csr_s* h, cudaStream_t s, const void* x, voi
   SellArgs a;
   a.m = h->m_loc;
   a.nchunks = h->sl.nchunks;
+  a.perm = h->sl.perm;
+  a.nlong = h->sl.nlong;
+  a.nseg = h->sl.nseg;
+  a.seg = h->sl.seg;
+  a.seg_part = h->sl.seg_part;
+  a.seg_cnt = h->sl.seg_cnt;
+  a.colidx = h->ci_loc;
+  a.csr_vals = h->vals;
   a.vals = h->sl.vals;
   a.cols = reinterpret_cast<const int2*>(h->sl.cols);
   a.pair_off = h->sl.pair_off;
@@ -660,8 +742,22 @@ static spmv_status launch_sell(spmv_csr_s* h, cudaStream_t s, const void* x, voi
   a.hk = hook;
   const unsigned g = (unsigned)h->sl.grid;
   if (h->dt == SPMV_F64) {
-    if (part) k_spmv_sell<double, true><<<g, SELL_NT, 0, s>>>(a);
-    else k_spmv_sell<double, false><<<g, SELL_NT, 0, s>>>(a);
+    if (part && h->sl.nmulti > 0) {
+      // multi-segment rows are finished by whichever warp completes them: the dot
+      // runs as a separate pass so its per-CTA partials stay deterministic
+      P2PHook wait_only = hook;
+      wait_only.push_slot = -1;
+      a.hk = wait_only;
+      k_spmv_sell<double, false><<<g, SELL_NT, 0, s>>>(a);
+      LAUNCHED();
+      P2PHook push_only = hook;
+      push_only.wait_x = 0;
+      k_dot_partials<<<(int)h->vgrid, 256, 0, s>>>(h->m_loc, w, (const double*)y, part, push_only);
+    } else if (part) {
+      k_spmv_sell<double, true><<<g, SELL_NT, 0, s>>>(a);
+    } else {
+      k_spmv_sell<double, false><<<g, SELL_NT, 0, s>>>(a);
+    }
   } else {
     a.alpha = (double)(float)alpha;
     a.beta = (double)(float)beta;
@@ -741,9 +837,9 @@ static spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, con
     return SPMV_OK;
   }
   if (h->kernel == SPMV_KERNEL_XPLAN && vals == h->vals) return launch_xplan(h, s, x, y, alpha, beta, w, part, hook);
-  if (h->kernel == SPMV_KERNEL_SELL && vals == h->vals) return launch_sell(h, s, x, y, alpha, beta, w, part, hook);
-  const int64_t vgrid_spmv =
-      (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_SELL) ? h->grid_vec : h->grid;
+  const bool sell = h->kernel == SPMV_KERNEL_SELL || h->kernel == SPMV_KERNEL_SELL_SORTED;
+  if (sell && vals == h->vals) return launch_sell(h, s, x, y, alpha, beta, w, part, hook);
+  const int64_t vgrid_spmv = (h->kernel == SPMV_KERNEL_XPLAN || sell) ? h->grid_vec : h->grid;
   if (h->kernel == SPMV_KERNEL_XSTAT) return launch_xstat(h, s, vals, x, y, alpha, beta, w, part, hook);
   if (h->kernel == SPMV_KERNEL_MERGE) {
     P2PHook wait_only = hook;
@@ -1036,29 +1132,33 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
       }
     }
   }
-  if (h->kernel != SPMV_KERNEL_XPLAN && (rk == SPMV_KERNEL_SELL || (rk == SPMV_KERNEL_AUTO && plan))) {
-    // auto + plan, x too large for the clusters (or short rows): the SELL-32
-    // plan with global x gathers when the rows are regular enough that the
-    // 32-row chunks pad little (the 27-point stencil); forced: any padding
+  const bool skewed = (double)h->row_max > 32.0 * std::max(h->row_mean, 1.0);
+  if (h->kernel != SPMV_KERNEL_XPLAN && (rk == SPMV_KERNEL_SELL || rk == SPMV_KERNEL_SELL_SORTED ||
+                                         (rk == SPMV_KERNEL_AUTO && plan))) {
+    // auto + plan, x too large for the clusters (or short rows): a SELL-32 plan
+    // with global x gathers -- chunks of consecutive rows when they pad by
+    // <= 20 % (the 27-point stencil), else (skewed rows: the power law) the
+    // length-sorted chunks with the long rows warp-per-row; forced: any padding
+    const int sorted = rk == SPMV_KERNEL_SELL_SORTED || (rk == SPMV_KERNEL_AUTO && skewed);
     bool ok = false;
-    spmv_status st = sell_build(h, rk == SPMV_KERNEL_SELL ? 1e30 : 1.2, &ok);
+    spmv_status st = sell_build(h, rk == SPMV_KERNEL_AUTO ? 1.2 : 1e30, sorted, &ok);
     if (st != SPMV_OK) return fail(st);
     if (ok) {
-      h->kernel = SPMV_KERNEL_SELL;
-      h->grid = h->sl.grid;
+      h->kernel = sorted ? SPMV_KERNEL_SELL_SORTED : SPMV_KERNEL_SELL;
+      h->grid = h->sl.nmulti > 0 ? h->vgrid : h->sl.grid;  // dot partials: k_dot_partials or fused
     }
   }
-  if (h->kernel != SPMV_KERNEL_XPLAN && h->kernel != SPMV_KERNEL_SELL && rk != SPMV_KERNEL_VECTOR &&
-      rk != SPMV_KERNEL_SCALAR && rk != SPMV_KERNEL_XSTAT &&
-      h->m_loc > 0 &&
-      (rk == SPMV_KERNEL_MERGE || (double)h->row_max > 32.0 * std::max(h->row_mean, 1.0))) {
-    // skewed rows (a long row would pin one warp of the vector kernel): merge path
+  if (h->kernel != SPMV_KERNEL_XPLAN && h->kernel != SPMV_KERNEL_SELL && h->kernel != SPMV_KERNEL_SELL_SORTED &&
+      rk != SPMV_KERNEL_VECTOR && rk != SPMV_KERNEL_SCALAR && rk != SPMV_KERNEL_XSTAT && h->m_loc > 0 &&
+      (rk == SPMV_KERNEL_MERGE || skewed)) {
+    // skewed rows without a plan (a long row would pin one warp of the vector kernel): merge path
     spmv_status st = merge_setup(h);
     if (st != SPMV_OK) return fail(st);
     h->kernel = SPMV_KERNEL_MERGE;
     h->grid = h->vgrid;  // dot partials come from k_dot_partials
   }
-  if (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_MERGE || h->kernel == SPMV_KERNEL_SELL) {
+  if (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_MERGE || h->kernel == SPMV_KERNEL_SELL ||
+      h->kernel == SPMV_KERNEL_SELL_SORTED) {
   } else if (rk == SPMV_KERNEL_XSTAT) {
     bool ok = false;
     spmv_status st = xstat_setup(h, &ok);
@@ -1089,7 +1189,7 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
     if (h->xpad == h->fabric) h->xpad = nullptr;
   }
   void* bufs[] = {h->p2p_local, h->peer_table, h->mg.split_row, h->mg.split_nz, h->mg.head, h->mg.carry, h->mg.head_flag, h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
-                  h->xp.chunk_row, h->xp.plan, h->sl.pair_off, h->sl.vals, h->sl.cols,
+                  h->xp.chunk_row, h->xp.plan, h->sl.pair_off, h->sl.vals, h->sl.cols, h->sl.perm, h->sl.seg, h->sl.seg_part, h->sl.seg_cnt,
                   h->seg, h->crow, h->ci_own, h->send_iv, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
                   h->stage_x, h->stage_z};

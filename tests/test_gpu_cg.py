@@ -154,7 +154,7 @@ def test_npb_graph_vs_eager_bitexact(sp, torch_dev, monkeypatch):
     assert np.array_equal(z1, z2) and np.array_equal(r1, r2)
 
 
-@pytest.mark.parametrize("kernel", ["merge", "vector", "xstat", "xplan", "sell"])
+@pytest.mark.parametrize("kernel", ["merge", "vector", "xstat", "xplan", "sell", "sellsort"])
 def test_npb_s_every_kernel(sp, torch_dev, kernel):
     """NPB class S zeta with every SpMV kernel inside CG (fused or separate dot)."""
     torch, dev = torch_dev
@@ -170,3 +170,30 @@ def test_npb_s_every_kernel(sp, torch_dev, kernel):
             M.npb_outer(x, z, 25, shift, out)
         zeta = float(out[0].item())
     assert abs(zeta - gen.NPB_ZETA["S"]) / gen.NPB_ZETA["S"] <= 1e-10
+
+
+def test_cg_sellsort_multisegment_rows(sp, torch_dev):
+    """Length-sorted SELL with rows split into several warp segments (arrowhead
+    matrix: dense first row/column of 3000 entries): CG iterates match the
+    oracle, and two identical solves are bit-identical (the separate dot pass
+    keeps the scalars deterministic although segment completion order varies)."""
+    torch, dev = torch_dev
+    n = 3000
+    rows = np.concatenate([np.zeros(n, np.int64), np.arange(1, n), np.arange(1, n)])
+    cols = np.concatenate([np.arange(n), np.zeros(n - 1, np.int64), np.arange(1, n)])
+    vals = np.concatenate([np.full(n, 0.5), np.full(n - 1, 0.5), np.full(n - 1, 4.0)])
+    vals[0] = float(n)  # A[0,0]: diagonally dominant -> SPD
+    A = gen.from_coo(n, n, rows, cols, vals)
+    rp, ci, va = to_dev(A, dev)
+    b_h = gen.uniform(n, seed=12)
+    b = torch.from_numpy(b_h).to(dev)
+    xs = []
+    with sp.CSRMatrix(rp, ci, va, n, kernel="sellsort") as M:
+        assert M.info()["kernel_name"] == "sellsort"
+        for _ in range(2):
+            x = torch.empty_like(b)
+            its, rn = M.cg_solve(b, x, max_iter=20)
+            xs.append(x.cpu().numpy())
+    z_ref, its_ref, rn_ref, st = oracle.cg(A.rowptr, A.colidx, A.vals, b_h, 20)
+    assert np.allclose(xs[0], z_ref, rtol=1e-10, atol=1e-13)
+    assert np.array_equal(xs[0], xs[1])

@@ -444,9 +444,47 @@ def test_sell_auto_update_values_and_vals_override(sp, torch_dev):
         check_rows(y.cpu().numpy(), y_ref, bound, np.float64, "sell vals override")
 
 
-def test_parboil_auto_is_merge(sp, torch_dev):
+def test_parboil_auto_kernels(sp, torch_dev):
+    """BJ.cfg[2] (power law, fp32): auto picks the length-sorted SELL plan, and
+    the merge path without a plan; both every row against the oracle."""
     torch, dev = torch_dev
     A = gen.powerlaw()
     x = gen.uniform(A.n, seed=42, f32=True)
     info = run_case(sp, torch, dev, A, x, what="parboil auto")
-    assert info["kernel_name"] == "merge"
+    assert info["kernel_name"] == "sellsort"
+    rp, ci, va = to_dev(A, dev)
+    with sp.CSRMatrix(rp, ci, va, A.n, plan=False) as M:
+        assert M.info()["kernel_name"] == "merge"
+
+
+@pytest.mark.parametrize("name,A", ZOO, ids=[c[0] for c in ZOO])
+def test_zoo_sellsort(sp, torch_dev, name, A):
+    """Length-sorted SELL (forced: any padding), long rows (> 64) warp-per-row
+    from the CSR, y through the permutation: fp64, fp32, alpha/beta."""
+    torch, dev = torch_dev
+    x = gen.uniform(A.n, seed=31)
+    info = run_case(sp, torch, dev, A, x, kernel="sellsort", what=f"{name} sellsort")
+    if A.m > 0 and A.nnz > 0:
+        assert info["kernel_name"] == "sellsort"
+    A32 = A.astype(np.float32)
+    run_case(sp, torch, dev, A32, gen.uniform(A.n, seed=32, f32=True), kernel="sellsort",
+             what=f"{name} sellsort fp32")
+    y0 = gen.uniform(A.m, seed=33)
+    run_case(sp, torch, dev, A, x, alpha=1.5, beta=-0.5, y0=y0, kernel="sellsort", what=f"{name} sellsort a/b")
+
+
+def test_sellsort_update_values(sp, torch_dev):
+    torch, dev = torch_dev
+    A = gen.powerlaw(m=50000, lmax=5000.0, seed=9, f32=False)
+    x_h = gen.uniform(A.n, seed=34)
+    rp, ci, va = to_dev(A, dev)
+    y = torch.empty(A.m, dtype=torch.float64, device=dev)
+    v2_h = gen.uniform(A.nnz, seed=35)
+    with sp.CSRMatrix(rp, ci, va, A.n, kernel="sellsort") as M:
+        assert M.info()["kernel_name"] == "sellsort"
+        va.copy_(torch.from_numpy(v2_h))
+        M.update_values(va)
+        M.spmv(torch.from_numpy(x_h).to(dev), y)
+        torch.cuda.synchronize()
+    y_ref, bound = oracle.spmv(A.rowptr, A.colidx, v2_h, x_h)
+    check_rows(y.cpu().numpy(), y_ref, bound, np.float64, "sellsort update_values")

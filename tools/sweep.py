@@ -19,7 +19,7 @@ import paper_conf_asplos_ginsbachrsbdo18_b200 as sp
 VARIANTS = [("auto", {}, {}), ("auto_noplan", {"plan": False}, {})] + \
     [(f"xplan_B{b}", {"kernel": "xplan"}, {"SPMV_XPLAN_B": str(b)}) for b in (4, 8)] + \
     [("xplan_pf", {"kernel": "xplan"}, {"SPMV_XPLAN_PF": "1"})] + \
-    [("sell", {"kernel": "sell"}, {})] + \
+    [("sell", {"kernel": "sell"}, {}), ("sellsort", {"kernel": "sellsort"}, {}), ("merge", {"kernel": "merge"}, {})] + \
     [(f"vector{g}", {"kernel": "vector", "vec_lanes": g, "plan": False}, {}) for g in (8, 16, 32)] + \
     [(f"vector32_u{u}", {"kernel": "vector", "vec_lanes": 32, "plan": False}, {"SPMV_UNROLL": str(u)}) for u in (2, 8)] + \
     [(f"xstat_B8_G{g}_U8", {"kernel": "xstat", "plan": False}, {"SPMV_XSTAT_B": "8", "SPMV_XSTAT_G": str(g),
