@@ -81,6 +81,10 @@ def _L():
         L.gen_uniform_f64.restype = None
         L.gen_uniform_f32.argtypes = [U64, U64, I64, P]
         L.gen_uniform_f32.restype = None
+        L.gen_is_keys.argtypes = [I64, I64, U64, U64, P]
+        L.gen_is_keys.restype = None
+        L.gen_histo_image.argtypes = [I64, I64, I32, U64, P]
+        L.gen_histo_image.restype = None
         _lib = L
     return _lib
 
@@ -186,3 +190,34 @@ def from_coo(m: int, n: int, rows, cols, vals, dtype=np.float64) -> CSR:
     rowptr = np.cumsum(rowptr).astype(np.int32)
     return CSR(m, n, rowptr, np.asarray(cols, np.int32)[order],
                np.asarray(vals, dtype)[order], "coo")
+
+
+# ------------------------------------------------------------- idiom inputs
+# NPB IS class parameters [ext:NPB-IS]: (TOTAL_KEYS_LOG_2, MAX_KEY_LOG_2)
+NPB_IS_CLASSES = {"S": (16, 11), "W": (20, 16), "A": (23, 19), "B": (25, 21), "C": (27, 23)}
+# NPB EP classes [ext:NPB-EP]: M (2^M Gaussian pairs)
+NPB_EP_CLASSES = {"S": 24, "W": 25, "A": 28, "B": 30, "C": 32}
+# Parboil-histo-shaped image (reading R32): 996x1040 pixels, 4096x256 uint8 bins
+HISTO_NPIX = 996 * 1040
+HISTO_NBINS = 4096 * 256
+HISTO_HOT = 64
+HISTO_SEED = 20180324
+
+
+def is_keys(cls: str | None = None, *, n: int | None = None, max_key: int | None = None,
+            seed: int = 314159265, a: int = 1220703125) -> np.ndarray:
+    """NPB IS create_seq keys (int32) of a class or of explicit (n, max_key)."""
+    if cls is not None:
+        lk, lm = NPB_IS_CLASSES[cls]
+        n, max_key = 1 << lk, 1 << lm
+    out = np.empty(n, np.int32)
+    _L().gen_is_keys(int(n), int(max_key), int(seed), int(a), out.ctypes.data)
+    return out
+
+
+def histo_image(npix: int = HISTO_NPIX, nbins: int = HISTO_NBINS, hot: int = HISTO_HOT,
+                seed: int = HISTO_SEED) -> np.ndarray:
+    """Parboil-histo-shaped pixel values in [0, nbins) with hot spots (int32)."""
+    out = np.empty(npix, np.int32)
+    _L().gen_histo_image(int(npix), int(nbins), int(hot), int(seed), out.ctypes.data)
+    return out

@@ -353,3 +353,47 @@ gen_csr *gen_laplace1d(int64_t n)
     }
     return g;
 }
+
+/* ----------------------------------------------------------------------- */
+/* NAS IS keys [ext:NPB-IS] create_seq(seed=314159265, a=1220703125):
+ *   k = max_key/4;  key[i] = (int)(k * (u1 + u2 + u3 + u4)),
+ * four consecutive randlc draws per key, summed left to right in double
+ * (k is a power of two, so k*x is exact and the truncation is NPB's).       */
+void gen_is_keys(int64_t n, int64_t max_key, uint64_t seed, uint64_t a, int32_t *keys)
+{
+    uint64_t s = seed;
+    const double k = (double)(max_key / 4);
+    for (int64_t i = 0; i < n; i++) {
+        double x = randlc(&s, a);
+        x += randlc(&s, a);
+        x += randlc(&s, a);
+        x += randlc(&s, a);
+        keys[i] = (int32_t)(k * x);
+    }
+}
+
+/* Parboil-histo-shaped image (reading R32; the paper's histo input is not
+ * described): npix values in [0, nbins).  With probability 5/8 a pixel sits
+ * near one of `hot` seeded centres (offset = sum of two uniform integers in
+ * [-8, 8], triangular, wrapped into range) -- the hot spots that make the
+ * saturating uint8 counters of Parboil histo matter; otherwise uniform.
+ * splitmix64 streams: 11 = centres, 12 = per-pixel draws.                   */
+void gen_histo_image(int64_t npix, int64_t nbins, int32_t hot, uint64_t seed, int32_t *img)
+{
+    if (hot < 1) hot = 1;
+    int64_t *cen = (int64_t *)malloc(sizeof(int64_t) * (size_t)hot);
+    for (int32_t h = 0; h < hot; h++) cen[h] = (int64_t)(rng(seed, 11, (uint64_t)h) % (uint64_t)nbins);
+    for (int64_t i = 0; i < npix; i++) {
+        uint64_t r = rng(seed, 12, (uint64_t)i);
+        int64_t v;
+        if ((r & 7) < 5) {
+            int64_t c = cen[(r >> 3) % (uint64_t)hot];
+            int64_t o = (int64_t)((r >> 24) % 17) + (int64_t)((r >> 40) % 17) - 16;
+            v = ((c + o) % nbins + nbins) % nbins;
+        } else {
+            v = (int64_t)((r >> 8) % (uint64_t)nbins);
+        }
+        img[i] = (int32_t)v;
+    }
+    free(cen);
+}

@@ -21,6 +21,7 @@ import numpy as np
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
 _SRC = os.path.join(_HERE, "oracle_spmv.c")
+_SRCS = [_SRC, os.path.join(_HERE, "oracle_idioms.c")]
 _LIB = os.path.join(_HERE, "liboracle_spmv.so")
 _lib = None
 
@@ -32,11 +33,11 @@ _D = ctypes.c_double
 
 def build(force: bool = False) -> str:
     """Compile the oracle (gcc, no FMA contraction).  Returns the .so path."""
-    if force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < os.path.getmtime(_SRC):
+    if force or not os.path.exists(_LIB) or any(os.path.getmtime(_LIB) < os.path.getmtime(f) for f in _SRCS):
         tmp = _LIB + f".tmp{os.getpid()}"
         subprocess.check_call(
             ["gcc", "-O3", "-march=native", "-ffp-contract=off", "-std=c11", "-fPIC",
-             "-shared", "-o", tmp, _SRC, "-lm"])
+             "-shared", "-o", tmp, *_SRCS, "-lm"])
         os.replace(tmp, _LIB)
     return _LIB
 
@@ -60,6 +61,20 @@ def lib():
         L.oracle_stencil27.argtypes = [_I64, _I64, _I64, _P, _P, _P, _D, _D, _P, _P]
         L.oracle_stencil27.restype = None
         L.oracle_merge_path.restype = None
+        L.oracle_reduce_f64.argtypes = [_I64, _P, _P, _P, _P]
+        L.oracle_reduce_f64.restype = None
+        L.oracle_reduce_f32.argtypes = [_I64, _P, _P, _P, _P]
+        L.oracle_reduce_f32.restype = None
+        L.oracle_hist_count_u32.argtypes = [_I64, _P, _I64, _P]
+        L.oracle_hist_count_u32.restype = None
+        L.oracle_hist_sat_u8.argtypes = [_I64, _P, _I64, _P]
+        L.oracle_hist_sat_u8.restype = None
+        L.oracle_hist_sum_f64.argtypes = [_I64, _P, _P, _I64, _P, _P]
+        L.oracle_hist_sum_f64.restype = None
+        L.oracle_npb_randlc_stream.argtypes = [_D, _D, _I64, _P]
+        L.oracle_npb_randlc_stream.restype = None
+        L.oracle_ep.argtypes = [_I32, _I64, _I64, _P, _P, _P]
+        L.oracle_ep.restype = ctypes.c_int
         _lib = L
     return _lib
 
@@ -176,3 +191,64 @@ def stencil27(nx, ny, nz, x, w=None, y_old=None, alpha=1.0, beta=0.0):
     b = np.empty(n)
     lib().oracle_stencil27(nx, ny, nz, _ptr(w), _ptr(x), _ptr(yo), alpha, beta, _ptr(y), _ptr(b))
     return y, b
+
+
+# ---------------------------------------------------------------- idioms
+# Scalar reduction (Fig. 14), generalised histogram (Fig. 11), NAS EP.
+
+def reduce(a, b=None):
+    """(sum, bound): sequential sum of a[i] (or a[i]*b[i]) in fp64 and sum|term|."""
+    f32 = np.asarray(a).dtype == np.float32
+    dt = np.float32 if f32 else np.float64
+    a = _c(a, dt)
+    b = _c(b, dt) if b is not None else None
+    s = ctypes.c_double(0.0)
+    bd = ctypes.c_double(0.0)
+    fn = lib().oracle_reduce_f32 if f32 else lib().oracle_reduce_f64
+    fn(a.shape[0], _ptr(a), _ptr(b), ctypes.byref(s), ctypes.byref(bd))
+    return s.value, bd.value
+
+
+def hist_count_u32(keys, nbins, bins=None):
+    keys = _c(keys, np.int32)
+    out = np.zeros(max(nbins, 1), np.uint32) if bins is None else _c(bins, np.uint32).copy()
+    lib().oracle_hist_count_u32(keys.shape[0], _ptr(keys), int(nbins), _ptr(out))
+    return out[:nbins]
+
+
+def hist_sat_u8(keys, nbins, bins=None):
+    keys = _c(keys, np.int32)
+    out = np.zeros(max(nbins, 1), np.uint8) if bins is None else _c(bins, np.uint8).copy()
+    lib().oracle_hist_sat_u8(keys.shape[0], _ptr(keys), int(nbins), _ptr(out))
+    return out[:nbins]
+
+
+def hist_sum_f64(keys, w, nbins, bins=None):
+    """(bins, bound): weighted histogram and the per-bin sum of |w| (+|old|)."""
+    keys = _c(keys, np.int32)
+    w = _c(w, np.float64)
+    out = np.zeros(max(nbins, 1)) if bins is None else _c(bins, np.float64).copy()
+    bound = np.zeros(max(nbins, 1))
+    lib().oracle_hist_sum_f64(keys.shape[0], _ptr(keys), _ptr(w), int(nbins), _ptr(out), _ptr(bound))
+    return out[:nbins], bound[:nbins]
+
+
+def npb_randlc_stream(count, seed=314159265.0, a=1220703125.0):
+    out = np.empty(count)
+    lib().oracle_npb_randlc_stream(float(seed), float(a), int(count), _ptr(out))
+    return out
+
+
+def ep(M, pair_begin=0, pair_count=None):
+    """NAS EP over pairs [pair_begin, pair_begin+pair_count) of class 2^M.
+
+    Returns (q[10], sx, sy)."""
+    if pair_count is None:
+        pair_count = (1 << M) - pair_begin
+    q = np.zeros(10)
+    sx = ctypes.c_double(0.0)
+    sy = ctypes.c_double(0.0)
+    st = lib().oracle_ep(int(M), int(pair_begin), int(pair_count), _ptr(q), ctypes.byref(sx), ctypes.byref(sy))
+    if st != 0:
+        raise ValueError(f"oracle_ep: bad arguments (status {st})")
+    return q, sx.value, sy.value
