@@ -82,6 +82,14 @@ spmv_dist_colidx_c = _decl("spmv_dist_colidx", [_P, _P])
 spmv_dist_halo_host_c = _decl("spmv_dist_halo_host", [_P, _P, _I64, _I32, _P])
 spmv_dist_halo_c = _decl("spmv_dist_halo", [_P, _P, _P])
 stencil27_apply_c = _decl("stencil27_apply", [_ST, _I64, _I64, _I64, _P, _P, _P, _D, _D, _P])
+# include/idioms.h (histogram, scalar reduction, NAS EP)
+_SZ = ctypes.c_size_t
+idl_reduce_workspace_c = _decl("idl_reduce_workspace", [_I64, ctypes.POINTER(_SZ)])
+idl_reduce_c = _decl("idl_reduce", [_ST, _ST, _P, _P, _I64, _P, _P, _SZ, _P])
+idl_histogram_workspace_c = _decl("idl_histogram_workspace", [_ST, _I64, _I64, ctypes.POINTER(_SZ)])
+idl_histogram_c = _decl("idl_histogram", [_ST, _P, _P, _I64, _I64, _P, _P, _SZ, _P])
+ep_npb_workspace_c = _decl("ep_npb_workspace", [ctypes.POINTER(_SZ)])
+ep_npb_c = _decl("ep_npb", [_I32, _I64, _I64, _P, _P, _SZ, _P])
 
 # every symbol include/spmv.h declares (checked by tests/test_abi.py)
 EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_status",
@@ -91,6 +99,12 @@ EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_s
            "spmv_dist_get_unique_id", "spmv_dist_init", "spmv_dist_destroy", "spmv_dist_plan_host",
            "spmv_dist_colidx", "spmv_dist_init_p2p", "spmv_csr_p2p_handle", "spmv_csr_p2p_connect",
            "spmv_dist_halo_host", "spmv_dist_halo", "stencil27_apply"]
+# every symbol include/idioms.h declares
+IDIOM_EXPORTS = ["idl_reduce_workspace", "idl_reduce", "idl_histogram_workspace", "idl_histogram",
+                 "ep_npb_workspace", "ep_npb"]
+IDL_RED_SUM, IDL_RED_DOT = 0, 1
+IDL_HIST_COUNT_U32, IDL_HIST_SAT_U8, IDL_HIST_SUM_F64 = 0, 1, 2
+HIST_KINDS = {"count": IDL_HIST_COUNT_U32, "sat_u8": IDL_HIST_SAT_U8, "sum_f64": IDL_HIST_SUM_F64}
 
 
 class SpmvError(RuntimeError):
@@ -376,3 +390,85 @@ class CSRMatrix:
 
 def launch_count() -> int:
     return int(spmv_launch_count())
+
+
+# ------------------------------------------------------------------ idioms
+# include/idioms.h: the histogram (Fig. 11), scalar reduction (Fig. 14) and
+# NAS EP.  Workspaces are zero-filled device buffers (torch.zeros); pass one
+# back in to avoid the allocation (bench loops do).
+
+def _stream_of(t):
+    import torch
+    return torch.cuda.current_stream(t.device).cuda_stream
+
+
+def _workspace(nbytes, device):
+    import torch
+    return torch.zeros(max(int(nbytes), 16), dtype=torch.uint8, device=device)
+
+
+def idl_reduce_workspace(n: int) -> int:
+    b = ctypes.c_size_t(0)
+    _check(idl_reduce_workspace_c(int(n), ctypes.byref(b)), "idl_reduce_workspace")
+    return b.value
+
+
+def idl_reduce(a, b=None, out=None, workspace=None, stream=None):
+    """Scalar reduction: sum(a) or dot(a, b) into a device float64 tensor of
+    one element (returned).  fp32 inputs are summed in double.  Asynchronous."""
+    import torch
+    dt = SPMV_F64 if a.dtype == torch.float64 else SPMV_F32
+    n = a.numel()
+    if out is None:
+        out = torch.empty(1, dtype=torch.float64, device=a.device)
+    if workspace is None:
+        workspace = _workspace(idl_reduce_workspace(n), a.device)
+    op = IDL_RED_SUM if b is None else IDL_RED_DOT
+    st = idl_reduce_c(dt, op, _ptr(a), _ptr(b), n, _ptr(out), _ptr(workspace), workspace.numel(),
+                      _stream_of(out) if stream is None else stream)
+    _check(st, "idl_reduce")
+    return out
+
+
+def idl_histogram_workspace(kind, n: int, nbins: int) -> int:
+    k = HIST_KINDS[kind] if isinstance(kind, str) else int(kind)
+    b = ctypes.c_size_t(0)
+    _check(idl_histogram_workspace_c(k, int(n), int(nbins), ctypes.byref(b)), "idl_histogram_workspace")
+    return b.value
+
+
+def idl_histogram(kind, keys, bins, w=None, workspace=None, stream=None):
+    """Generalised histogram accumulating into `bins` (uint32 / uint8 / float64
+    device tensor for kind "count" / "sat_u8" / "sum_f64"); keys int32.
+    Keys outside [0, len(bins)) are skipped.  Asynchronous; returns bins."""
+    k = HIST_KINDS[kind] if isinstance(kind, str) else int(kind)
+    n, nbins = keys.numel(), bins.numel()
+    if workspace is None:
+        workspace = _workspace(idl_histogram_workspace(k, n, nbins), bins.device)
+    st = idl_histogram_c(k, _ptr(keys), _ptr(w), n, nbins, _ptr(bins), _ptr(workspace), workspace.numel(),
+                         _stream_of(bins) if stream is None else stream)
+    _check(st, "idl_histogram")
+    return bins
+
+
+def ep_npb_workspace() -> int:
+    b = ctypes.c_size_t(0)
+    _check(ep_npb_workspace_c(ctypes.byref(b)), "ep_npb_workspace")
+    return b.value
+
+
+def ep_npb(M: int, pair_begin: int = 0, pair_count: int | None = None, out=None, workspace=None,
+           device=None, stream=None):
+    """NAS EP over pairs [pair_begin, pair_begin+pair_count) of class 2^M into a
+    device float64[12] tensor: q[0..9], sx, sy (returned).  Asynchronous."""
+    import torch
+    if pair_count is None:
+        pair_count = (1 << M) - pair_begin
+    if out is None:
+        out = torch.empty(12, dtype=torch.float64, device=device or torch.device("cuda", torch.cuda.current_device()))
+    if workspace is None:
+        workspace = _workspace(ep_npb_workspace(), out.device)
+    st = ep_npb_c(int(M), int(pair_begin), int(pair_count), _ptr(out), _ptr(workspace), workspace.numel(),
+                  _stream_of(out) if stream is None else stream)
+    _check(st, "ep_npb")
+    return out

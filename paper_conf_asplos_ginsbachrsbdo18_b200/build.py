@@ -29,7 +29,7 @@ def nccl_dir() -> str:
 
 def sources():
     return sorted(glob.glob(os.path.join(CSRC, "*.cu")) + glob.glob(os.path.join(CSRC, "*.cuh"))
-                  + [os.path.join(ROOT, "include", "spmv.h")])
+                  + glob.glob(os.path.join(ROOT, "include", "*.h")))
 
 
 def stale() -> bool:

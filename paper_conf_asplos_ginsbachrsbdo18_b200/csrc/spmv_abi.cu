@@ -1907,3 +1907,6 @@ extern "C" spmv_status spmv_dist_destroy(spmv_dist_t d) {
   delete d;
   return st;
 }
+
+// ------------------------------------------------------------------ idioms (NEXT-4)
+#include "idioms_abi.cuh"

@@ -21,8 +21,8 @@ def sp():
     return sp
 
 
-def _declared_functions():
-    txt = open(os.path.join(ROOT, "include", "spmv.h")).read()
+def _declared_functions(header="spmv.h"):
+    txt = open(os.path.join(ROOT, "include", header)).read()
     txt = re.sub(r"/\*.*?\*/", "", txt, flags=re.S)
     names = re.findall(r"^\s*(?:const\s+)?[a-z_0-9]+\s*\*?\s*([a-z_0-9]+)\s*\(", txt, flags=re.M)
     return sorted(set(names))
@@ -40,6 +40,23 @@ def test_library_exports_every_declared_symbol(sp):
     for name in _declared_functions():
         assert hasattr(lib, name), f"{name} declared in include/spmv.h but not exported"
     assert sorted(sp.EXPORTS) == _declared_functions()
+    for name in _declared_functions("idioms.h"):
+        assert hasattr(lib, name), f"{name} declared in include/idioms.h but not exported"
+    assert sorted(sp.IDIOM_EXPORTS) == _declared_functions("idioms.h")
+
+
+def test_idiom_workspace_queries_and_argument_errors(sp):
+    """Host-side checks of include/idioms.h (no kernel is launched)."""
+    assert sp.idl_reduce_workspace(0) >= 16 and sp.idl_reduce_workspace(10**9) == sp.idl_reduce_workspace(1)
+    assert sp.idl_histogram_workspace("sat_u8", 10, 1000) >= 4000
+    assert sp.ep_npb_workspace() >= 16 + 12 * 8
+    with pytest.raises(sp.SpmvError):
+        sp.idl_histogram_workspace("count", 10, 0)
+    assert sp.idl_reduce_c(7, 0, None, None, 0, None, None, 0, None) == sp.SPMV_ERR_ARG
+    assert sp.idl_reduce_c(sp.SPMV_F64, 0, None, None, -1, None, None, 0, None) == sp.SPMV_ERR_ARG
+    assert sp.ep_npb_c(23, 0, 1, None, None, 0, None) == sp.SPMV_ERR_ARG
+    assert sp.ep_npb_c(24, (1 << 24) - 1, 2, None, None, 1 << 20, None) == sp.SPMV_ERR_ARG
+    assert sp.idl_histogram_c(1, None, None, 1 << 33, 10, None, None, 1 << 20, None) == sp.SPMV_ERR_ARG
 
 
 def test_library_is_sm100a(sp):
