@@ -55,6 +55,10 @@ def lib():
         L.oracle_cg.restype = ctypes.c_int
         L.oracle_npb_outer.argtypes = [_I64, _P, _P, _P, _P, _P, _I32, _D, _P, _P]
         L.oracle_npb_outer.restype = ctypes.c_int
+        L.oracle_cg_cgcg.argtypes = [_I64, _P, _P, _P, _P, _P, _I32, _D, _P, _P]
+        L.oracle_cg_cgcg.restype = ctypes.c_int
+        L.oracle_npb_outer_v.argtypes = [_I64, _P, _P, _P, _P, _P, _I32, _D, _P, _P, _I32]
+        L.oracle_npb_outer_v.restype = ctypes.c_int
         L.oracle_partition.argtypes = [_P, _I64, _I32, _P]
         L.oracle_partition.restype = None
         L.oracle_merge_path.argtypes = [_P, _I64, _I64, _P, _P]
@@ -109,8 +113,9 @@ def spmv(rowptr, colidx, vals, x, y_old=None, alpha=1.0, beta=0.0):
     return y_ref[:m], bound[:m]
 
 
-def cg(rowptr, colidx, vals, b, max_iter, tol=0.0):
-    """Textbook CG from x0=0 (NPB conj_grad).  Returns (z, iters, rnorm, status)."""
+def cg(rowptr, colidx, vals, b, max_iter, tol=0.0, variant=0):
+    """CG from x0=0: variant 0 textbook (NPB conj_grad), 1 Chronopoulos-Gear
+    single reduction.  Returns (z, iters, rnorm, status)."""
     rowptr = _c(rowptr, np.int32)
     colidx = _c(colidx, np.int32)
     vals = _c(vals, np.float64)
@@ -119,15 +124,15 @@ def cg(rowptr, colidx, vals, b, max_iter, tol=0.0):
     z = np.zeros(max(n, 1))
     its = ctypes.c_int32(0)
     rn = ctypes.c_double(0.0)
-    st = lib().oracle_cg(n, _ptr(rowptr), _ptr(colidx), _ptr(vals), _ptr(b), _ptr(z),
-                         int(max_iter), float(tol), ctypes.byref(its), ctypes.byref(rn))
+    fn = lib().oracle_cg_cgcg if variant == 1 else lib().oracle_cg
+    st = fn(n, _ptr(rowptr), _ptr(colidx), _ptr(vals), _ptr(b), _ptr(z),
+            int(max_iter), float(tol), ctypes.byref(its), ctypes.byref(rn))
     return z[:n], its.value, rn.value, st
 
 
-def npb_outer(rowptr, colidx, vals, x, cgitmax, shift):
+def npb_outer(rowptr, colidx, vals, x, cgitmax, shift, variant=0):
     """One NAS CG outer iteration; x (float64, contiguous) updated in place.
-
-    Returns (z, zeta, rnorm).
+    variant: 0 textbook CG, 1 Chronopoulos-Gear.  Returns (z, zeta, rnorm).
     """
     assert x.dtype == np.float64 and x.flags.c_contiguous
     rowptr = _c(rowptr, np.int32)
@@ -137,12 +142,12 @@ def npb_outer(rowptr, colidx, vals, x, cgitmax, shift):
     z = np.zeros(n)
     zeta = ctypes.c_double(0.0)
     rn = ctypes.c_double(0.0)
-    lib().oracle_npb_outer(n, _ptr(rowptr), _ptr(colidx), _ptr(vals), _ptr(x), _ptr(z),
-                           int(cgitmax), float(shift), ctypes.byref(zeta), ctypes.byref(rn))
+    lib().oracle_npb_outer_v(n, _ptr(rowptr), _ptr(colidx), _ptr(vals), _ptr(x), _ptr(z),
+                             int(cgitmax), float(shift), ctypes.byref(zeta), ctypes.byref(rn), int(variant))
     return z, zeta.value, rn.value
 
 
-def npb_run(rowptr, colidx, vals, niter, shift, cgitmax=25, on_iter=None):
+def npb_run(rowptr, colidx, vals, niter, shift, cgitmax=25, on_iter=None, variant=0):
     """NPB CG benchmark driver: x=1; NITER outer iterations; returns zetas, rnorms.
 
     (The untimed warm-up iteration of NPB resets x=1 afterwards and so does not
@@ -152,7 +157,7 @@ def npb_run(rowptr, colidx, vals, niter, shift, cgitmax=25, on_iter=None):
     x = np.ones(n)
     zetas, rnorms = [], []
     for it in range(niter):
-        _, zeta, rn = npb_outer(rowptr, colidx, vals, x, cgitmax, shift)
+        _, zeta, rn = npb_outer(rowptr, colidx, vals, x, cgitmax, shift, variant)
         zetas.append(zeta)
         rnorms.append(rn)
         if on_iter:

@@ -169,6 +169,64 @@ def test_cg_breakdown_zero_rhs():
     assert st == 7 and its == 0
 
 
+# Single-reduction (Chronopoulos-Gear) CG oracle, NEXT-1: pinned to the same
+# closed forms, to exact termination, and to the textbook oracle's iterates.
+@pytest.mark.parametrize("n", [1, 2, 5, 16, 64])
+def test_cgcg_laplace1d_closed_form(n):
+    A = gen.laplace1d(n)
+    z, its, rn, st = oracle.cg(A.rowptr, A.colidx, A.vals, np.ones(n), max_iter=n, tol=1e-14, variant=1)
+    j = np.arange(n)
+    ref = (j + 1) * (n - j) / 2.0
+    assert st == 0
+    assert np.allclose(z, ref, rtol=1e-10, atol=0)
+
+
+def test_cgcg_small_integer_spd_exact_solution():
+    """A = B^T B + n I with small integers, x* integer: n steps reach x* (rounding only)."""
+    rng = np.random.default_rng(3)
+    n = 12
+    B = rng.integers(-3, 4, size=(n, n)).astype(np.float64)
+    Ad = B.T @ B + n * np.eye(n)
+    xs = rng.integers(-5, 6, size=n).astype(np.float64)
+    b = Ad @ xs
+    A = gen.from_dense(Ad)
+    z, its, rn, st = oracle.cg(A.rowptr, A.colidx, A.vals, b, max_iter=n, variant=1)
+    assert st == 0 and its == n
+    assert np.allclose(z, xs, rtol=0, atol=1e-9)
+
+
+@pytest.mark.parametrize("k", [1, 2, 3, 10, 25])
+def test_cgcg_iterates_equal_textbook(k):
+    """Mathematically identical iterates: z_k of both oracles agree to rounding on makea S."""
+    A = gen.makea("S")
+    b = np.ones(A.n)
+    z0, _, _, _ = oracle.cg(A.rowptr, A.colidx, A.vals, b, max_iter=k)
+    z1, its, _, st = oracle.cg(A.rowptr, A.colidx, A.vals, b, max_iter=k, variant=1)
+    assert st == 0 and its == k
+    assert np.max(np.abs(z1 - z0)) <= 1e-12 * np.max(np.abs(z0))
+
+
+def test_cgcg_one_step_and_breakdown():
+    n = 40
+    A = gen.from_coo(n, n, np.arange(n), np.arange(n), np.full(n, 4.0))
+    b = gen.uniform(n, seed=9)
+    z, its, rn, st = oracle.cg(A.rowptr, A.colidx, A.vals, b, max_iter=1, variant=1)
+    assert st == 0 and its == 1 and np.allclose(z, b / 4.0, rtol=1e-15, atol=0)
+    L = gen.laplace1d(8)
+    z, its, rn, st = oracle.cg(L.rowptr, L.colidx, L.vals, np.zeros(8), max_iter=5, variant=1)
+    assert st == 7 and its == 0
+
+
+@pytest.mark.parametrize("cls", ["S", "W"])
+def test_cgcg_npb_zeta_published(cls):
+    g = {r[0]: r[1:] for r in _read_golden("npb_zeta.txt")}[cls]
+    niter, shift, zeta_ref = int(g[2]), float(g[3]), float(g[4])
+    A = gen.makea(cls)
+    zetas, rnorms = oracle.npb_run(A.rowptr, A.colidx, A.vals, niter, shift, variant=1)
+    assert abs(zetas[-1] - zeta_ref) / zeta_ref <= 1e-10
+    assert rnorms.max() <= 1e-11
+
+
 def test_randlc_against_bigint():
     """NPB randlc: x <- 5^13 x mod 2^46 (exact integer recurrence)."""
     vals = gen.randlc_stream(2000)
