@@ -191,6 +191,7 @@ def run_ours(args):
         with stdout_to_stderr():
             d = sp.Dist(rank, world, local, transport="nccl")
         M = sp.CSRMatrix(rp, ci, va, A.n, dist=d)
+    M.set_cg_variant(args.cg_variant)
     info = M.info()
     b0, b1 = info["row_begin"], info["row_end"]
     nl = b1 - b0
@@ -236,6 +237,25 @@ def run_ours(args):
     t_ms = max_over_ranks(ev0.elapsed_time(ev1))
     zeta_last = float(out2[0].item())
     value = 25.0 * args.steps / (t_ms / 1e3)
+
+    # the other CG variant (NEXT-1), same protocol, reported beside the headline
+    other = "cgcg" if args.cg_variant == "textbook" else "textbook"
+    M.set_cg_variant(other)
+    x.fill_(1.0)
+    for _ in range(args.warmup):
+        M.npb_outer(x, z, 25, shift, out2)
+    x.fill_(1.0)
+    barrier()
+    ev0.record(stream)
+    for k in range(args.steps):
+        M.npb_outer(x, z, 25, shift, out2)
+    ev1.record(stream)
+    barrier()
+    M.cg_status()
+    t_other = max_over_ranks(ev0.elapsed_time(ev1))
+    variants = {args.cg_variant: round(value, 2), other: round(25.0 * args.steps / (t_other / 1e3), 2),
+                f"zeta_last_{other}": float(out2[0].item())}
+    M.set_cg_variant(args.cg_variant)
 
     # ---------------- e2e through the public API with host buffers
     xh = torch.ones(nl, dtype=torch.float64).pin_memory()
@@ -325,6 +345,8 @@ def run_ours(args):
             "gpu_launches": int(launches),
             "clocks": clk,
             "zeta_last": zeta_last,
+            "cg_variant": args.cg_variant,
+            "cg_variants": variants,
             "cpu_baseline": cpu,
         }
         print(json.dumps(line), flush=True)
@@ -411,6 +433,9 @@ def main():
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
     ap.add_argument("--no-cpu", action="store_true", help="skip the cpu_baseline leg")
     ap.add_argument("--cpu-budget", type=float, default=15.0)
+    ap.add_argument("--cg-variant", choices=["textbook", "cgcg"],
+                    default=os.environ.get("SPMV_CG_VARIANT", "textbook"),
+                    help="CG inside the NAS step: textbook (NPB conj_grad) or cgcg (single reduction)")
     args = ap.parse_args()
     if args.warmup < 3:
         log("warmup < 3 is not allowed by the timing rules; using 3")

@@ -62,6 +62,7 @@ spmv_csr_c = _decl("spmv_csr", [_P, _I64, _I64, _I64, _P, _P, _P, _P, _P, _D, _D
 cg_solve_c = _decl("cg_solve", [_P, _P, _P, _I32, _D, ctypes.POINTER(_I32), ctypes.POINTER(_D)])
 cg_npb_outer_c = _decl("cg_npb_outer", [_P, _P, _P, _I32, _D, _P])
 spmv_cg_status_c = _decl("spmv_cg_status", [_P])
+spmv_csr_set_cg_variant_c = _decl("spmv_csr_set_cg_variant", [_P, _I32])
 spmv_csr_update_values_c = _decl("spmv_csr_update_values", [_P, _P])
 spmv_csr_merge_splits_device_c = _decl("spmv_csr_merge_splits_device", [_P, _P, _P, _I64, ctypes.POINTER(_I64)])
 spmv_csr_destroy_c = _decl("spmv_csr_destroy", [_P])
@@ -92,7 +93,7 @@ ep_npb_workspace_c = _decl("ep_npb_workspace", [ctypes.POINTER(_SZ)])
 ep_npb_c = _decl("ep_npb", [_I32, _I64, _I64, _P, _P, _SZ, _P])
 
 # every symbol include/spmv.h declares (checked by tests/test_abi.py)
-EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_status",
+EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_status", "spmv_csr_set_cg_variant",
            "spmv_csr_update_values", "spmv_csr_merge_splits_device",
            "spmv_csr_destroy", "spmv_csr_partition", "spmv_csr_merge_splits", "spmv_csr_info",
            "spmv_launch_count", "spmv_status_string", "spmv_last_error_string",
@@ -250,7 +251,7 @@ class CSRMatrix:
 
     def __init__(self, rowptr, colidx, vals, n: int | None = None, *, kernel: str = "auto",
                  vec_lanes: int = 0, validate: bool = False, stream=None, dist: Dist | None = None,
-                 plan: bool = True):
+                 plan: bool = True, cg_variant: str = "textbook"):
         import torch
         assert rowptr.dtype == torch.int32 and colidx.dtype == torch.int32
         assert vals.dtype in (torch.float64, torch.float32)
@@ -296,6 +297,15 @@ class CSRMatrix:
                 raise err
             tdist.barrier(group=dist.group)
         self._info = self.info()
+        if cg_variant != "textbook":
+            self.set_cg_variant(cg_variant)
+
+    CG_VARIANTS = {"textbook": 0, "cgcg": 1}
+
+    def set_cg_variant(self, variant: str):
+        """'textbook' (NPB conj_grad) or 'cgcg' (single-reduction Chronopoulos-Gear)."""
+        _check(spmv_csr_set_cg_variant_c(self.handle, self.CG_VARIANTS[variant]), "spmv_csr_set_cg_variant")
+        self.cg_variant = variant
 
     # -- calls ------------------------------------------------------------
     def spmv(self, x, y, alpha: float = 1.0, beta: float = 0.0, vals=None):

@@ -133,6 +133,100 @@ k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
   }
 }
 
+// ------------------------------------------------------------ NEXT-1
+// Single-reduction CG (Chronopoulos & Gear).  In exact
+// arithmetic it produces the iterates z_k of NPB conj_grad, with one
+// reduction point per iteration instead of two.  Iteration k:
+//   K1  w = A r  and partial d = w.r        (the SpMV with x = r, DOT fused)
+//   K2  (this kernel)  g = r.r (from the previous K2), d:
+//        k == 0: beta = 0, alpha = g/d
+//        else  : beta = g/g_old, alpha = g/(d - beta*g/alpha_old)
+//       p = r + beta p;  s = w + beta s;  z += alpha p;  r -= alpha s;
+//       partial r.r of the new r.
+// (s = A p is carried by recurrence, so p.Ap = d - beta*g/alpha_old.)
+// alpha is handed to the next K2 through alpha2[k & 1] (written by CTA 0;
+// every CTA computes the same value from the same partials in the same
+// order).  tol > 0: the check sqrt(g) <= tol*||b|| is made on entry, before
+// the update, so the solve stops with the same z_k as the textbook loop.
+__global__ void __launch_bounds__(256)
+k_cgcg(int64_t n, int k, SumSrc gam, SumSrc gam_old, SumSrc del, double* __restrict__ alpha2,
+       double* __restrict__ p, double* __restrict__ sv, const double* __restrict__ w,
+       double* __restrict__ z, double* __restrict__ r, double* __restrict__ part_rr_new,
+       int* __restrict__ flags, double tol, SumSrc rr_b, P2PHook hk, int64_t xoff) {
+  __shared__ double red[8];
+  __shared__ double s_g, s_go, s_d, s_b;
+  if (flags[1]) return;  // converged (tol mode): no-op
+  const double g = read_sum(gam, &s_g);
+  if (tol > 0.0) {
+    const double bb = read_sum(rr_b, &s_b);
+    if (sqrt(g) <= tol * sqrt(bb)) {
+      if (blockIdx.x == 0 && threadIdx.x == 0) flags[1] = 1;
+      return;
+    }
+  }
+  const double d = read_sum(del, &s_d);
+  double beta = 0.0, alpha, pap;
+  if (k == 0) {
+    pap = d;
+  } else {
+    const double go = read_sum(gam_old, &s_go);
+    beta = g / go;
+    pap = d - beta * g / __ldcg(alpha2 + ((k - 1) & 1));
+  }
+  alpha = g / pap;
+  if (blockIdx.x == 0 && threadIdx.x == 0) {
+    if (pap == 0.0 || !isfinite(pap)) flags[0] = 1;
+    alpha2[k & 1] = alpha;
+    flags[2] = k + 1;
+  }
+  double acc = 0.0;
+  const int64_t stride = int64_t(gridDim.x) * blockDim.x;
+  for (int64_t j0 = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j0 < n; j0 += CG_U * stride) {
+    double pr[CG_U], pw[CG_U], pp[CG_U], ps[CG_U], pz[CG_U];
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) {
+        pr[u] = r[j]; pw[u] = w[j]; pz[u] = z[j];
+        if (k > 0) { pp[u] = p[j]; ps[u] = sv[j]; }
+      }
+    }
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) {
+        const double pj = k > 0 ? pr[u] + beta * pp[u] : pr[u];
+        const double sj = k > 0 ? pw[u] + beta * ps[u] : pw[u];
+        const double rj = pr[u] - alpha * sj;
+        p[j] = pj;
+        sv[j] = sj;
+        z[j] = pz[u] + alpha * pj;
+        r[j] = rj;
+        acc += rj * rj;
+        if (hk.enabled)  // fused all-gather of the next SpMV's x (= r)
+          for (int q = 0; q < hk.c.P; ++q)
+            if (q != hk.c.me && p2p_sends(hk.c, q, j)) reinterpret_cast<double*>(hk.c.peer[q])[xoff + j] = rj;
+      }
+    }
+  }
+  const double t = block_sum(acc, red);
+  if (threadIdx.x == 0) part_rr_new[blockIdx.x] = t;
+  p2p_push_partials_last(hk, part_rr_new, gridDim.x);
+  if (hk.enabled) {
+    // publication of x uses its own ticket (the next u64 slot): the partials
+    // push above re-arms hk.c.ticket while other CTAs may already be here
+    int* tk2 = hk.c.ticket + 2;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+      __threadfence_system();
+      if (atomicAdd(tk2, 1) == int(gridDim.x) - 1) {
+        *tk2 = 0;
+        p2p_signal(hk.c, P2P_XSLOT);
+      }
+    }
+  }
+}
+
 // Residual / NPB norms: partials of ||b - Az||^2 and (NPB) x.z, z.z.
 // b is the right-hand side (NPB: x), az = A z.
 template <bool NPB>

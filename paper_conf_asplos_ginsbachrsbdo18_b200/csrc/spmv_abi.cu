@@ -172,6 +172,8 @@ struct spmv_csr_s {
   bool p2p_connected = false;
   // CG workspace (lazy)
   double *z = nullptr, *r = nullptr, *q = nullptr, *p_single = nullptr;
+  double *s_vec = nullptr, *alpha2 = nullptr;  // single-reduction CG (NEXT-1): s = A p, alpha_{k-1}
+  int cg_variant = 0;                          // 0 textbook (NPB conj_grad), 1 Chronopoulos-Gear
   double *part_pq = nullptr, *part_rr = nullptr, *part_res = nullptr, *part_xz = nullptr,
          *part_zz = nullptr, *scal = nullptr, *out2 = nullptr;
   int* flags = nullptr;
@@ -1191,7 +1193,7 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   void* bufs[] = {h->p2p_local, h->peer_table, h->mg.split_row, h->mg.split_nz, h->mg.head, h->mg.carry, h->mg.head_flag, h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
                   h->xp.chunk_row, h->xp.plan, h->sl.pair_off, h->sl.vals, h->sl.cols, h->sl.perm, h->sl.seg, h->sl.seg_part, h->sl.seg_cnt,
                   h->seg, h->crow, h->ci_own, h->send_iv, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
-                  h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags,
+                  h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags, h->s_vec, h->alpha2,
                   h->stage_x, h->stage_z};
   for (void* b : bufs)
     if (b) cudaFree(b);
@@ -1251,7 +1253,10 @@ static spmv_status cg_alloc(spmv_csr_s* h) {
   ST(ensure_buf((void**)&h->q, nb));
   if (!h->dist) ST(ensure_buf((void**)&h->p_single, nb));
   ST(ensure_buf((void**)&h->part_pq, pb));
-  ST(ensure_buf((void**)&h->part_rr, 3 * pb));  // [0],[1]: parity slots; [2]: ||b||^2 (init)
+  // [0],[1]: parity slots; [2]: ||b||^2 (init); [3..5]: rotating r.r of the single-reduction CG
+  ST(ensure_buf((void**)&h->part_rr, 6 * pb));
+  ST(ensure_buf((void**)&h->s_vec, nb));
+  ST(ensure_buf((void**)&h->alpha2, sizeof(double) * 2));
   ST(ensure_buf((void**)&h->part_res, pb));
   ST(ensure_buf((void**)&h->part_xz, pb));
   ST(ensure_buf((void**)&h->part_zz, pb));
@@ -1358,7 +1363,7 @@ static spmv_status gather_p(spmv_csr_s* h, cudaStream_t s) {
 
 // CG enqueue state: the scalar sources carried between iterations.
 struct CgRun {
-  SumSrc rr_b, rr_old;
+  SumSrc rr_b, rr_old, rr_prev;  // rr_prev: gamma_{k-1} of the single-reduction CG
   int it = 0;
 };
 
@@ -1367,10 +1372,14 @@ static spmv_status cg_enqueue_init(spmv_csr_s* h, cudaStream_t s, const double* 
                                    CgRun* run) {
   const int vg = (int)h->vgrid;
   double* prb = h->part_rr + 2 * std::max(std::max(h->grid, h->grid_vec), h->vgrid);
-  k_cg_init<<<vg, 256, 0, s>>>(h->m_loc, b, z, h->r, cg_p(h), prb);
+  // textbook: r = h->r, p = the SpMV input (cg_p); single-reduction: the SpMV
+  // input is r (cg_p) and h->r holds p (overwritten before it is read)
+  if (h->cg_variant == 1) k_cg_init<<<vg, 256, 0, s>>>(h->m_loc, b, z, cg_p(h), h->r, prb);
+  else k_cg_init<<<vg, 256, 0, s>>>(h->m_loc, b, z, h->r, cg_p(h), prb);
   LAUNCHED();
   ST(reduce_src(h, s, SumSrc{prb, vg}, 0, &run->rr_b));
   run->rr_old = run->rr_b;
+  run->rr_prev = run->rr_b;
   run->it = 0;
   if (use_p2p(h)) ST(exchange_x(h, s));  // p = b to every peer; later rounds are fused into k_cg_p
   return SPMV_OK;
@@ -1390,6 +1399,40 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
   if (p2p) {
     base.c = p2p_ctx(h);
     base.enabled = 1;
+  }
+  if (h->cg_variant == 1) {
+    // single-reduction CG (cg_kernels.cuh k_cgcg): SpMV w = A r with w.r fused, then one update
+    double* rv = p;  // the SpMV input slice holds r
+    static const int kGamSlot[3] = {2, 3, 7};
+    for (int c = 0; c < iters; ++c) {
+      const int k = run->it++;
+      SumSrc del;
+      if (p2p) {
+        P2PHook hs = base;
+        hs.wait_x = 1;
+        hs.push_slot = 1;
+        ST(run_spmv(h, s, h->vals, xg, h->q, 1.0, 0.0, rv, h->part_pq, &hs));
+        del = p2p_src(h, 1);
+      } else {
+        ST(gather_p(h, s));
+        ST(run_spmv(h, s, h->vals, xg, h->q, 1.0, 0.0, rv, h->part_pq));
+        ST(reduce_src(h, s, SumSrc{h->part_pq, sg}, 1, &del));
+      }
+      double* gnew = h->part_rr + (3 + (k + 1) % 3) * pstride;
+      const int gslot = kGamSlot[(k + 1) % 3];
+      P2PHook hz = base;
+      hz.push_slot = p2p ? gslot : -1;
+      const int64_t xoff = h->dist ? (int64_t)h->dist->rank * h->maxlen : 0;
+      k_cgcg<<<vg, 256, 0, s>>>(n, k, run->rr_old, run->rr_prev, del, h->alpha2, h->r, h->s_vec, h->q, z, rv,
+                                gnew, h->flags, tol, run->rr_b, hz, xoff);
+      LAUNCHED();
+      SumSrc g1;
+      if (p2p) g1 = p2p_src(h, gslot);
+      else ST(reduce_src(h, s, SumSrc{gnew, vg}, gslot, &g1));
+      run->rr_prev = run->rr_old;
+      run->rr_old = g1;
+    }
+    return SPMV_OK;
   }
   for (int c = 0; c < iters; ++c) {
     const int it = run->it++;
@@ -1469,6 +1512,10 @@ extern "C" spmv_status cg_solve(spmv_csr_t h, const void* b, void* x, int32_t ma
   ST(stage_in(h, s, b, &h->stage_x, &bd, true));
   ST(stage_in(h, s, x, &h->stage_z, &xd, false));
   double* xw = const_cast<double*>(xd);
+  if (tol > 0.0 && h->cg_variant == 1 && use_p2p(h)) {
+    g_err = "tol > 0 with the single-reduction CG needs the NCCL or single-GPU transport";
+    return SPMV_ERR_UNSUPPORTED;
+  }
   CK(cudaMemsetAsync(h->flags, 0, sizeof(int) * 4, s));
   CgRun run;
   ST(cg_enqueue_init(h, s, bd, xw, &run));
@@ -1599,6 +1646,16 @@ extern "C" spmv_status spmv_csr_update_values(spmv_csr_t h, const void* vals) {
   if (h->xp.built) ST(xplan_pack(h, vals, 1));
   if (h->sl.built) ST(sell_pack(h, vals, 1));
   h->g_npb.reset();
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_csr_set_cg_variant(spmv_csr_t h, int32_t variant) {
+  if (!h) return arg_fail("handle is NULL");
+  if (variant != 0 && variant != 1) return arg_fail("variant must be 0 (textbook) or 1 (single reduction)");
+  if (h->cg_variant != variant) {
+    h->cg_variant = variant;
+    h->g_npb.reset();  // the captured NPB graph belongs to the other variant
+  }
   return SPMV_OK;
 }
 

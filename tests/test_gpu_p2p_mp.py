@@ -55,6 +55,14 @@ def _worker(rank, world, port, q):
                             M.npb_outer(xs, z, 25, shift, o2)
                         torch.cuda.synchronize()
                         out[kernel] = float(o2[0].item())
+                        if kernel == "auto":  # NEXT-1: single-reduction CG over the p2p transport
+                            M.set_cg_variant("cgcg")
+                            xs.fill_(1.0)
+                            for _ in range(niter):
+                                M.npb_outer(xs, z, 25, shift, o2)
+                            torch.cuda.synchronize()
+                            out["cgcg"] = float(o2[0].item())
+                            M.set_cg_variant("textbook")
         # halo exchange (NEXT-2): the stencil's ranks only exchange boundary planes
         A = gen.stencil27(20)
         rp = torch.from_numpy(A.rowptr).to(dev)
