@@ -434,7 +434,7 @@ def main():
     ap.add_argument("--no-cpu", action="store_true", help="skip the cpu_baseline leg")
     ap.add_argument("--cpu-budget", type=float, default=15.0)
     ap.add_argument("--cg-variant", choices=["textbook", "cgcg"],
-                    default=os.environ.get("SPMV_CG_VARIANT", "textbook"),
+                    default=os.environ.get("SPMV_CG_VARIANT", "cgcg"),
                     help="CG inside the NAS step: textbook (NPB conj_grad) or cgcg (single reduction)")
     args = ap.parse_args()
     if args.warmup < 3:
