@@ -221,3 +221,55 @@ def histo_image(npix: int = HISTO_NPIX, nbins: int = HISTO_NBINS, hot: int = HIS
     out = np.empty(npix, np.int32)
     _L().gen_histo_image(int(npix), int(nbins), int(hot), int(seed), out.ctypes.data)
     return out
+
+
+# --------------------------------------------------- JDS-32 layout (R34)
+@dataclass
+class JDS:
+    """Jagged-diagonal layout of a CSR matrix (Parboil spmv's format, reading R34).
+
+    perm[i]   original row at sorted position i (decreasing length, stable)
+    zcnt[s]   diagonal steps of slice s = positions [32s, 32s+32) (its longest row)
+    jds_ptr   int64[depth+1]: diagonal k occupies [jds_ptr[k], jds_ptr[k+1]) and holds
+              positions 0 .. jds_ptr[k+1]-jds_ptr[k]-1 (whole slices with zcnt > k)
+    indices, data: entry jds_ptr[k]+i = step k of position i (value 0, column 0 padding)
+    """
+    m: int
+    n: int
+    perm: np.ndarray
+    zcnt: np.ndarray
+    jds_ptr: np.ndarray
+    indices: np.ndarray
+    data: np.ndarray
+
+    @property
+    def depth(self) -> int:
+        return len(self.jds_ptr) - 1
+
+
+def csr_to_jds(A: CSR) -> JDS:
+    """Pure layout transform (no arithmetic): CSR -> JDS-32, entries in CSR order per row."""
+    m = A.m
+    L = A.row_lengths().astype(np.int64)
+    perm = np.argsort(-L, kind="stable").astype(np.int32)
+    Ls = L[perm]
+    ns = (m + 31) // 32
+    zcnt = Ls[0::32].astype(np.int32) if m else np.zeros(0, np.int32)
+    depth = int(zcnt[0]) if ns else 0
+    # positions covered by diagonal k: 32 * #{slices with zcnt > k} (zcnt is non-increasing)
+    cover = np.array([32 * int(np.searchsorted(-zcnt, -k, side="left")) for k in range(depth)], np.int64)
+    jds_ptr = np.zeros(depth + 1, np.int64)
+    jds_ptr[1:] = np.cumsum(cover)
+    tot = int(jds_ptr[-1])
+    indices = np.zeros(tot, np.int32)
+    data = np.zeros(tot, A.vals.dtype)
+    start = A.rowptr[:-1].astype(np.int64)[perm] if m else np.zeros(0, np.int64)
+    for k in range(depth):
+        c = int(cover[k])
+        i = np.arange(min(c, m))
+        ok = Ls[i] > k
+        src = start[i[ok]] + k
+        dst = jds_ptr[k] + i[ok]
+        indices[dst] = A.colidx[src]
+        data[dst] = A.vals[src]
+    return JDS(m, A.n, perm, zcnt, jds_ptr, indices, data)

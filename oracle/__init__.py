@@ -55,6 +55,8 @@ def lib():
         L.oracle_cg.restype = ctypes.c_int
         L.oracle_npb_outer.argtypes = [_I64, _P, _P, _P, _P, _P, _I32, _D, _P, _P]
         L.oracle_npb_outer.restype = ctypes.c_int
+        L.oracle_spmv_jds.argtypes = [_I64, _P, _P, _P, _P, _P, _P, _P, _D, _D, _I32, _P, _P]
+        L.oracle_spmv_jds.restype = None
         L.oracle_cg_cgcg.argtypes = [_I64, _P, _P, _P, _P, _P, _I32, _D, _P, _P]
         L.oracle_cg_cgcg.restype = ctypes.c_int
         L.oracle_npb_outer_v.argtypes = [_I64, _P, _P, _P, _P, _P, _I32, _D, _P, _P, _I32]
@@ -257,3 +259,17 @@ def ep(M, pair_begin=0, pair_count=None):
     if st != 0:
         raise ValueError(f"oracle_ep: bad arguments (status {st})")
     return q, sx.value, sy.value
+
+
+def spmv_jds(J, x, y_old=None, alpha=1.0, beta=0.0):
+    """y_ref, bound on the JDS-32 layout J (gen.JDS): y indexed by ORIGINAL row."""
+    f32 = J.data.dtype == np.float32
+    dt = np.float32 if f32 else np.float64
+    x = _c(x, dt)
+    yo = _c(y_old, dt) if y_old is not None else np.zeros(max(J.m, 1), dtype=dt)
+    y_ref = np.empty(max(J.m, 1))
+    bound = np.empty(max(J.m, 1))
+    lib().oracle_spmv_jds(J.m, _ptr(_c(J.perm, np.int32)), _ptr(_c(J.jds_ptr, np.int64)), _ptr(_c(J.zcnt, np.int32)),
+                          _ptr(_c(J.indices, np.int32)), _ptr(_c(J.data, dt)), _ptr(x), _ptr(yo),
+                          float(alpha), float(beta), int(f32), _ptr(y_ref), _ptr(bound))
+    return y_ref[:J.m], bound[:J.m]

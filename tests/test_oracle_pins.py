@@ -355,3 +355,37 @@ def test_stencil27_equals_csr_oracle_bitwise(N):
         ys, bs = oracle.stencil27(N, N, N, x, y_old=y0, alpha=a, beta=b)
         yc, bc = oracle.spmv(A.rowptr, A.colidx, A.vals, x, y0, a, b)
         assert np.array_equal(ys, yc) and np.array_equal(bs, bc)
+
+
+# ------------------------------------------------- JDS-32 (Parboil format, R34)
+def _jds_cases():
+    cases = [gen.makea("S"), gen.powerlaw(m=5000, lmax=700.0, seed=4), gen.laplace1d(33),
+             gen.from_dense(np.zeros((3, 4))), gen.from_dense(np.eye(1))]
+    rows = np.array([0, 0, 2, 5, 5, 5, 40]); cols = np.array([3, 1, 0, 2, 9, 4, 7])
+    cases.append(gen.from_coo(41, 10, rows, cols, np.arange(1.0, 8.0)))   # empty rows, m % 32 != 0
+    return cases
+
+
+@pytest.mark.parametrize("f32", [False, True])
+def test_jds_oracle_equals_csr_oracle(f32):
+    """The JDS layout changes only the storage order: per row the same terms in
+    the same order (padding adds exact zeros), so the results are bit-identical."""
+    for A in _jds_cases():
+        A = A.astype(np.float32) if f32 else A
+        J = gen.csr_to_jds(A)
+        assert np.all(np.diff(J.zcnt) <= 0) and sorted(J.perm.tolist()) == list(range(A.m))
+        x = gen.uniform(A.n, seed=2, f32=f32)
+        yo = gen.uniform(A.m, seed=3, f32=f32)
+        for al, be in ((1.0, 0.0), (-2.5, 0.5), (0.0, 3.0)):
+            y1, b1 = oracle.spmv(A.rowptr, A.colidx, A.vals, x, yo, al, be)
+            y2, b2 = oracle.spmv_jds(J, x, yo, al, be)
+            assert np.array_equal(y1, y2) and np.array_equal(b1, b2), (A.name, al, be)
+
+
+def test_jds_tiny_by_hand():
+    """3x3 [[1,0,2],[0,0,0],[3,4,5]] x=(1,10,100): rows sorted (2,0,1); y = (201, 0, 543)."""
+    A = gen.from_dense(np.array([[1.0, 0, 2], [0, 0, 0], [3, 4, 5]]))
+    J = gen.csr_to_jds(A)
+    assert J.perm.tolist() == [2, 0, 1] and J.zcnt.tolist() == [3] and J.jds_ptr.tolist() == [0, 32, 64, 96]
+    y, _ = oracle.spmv_jds(J, np.array([1.0, 10.0, 100.0]))
+    assert y.tolist() == [201.0, 0.0, 543.0]
