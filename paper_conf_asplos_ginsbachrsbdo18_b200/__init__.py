@@ -83,6 +83,9 @@ spmv_dist_colidx_c = _decl("spmv_dist_colidx", [_P, _P])
 spmv_dist_halo_host_c = _decl("spmv_dist_halo_host", [_P, _P, _I64, _I32, _P])
 spmv_dist_halo_c = _decl("spmv_dist_halo", [_P, _P, _P])
 stencil27_apply_c = _decl("stencil27_apply", [_ST, _I64, _I64, _I64, _P, _P, _P, _D, _D, _P])
+spmv_jds_create_c = _decl("spmv_jds_create", [ctypes.POINTER(_P), _ST, _I64, _I64, _I64, _P, _P, _P, _P, _P, _P])
+spmv_jds_c = _decl("spmv_jds", [_P, _P, _P, _D, _D])
+spmv_jds_destroy_c = _decl("spmv_jds_destroy", [_P])
 # include/idioms.h (histogram, scalar reduction, NAS EP)
 _SZ = ctypes.c_size_t
 idl_reduce_workspace_c = _decl("idl_reduce_workspace", [_I64, ctypes.POINTER(_SZ)])
@@ -99,7 +102,8 @@ EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_s
            "spmv_launch_count", "spmv_status_string", "spmv_last_error_string",
            "spmv_dist_get_unique_id", "spmv_dist_init", "spmv_dist_destroy", "spmv_dist_plan_host",
            "spmv_dist_colidx", "spmv_dist_init_p2p", "spmv_csr_p2p_handle", "spmv_csr_p2p_connect",
-           "spmv_dist_halo_host", "spmv_dist_halo", "stencil27_apply"]
+           "spmv_dist_halo_host", "spmv_dist_halo", "stencil27_apply",
+           "spmv_jds_create", "spmv_jds", "spmv_jds_destroy"]
 # every symbol include/idioms.h declares
 IDIOM_EXPORTS = ["idl_reduce_workspace", "idl_reduce", "idl_histogram_workspace", "idl_histogram",
                  "ep_npb_workspace", "ep_npb"]
@@ -482,3 +486,48 @@ def ep_npb(M: int, pair_begin: int = 0, pair_count: int | None = None, out=None,
                   _stream_of(out) if stream is None else stream)
     _check(st, "ep_npb")
     return out
+
+
+# ------------------------------------------------------------------ JDS-32
+class JDSMatrix:
+    """Handle of spmv_jds_create (Parboil's jagged-diagonal layout, reading R34).
+
+    perm/zcnt/indices int32, jds_ptr int64, data float64/float32: device tensors
+    the caller keeps alive.  ``spmv(x, y)``: y (original row order) <- alpha*A x + beta*y.
+    """
+
+    def __init__(self, perm, jds_ptr, zcnt, indices, data, m: int, n: int, stream=None):
+        import torch
+        assert jds_ptr.dtype == torch.int64 and perm.dtype == torch.int32 and zcnt.dtype == torch.int32
+        self._keep = (perm, jds_ptr, zcnt, indices, data)
+        self.m, self.n = int(m), int(n)
+        self.dtype = data.dtype
+        if stream is None:
+            stream = torch.cuda.current_stream(data.device)
+        h = _P()
+        _check(spmv_jds_create_c(ctypes.byref(h), SPMV_F64 if data.dtype == torch.float64 else SPMV_F32,
+                                 self.m, self.n, jds_ptr.numel() - 1, _ptr(perm), _ptr(jds_ptr), _ptr(zcnt),
+                                 _ptr(indices), _ptr(data), stream.cuda_stream), "spmv_jds_create")
+        self.handle = h
+
+    def spmv(self, x, y, alpha: float = 1.0, beta: float = 0.0):
+        _check(spmv_jds_c(self.handle, _ptr(x), _ptr(y), float(alpha), float(beta)), "spmv_jds")
+        return y
+
+    def destroy(self):
+        if getattr(self, "handle", None):
+            st = spmv_jds_destroy_c(self.handle)
+            self.handle = None
+            _check(st, "spmv_jds_destroy")
+
+    def __del__(self):
+        try:
+            self.destroy()
+        except Exception:
+            pass
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *a):
+        self.destroy()

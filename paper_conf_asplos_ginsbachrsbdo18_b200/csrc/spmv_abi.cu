@@ -1967,3 +1967,5 @@ extern "C" spmv_status spmv_dist_destroy(spmv_dist_t d) {
 
 // ------------------------------------------------------------------ idioms (NEXT-4)
 #include "idioms_abi.cuh"
+// ------------------------------------------------------------------ JDS-32 (NEXT-4, Parboil format)
+#include "jds_abi.cuh"

@@ -73,7 +73,7 @@ def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--reps", type=int, default=20)
     ap.add_argument("--no-cpu", action="store_true")
-    ap.add_argument("which", nargs="*", default=["ep_C", "is_C", "histo", "dot_2p27"])
+    ap.add_argument("which", nargs="*", default=["ep_C", "is_C", "histo", "dot_2p27", "jds_parboil"])
     args = ap.parse_args()
     dev = torch.device("cuda:0")
     torch.cuda.set_device(dev)
@@ -148,6 +148,20 @@ def main():
             cpu = {"value": round(16 * ah.size / dt / 1e9, 2), "unit": "GB/s", "cores": 1, "kind": "oracle",
                    "sample": f"2^24-element dot in {dt * 1e3:.1f} ms, 1 thread"}
         line("scalar reduction: fp64 dot, 2^27 elements", us, us_min, 16.0 * n / 1e9, "GB/s", 16 * n, {}, cpu)
+
+    if "jds_parboil" in args.which:
+        A = gen.powerlaw()
+        J = gen.csr_to_jds(A)
+        dv = lambda a: torch.from_numpy(np.ascontiguousarray(a)).to(dev)
+        M = sp.JDSMatrix(dv(J.perm), dv(J.jds_ptr), dv(J.zcnt), dv(J.indices), dv(J.data), J.m, J.n)
+        x = dv(gen.uniform(A.n, seed=5, f32=True))
+        y = torch.empty(A.m, dtype=torch.float32, device=dev)
+        us, us_min = timed(lambda: M.spmv(x, y), args.reps, flush)
+        # the method's algorithmic bytes of the CSR SpMV: nnz*8 + 4(m+1) + 4n + 4m
+        alg = A.nnz * 8 + 4 * (A.m + 1) + 4 * A.n + 4 * A.m
+        line("Parboil-shaped SpMV on the JDS-32 layout (fp32, 2^20 rows, 11.5M nnz)", us, us_min, 2.0 * A.nnz / 1e9,
+             "GFLOP/s", alg, {"jds_entries": int(J.jds_ptr[-1]), "depth": J.depth})
+        M.destroy()
 
 
 if __name__ == "__main__":
