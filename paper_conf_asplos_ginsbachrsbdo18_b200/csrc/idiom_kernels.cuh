@@ -260,11 +260,13 @@ k_ep(int64_t p0, int64_t count, int64_t chunk, double* __restrict__ out, unsigne
   double sx = 0.0, sy = 0.0;
   unsigned q0 = 0, q1 = 0, q2 = 0, q3 = 0;
   for (int64_t p = lo; p < hi; ++p) {
+    // x = 2u - 1 with u = s * 2^-46, exactly, without an int->double convert:
+    // the bits 0x3FF.. | s << 6 are the double 1 + s * 2^-46, and 2v - 3 = 2u - 1
     s = mul46(s, kEpA);
-    const double u1 = (double)s * 0x1.0p-46;
+    const double v1 = __longlong_as_double((long long)(0x3FF0000000000000ULL | (s << 6)));
     s = mul46(s, kEpA);
-    const double u2 = (double)s * 0x1.0p-46;
-    const double x1 = 2.0 * u1 - 1.0, x2 = 2.0 * u2 - 1.0;     // exact
+    const double v2 = __longlong_as_double((long long)(0x3FF0000000000000ULL | (s << 6)));
+    const double x1 = fma(2.0, v1, -3.0), x2 = fma(2.0, v2, -3.0);   // exact
     const double tt = __dadd_rn(__dmul_rn(x1, x1), __dmul_rn(x2, x2));  // NPB's rounding, no FMA
     if (tt <= 1.0) {
       const double f = sqrt(-2.0 * log(tt) / tt);
