@@ -82,21 +82,40 @@ static const int kHistSmemMax = 200 * 1024;  // dynamic shared memory of one 102
 
 static size_t hist_bin_bytes(idl_hist_kind kind) { return kind == IDL_HIST_SUM_F64 ? 8 : 4; }
 
+// Bucketed counting (idiom_kernels.cuh K1-K4): eligible for the counting kinds
+// when the bins exceed one CTA's shared memory, fit HB_MAXB buckets, and there
+// are >= 2 keys per bin.  Workspace: [fixed part | cnt nb*G u32 | total nb u32 | keys n u16].
+static int hb_grid(int sms) { return std::min(2 * sms, HB_THREADS); }
+static bool hb_eligible(idl_hist_kind kind, int64_t n, int64_t nbins) {
+  return kind != IDL_HIST_SUM_F64 && (size_t)4 * (size_t)nbins > (size_t)kHistSmemMax &&
+         nbins <= (int64_t)HB_MAXB * HB_BW && n >= 2 * nbins && n < 4294967295LL;
+}
+static size_t hist_fixed_bytes(idl_hist_kind kind, int64_t nbins) {
+  // saturating bins are counted in a uint32 workspace first (then min(255, old + count))
+  return kind == IDL_HIST_SAT_U8 ? (((size_t)4 * (size_t)nbins + 255) & ~size_t(255)) : 256;
+}
+static size_t hb_bytes(int64_t n, int64_t nbins, int G) {
+  const size_t nb = (size_t)cdiv(nbins, HB_BW);
+  return ((4 * nb * (size_t)G + 4 * nb + 255) & ~size_t(255)) + 2 * (size_t)n + 256;
+}
+
 extern "C" spmv_status idl_histogram_workspace(idl_hist_kind kind, int64_t n, int64_t nbins, size_t* bytes) {
   if (!bytes) return arg_fail("bytes is NULL");
   if (kind < IDL_HIST_COUNT_U32 || kind > IDL_HIST_SUM_F64) return arg_fail("unknown histogram kind");
   if (n < 0 || nbins < 1 || nbins > 2147483647LL) return arg_fail("need n >= 0 and 1 <= nbins <= 2^31-1");
-  // saturating bins are counted in a uint32 workspace first (then min(255, old + count))
-  *bytes = kind == IDL_HIST_SAT_U8 ? (size_t)4 * (size_t)nbins : 16;
+  size_t b = hist_fixed_bytes(kind, nbins);
+  if (hb_eligible(kind, n, nbins)) b += hb_bytes(n, nbins, HB_THREADS);  // any grid up to HB_THREADS
+  *bytes = b;
   return SPMV_OK;
 }
 
-static int hist_mode() {  // SPMV_HIST=smem|global|agg forces a variant (kernel sweeps), else auto
+static int hist_mode() {  // SPMV_HIST=smem|global|agg|bucket forces a variant (kernel sweeps), else auto
   const char* v = getenv("SPMV_HIST");
   if (!v) return 0;
   if (!strcmp(v, "smem")) return 1;
   if (!strcmp(v, "global")) return 2;
   if (!strcmp(v, "agg")) return 3;
+  if (!strcmp(v, "bucket")) return 4;
   return 0;
 }
 
@@ -107,11 +126,19 @@ extern "C" spmv_status idl_histogram(idl_hist_kind kind, const int32_t* keys, co
   ST(idl_histogram_workspace(kind, n, nbins, &need));
   if (kind == IDL_HIST_SUM_F64 ? false : w != nullptr) return arg_fail("w must be NULL for the counting kinds");
   if (kind == IDL_HIST_SAT_U8 && n > 4294967295LL) return arg_fail("IDL_HIST_SAT_U8 needs n < 2^32");
-  if (kind == IDL_HIST_SAT_U8 && workspace_bytes < need) return arg_fail("workspace too small (idl_histogram_workspace)");
+  const size_t fixed = hist_fixed_bytes(kind, nbins);
+  if (kind == IDL_HIST_SAT_U8 && workspace_bytes < fixed) return arg_fail("workspace too small (idl_histogram_workspace)");
   int dev = 0;
   if (cur_device(&dev)) return arg_fail("no current CUDA device");
   ST(need_device(bins, dev, "bins must be a device pointer on the current device", false));
-  if (kind == IDL_HIST_SAT_U8)
+  const int sms_ = num_sms(dev);
+  const int hbG = hb_grid(sms_);
+  const int mode0 = hist_mode();
+  // bucketed counting when eligible and the caller's workspace holds it (older
+  // callers that pass the fixed part only keep the atomic paths)
+  const bool use_hb = hb_eligible(kind, n, nbins) && workspace && workspace_bytes >= fixed + hb_bytes(n, nbins, hbG) &&
+                      mode0 != 1 && mode0 != 2 && mode0 != 3;
+  if (kind == IDL_HIST_SAT_U8 || use_hb)
     ST(need_device(workspace, dev, "workspace must be a device pointer on the current device", false));
   if (n > 0) {
     ST(need_device(keys, dev, "keys must be a device pointer on the current device", false));
@@ -130,6 +157,36 @@ extern "C" spmv_status idl_histogram(idl_hist_kind kind, const int32_t* keys, co
   if (n == 0) return SPMV_OK;
   cudaStream_t s = (cudaStream_t)stream;
   const int sms = num_sms(dev);
+  if (use_hb) {
+    if (overlap(workspace, fixed + hb_bytes(n, nbins, hbG), bins, (kind == IDL_HIST_SAT_U8 ? 1 : 4) * (size_t)nbins) ||
+        overlap(workspace, fixed + hb_bytes(n, nbins, hbG), keys, 4 * (size_t)n)) {
+      g_err = "workspace overlaps bins or keys";
+      return SPMV_ERR_ALIAS;
+    }
+    const int nb = (int)cdiv(nbins, HB_BW);
+    const int64_t chunk = cdiv(cdiv(n, hbG), 4) * 4;
+    const int G = (int)cdiv(n, chunk);
+    char* wb = (char*)workspace + fixed;
+    unsigned* cnt = (unsigned*)wb;
+    unsigned* total = cnt + (size_t)nb * G;
+    uint16_t* sorted = (uint16_t*)(wb + ((4 * (size_t)nb * G + 4 * (size_t)nb + 255) & ~size_t(255)));
+    k_hb_count<<<G, HB_THREADS, 0, s>>>(n, chunk, (int)nbins, nb, keys, cnt, aligned16(keys) ? 1 : 0);
+    LAUNCHED();
+    k_hb_scan<<<nb, HB_THREADS, 0, s>>>(G, cnt, total);
+    LAUNCHED();
+    k_hb_scatter<<<G, HB_THREADS, 0, s>>>(n, chunk, (int)nbins, nb, keys, cnt, total, sorted);
+    LAUNCHED();
+    const size_t sm4 = (size_t)4 * HB_BW;
+    if (kind == IDL_HIST_COUNT_U32) {
+      CK(cudaFuncSetAttribute(k_hb_bins<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm4));
+      k_hb_bins<0><<<nb, HB_THREADS, sm4, s>>>((int)nbins, nb, total, sorted, bins);
+    } else {
+      CK(cudaFuncSetAttribute(k_hb_bins<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm4));
+      k_hb_bins<1><<<nb, HB_THREADS, sm4, s>>>((int)nbins, nb, total, sorted, bins);
+    }
+    LAUNCHED();
+    return SPMV_OK;
+  }
   const int nb = (int)nbins;
   const int vec = aligned16(keys) ? 1 : 0;
   void* dst = kind == IDL_HIST_SAT_U8 ? workspace : bins;

@@ -234,3 +234,25 @@ def test_ep_ranges_shards_and_determinism(sp):
     assert len(set(runs)) == 1
     z = sp.ep_npb(M, 5, 0).cpu().numpy()
     assert not z.any()
+
+
+@pytest.mark.parametrize("kind", ["count", "sat_u8"])
+@pytest.mark.parametrize("n,nbins", [(3_000_001, 1_000_003), (600_000, 65_537), (5_000_000, 2_000_000)])
+def test_hist_bucketed_exact(sp, kind, n, nbins):
+    """Bucketed counting (partition by key >> 15, shared-memory counts per bucket):
+    out-of-range keys skipped, accumulation onto old bins, unaligned key views."""
+    import torch
+    r = np.random.default_rng(n)
+    hot = r.integers(0, nbins, size=16)
+    k = np.where(r.random(n) < 0.3, hot[r.integers(0, 16, size=n)], r.integers(-7, nbins + 7, size=n)).astype(np.int32)
+    dt = np.uint32 if kind == "count" else np.uint8
+    old = (np.arange(nbins) % (7 if kind == "count" else 200)).astype(dt)
+    for view in (slice(None), slice(1, None)):
+        kk = k[view]
+        ref = (oracle.hist_count_u32(kk, nbins, old) if kind == "count" else oracle.hist_sat_u8(kk, nbins, old))
+        bins = _dev(old)
+        wsb = sp.idl_histogram_workspace(kind, kk.size, nbins)
+        assert wsb > 2 * kk.size                                   # the bucketed path's scratch is offered
+        ws = torch.zeros(wsb, dtype=torch.uint8, device="cuda")
+        sp.idl_histogram(kind, _dev(k)[view], bins, workspace=ws)
+        assert np.array_equal(bins.cpu().numpy(), ref), (kind, n, nbins, view)
