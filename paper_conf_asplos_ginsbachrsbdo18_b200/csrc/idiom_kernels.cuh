@@ -245,7 +245,7 @@ constexpr int HB_SHIFT = 15;               // 32768 bins per bucket (128 KB of u
 constexpr int HB_BW = 1 << HB_SHIFT;
 constexpr int HB_MAXB = 1024;              // buckets (nbins <= 2^25)
 constexpr int HB_THREADS = 1024;
-constexpr int HB_TILE = 4096;              // keys staged per tile in K3
+constexpr int HB_TILE = 4096;              // keys staged per tile in K3 (16 KB of shared memory)
 
 __global__ void __launch_bounds__(HB_THREADS)
 k_hb_count(int64_t n, int64_t chunk, int nbins, int nb, const int32_t* __restrict__ keys,
@@ -321,7 +321,7 @@ k_hb_scatter(int64_t n, int64_t chunk, int nbins, int nb, const int32_t* __restr
              const unsigned* __restrict__ off /* [nb][G] exclusive */, const unsigned* __restrict__ total,
              uint16_t* __restrict__ out) {
   __shared__ unsigned cursor[HB_MAXB], tcnt[HB_MAXB], tbase[HB_MAXB], ws[32];
-  __shared__ unsigned stage[HB_TILE];
+  extern __shared__ __align__(16) unsigned stage[];  // HB_TILE entries (dynamic)
   const int t = threadIdx.x;
   // global start of bucket b = sum of the totals before it; cursor = start + this CTA's offset
   for (int b = t; b < HB_MAXB; b += HB_THREADS) cursor[b] = b < nb ? total[b] : 0u;

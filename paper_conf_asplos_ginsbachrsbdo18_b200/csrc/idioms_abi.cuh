@@ -136,8 +136,10 @@ extern "C" spmv_status idl_histogram(idl_hist_kind kind, const int32_t* keys, co
   const int mode0 = hist_mode();
   // bucketed counting when eligible and the caller's workspace holds it (older
   // callers that pass the fixed part only keep the atomic paths)
+  // opt-in (SPMV_HIST=bucket): measured slower than the L2 atomics on NAS IS
+  // class C (878 vs 748 us; its tile-staged scatter pass alone takes 566 us)
   const bool use_hb = hb_eligible(kind, n, nbins) && workspace && workspace_bytes >= fixed + hb_bytes(n, nbins, hbG) &&
-                      mode0 != 1 && mode0 != 2 && mode0 != 3;
+                      mode0 == 4;
   if (kind == IDL_HIST_SAT_U8 || use_hb)
     ST(need_device(workspace, dev, "workspace must be a device pointer on the current device", false));
   if (n > 0) {
@@ -174,7 +176,8 @@ extern "C" spmv_status idl_histogram(idl_hist_kind kind, const int32_t* keys, co
     LAUNCHED();
     k_hb_scan<<<nb, HB_THREADS, 0, s>>>(G, cnt, total);
     LAUNCHED();
-    k_hb_scatter<<<G, HB_THREADS, 0, s>>>(n, chunk, (int)nbins, nb, keys, cnt, total, sorted);
+    CK(cudaFuncSetAttribute(k_hb_scatter, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 * HB_TILE));
+    k_hb_scatter<<<G, HB_THREADS, 4 * HB_TILE, s>>>(n, chunk, (int)nbins, nb, keys, cnt, total, sorted);
     LAUNCHED();
     const size_t sm4 = (size_t)4 * HB_BW;
     if (kind == IDL_HIST_COUNT_U32) {

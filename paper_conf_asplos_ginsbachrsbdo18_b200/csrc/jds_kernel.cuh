@@ -21,7 +21,6 @@ namespace spmv {
 
 constexpr int JDS_SEG = 256;      // diagonal steps per warp unit
 constexpr int JDS_THREADS = 256;
-constexpr int JDS_U = 8;         // diagonal steps in flight per lane
 
 // unit: {slice, k0, k1, part}; part < 0: the slice's only unit (writes y)
 template <typename T>
@@ -36,28 +35,25 @@ k_spmv_jds(const int4* __restrict__ units, int nunits, int64_t m, const long lon
   const int4 u = units[warp];
   const int64_t i = (int64_t)u.x * 32 + lane;
   double acc = 0.0;
-  // batches of JDS_U steps with every load of the batch issued before the
-  // first use (predicated tail): most slices of a power-law matrix have < 16
-  // steps, so a whole slice is one or two memory round trips
-  for (int k = u.y; k < u.z; k += JDS_U) {
-    T d[JDS_U];
-    int c[JDS_U];
+  int k = u.y;
+  for (; k + 4 <= u.z; k += 4) {
+    T d[4];
+    int c[4];
 #pragma unroll
-    for (int q = 0; q < JDS_U; ++q) {
-      d[q] = T(0);
-      c[q] = 0;
-      if (k + q < u.z) {
-        const int64_t j = __ldg(jds_ptr + k + q) + i;
-        d[q] = ld_stream(data + j);
-        c[q] = ld_stream(idx + j);
-      }
+    for (int q = 0; q < 4; ++q) {
+      const int64_t j = __ldg(jds_ptr + k + q) + i;
+      d[q] = ld_stream(data + j);
+      c[q] = ld_stream(idx + j);
     }
-    T xv[JDS_U];
+    T xv[4];
 #pragma unroll
-    for (int q = 0; q < JDS_U; ++q) xv[q] = k + q < u.z ? ld_x(x + c[q]) : T(0);
+    for (int q = 0; q < 4; ++q) xv[q] = ld_x(x + c[q]);
 #pragma unroll
-    for (int q = 0; q < JDS_U; ++q)
-      if (k + q < u.z) acc = fma((double)d[q], (double)xv[q], acc);
+    for (int q = 0; q < 4; ++q) acc = fma((double)d[q], (double)xv[q], acc);
+  }
+  for (; k < u.z; ++k) {
+    const int64_t j = __ldg(jds_ptr + k) + i;
+    acc = fma((double)ld_stream(data + j), (double)ld_x(x + ld_stream(idx + j)), acc);
   }
   if (u.w < 0) {
     if (i < m) {

@@ -238,10 +238,12 @@ def test_ep_ranges_shards_and_determinism(sp):
 
 @pytest.mark.parametrize("kind", ["count", "sat_u8"])
 @pytest.mark.parametrize("n,nbins", [(3_000_001, 1_000_003), (600_000, 65_537), (5_000_000, 2_000_000)])
-def test_hist_bucketed_exact(sp, kind, n, nbins):
-    """Bucketed counting (partition by key >> 15, shared-memory counts per bucket):
-    out-of-range keys skipped, accumulation onto old bins, unaligned key views."""
+def test_hist_bucketed_exact(sp, monkeypatch, kind, n, nbins):
+    """Bucketed counting (partition by key >> 15, shared-memory counts per bucket;
+    opt-in via SPMV_HIST=bucket): out-of-range keys skipped, accumulation onto
+    old bins, unaligned key views."""
     import torch
+    monkeypatch.setenv("SPMV_HIST", "bucket")
     r = np.random.default_rng(n)
     hot = r.integers(0, nbins, size=16)
     k = np.where(r.random(n) < 0.3, hot[r.integers(0, 16, size=n)], r.integers(-7, nbins + 7, size=n)).astype(np.int32)
