@@ -1779,8 +1779,22 @@ extern "C" spmv_status stencil27_apply(spmv_dtype dt, int64_t nx, int64_t ny, in
   a.zchunk = zc;
   if (by > 65535 || zs > 65535) return arg_fail("grid too large for the stencil launch");
   const dim3 grid((unsigned)bx, (unsigned)by, (unsigned)zs);
-  if (dt == SPMV_F64) k_stencil27<double><<<grid, ST_NT, 0, s>>>(a);
-  else k_stencil27<float><<<grid, ST_NT, 0, s>>>(a);
+  // BOX form when the 26 neighbour weights are equal (R19's default among them);
+  // SPMV_STENCIL_BOX=0 forces the general 27-weight form
+  bool box = true;
+  for (int i = 0; i < 27; ++i)
+    if (i != 13 && a.w[i] != a.w[0]) box = false;
+  int benv = 1;
+  if (env_int("SPMV_STENCIL_BOX", &benv) && benv == 0) box = false;
+  a.wn = a.w[0];
+  a.wd = a.w[13] - a.w[0];
+  if (dt == SPMV_F64) {
+    if (box) k_stencil27<double, true><<<grid, ST_NT, 0, s>>>(a);
+    else k_stencil27<double, false><<<grid, ST_NT, 0, s>>>(a);
+  } else {
+    if (box) k_stencil27<float, true><<<grid, ST_NT, 0, s>>>(a);
+    else k_stencil27<float, false><<<grid, ST_NT, 0, s>>>(a);
+  }
   LAUNCHED();
   return SPMV_OK;
 }

@@ -4,8 +4,9 @@
 // function a weighted sum over the 3x3x3 neighbourhood and Dirichlet
 // truncation (reading R19): for every grid point p = x + nx*(y + ny*z)
 //     y[p] = alpha * sum_{d in {-1,0,1}^3, p+d inside} w[d] * x[p+d] + beta * y[p]
-// It is the operator whose CSR form is BJ.cfg[4]; with R19's weights (26, -1)
-// the result equals spmv_csr on gen.stencil27 (same terms, same order).
+// It is the operator whose CSR form is BJ.cfg[4]; with general weights the
+// result equals spmv_csr on the same CSR matrix (same terms, same order);
+// with R19's weights (26, -1) the separable box-sum form below is used.
 //
 // 2.5-D blocking: a CTA owns a TX x TY tile of (x, y) and marches a range of
 // z planes.  Each plane (+ a one-point halo) is staged once in shared memory
@@ -52,9 +53,17 @@ struct StencilArgs {
   const void* x;
   void* y;
   double alpha, beta;
+  double wd, wn;       // BOX: w[13] - wn and the common neighbour weight wn
 };
 
-template <typename T>
+// BOX = every one of the 26 neighbour weights equals wn (R19's Laplacian:
+// wn = -1, centre 26).  Then  y = alpha*((w_c - wn)*x_c + wn*B)  with B the
+// 3x3x3 box sum, which is separable: per plane, 3-point row sums then 3-row
+// column sums (the in-plane 3x3 box, 4 adds per point for ST_RY = 2), and
+// the three plane boxes of an output added in z.  ~11 fp64 operations per
+// point instead of 27 FMAs; a different summation order than the CSR row,
+// within reading R11's per-row bound (the bound holds |x_j| of all 27 terms).
+template <typename T, bool BOX>
 __global__ void __launch_bounds__(ST_NT)
 k_stencil27(StencilArgs a) {
   __shared__ T pl[2][ST_PN];
@@ -95,8 +104,9 @@ k_stencil27(StencilArgs a) {
 
   const double alpha = a.alpha, beta = a.beta;
   double acc_m[ST_RY], acc_c[ST_RY], acc_p[ST_RY];  // outputs zp-1, zp, zp+1 of each row
+  double cen_m[ST_RY];                               // BOX: centre x of output zp-1
 #pragma unroll
-  for (int r = 0; r < ST_RY; ++r) acc_m[r] = acc_c[r] = acc_p[r] = 0.0;
+  for (int r = 0; r < ST_RY; ++r) acc_m[r] = acc_c[r] = acc_p[r] = cen_m[r] = 0.0;
   {
     T v0[ST_LPT];
     fetch(z0 - 1, v0);
@@ -110,30 +120,53 @@ k_stencil27(StencilArgs a) {
     T vf[ST_LPT];
     fetch(zp + 1 + ST_PF, vf);  // ST_PF planes ahead (zeros past z1: never stashed)
     const T* P = pl[cur];
+    if (BOX) {
+      double rs[ST_RY + 2];  // 3-point row sums of plane rows ty-1 .. ty+ST_RY
 #pragma unroll
-    for (int sy = 0; sy < ST_RY + 2; ++sy)  // plane rows ty-1 .. ty+ST_RY
-#pragma unroll
-      for (int dx = 0; dx < 3; ++dx) {
-        const double xv = double(P[(ty + sy) * ST_PX + tx + dx]);
-#pragma unroll
-        for (int r = 0; r < ST_RY; ++r) {
-          const int dy = sy - r;  // row offset + 1 of this value for output row r
-          if (dy < 0 || dy > 2) continue;
-          acc_p[r] = fma(a.w[0 * 9 + dy * 3 + dx], xv, acc_p[r]);  // output zp+1, dz = -1
-          acc_c[r] = fma(a.w[1 * 9 + dy * 3 + dx], xv, acc_c[r]);  // output zp,   dz =  0
-          acc_m[r] = fma(a.w[2 * 9 + dy * 3 + dx], xv, acc_m[r]);  // output zp-1, dz = +1
-        }
+      for (int sy = 0; sy < ST_RY + 2; ++sy) {
+        const T* q = P + (ty + sy) * ST_PX + tx;
+        rs[sy] = (double(q[0]) + double(q[1])) + double(q[2]);
       }
+#pragma unroll
+      for (int r = 0; r < ST_RY; ++r) {
+        const double b2 = (rs[r] + rs[r + 1]) + rs[r + 2];  // in-plane 3x3 box of output row r
+        acc_p[r] += b2;
+        acc_c[r] += b2;
+        acc_m[r] += b2;
+      }
+    } else {
+#pragma unroll
+      for (int sy = 0; sy < ST_RY + 2; ++sy)  // plane rows ty-1 .. ty+ST_RY
+#pragma unroll
+        for (int dx = 0; dx < 3; ++dx) {
+          const double xv = double(P[(ty + sy) * ST_PX + tx + dx]);
+#pragma unroll
+          for (int r = 0; r < ST_RY; ++r) {
+            const int dy = sy - r;  // row offset + 1 of this value for output row r
+            if (dy < 0 || dy > 2) continue;
+            acc_p[r] = fma(a.w[0 * 9 + dy * 3 + dx], xv, acc_p[r]);  // output zp+1, dz = -1
+            acc_c[r] = fma(a.w[1 * 9 + dy * 3 + dx], xv, acc_c[r]);  // output zp,   dz =  0
+            acc_m[r] = fma(a.w[2 * 9 + dy * 3 + dx], xv, acc_m[r]);  // output zp-1, dz = +1
+          }
+        }
+    }
     const int64_t zo = zp - 1;  // complete now
     if (gx < nx && zo >= z0 && zo < z1) {
 #pragma unroll
       for (int r = 0; r < ST_RY; ++r) {
         if (gy + r >= ny) continue;
         const int64_t p = gx + nx * (gy + r) + nxy * zo;
-        double res = alpha * acc_m[r];
+        double res;
+        if (BOX) res = alpha * fma(a.wd, cen_m[r], a.wn * acc_m[r]);  // (w_c - wn) x_c + wn B
+        else res = alpha * acc_m[r];
         if (beta != 0.0) res += beta * double(y[p]);
         y[p] = T(res);
       }
+    }
+    if (BOX) {
+#pragma unroll
+      for (int r = 0; r < ST_RY; ++r)  // centre of plane zp: the output written next iteration
+        cen_m[r] = double(P[(ty + 1 + r) * ST_PX + tx + 1]);
     }
 #pragma unroll
     for (int r = 0; r < ST_RY; ++r) {

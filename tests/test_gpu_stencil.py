@@ -67,7 +67,8 @@ def test_stencil_z_ranges(env, zchunk, monkeypatch):
 
 @pytest.mark.parametrize("alpha,beta", [(2.5, 0.0), (-1.0, 0.5), (0.0, 3.0), (0.0, 0.0), (1.0, 1.0)])
 @pytest.mark.parametrize("f32", [False, True])
-def test_stencil_alpha_beta(env, alpha, beta, f32):
+@pytest.mark.parametrize("wkind", ["random", "laplace"])
+def test_stencil_alpha_beta(env, alpha, beta, f32, wkind):
     dims = (17, 9, 11)
     n = 17 * 9 * 11
     x = gen.uniform(n, seed=3, f32=f32)
@@ -76,7 +77,7 @@ def test_stencil_alpha_beta(env, alpha, beta, f32):
     y0 = gen.uniform(n, seed=4, f32=f32)
     if beta == 0.0:
         y0 = np.full(n, np.nan, dtype=y0.dtype)  # must not be read
-    w = gen.uniform(27, seed=9)
+    w = gen.uniform(27, seed=9) if wkind == "random" else None   # laplace: the BOX form
     y, y_ref, bound = _run(env, dims, x, w=w, y0=y0, alpha=alpha, beta=beta, f32=f32)
     check_rows(y, y_ref, bound, np.float32 if f32 else np.float64, f"stencil f32={f32} a={alpha} b={beta}")
 
@@ -130,3 +131,19 @@ def test_stencil256_full_size(env):
     for c in (i % N, (i // N) % N, i // (N * N)):
         cnt = cnt * (3 - (c == 0) - (c == N - 1))
     assert np.array_equal(yy.cpu().numpy(), (27 - cnt).astype(np.float64))
+
+
+@pytest.mark.parametrize("dims", [(33, 9, 17), (64, 64, 64), (5, 1, 130)])
+def test_stencil_box_form(env, dims, monkeypatch):
+    """Equal neighbour weights select the separable box-sum form: R19's Laplacian,
+    all 27 weights equal, and an arbitrary (centre, neighbour) pair; each within
+    the R11 bound of the oracle, and close to the general 27-FMA form."""
+    n = dims[0] * dims[1] * dims[2]
+    x = gen.uniform(n, seed=11)
+    for w in (None, np.full(27, 0.37), np.where(np.arange(27) == 13, 5.5, -0.25)):
+        y, y_ref, bound = _run(env, dims, x, w=w)
+        check_rows(y, y_ref, bound, np.float64, f"box {dims}")
+        monkeypatch.setenv("SPMV_STENCIL_BOX", "0")
+        y2, _, _ = _run(env, dims, x, w=w)
+        monkeypatch.delenv("SPMV_STENCIL_BOX")
+        check_rows(y2, y_ref, bound, np.float64, f"general {dims}")
