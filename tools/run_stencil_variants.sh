@@ -2,8 +2,8 @@ L=paper_conf_asplos_ginsbachrsbdo18_b200/libspmv_b200.so
 cp $L /tmp/orig_lib.so
 for v in tools/variants/lib_*.so; do
   cp $v $L
-  for z in 0 24 48; do
-    if [ $z = 0 ]; then timeout 60 python tools/time_stencil.py $(basename $v .so) 256; else timeout 60 python tools/time_stencil.py $(basename $v .so) 256 SPMV_STENCIL_ZCHUNK=$z; fi
+  for e in "SPMV_STENCIL_BOX=1" "SPMV_STENCIL_BOX=0" "SPMV_STENCIL_ZCHUNK=32" "SPMV_STENCIL_ZCHUNK=43"; do
+    timeout 60 python tools/time_stencil.py $(basename $v .so) 256 $e
   done
 done
 cp /tmp/orig_lib.so $L
