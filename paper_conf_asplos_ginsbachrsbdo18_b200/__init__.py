@@ -465,6 +465,15 @@ def idl_histogram(kind, keys, bins, w=None, workspace=None, stream=None):
     return bins
 
 
+def ep_shard_range(M: int, rank: int, nranks: int):
+    """Reading R33: rank r of P owns pairs [floor(r*2^M/P), floor((r+1)*2^M/P)).
+    Returns (pair_begin, pair_count); host-only."""
+    total = 1 << M
+    b0 = rank * total // nranks
+    b1 = (rank + 1) * total // nranks
+    return b0, b1 - b0
+
+
 def ep_npb_workspace() -> int:
     b = ctypes.c_size_t(0)
     _check(ep_npb_workspace_c(ctypes.byref(b)), "ep_npb_workspace")

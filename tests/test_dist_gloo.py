@@ -125,3 +125,56 @@ def test_dist_plan_gloo(world, cls):
         p.join(timeout=60)
     for r, msg in res:
         assert msg == "ok", f"rank {r}: {msg}"
+
+
+def _ep_worker(rank, world, port, q):
+    import sys
+    sys.path.insert(0, ROOT)
+    import numpy as np
+    import torch
+    import torch.distributed as dist
+
+    import oracle
+    from paper_conf_asplos_ginsbachrsbdo18_b200 import ep_shard_range
+    try:
+        dist.init_process_group("gloo", init_method=f"tcp://127.0.0.1:{port}", rank=rank, world_size=world)
+        M = 24
+        b0, cnt = ep_shard_range(M, rank, world)
+        qq, sx, sy = oracle.ep(M, b0, cnt)
+        mine = torch.tensor(np.concatenate([qq, [sx, sy]]), dtype=torch.float64)
+        parts = [torch.zeros(12, dtype=torch.float64) for _ in range(world)]
+        dist.all_gather(parts, mine)
+        tot = torch.zeros(12, dtype=torch.float64)
+        for p in parts:           # rank order: every rank gets the same sums
+            tot += p
+        dist.destroy_process_group()
+        q.put((rank, "ok", tot.numpy().tolist(), (b0, cnt)))
+    except Exception as e:  # pragma: no cover
+        import traceback
+        q.put((rank, "".join(traceback.format_exception(e)), None, None))
+
+
+@pytest.mark.parametrize("world", [2, 3])
+def test_ep_sharded_gloo(world):
+    """NAS EP sharded by pair ranges (R33) over gloo ranks: the rank-order sum of
+    the per-rank tallies equals the single-process oracle (q exactly)."""
+    import oracle
+    port = _free_port()
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    ps = [ctx.Process(target=_ep_worker, args=(r, world, port, q)) for r in range(world)]
+    for p in ps:
+        p.start()
+    res = [q.get(timeout=300) for _ in ps]
+    for p in ps:
+        p.join(timeout=60)
+    ranges = sorted(r[3] for r in res)
+    assert ranges[0][0] == 0 and sum(c for _, c in ranges) == 1 << 24
+    assert all(ranges[i][0] + ranges[i][1] == ranges[i + 1][0] for i in range(world - 1))
+    qf, sxf, syf = oracle.ep(24)
+    for rank, msg, tot, _ in res:
+        assert msg == "ok", msg
+        tot = np.array(tot)
+        assert np.array_equal(tot[:10], qf)
+        assert abs(tot[10] - sxf) <= 1e-10 * abs(sxf) and abs(tot[11] - syf) <= 1e-10 * abs(syf)
+    assert res[0][2] == res[-1][2]
