@@ -19,7 +19,10 @@
 
 namespace spmv {
 
-constexpr int JDS_SEG = 256;      // diagonal steps per warp unit
+#ifndef JDS_SEG_DEF
+#define JDS_SEG_DEF 256
+#endif
+constexpr int JDS_SEG = JDS_SEG_DEF;  // diagonal steps per warp unit
 constexpr int JDS_THREADS = 256;
 
 // unit: {slice, k0, k1, part}; part < 0: the slice's only unit (writes y)

@@ -475,38 +475,51 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   const size_t xbudget = smem_cap - recv - 64;
   const int64_t Bneed = cdiv((int64_t)(ts * h->nx), (int64_t)xbudget);
   if (Bneed > 16) return SPMV_OK;  // x does not fit the shared memory of a 16-CTA cluster
-  int B = Bneed <= 1 ? 1 : Bneed <= 2 ? 2 : Bneed <= 4 ? 4 : Bneed <= 8 ? 8 : 16;
-  int forced = 0;
-  if (env_int("SPMV_XPLAN_B", &forced) && forced >= B && forced <= 16 && (forced & (forced - 1)) == 0) B = forced;
-  if (B > 16) return SPMV_OK;
-  int W = (int)cdiv(h->nx, B);
-  W = (W + 7) & ~7;
-  if (W > 65534) return SPMV_OK;  // 16-bit column offsets, pad column W
-  const size_t xbytes = ((size_t)(W + 1) * ts + 15) & ~size_t(15);
-  const size_t smem = xbytes + recv;
-  if (smem > smem_cap) return SPMV_OK;
   void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, false> : k_spmv_xplan<float, false>;
   void (*fnd)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, true> : nullptr;
+  // cluster size: any B >= Bneed that divides the tile height R (rows are
+  // owned in R/B blocks); among those, the one whose resident clusters cover
+  // the most SMs (ties: the smaller B, whose x blocks are larger); clusters of
+  // 16 only when nothing smaller fits.  SPMV_XPLAN_B forces a size.
+  int forced = 0;
+  env_int("SPMV_XPLAN_B", &forced);
+  int B = 0, W = 0, ncl = 0;
+  size_t smem = 0;
+  for (int cand = (int)std::max<int64_t>(1, Bneed); cand <= 16; ++cand) {
+    if (XP_R % cand) continue;
+    if (forced && cand != forced) continue;
+    if (cand > 8 && B > 0) break;  // non-portable sizes only as the last resort
+    int Wc = (int)cdiv(h->nx, cand);
+    Wc = (Wc + 7) & ~7;
+    if (Wc > 65534) continue;  // 16-bit column offsets, pad column W
+    const size_t sm = (((size_t)(Wc + 1) * ts + 15) & ~size_t(15)) + recv;
+    if (sm > smem_cap) continue;
+    CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm));
+    if (cand > 8) CK(cudaFuncSetAttribute(fn, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3((unsigned)cand, 1, 1);
+    cfg.blockDim = dim3(XP_THREADS, 1, 1);
+    cfg.dynamicSmemBytes = sm;
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeClusterDimension;
+    at[0].val.clusterDim.x = (unsigned)cand;
+    at[0].val.clusterDim.y = 1;
+    at[0].val.clusterDim.z = 1;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    int nc = 0;
+    cudaError_t e = cudaOccupancyMaxActiveClusters(&nc, fn, &cfg);
+    if (e != cudaSuccess || nc < 1) { cudaGetLastError(); continue; }
+    DBG("candidate B=%d W=%d clusters=%d SMs=%d", cand, Wc, nc, nc * cand);
+    if (B == 0 || nc * cand > ncl * B) { B = cand; W = Wc; ncl = nc; smem = sm; }
+  }
+  if (B == 0) return SPMV_OK;
   CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
   if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
   if (B > 8) {  // clusters of 16 need the non-portable size
     CK(cudaFuncSetAttribute(fn, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
     if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
   }
-  cudaLaunchConfig_t cfg = {};
-  cfg.gridDim = dim3((unsigned)B, 1, 1);
-  cfg.blockDim = dim3(XP_THREADS, 1, 1);
-  cfg.dynamicSmemBytes = smem;
-  cudaLaunchAttribute at[1];
-  at[0].id = cudaLaunchAttributeClusterDimension;
-  at[0].val.clusterDim.x = (unsigned)B;
-  at[0].val.clusterDim.y = 1;
-  at[0].val.clusterDim.z = 1;
-  cfg.attrs = at;
-  cfg.numAttrs = 1;
-  int ncl = 0;
-  cudaError_t e = cudaOccupancyMaxActiveClusters(&ncl, fn, &cfg);
-  if (e != cudaSuccess || ncl < 1) { cudaGetLastError(); return SPMV_OK; }
   int nc_env = 0;
   if (env_int("SPMV_XPLAN_CLUSTERS", &nc_env) && nc_env >= 1 && nc_env <= ncl) ncl = nc_env;
   cudaStream_t s = h->stream;

@@ -329,8 +329,12 @@ __global__ void __launch_bounds__(XP_THREADS)
 k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_t m, int B,
              const long long* __restrict__ crow, const int* __restrict__ tile0, int ncl, int* __restrict__ chunk_len,
              uint16_t* __restrict__ chunk_row, int* __restrict__ row_slot) {
-  __shared__ unsigned long long key[XP_R];
-  constexpr int PER = XP_R / XP_THREADS;
+  // bitonic sort over the next power of two >= R (XP_R need not be one: the
+  // tile height must be a multiple of the cluster size B); padding sorts last
+  constexpr int PR = XP_R <= 1024 ? 1024 : XP_R <= 2048 ? 2048 : 4096;
+  static_assert(XP_R <= PR, "tile too tall");
+  __shared__ unsigned long long key[PR];
+  constexpr int PER = (PR + XP_THREADS - 1) / XP_THREADS;
   const int tg = blockIdx.x / B, b = blockIdx.x % B;
   int c = 0;
   while (c + 1 < ncl && tile0[c + 1] <= tg) ++c;
@@ -339,6 +343,11 @@ k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_
   const int nrows = int(cmin64(XP_R, crow[c + 1] - rt));
   for (int e = 0; e < PER; ++e) {
     const int j = threadIdx.x + e * XP_THREADS;
+    if (j >= PR) continue;
+    if (j >= XP_R) {
+      key[j] = ~0ull;  // power-of-two padding
+      continue;
+    }
     int L = -1;  // absent rows sort last
     if (j < nrows) {
       int k0, k1;
@@ -349,10 +358,11 @@ k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_
     key[j] = (static_cast<unsigned long long>(~static_cast<uint32_t>(L + 1)) << 32) | uint32_t(j);
   }
   __syncthreads();
-  for (int k = 2; k <= XP_R; k <<= 1)
+  for (int k = 2; k <= PR; k <<= 1)
     for (int s = k >> 1; s > 0; s >>= 1) {
       for (int e = 0; e < PER; ++e) {
         const int j = threadIdx.x + e * XP_THREADS;
+        if (j >= PR) continue;
         const int p = j ^ s;
         if (p > j) {
           const bool up = (j & k) == 0;
@@ -364,6 +374,7 @@ k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_
     }
   for (int e = 0; e < PER; ++e) {
     const int j = threadIdx.x + e * XP_THREADS;
+    if (j >= XP_R) continue;
     const unsigned long long kk = key[j];
     const int row = int(kk & 0xffffffffu);
     const int Ls = int(~uint32_t(kk >> 32)) - 1;
