@@ -20,7 +20,7 @@
 namespace spmv {
 
 #ifndef JDS_SEG_DEF
-#define JDS_SEG_DEF 256
+#define JDS_SEG_DEF 64
 #endif
 constexpr int JDS_SEG = JDS_SEG_DEF;  // diagonal steps per warp unit
 constexpr int JDS_THREADS = 256;
