@@ -45,6 +45,27 @@ constexpr int ST_LPT = (ST_PN + ST_NT - 1) / ST_NT;  // plane elements staged pe
 #define ST_PF_DEF 1
 #endif
 constexpr int ST_PF = ST_PF_DEF;  // planes whose loads are in flight (register ring)
+#ifndef ST_ASYNC_DEF
+#define ST_ASYNC_DEF 1
+#endif
+#ifndef ST_NS_DEF
+#define ST_NS_DEF 3
+#endif
+// ST_ASYNC: planes are copied global -> shared with cp.async (zero-fill for
+// the halo outside the grid) into a ring of ST_NS plane buffers, so ST_NS-1
+// planes are in flight per CTA without holding them in registers
+constexpr bool ST_ASYNC = ST_ASYNC_DEF != 0;
+constexpr int ST_NS = ST_NS_DEF;
+
+template <int BYTES>
+__device__ __forceinline__ void cp_async_zfill(void* sdst, const void* gsrc, int src_bytes) {
+  const uint32_t d = static_cast<uint32_t>(__cvta_generic_to_shared(sdst));
+  asm volatile("cp.async.ca.shared.global [%0], [%1], %2, %3;\n" ::"r"(d), "l"(gsrc), "n"(BYTES), "r"(src_bytes)
+               : "memory");
+}
+__device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;\n" ::: "memory"); }
+template <int N>
+__device__ __forceinline__ void cp_async_wait() { asm volatile("cp.async.wait_group %0;\n" ::"n"(N) : "memory"); }
 
 struct StencilArgs {
   int64_t nx, ny, nz;
@@ -66,7 +87,7 @@ struct StencilArgs {
 template <typename T, bool BOX>
 __global__ void __launch_bounds__(ST_NT)
 k_stencil27(StencilArgs a) {
-  __shared__ T pl[2][ST_PN];
+  __shared__ __align__(16) T pl[ST_ASYNC ? ST_NS : 2][ST_PN];
   const T* __restrict__ x = static_cast<const T*>(a.x);
   T* __restrict__ y = static_cast<T*>(a.y);
   const int tx = threadIdx.x % ST_TX, ty = (threadIdx.x / ST_TX) * ST_RY;  // first of ST_RY rows
@@ -107,18 +128,43 @@ k_stencil27(StencilArgs a) {
   double cen_m[ST_RY];                               // BOX: centre x of output zp-1
 #pragma unroll
   for (int r = 0; r < ST_RY; ++r) acc_m[r] = acc_c[r] = acc_p[r] = cen_m[r] = 0.0;
-  {
-    T v0[ST_LPT];
-    fetch(z0 - 1, v0);
-    stash(0, v0);
-  }
+  // cp.async staging of plane zp into ring slot `slot` (always one commit group)
+  auto issue = [&](int64_t zp, int slot) {
+    const bool zin = zp >= 0 && zp < nz && zp <= z1;
 #pragma unroll
-  for (int k = 0; k < ST_PF; ++k) fetch(z0 + k, v[k]);
-  __syncthreads();
+    for (int u = 0; u < ST_LPT; ++u) {
+      const int e = threadIdx.x + u * ST_NT;
+      if (e < ST_PN) {
+        const bool ok = zin && off[u] >= 0;
+        cp_async_zfill<sizeof(T)>(&pl[slot][e], ok ? x + zp * nxy + off[u] : x, ok ? int(sizeof(T)) : 0);
+      }
+    }
+    cp_async_commit();
+  };
   int cur = 0;
+  if (ST_ASYNC) {
+#pragma unroll
+    for (int k = 0; k < ST_NS - 1; ++k) issue(z0 - 1 + k, k);
+  } else {
+    {
+      T v0[ST_LPT];
+      fetch(z0 - 1, v0);
+      stash(0, v0);
+    }
+#pragma unroll
+    for (int k = 0; k < ST_PF; ++k) fetch(z0 + k, v[k]);
+    __syncthreads();
+  }
   for (int64_t zp = z0 - 1; zp <= z1; ++zp) {
     T vf[ST_LPT];
-    fetch(zp + 1 + ST_PF, vf);  // ST_PF planes ahead (zeros past z1: never stashed)
+    if (ST_ASYNC) {
+      // slot (cur + NS - 1) % NS was consumed in the previous iteration (barrier at its end)
+      issue(zp + ST_NS - 1, (cur + ST_NS - 1) % ST_NS);
+      cp_async_wait<ST_NS - 1>();  // plane zp has landed (the newest NS-1 groups may be in flight)
+      __syncthreads();
+    } else {
+      fetch(zp + 1 + ST_PF, vf);  // ST_PF planes ahead (zeros past z1: never stashed)
+    }
     const T* P = pl[cur];
     if (BOX) {
       double rs[ST_RY + 2];  // 3-point row sums of plane rows ty-1 .. ty+ST_RY
@@ -174,16 +220,22 @@ k_stencil27(StencilArgs a) {
       acc_c[r] = acc_p[r];
       acc_p[r] = 0.0;
     }
-    if (zp + 1 <= z1) stash(cur ^ 1, v[0]);
-    __syncthreads();
-    cur ^= 1;
+    if (ST_ASYNC) {
+      __syncthreads();  // every thread is done with slot cur before it is refilled
+      cur = (cur + 1) % ST_NS;
+    } else {
+      if (zp + 1 <= z1) stash(cur ^ 1, v[0]);
+      __syncthreads();
+      cur ^= 1;
 #pragma unroll
-    for (int k = 0; k + 1 < ST_PF; ++k)
+      for (int k = 0; k + 1 < ST_PF; ++k)
 #pragma unroll
-      for (int u = 0; u < ST_LPT; ++u) v[k][u] = v[k + 1][u];
+        for (int u = 0; u < ST_LPT; ++u) v[k][u] = v[k + 1][u];
 #pragma unroll
-    for (int u = 0; u < ST_LPT; ++u) v[ST_PF - 1][u] = vf[u];
+      for (int u = 0; u < ST_LPT; ++u) v[ST_PF - 1][u] = vf[u];
+    }
   }
+  if (ST_ASYNC) cp_async_wait<0>();  // no copy may outlive the CTA's shared memory
 }
 
 }  // namespace spmv
