@@ -132,7 +132,13 @@ struct spmv_csr_s {
     unsigned char* plan = nullptr;
     void (*k)(XplanArgs) = nullptr;
     void (*kdot)(XplanArgs) = nullptr;
+    // side split (SPMV_XPLAN_SIDE): rows [mplan, m) run concurrently in the
+    // vector kernel on the SMs the clusters leave idle
+    int64_t mplan = -1;
+    int g2 = 0;
   } xp;
+  cudaStream_t side = nullptr;
+  cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
   // SELL (SELL-32 device plan, x gathered from global memory)
   struct Sell {
     bool built = false;
@@ -429,8 +435,44 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
     CK(cudaMalloc(&a.tstamp, nb));
     CK(cudaMemsetAsync(a.tstamp, 0, nb, s));
   }
+  const bool side = h->xp.mplan >= 0 && h->xp.mplan < h->m_loc;
+  if (side) {
+    if (!h->side) {
+      CK(cudaStreamCreateWithFlags(&h->side, cudaStreamNonBlocking));
+      CK(cudaEventCreateWithFlags(&h->ev_fork, cudaEventDisableTiming));
+      CK(cudaEventCreateWithFlags(&h->ev_join, cudaEventDisableTiming));
+    }
+    CK(cudaEventRecord(h->ev_fork, s));
+    CK(cudaStreamWaitEvent(h->side, h->ev_fork, 0));
+  }
   CK(cudaLaunchKernelEx(&cfg, part ? h->xp.kdot : h->xp.k, a));
   LAUNCHED();
+  if (side) {
+    // rows [mplan, m) in the vector kernel, launched after the clusters so it
+    // takes the SMs they leave idle; its dot partials follow the clusters'
+    const int64_t ms = h->m_loc - h->xp.mplan;
+    SpmvArgs sa;
+    sa.m = ms;
+    sa.rowptr = h->rp_loc + h->xp.mplan;
+    sa.colidx = h->ci_loc;
+    sa.vals = h->vals;
+    sa.x = x;
+    sa.y = (char*)y + h->ts * (size_t)h->xp.mplan;
+    sa.alpha = a.alpha;
+    sa.beta = a.beta;
+    sa.w = w ? (const void*)(w + h->xp.mplan) : nullptr;
+    sa.part = part ? part + cfg.gridDim.x : nullptr;
+    sa.hk = P2PHook();
+    if (h->dt == SPMV_F64) {
+      if (part) launch_vec<double, true>(h->lanes, h->unroll, h->xp.g2, h->side, sa);
+      else launch_vec<double, false>(h->lanes, h->unroll, h->xp.g2, h->side, sa);
+    } else {
+      launch_vec<float, false>(h->lanes, h->unroll, h->xp.g2, h->side, sa);
+    }
+    LAUNCHED();
+    CK(cudaEventRecord(h->ev_join, h->side));
+    CK(cudaStreamWaitEvent(s, h->ev_join, 0));
+  }
   if (a.tstamp) {
     std::vector<unsigned long long> t(4 * cfg.gridDim.x);
     CK(cudaMemcpyAsync(t.data(), a.tstamp, sizeof(unsigned long long) * t.size(), cudaMemcpyDeviceToHost, s));
@@ -455,11 +497,11 @@ static spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only) 
   if (h->dt == SPMV_F64)
     k_xplan_pack<double><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const double*)vals, P.seg, h->m_loc, P.B, P.W,
                                           P.crow, P.tile0, P.ncl, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
-                                          values_only);
+                                          values_only, P.mplan);
   else
     k_xplan_pack<float><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const float*)vals, P.seg, h->m_loc, P.B, P.W,
                                          P.crow, P.tile0, P.ncl, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
-                                         values_only);
+                                         values_only, P.mplan);
   LAUNCHED();
   return SPMV_OK;
 }
@@ -533,8 +575,27 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   P.B = B; P.W = W; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd;
   DBG("B=%d W=%d ncl=%d smem=%zu", B, W, ncl, smem);
   const int64_t m = h->m_loc;
+  // side split: the last SPMV_XPLAN_SIDE per mille of the nonzeros go to the
+  // vector kernel on the idle SMs (single GPU only)
+  P.mplan = m;
+  {
+    int side_pm = 0;
+    env_int("SPMV_XPLAN_SIDE", &side_pm);
+    const int idle = num_sms(h->device) - ncl * B;
+    if (side_pm > 0 && side_pm < 500 && !h->dist && idle > 0) {
+      std::vector<int> rph((size_t)m + 1);
+      CK(cudaMemcpyAsync(rph.data(), h->rp_loc, sizeof(int) * (m + 1), cudaMemcpyDeviceToHost, s));
+      CK(cudaStreamSynchronize(s));
+      const long long nz = (long long)rph[m] - rph[0];
+      const long long target = rph[0] + nz - nz * side_pm / 1000;
+      P.mplan = std::lower_bound(rph.begin(), rph.end(), (int)target) - rph.begin();
+      P.mplan = std::min<int64_t>(std::max<int64_t>(P.mplan, 1), m);
+      P.g2 = idle * 8;
+      DBG("side split: plan rows %lld of %lld, side grid %d", (long long)P.mplan, (long long)m, P.g2);
+    }
+  }
   CK(cudaMalloc(&P.crow, sizeof(long long) * (ncl + 1)));
-  k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(m, h->rp_loc, ncl, P.crow);
+  k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(P.mplan, h->rp_loc, ncl, P.crow);
   LAUNCHED();
   std::vector<long long> crow(ncl + 1);
   CK(cudaMemcpyAsync(crow.data(), P.crow, sizeof(long long) * (ncl + 1), cudaMemcpyDeviceToHost, s));
@@ -1144,6 +1205,7 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
       if (ok) {
         h->kernel = SPMV_KERNEL_XPLAN;
         h->grid = (int64_t)h->xp.ncl * h->xp.B;
+        if (h->xp.mplan < h->m_loc) h->grid += h->xp.g2;  // dot partials: clusters, then the side kernel
       }
     }
   }
@@ -1211,6 +1273,9 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   for (void* b : bufs)
     if (b) cudaFree(b);
   if (h->cap) cudaStreamDestroy(h->cap);
+  if (h->side) cudaStreamDestroy(h->side);
+  if (h->ev_fork) cudaEventDestroy(h->ev_fork);
+  if (h->ev_join) cudaEventDestroy(h->ev_join);
   if (h->ev_a) cudaEventDestroy(h->ev_a);
   if (h->ev_b) cudaEventDestroy(h->ev_b);
   delete h;

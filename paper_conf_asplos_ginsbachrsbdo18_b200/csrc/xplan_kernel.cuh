@@ -394,9 +394,9 @@ k_xplan_pack(const int* __restrict__ rowptr, const int* __restrict__ colidx, con
              const int* __restrict__ seg, int64_t m, int B, int W, const long long* __restrict__ crow,
              const int* __restrict__ tile0, int ncl, const long long* __restrict__ chunk_off,
              const int* __restrict__ chunk_len, const int* __restrict__ row_slot, unsigned char* __restrict__ plan,
-             int values_only) {
+             int values_only, int64_t mplan /* rows [0, mplan) are in the plan */) {
   const int lane = threadIdx.x & 31;
-  for (int64_t i = (int64_t(blockIdx.x) * blockDim.x + threadIdx.x) / 32; i < m;
+  for (int64_t i = (int64_t(blockIdx.x) * blockDim.x + threadIdx.x) / 32; i < mplan;
        i += int64_t(gridDim.x) * blockDim.x / 32) {
     int lo = 0, hi = ncl - 1;
     while (lo < hi) {
