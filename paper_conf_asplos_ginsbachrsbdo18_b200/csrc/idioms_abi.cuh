@@ -123,7 +123,8 @@ extern "C" spmv_status idl_histogram(idl_hist_kind kind, const int32_t* keys, co
                                      int64_t nbins, void* bins, void* workspace, size_t workspace_bytes,
                                      void* stream) {
   size_t need = 0;
-  ST(idl_histogram_workspace(kind, n, nbins, &need));
+  ST(idl_histogram_workspace(kind, n, nbins, &need));  // validates kind, n, nbins
+  (void)need;
   if (kind == IDL_HIST_SUM_F64 ? false : w != nullptr) return arg_fail("w must be NULL for the counting kinds");
   if (kind == IDL_HIST_SAT_U8 && n > 4294967295LL) return arg_fail("IDL_HIST_SAT_U8 needs n < 2^32");
   const size_t fixed = hist_fixed_bytes(kind, nbins);
