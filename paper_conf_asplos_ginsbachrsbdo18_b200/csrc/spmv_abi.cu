@@ -978,7 +978,11 @@ static void choose_kernel(spmv_csr_s* h, int req_kernel, int req_lanes) {
   const int64_t groups_per_cta = 256 / lanes;
   h->grid = std::max<int64_t>(1, std::min<int64_t>(cdiv(h->m_loc, groups_per_cta), 8LL * sms));
   h->grid_vec = h->grid;
-  h->vgrid = std::max<int64_t>(1, std::min<int64_t>(cdiv(h->m_loc, 1024), 4LL * sms));
+  // CG vector kernels: elements per CTA (SPMV_VGRID_ELEMS overrides, for sweeps)
+  int vel = 1024;
+  env_int("SPMV_VGRID_ELEMS", &vel);
+  vel = std::max(vel, 32);
+  h->vgrid = std::max<int64_t>(1, std::min<int64_t>(cdiv(h->m_loc, vel), 4LL * sms));
 }
 
 // ----------------------------------------------------------------- create

@@ -73,7 +73,8 @@ def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--reps", type=int, default=20)
     ap.add_argument("--no-cpu", action="store_true")
-    ap.add_argument("which", nargs="*", default=["ep_C", "is_C", "histo", "dot_2p27", "jds_parboil"])
+    ap.add_argument("which", nargs="*", default=["ep_C", "is_C", "histo", "dot_2p27", "jds_parboil", "stencil256",
+                                                 "spmv_B", "spmv_parboil", "spmv_stencil256"])
     args = ap.parse_args()
     dev = torch.device("cuda:0")
     torch.cuda.set_device(dev)
@@ -162,6 +163,29 @@ def main():
         line("Parboil-shaped SpMV on the JDS-32 layout (fp32, 2^20 rows, 11.5M nnz)", us, us_min, 2.0 * A.nnz / 1e9,
              "GFLOP/s", alg, {"jds_entries": int(J.jds_ptr[-1]), "depth": J.depth})
         M.destroy()
+
+    if "stencil256" in args.which:
+        N = 256
+        x = torch.rand(N ** 3, dtype=torch.float64, device=dev)
+        y = torch.empty_like(x)
+        us, us_min = timed(lambda: sp.stencil27_apply(N, N, N, x, y), args.reps, flush)
+        # the matrix-free operator's own bytes: x once + y once (16 B per point, fp64)
+        line("matrix-free 27-point stencil 256^3 fp64 (R19 weights)", us, us_min, float(N ** 3), "points/s",
+             16 * N ** 3, {}, None)
+
+    for w in ("B", "parboil", "stencil256"):
+        if f"spmv_{w}" not in args.which:
+            continue
+        A = gen.powerlaw() if w == "parboil" else gen.stencil27(256) if w == "stencil256" else gen.makea(w)
+        dv = lambda a: torch.from_numpy(np.ascontiguousarray(a)).to(dev)
+        M = sp.CSRMatrix(dv(A.rowptr), dv(A.colidx), dv(A.vals), A.n)
+        x = dv(gen.uniform(A.n, seed=1, f32=A.vals.dtype == np.float32))
+        y = torch.empty(A.m, dtype=x.dtype, device=dev)
+        us, us_min = timed(lambda: M.spmv(x, y), args.reps, flush)
+        line(f"CSR SpMV {w} ({M.info()['kernel_name']}, {'fp32' if A.vals.dtype == np.float32 else 'fp64'})", us,
+             us_min, 2.0 * A.nnz / 1e9, "GFLOP/s", A.bytes_per_spmv(), {"nnz": int(A.nnz)}, None)
+        M.destroy()
+        del A
 
 
 if __name__ == "__main__":
