@@ -4,6 +4,7 @@
 mkdir -p gpurun_out
 timeout 900 python -m pytest tests/test_gpu_idioms.py -x -q > gpurun_out/pytest_idioms.log 2>&1
 echo "pytest exit $?" >> gpurun_out/pytest_idioms.log
+[ -x tools/microbench/dfma ] || nvcc -gencode arch=compute_100a,code=sm_100a -O3 -o tools/microbench/dfma tools/microbench/dfma.cu
 tools/microbench/dfma > gpurun_out/dfma.json 2>&1
 timeout 600 python tools/bench_idioms.py > gpurun_out/idioms.jsonl 2> gpurun_out/idioms.err
 if [ -n "$NCU" ]; then
