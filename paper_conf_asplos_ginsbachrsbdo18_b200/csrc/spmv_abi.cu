@@ -525,6 +525,7 @@ static spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   // 16 only when nothing smaller fits.  SPMV_XPLAN_B forces a size.
   int forced = 0;
   env_int("SPMV_XPLAN_B", &forced);
+  if (forced < Bneed || forced > 16 || XP_R % std::max(forced, 1)) forced = 0;  // infeasible request: ignored
   int B = 0, W = 0, ncl = 0;
   size_t smem = 0;
   for (int cand = (int)std::max<int64_t>(1, Bneed); cand <= 16; ++cand) {
