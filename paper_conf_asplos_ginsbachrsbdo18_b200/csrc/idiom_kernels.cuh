@@ -421,6 +421,7 @@ __device__ __forceinline__ uint64_t pow46(uint64_t base, uint64_t e) {
 
 // Thread t of the grid owns pairs [p0 + t*chunk, ...); out of the CTA: 12
 // partial sums (q[0..9] as exact integer-valued doubles, sx, sy) in part[c*12].
+template <bool EP_COMPACT>
 __global__ void __launch_bounds__(kEpThreads)
 k_ep(int64_t p0, int64_t count, int64_t chunk, double* __restrict__ out, unsigned* __restrict__ ticket,
      double* __restrict__ part) {
@@ -434,26 +435,68 @@ k_ep(int64_t p0, int64_t count, int64_t chunk, double* __restrict__ out, unsigne
   uint64_t s = mul46(kEpS, pow46(kEpA, 2ull * (uint64_t)(p0 + lo)));
   double sx = 0.0, sy = 0.0;
   unsigned q0 = 0, q1 = 0, q2 = 0, q3 = 0;
-  for (int64_t p = lo; p < hi; ++p) {
-    // x = 2u - 1 with u = s * 2^-46, exactly, without an int->double convert:
-    // the bits 0x3FF.. | s << 6 are the double 1 + s * 2^-46, and 2v - 3 = 2u - 1
+  // x = 2u - 1 with u = s * 2^-46, exactly, without an int->double convert:
+  // the bits 0x3FF.. | s << 6 are the double 1 + s * 2^-46, and 2v - 3 = 2u - 1
+  auto draw = [&](double& x1, double& x2) {
     s = mul46(s, kEpA);
     const double v1 = __longlong_as_double((long long)(0x3FF0000000000000ULL | (s << 6)));
     s = mul46(s, kEpA);
     const double v2 = __longlong_as_double((long long)(0x3FF0000000000000ULL | (s << 6)));
-    const double x1 = fma(2.0, v1, -3.0), x2 = fma(2.0, v2, -3.0);   // exact
+    x1 = fma(2.0, v1, -3.0);   // exact
+    x2 = fma(2.0, v2, -3.0);
+  };
+  auto tally = [&](double x1, double x2) {
     const double tt = __dadd_rn(__dmul_rn(x1, x1), __dmul_rn(x2, x2));  // NPB's rounding, no FMA
-    if (tt <= 1.0) {
-      const double f = sqrt(-2.0 * log(tt) / tt);
-      const double X = x1 * f, Y = x2 * f;
-      const int l = (int)fmax(fabs(X), fabs(Y));
-      q0 += (l == 0);
-      q1 += (l == 1);
-      q2 += (l == 2);
-      q3 += (l == 3);
-      if (l >= 4 && l < 10) atomicAdd(&qrare[l], 1ull);
-      sx += X;
-      sy += Y;
+    const double f = sqrt(-2.0 * log(tt) / tt);
+    const double X = x1 * f, Y = x2 * f;
+    const int l = (int)fmax(fabs(X), fabs(Y));
+    q0 += (l == 0);
+    q1 += (l == 1);
+    q2 += (l == 2);
+    q3 += (l == 3);
+    if (l >= 4 && l < 10) atomicAdd(&qrare[l], 1ull);
+    sx += X;
+    sy += Y;
+  };
+  if (EP_COMPACT) {
+    // warp-level compaction: accepted pairs (t <= 1, ~pi/4 of them) are queued
+    // in shared memory and tallied 32 at a time by the whole warp, so the
+    // log/div/sqrt body never runs with idle lanes
+    __shared__ double2 queue[kEpThreads / 32][64];
+    double2* qw = queue[threadIdx.x >> 5];
+    const int lane = threadIdx.x & 31;
+    const unsigned lt = (1u << lane) - 1u;
+    int cnt = 0;  // warp-uniform
+    for (int64_t it = 0; it < chunk; ++it) {
+      double x1 = 0.0, x2 = 0.0;
+      bool acc = false;
+      if (lo + it < hi) {
+        draw(x1, x2);
+        acc = __dadd_rn(__dmul_rn(x1, x1), __dmul_rn(x2, x2)) <= 1.0;
+      }
+      const unsigned m = __ballot_sync(0xffffffffu, acc);
+      if (acc) qw[cnt + __popc(m & lt)] = make_double2(x1, x2);
+      cnt += __popc(m);
+      if (cnt >= 32) {
+        __syncwarp();
+        const double2 e = qw[lane];
+        tally(e.x, e.y);
+        __syncwarp();
+        if (lane < cnt - 32) qw[lane] = qw[32 + lane];
+        __syncwarp();
+        cnt -= 32;
+      }
+    }
+    __syncwarp();
+    if (lane < cnt) {
+      const double2 e = qw[lane];
+      tally(e.x, e.y);
+    }
+  } else {
+    for (int64_t p = lo; p < hi; ++p) {
+      double x1, x2;
+      draw(x1, x2);
+      if (__dadd_rn(__dmul_rn(x1, x1), __dmul_rn(x2, x2)) <= 1.0) tally(x1, x2);
     }
   }
   double v[12];

@@ -272,8 +272,14 @@ extern "C" spmv_status ep_npb(int32_t M, int64_t pair_begin, int64_t pair_count,
   const int64_t T = std::max<int64_t>(1, std::min<int64_t>(8LL * sms * kEpThreads, cdiv(pair_count, 64)));
   const int64_t chunk = std::max<int64_t>(1, cdiv(pair_count, T));
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(kEpMaxGrid, cdiv(cdiv(pair_count, chunk), kEpThreads)));
-  k_ep<<<(int)grid, kEpThreads, 0, s>>>(pair_begin, pair_count, chunk, out, (unsigned*)workspace,
-                                        (double*)((char*)workspace + kWsHeader));
+  int compact = 1;  // SPMV_EP_COMPACT=0: per-thread tally without the warp queue
+  env_int("SPMV_EP_COMPACT", &compact);
+  if (compact)
+    k_ep<true><<<(int)grid, kEpThreads, 0, s>>>(pair_begin, pair_count, chunk, out, (unsigned*)workspace,
+                                               (double*)((char*)workspace + kWsHeader));
+  else
+    k_ep<false><<<(int)grid, kEpThreads, 0, s>>>(pair_begin, pair_count, chunk, out, (unsigned*)workspace,
+                                                (double*)((char*)workspace + kWsHeader));
   LAUNCHED();
   return SPMV_OK;
 }
