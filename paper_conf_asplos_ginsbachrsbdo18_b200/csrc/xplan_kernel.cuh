@@ -266,17 +266,29 @@ k_spmv_xplan(XplanArgs a) {
     const double* rv = recv + (t % XP_K) * R;
     const int64_t rt = r0c + int64_t(t) * R;
     const int nrows = int(cmin64(R, r1c - rt));
+    // the fused dot's w[i] (and beta*y[i]) do not depend on the partials: for
+    // the first row of each finalizer thread (all of them when RB <= nfin) the
+    // loads are issued before the wait so their latency hides behind it
+    const int jl0 = threadIdx.x;
+    const bool has0 = jl0 < RB && b * RB + jl0 < nrows;
+    double w0 = 0.0, y0 = 0.0;
+    if (has0) {
+      const int64_t i0 = rt + b * RB + jl0;
+      if (DOT) w0 = double(static_cast<const T*>(a.w)[i0]);
+      if (beta != 0.0) y0 = double(static_cast<const T*>(a.y)[i0]);
+    }
     mbar_wait(&tbar[t % XP_K], (t / XP_K) & 1, 1000000 * ntiles + 1000 * t + int(recv_bytes(t) / 8));
     for (int jl = threadIdx.x; jl < RB && b * RB + jl < nrows; jl += nfin) {
       double sum = 0.0;
       for (int q = 0; q < B; ++q) sum += rv[q * RB + jl];
       const int64_t i = rt + b * RB + jl;
       T* y = static_cast<T*>(a.y);
+      const bool first = jl == jl0;
       double r = alpha * sum;
-      if (beta != 0.0) r += beta * double(y[i]);
+      if (beta != 0.0) r += beta * (first ? y0 : double(y[i]));
       const T out = T(r);
       y[i] = out;
-      if (DOT) dacc += double(static_cast<const T*>(a.w)[i]) * double(out);
+      if (DOT) dacc += (first ? w0 : double(static_cast<const T*>(a.w)[i])) * double(out);
     }
     asm volatile("bar.sync 2, %0;\n" ::"r"(nfin) : "memory");
     if (threadIdx.x == 0 && t + XP_K < ntiles) mbar_expect_tx(&tbar[t % XP_K], recv_bytes(t + XP_K));
