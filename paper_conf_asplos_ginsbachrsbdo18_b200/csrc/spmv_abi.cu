@@ -1863,15 +1863,11 @@ extern "C" spmv_status stencil27_apply(spmv_dtype dt, int64_t nx, int64_t ny, in
   a.wd = a.w[13] - a.w[0];
   void (*kfn)(StencilArgs) = dt == SPMV_F64 ? (box ? k_stencil27<double, true> : k_stencil27<double, false>)
                                             : (box ? k_stencil27<float, true> : k_stencil27<float, false>);
-  // z ranges: ONE wave of resident CTAs (a partial second wave measured ~10 % slower
-  // on 256^3: 1280 CTAs for 1184 slots), each marching >= 16 planes (2 halo planes per range)
-  int per_sm = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kfn, ST_NT, 0) != cudaSuccess || per_sm < 1) {
-    cudaGetLastError();
-    per_sm = 8;
-  }
+  // z ranges: ~8 CTAs per SM, each marching >= 16 planes (2 halo planes per range).
+  // 256^3 with the cp.async ring (5 CTAs of 256 resident per SM, register-limited):
+  // 52 planes per CTA 70.7 us, 26 (this rule) 66.6 us, 24 70.7 us, 13 70.7 us, 7 76.8 us
   const int64_t bx = cdiv(nx, ST_TX), by = cdiv(ny, ST_TY);
-  int64_t zs = std::max<int64_t>(1, std::min<int64_t>((int64_t)per_sm * sms / (bx * by), cdiv(nz, 16)));
+  int64_t zs = std::max<int64_t>(1, std::min<int64_t>(cdiv(8LL * sms, bx * by), cdiv(nz, 16)));
   int zc = (int)cdiv(nz, zs);
   int env = 0;
   if (env_int("SPMV_STENCIL_ZCHUNK", &env) && env > 0) zc = env;

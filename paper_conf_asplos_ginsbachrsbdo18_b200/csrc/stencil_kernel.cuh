@@ -84,8 +84,11 @@ struct StencilArgs {
 // the three plane boxes of an output added in z.  ~11 fp64 operations per
 // point instead of 27 FMAs; a different summation order than the CSR row,
 // within reading R11's per-row bound (the bound holds |x_j| of all 27 terms).
+#ifndef ST_MINB_DEF
+#define ST_MINB_DEF 1
+#endif
 template <typename T, bool BOX>
-__global__ void __launch_bounds__(ST_NT)
+__global__ void __launch_bounds__(ST_NT, ST_MINB_DEF)
 k_stencil27(StencilArgs a) {
   __shared__ __align__(16) T pl[ST_ASYNC ? ST_NS : 2][ST_PN];
   const T* __restrict__ x = static_cast<const T*>(a.x);
