@@ -1866,7 +1866,12 @@ extern "C" spmv_status stencil27_apply(spmv_dtype dt, int64_t nx, int64_t ny, in
   // z ranges: ~8 CTAs per SM, each marching >= 16 planes (2 halo planes per range).
   // 256^3 with the cp.async ring (5 CTAs of 256 resident per SM, register-limited):
   // 52 planes per CTA 70.7 us, 26 (this rule) 66.6 us, 24 70.7 us, 13 70.7 us, 7 76.8 us
-  const int64_t bx = cdiv(nx, ST_TX), by = cdiv(ny, ST_TY);
+  // BOX with two columns per thread (k_stencil27_box2) unless SPMV_STENCIL_BOX2=0
+  int b2env = 1;
+  env_int("SPMV_STENCIL_BOX2", &b2env);
+  const bool box2 = box && b2env != 0;
+  if (box2) kfn = dt == SPMV_F64 ? k_stencil27_box2<double> : k_stencil27_box2<float>;
+  const int64_t bx = cdiv(nx, box2 ? SB_TX : ST_TX), by = cdiv(ny, box2 ? SB_TY : ST_TY);
   int64_t zs = std::max<int64_t>(1, std::min<int64_t>(cdiv(8LL * sms, bx * by), cdiv(nz, 16)));
   int zc = (int)cdiv(nz, zs);
   int env = 0;
@@ -1875,7 +1880,7 @@ extern "C" spmv_status stencil27_apply(spmv_dtype dt, int64_t nx, int64_t ny, in
   a.zchunk = zc;
   if (by > 65535 || zs > 65535) return arg_fail("grid too large for the stencil launch");
   const dim3 grid((unsigned)bx, (unsigned)by, (unsigned)zs);
-  kfn<<<grid, ST_NT, 0, s>>>(a);
+  kfn<<<grid, box2 ? SB_NT : ST_NT, 0, s>>>(a);
   LAUNCHED();
   return SPMV_OK;
 }

@@ -242,3 +242,127 @@ k_stencil27(StencilArgs a) {
 }
 
 }  // namespace spmv
+
+namespace spmv {
+
+// ---------------------------------------------------------------------------
+// BOX form with two adjacent columns per thread (k_stencil27_box2): the
+// x-direction row sums of columns 2c and 2c+1 share the plane values
+// x[2c-1..2c+2], read as two 16-B (fp64) / 8-B (fp32) shared loads instead
+// of six scalar ones, and the two centre values come out of the same loads.
+// Same staging (cp.async ring, zero-filled halo), same z marching and
+// summation order as the BOX form of k_stencil27.
+constexpr int SB_CX = 32;                  // column pairs per CTA row (warp)
+constexpr int SB_TX = 2 * SB_CX;           // 64 columns per tile
+constexpr int SB_NT = 256, SB_RY = 2;
+constexpr int SB_TY = (SB_NT / SB_CX) * SB_RY;  // 16 rows per tile
+constexpr int SB_PX = SB_TX + 2, SB_PY = SB_TY + 2, SB_PN = SB_PX * SB_PY;  // 66 x 18 (rows 16-B aligned)
+constexpr int SB_LPT = (SB_PN + SB_NT - 1) / SB_NT;
+
+template <typename T> struct V2;
+template <> struct V2<double> { using t = double2; };
+template <> struct V2<float> { using t = float2; };
+
+template <typename T>
+__global__ void __launch_bounds__(SB_NT)
+k_stencil27_box2(StencilArgs a) {
+  using V = typename V2<T>::t;
+  __shared__ __align__(16) T pl[ST_NS][SB_PN];
+  const T* __restrict__ x = static_cast<const T*>(a.x);
+  T* __restrict__ y = static_cast<T*>(a.y);
+  const int cx = threadIdx.x % SB_CX, ty = (threadIdx.x / SB_CX) * SB_RY;
+  const int64_t nx = a.nx, ny = a.ny, nz = a.nz, nxy = nx * ny;
+  const int64_t x0 = int64_t(blockIdx.x) * SB_TX, y0 = int64_t(blockIdx.y) * SB_TY;
+  const int64_t z0 = int64_t(blockIdx.z) * a.zchunk;
+  const int64_t z1 = cmin64(nz, z0 + a.zchunk);
+  const int64_t gx = x0 + 2 * cx, gy = y0 + ty;
+
+  int64_t off[SB_LPT];
+#pragma unroll
+  for (int u = 0; u < SB_LPT; ++u) {
+    const int e = threadIdx.x + u * SB_NT;
+    off[u] = -1;
+    if (e < SB_PN) {
+      const int64_t X = x0 + (e % SB_PX) - 1, Y = y0 + (e / SB_PX) - 1;
+      if (X >= 0 && X < nx && Y >= 0 && Y < ny) off[u] = X + nx * Y;
+    }
+  }
+  auto issue = [&](int64_t zp, int slot) {
+    const bool zin = zp >= 0 && zp < nz && zp <= z1;
+#pragma unroll
+    for (int u = 0; u < SB_LPT; ++u) {
+      const int e = threadIdx.x + u * SB_NT;
+      if (e < SB_PN) {
+        const bool ok = zin && off[u] >= 0;
+        cp_async_zfill<sizeof(T)>(&pl[slot][e], ok ? x + zp * nxy + off[u] : x, ok ? int(sizeof(T)) : 0);
+      }
+    }
+    cp_async_commit();
+  };
+  const double alpha = a.alpha, beta = a.beta;
+  double acc_m[SB_RY][2], acc_c[SB_RY][2], acc_p[SB_RY][2], cen_m[SB_RY][2];
+#pragma unroll
+  for (int r = 0; r < SB_RY; ++r)
+#pragma unroll
+    for (int c = 0; c < 2; ++c) acc_m[r][c] = acc_c[r][c] = acc_p[r][c] = cen_m[r][c] = 0.0;
+#pragma unroll
+  for (int k = 0; k < ST_NS - 1; ++k) issue(z0 - 1 + k, k);
+  int cur = 0;
+  for (int64_t zp = z0 - 1; zp <= z1; ++zp) {
+    issue(zp + ST_NS - 1, (cur + ST_NS - 1) % ST_NS);
+    cp_async_wait<ST_NS - 1>();
+    __syncthreads();
+    const T* P = pl[cur];
+    double rs0[SB_RY + 2], rs1[SB_RY + 2], cc0[SB_RY], cc1[SB_RY];
+#pragma unroll
+    for (int sy = 0; sy < SB_RY + 2; ++sy) {
+      const V* q = reinterpret_cast<const V*>(P + (ty + sy) * SB_PX + 2 * cx);
+      const V lo = q[0], hi = q[1];  // x[2c-1], x[2c], x[2c+1], x[2c+2] of plane row ty+sy-1
+      const double e0 = double(lo.x), e1 = double(lo.y), e2 = double(hi.x), e3 = double(hi.y);
+      rs0[sy] = (e0 + e1) + e2;
+      rs1[sy] = (e1 + e2) + e3;
+      if (sy >= 1 && sy <= SB_RY) {
+        cc0[sy - 1] = e1;
+        cc1[sy - 1] = e2;
+      }
+    }
+#pragma unroll
+    for (int r = 0; r < SB_RY; ++r) {
+      const double b0 = (rs0[r] + rs0[r + 1]) + rs0[r + 2];
+      const double b1 = (rs1[r] + rs1[r + 1]) + rs1[r + 2];
+      acc_p[r][0] += b0; acc_c[r][0] += b0; acc_m[r][0] += b0;
+      acc_p[r][1] += b1; acc_c[r][1] += b1; acc_m[r][1] += b1;
+    }
+    const int64_t zo = zp - 1;
+    if (zo >= z0 && zo < z1) {
+#pragma unroll
+      for (int r = 0; r < SB_RY; ++r) {
+        if (gy + r >= ny) continue;
+#pragma unroll
+        for (int c = 0; c < 2; ++c) {
+          if (gx + c >= nx) continue;
+          const int64_t p = gx + c + nx * (gy + r) + nxy * zo;
+          double res = alpha * fma(a.wd, cen_m[r][c], a.wn * acc_m[r][c]);
+          if (beta != 0.0) res += beta * double(y[p]);
+          y[p] = T(res);
+        }
+      }
+    }
+#pragma unroll
+    for (int r = 0; r < SB_RY; ++r) {
+      cen_m[r][0] = cc0[r];
+      cen_m[r][1] = cc1[r];
+#pragma unroll
+      for (int c = 0; c < 2; ++c) {
+        acc_m[r][c] = acc_c[r][c];
+        acc_c[r][c] = acc_p[r][c];
+        acc_p[r][c] = 0.0;
+      }
+    }
+    __syncthreads();
+    cur = (cur + 1) % ST_NS;
+  }
+  cp_async_wait<0>();
+}
+
+}  // namespace spmv

@@ -133,7 +133,7 @@ def test_stencil256_full_size(env):
     assert np.array_equal(yy.cpu().numpy(), (27 - cnt).astype(np.float64))
 
 
-@pytest.mark.parametrize("dims", [(33, 9, 17), (64, 64, 64), (5, 1, 130)])
+@pytest.mark.parametrize("dims", [(33, 9, 17), (64, 64, 64), (5, 1, 130), (65, 17, 3), (2, 2, 2)])
 def test_stencil_box_form(env, dims, monkeypatch):
     """Equal neighbour weights select the separable box-sum form: R19's Laplacian,
     all 27 weights equal, and an arbitrary (centre, neighbour) pair; each within
@@ -143,6 +143,10 @@ def test_stencil_box_form(env, dims, monkeypatch):
     for w in (None, np.full(27, 0.37), np.where(np.arange(27) == 13, 5.5, -0.25)):
         y, y_ref, bound = _run(env, dims, x, w=w)
         check_rows(y, y_ref, bound, np.float64, f"box {dims}")
+        monkeypatch.setenv("SPMV_STENCIL_BOX2", "0")                    # one column per thread
+        y1, _, _ = _run(env, dims, x, w=w)
+        monkeypatch.delenv("SPMV_STENCIL_BOX2")
+        check_rows(y1, y_ref, bound, np.float64, f"box1 {dims}")
         monkeypatch.setenv("SPMV_STENCIL_BOX", "0")
         y2, _, _ = _run(env, dims, x, w=w)
         monkeypatch.delenv("SPMV_STENCIL_BOX")
