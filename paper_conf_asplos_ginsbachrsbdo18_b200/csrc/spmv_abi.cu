@@ -1869,7 +1869,7 @@ extern "C" spmv_status stencil27_apply(spmv_dtype dt, int64_t nx, int64_t ny, in
   // BOX with two columns per thread (k_stencil27_box2) unless SPMV_STENCIL_BOX2=0
   int b2env = 1;
   env_int("SPMV_STENCIL_BOX2", &b2env);
-  const bool box2 = box && b2env != 0;
+  const bool box2 = box && b2env != 0 && nx * ny < 2147483647LL;  // 32-bit in-plane offsets
   if (box2) kfn = dt == SPMV_F64 ? k_stencil27_box2<double> : k_stencil27_box2<float>;
   const int64_t bx = cdiv(nx, box2 ? SB_TX : ST_TX), by = cdiv(ny, box2 ? SB_TY : ST_TY);
   int64_t zs = std::max<int64_t>(1, std::min<int64_t>(cdiv(8LL * sms, bx * by), cdiv(nz, 16)));

@@ -254,7 +254,10 @@ namespace spmv {
 // summation order as the BOX form of k_stencil27.
 constexpr int SB_CX = 32;                  // column pairs per CTA row (warp)
 constexpr int SB_TX = 2 * SB_CX;           // 64 columns per tile
-constexpr int SB_NT = 256, SB_RY = 2;
+#ifndef SB_RY_DEF
+#define SB_RY_DEF 2
+#endif
+constexpr int SB_NT = 256, SB_RY = SB_RY_DEF;
 constexpr int SB_TY = (SB_NT / SB_CX) * SB_RY;  // 16 rows per tile
 constexpr int SB_PX = SB_TX + 2, SB_PY = SB_TY + 2, SB_PN = SB_PX * SB_PY;  // 66 x 18 (rows 16-B aligned)
 constexpr int SB_LPT = (SB_PN + SB_NT - 1) / SB_NT;
@@ -277,14 +280,14 @@ k_stencil27_box2(StencilArgs a) {
   const int64_t z1 = cmin64(nz, z0 + a.zchunk);
   const int64_t gx = x0 + 2 * cx, gy = y0 + ty;
 
-  int64_t off[SB_LPT];
+  int off[SB_LPT];  // in-plane offsets (the host guarantees nx*ny < 2^31); -1 = outside
 #pragma unroll
   for (int u = 0; u < SB_LPT; ++u) {
     const int e = threadIdx.x + u * SB_NT;
     off[u] = -1;
     if (e < SB_PN) {
       const int64_t X = x0 + (e % SB_PX) - 1, Y = y0 + (e / SB_PX) - 1;
-      if (X >= 0 && X < nx && Y >= 0 && Y < ny) off[u] = X + nx * Y;
+      if (X >= 0 && X < nx && Y >= 0 && Y < ny) off[u] = int(X + nx * Y);
     }
   }
   auto issue = [&](int64_t zp, int slot) {
