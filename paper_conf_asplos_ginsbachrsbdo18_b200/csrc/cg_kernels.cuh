@@ -154,22 +154,44 @@ k_cgcg(int64_t n, int k, SumSrc gam, SumSrc gam_old, SumSrc del, double* __restr
        double* __restrict__ z, double* __restrict__ r, double* __restrict__ part_rr_new,
        int* __restrict__ flags, double tol, SumSrc rr_b, P2PHook hk, int64_t xoff) {
   __shared__ double red[8];
-  __shared__ double s_g, s_go, s_d, s_b;
+  __shared__ double sc[4];
   if (flags[1]) return;  // converged (tol mode): no-op
-  const double g = read_sum(gam, &s_g);
-  if (tol > 0.0) {
-    const double bb = read_sum(rr_b, &s_b);
-    if (sqrt(g) <= tol * sqrt(bb)) {
-      if (blockIdx.x == 0 && threadIdx.x == 0) flags[1] = 1;
-      return;
+  const int64_t stride = int64_t(gridDim.x) * blockDim.x;
+  const int64_t jstart = int64_t(blockIdx.x) * blockDim.x + threadIdx.x;
+  double pr[CG_U], pw[CG_U], pp[CG_U], ps[CG_U], pz[CG_U];
+  auto load = [&](int64_t j0) {
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) {
+        pr[u] = r[j]; pw[u] = w[j]; pz[u] = z[j];
+        if (k > 0) { pp[u] = p[j]; ps[u] = sv[j]; }
+      }
     }
+  };
+  // the first batch of vector loads does not depend on the scalars: issue it,
+  // then read the (up to four) scalar sources concurrently, one warp each
+  if (jstart < n) load(jstart);
+  {
+    const int wid = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    double v = 0.0;
+    if (wid == 0) v = warp_read_sum(gam);
+    else if (wid == 1) v = warp_read_sum(del);
+    else if (wid == 2 && k > 0) v = warp_read_sum(gam_old);
+    else if (wid == 3 && tol > 0.0) v = warp_read_sum(rr_b);
+    if (wid < 4 && lane == 0) sc[wid] = v;
+    __syncthreads();
   }
-  const double d = read_sum(del, &s_d);
+  const double g = sc[0], d = sc[1];
+  if (tol > 0.0 && sqrt(g) <= tol * sqrt(sc[3])) {
+    if (blockIdx.x == 0 && threadIdx.x == 0) flags[1] = 1;
+    return;
+  }
   double beta = 0.0, alpha, pap;
   if (k == 0) {
     pap = d;
   } else {
-    const double go = read_sum(gam_old, &s_go);
+    const double go = sc[2];
     beta = g / go;
     pap = d - beta * g / __ldcg(alpha2 + ((k - 1) & 1));
   }
@@ -180,17 +202,8 @@ k_cgcg(int64_t n, int k, SumSrc gam, SumSrc gam_old, SumSrc del, double* __restr
     flags[2] = k + 1;
   }
   double acc = 0.0;
-  const int64_t stride = int64_t(gridDim.x) * blockDim.x;
-  for (int64_t j0 = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j0 < n; j0 += CG_U * stride) {
-    double pr[CG_U], pw[CG_U], pp[CG_U], ps[CG_U], pz[CG_U];
-#pragma unroll
-    for (int u = 0; u < CG_U; ++u) {
-      const int64_t j = j0 + u * stride;
-      if (j < n) {
-        pr[u] = r[j]; pw[u] = w[j]; pz[u] = z[j];
-        if (k > 0) { pp[u] = p[j]; ps[u] = sv[j]; }
-      }
-    }
+  for (int64_t j0 = jstart; j0 < n; j0 += CG_U * stride) {
+    if (j0 != jstart) load(j0);
 #pragma unroll
     for (int u = 0; u < CG_U; ++u) {
       const int64_t j = j0 + u * stride;

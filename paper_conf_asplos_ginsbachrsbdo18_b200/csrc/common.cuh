@@ -234,4 +234,24 @@ __device__ __forceinline__ double read_sum(SumSrc s, double* slot) {
   return v;
 }
 
+// The same sum as read_sum (same order, bit-identical), computed by ONE warp
+// without a block barrier, so several warps can read different sources at
+// once; the value is returned in every lane of the calling warp.
+__device__ __forceinline__ double warp_read_sum(SumSrc s) {
+  const int lane = threadIdx.x & 31;
+  int n = s.count;
+  double a = 0.0;
+  if (n < 0) {
+    n = -n;
+    if (lane == 0) {
+      p2p_wait_flags(s.flags, s.me, n, *s.epoch);
+      for (int i = 0; i < n; ++i) a += s.p[i];  // rank order
+    }
+    return __shfl_sync(0xffffffffu, a, 0);
+  }
+#pragma unroll 4
+  for (int i = lane; i < n; i += 32) a += s.p[i];
+  return warp_sum(a);
+}
+
 }  // namespace spmv
