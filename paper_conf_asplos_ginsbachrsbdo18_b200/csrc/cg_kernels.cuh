@@ -43,10 +43,17 @@ k_cg_zr(int64_t n, SumSrc pq, SumSrc rr_old, const double* __restrict__ p,
         const double* __restrict__ q, double* __restrict__ z, double* __restrict__ r,
         double* __restrict__ part_rr_new, int* __restrict__ flags, P2PHook hk) {
   __shared__ double red[8];
-  __shared__ double s_pq, s_rr;
+  __shared__ double sc[2];
   if (flags[1]) return;  // converged (tol mode): no-op
-  const double d = read_sum(pq, &s_pq);
-  const double rho = read_sum(rr_old, &s_rr);
+  {  // both scalar sources at once, one warp each (bit-identical to read_sum)
+    const int wid = threadIdx.x >> 5;
+    double v = 0.0;
+    if (wid == 0) v = warp_read_sum(pq);
+    else if (wid == 1) v = warp_read_sum(rr_old);
+    if (wid < 2 && (threadIdx.x & 31) == 0) sc[wid] = v;
+    __syncthreads();
+  }
+  const double d = sc[0], rho = sc[1];
   if (d == 0.0 || !isfinite(d)) {
     if (blockIdx.x == 0 && threadIdx.x == 0) flags[0] = 1;
   }
@@ -84,10 +91,18 @@ __global__ void __launch_bounds__(256)
 k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
        double* __restrict__ p, int* __restrict__ flags, double tol, SumSrc rr_b, int it, P2PHook hk,
        int64_t xoff) {
-  __shared__ double s_new, s_old, s_b;
+  __shared__ double s_b;
+  __shared__ double sc[2];
   if (flags[1]) return;
-  const double rho1 = read_sum(rr_new, &s_new);
-  const double rho0 = read_sum(rr_old, &s_old);
+  {  // both scalar sources at once, one warp each (bit-identical to read_sum)
+    const int wid = threadIdx.x >> 5;
+    double v = 0.0;
+    if (wid == 0) v = warp_read_sum(rr_new);
+    else if (wid == 1) v = warp_read_sum(rr_old);
+    if (wid < 2 && (threadIdx.x & 31) == 0) sc[wid] = v;
+    __syncthreads();
+  }
+  const double rho1 = sc[0], rho0 = sc[1];
   const double beta = rho1 / rho0;
   const int64_t stride = int64_t(gridDim.x) * blockDim.x;
   for (int64_t j0 = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j0 < n; j0 += CG_U * stride) {
