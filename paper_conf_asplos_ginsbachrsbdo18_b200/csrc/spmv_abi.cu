@@ -1595,10 +1595,6 @@ extern "C" spmv_status cg_solve(spmv_csr_t h, const void* b, void* x, int32_t ma
   ST(stage_in(h, s, b, &h->stage_x, &bd, true));
   ST(stage_in(h, s, x, &h->stage_z, &xd, false));
   double* xw = const_cast<double*>(xd);
-  if (tol > 0.0 && h->cg_variant == 1 && use_p2p(h)) {
-    g_err = "tol > 0 with the single-reduction CG needs the NCCL or single-GPU transport";
-    return SPMV_ERR_UNSUPPORTED;
-  }
   CK(cudaMemsetAsync(h->flags, 0, sizeof(int) * 4, s));
   CgRun run;
   ST(cg_enqueue_init(h, s, bd, xw, &run));

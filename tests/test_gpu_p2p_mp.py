@@ -88,6 +88,12 @@ def _worker(rank, world, port, q):
                 its, rn = M.cg_solve(bvec, xs, 200, tol=1e-10)
                 assert rn <= 1e-9 * np.sqrt(A.n), (kernel, its, rn)
                 out[f"stencil_{kernel}_its"] = its
+                if kernel == "auto":  # single-reduction CG with early stop over the p2p transport
+                    M.set_cg_variant("cgcg")
+                    its2, rn2 = M.cg_solve(bvec, xs, 200, tol=1e-10)
+                    M.set_cg_variant("textbook")
+                    assert rn2 <= 1e-9 * np.sqrt(A.n) and abs(its2 - its) <= 1, (its, its2, rn2)
+                    out["stencil_cgcg_its"] = its2
         dist.barrier()
         d.close()
         dist.destroy_process_group()
