@@ -49,7 +49,7 @@ constexpr int XP_R = 32 * XP_CPT;    // rows per tile
 constexpr int XP_THREADS = 32 * XP_NW;
 constexpr int XP_K = 3;              // receive buffers
 #ifndef XP_U_DEF
-#define XP_U_DEF 8
+#define XP_U_DEF 9
 #endif
 constexpr int XP_U = XP_U_DEF;       // step pairs (16-B loads) in flight per lane
 
