@@ -24,6 +24,9 @@ namespace spmv {
 #endif
 constexpr int JDS_SEG = JDS_SEG_DEF;  // diagonal steps per warp unit
 constexpr int JDS_THREADS = 256;
+#ifndef JDS_PRED
+#define JDS_PRED 1
+#endif
 
 // unit: {slice, k0, k1, part}; part < 0: the slice's only unit (writes y)
 template <typename T>
@@ -38,6 +41,31 @@ k_spmv_jds(const int4* __restrict__ units, int nunits, int64_t m, const long lon
   const int4 u = units[warp];
   const int64_t i = (int64_t)u.x * 32 + lane;
   double acc = 0.0;
+#if JDS_PRED
+  // batches of 4 steps, the tail batch predicated (no step-by-step tail)
+  for (int k = u.y; k < u.z; k += 4) {
+    long long jp[4];
+#pragma unroll
+    for (int q = 0; q < 4; ++q) jp[q] = k + q < u.z ? __ldg(jds_ptr + k + q) : 0;
+    T d[4];
+    int c[4];
+#pragma unroll
+    for (int q = 0; q < 4; ++q) {
+      d[q] = T(0);
+      c[q] = 0;
+      if (k + q < u.z) {
+        d[q] = ld_stream(data + jp[q] + i);
+        c[q] = ld_stream(idx + jp[q] + i);
+      }
+    }
+    T xv[4];
+#pragma unroll
+    for (int q = 0; q < 4; ++q) xv[q] = ld_x(x + c[q]);   // c = 0 on masked steps (x[0] valid)
+#pragma unroll
+    for (int q = 0; q < 4; ++q)
+      if (k + q < u.z) acc = fma((double)d[q], (double)xv[q], acc);
+  }
+#else
   int k = u.y;
   for (; k + 4 <= u.z; k += 4) {
     T d[4];
@@ -58,6 +86,7 @@ k_spmv_jds(const int4* __restrict__ units, int nunits, int64_t m, const long lon
     const int64_t j = __ldg(jds_ptr + k) + i;
     acc = fma((double)ld_stream(data + j), (double)ld_x(x + ld_stream(idx + j)), acc);
   }
+#endif
   if (u.w < 0) {
     if (i < m) {
       const int row = perm[i];
