@@ -41,7 +41,7 @@ namespace spmv {
 
 constexpr int SELL_NT = 256;  // threads per CTA
 #ifndef SELL_U_DEF
-#define SELL_U_DEF 4
+#define SELL_U_DEF 2
 #endif
 constexpr int SELL_U = SELL_U_DEF;  // step pairs in flight per lane
 
