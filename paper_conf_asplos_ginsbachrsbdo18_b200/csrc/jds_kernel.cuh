@@ -27,6 +27,9 @@ constexpr int JDS_THREADS = 256;
 #ifndef JDS_PRED
 #define JDS_PRED 1
 #endif
+#ifndef JDS_B
+#define JDS_B 4   // diagonal steps per predicated batch
+#endif
 
 // unit: {slice, k0, k1, part}; part < 0: the slice's only unit (writes y)
 template <typename T>
@@ -42,15 +45,15 @@ k_spmv_jds(const int4* __restrict__ units, int nunits, int64_t m, const long lon
   const int64_t i = (int64_t)u.x * 32 + lane;
   double acc = 0.0;
 #if JDS_PRED
-  // batches of 4 steps, the tail batch predicated (no step-by-step tail)
-  for (int k = u.y; k < u.z; k += 4) {
-    long long jp[4];
+  // batches of JDS_B steps, the tail batch predicated (no step-by-step tail)
+  for (int k = u.y; k < u.z; k += JDS_B) {
+    long long jp[JDS_B];
 #pragma unroll
-    for (int q = 0; q < 4; ++q) jp[q] = k + q < u.z ? __ldg(jds_ptr + k + q) : 0;
-    T d[4];
-    int c[4];
+    for (int q = 0; q < JDS_B; ++q) jp[q] = k + q < u.z ? __ldg(jds_ptr + k + q) : 0;
+    T d[JDS_B];
+    int c[JDS_B];
 #pragma unroll
-    for (int q = 0; q < 4; ++q) {
+    for (int q = 0; q < JDS_B; ++q) {
       d[q] = T(0);
       c[q] = 0;
       if (k + q < u.z) {
@@ -58,11 +61,11 @@ k_spmv_jds(const int4* __restrict__ units, int nunits, int64_t m, const long lon
         c[q] = ld_stream(idx + jp[q] + i);
       }
     }
-    T xv[4];
+    T xv[JDS_B];
 #pragma unroll
-    for (int q = 0; q < 4; ++q) xv[q] = ld_x(x + c[q]);   // c = 0 on masked steps (x[0] valid)
+    for (int q = 0; q < JDS_B; ++q) xv[q] = ld_x(x + c[q]);   // c = 0 on masked steps (x[0] valid)
 #pragma unroll
-    for (int q = 0; q < 4; ++q)
+    for (int q = 0; q < JDS_B; ++q)
       if (k + q < u.z) acc = fma((double)d[q], (double)xv[q], acc);
   }
 #else
