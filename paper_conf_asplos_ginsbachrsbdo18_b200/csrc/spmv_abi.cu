@@ -94,7 +94,8 @@ struct spmv_csr_s {
   int device = 0;
   cudaStream_t stream = nullptr;      // user stream (may be the legacy stream 0)
   cudaStream_t cap = nullptr;         // private stream used for graph capture
-  cudaEvent_t ev_a = nullptr, ev_b = nullptr;
+  cudaEvent_t ev_a = nullptr, ev_b = nullptr;  // ev_a: z final inside the NPB graph (external event)
+  cudaStream_t copy = nullptr;                 // D2H of z overlapping the residual SpMV
   spmv_dtype dt = SPMV_F64;
   size_t ts = 8;
   int64_t m = 0, n = 0, nnz = 0;
@@ -1282,6 +1283,7 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   if (h->ev_fork) cudaEventDestroy(h->ev_fork);
   if (h->ev_join) cudaEventDestroy(h->ev_join);
   if (h->ev_a) cudaEventDestroy(h->ev_a);
+  if (h->copy) cudaStreamDestroy(h->copy);
   if (h->ev_b) cudaEventDestroy(h->ev_b);
   delete h;
   return st;
@@ -1636,6 +1638,11 @@ static spmv_status npb_enqueue(spmv_csr_s* h, cudaStream_t s, double* x, double*
   CgRun run;
   ST(cg_enqueue_init(h, s, x, z, &run));
   ST(cg_enqueue_iters(h, s, z, cgitmax, 0.0, &run));
+  // z is final here: an external event lets the host copy of z overlap the residual
+  cudaStreamCaptureStatus cst = cudaStreamCaptureStatusNone;
+  CK(cudaStreamIsCapturing(s, &cst));
+  if (cst == cudaStreamCaptureStatusActive) CK(cudaEventRecordWithFlags(h->ev_a, s, cudaEventRecordExternal));
+  else CK(cudaEventRecord(h->ev_a, s));
   ST(cg_resid<true>(h, s, x, z));
   SumSrc res, xz, zz;
   const int vg = (int)h->vgrid;
@@ -1700,8 +1707,14 @@ extern "C" spmv_status cg_npb_outer(spmv_csr_t h, void* x, void* z, int32_t cgit
     CK(cudaMemcpyAsync(x, xd, sizeof(double) * h->m_loc, cudaMemcpyDeviceToHost, s));
     sync = true;
   }
+  bool copy_used = false;
   if (zd != z && h->m_loc > 0) {
-    CK(cudaMemcpyAsync(z, zd, sizeof(double) * h->m_loc, cudaMemcpyDeviceToHost, s));
+    // z (host) is copied on a side stream as soon as the CG loop wrote it,
+    // overlapping the residual SpMV and the finishing kernel
+    if (!h->copy) CK(cudaStreamCreateWithFlags(&h->copy, cudaStreamNonBlocking));
+    CK(cudaStreamWaitEvent(h->copy, h->ev_a, 0));
+    CK(cudaMemcpyAsync(z, zd, sizeof(double) * h->m_loc, cudaMemcpyDeviceToHost, h->copy));
+    copy_used = true;
     sync = true;
   }
   if (ok != 1) {
@@ -1712,6 +1725,7 @@ extern "C" spmv_status cg_npb_outer(spmv_csr_t h, void* x, void* z, int32_t cgit
     int hf[4];
     CK(cudaMemcpyAsync(hf, h->flags, sizeof(int) * 4, cudaMemcpyDeviceToHost, s));
     CK(cudaStreamSynchronize(s));
+    if (copy_used) CK(cudaStreamSynchronize(h->copy));
     if (hf[0]) { g_err = "CG breakdown"; return SPMV_ERR_BREAKDOWN; }
   }
   return SPMV_OK;

@@ -96,6 +96,27 @@ def test_cg_breakdown(sp, torch_dev):
         assert e.value.status == sp.SPMV_ERR_BREAKDOWN
 
 
+def test_npb_host_z_equals_device_z(sp, torch_dev):
+    """The host copy of z (made on a side stream after an event inside the NPB
+    graph, overlapping the residual) equals the device-path z bit for bit."""
+    torch, dev = torch_dev
+    A = gen.makea("S")
+    rp, ci, va = to_dev(A, dev)
+    with sp.CSRMatrix(rp, ci, va, A.n) as M:
+        xd = torch.ones(A.n, dtype=torch.float64, device=dev)
+        zd = torch.empty_like(xd)
+        od = torch.zeros(2, dtype=torch.float64, device=dev)
+        xh = torch.ones(A.n, dtype=torch.float64).pin_memory()
+        zh = torch.empty(A.n, dtype=torch.float64).pin_memory()
+        oh = torch.zeros(2, dtype=torch.float64).pin_memory()
+        for it in range(4):
+            M.npb_outer(xd, zd, 25, 10.0, od)
+            M.npb_outer(xh, zh, 25, 10.0, oh)
+            torch.cuda.synchronize()
+            assert torch.equal(zd.cpu(), zh) and torch.equal(xd.cpu(), xh), it
+            assert torch.equal(od.cpu(), oh)
+
+
 def _npb(sp, torch, dev, cls, niter=None, host=False):
     na, nonzer, NITER, shift = gen.NPB_CLASSES[cls]
     A = gen.makea(cls)
