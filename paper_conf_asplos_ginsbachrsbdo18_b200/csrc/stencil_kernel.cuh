@@ -29,7 +29,9 @@
 // uniform registers); 2 rows per thread 76-78 us (shared loads and loop
 // overhead amortised), 4 rows 80 us (register-limited occupancy).
 #pragma once
+#include <cuda.h>  // CUtensorMap (the TMA form of k_stencil27_box2)
 #include "common.cuh"
+#include "xstat_kernel.cuh"  // smem_u32 / mbarrier helpers
 
 namespace spmv {
 
@@ -259,48 +261,102 @@ constexpr int SB_TX = 2 * SB_CX;           // 64 columns per tile
 #endif
 constexpr int SB_NT = 256, SB_RY = SB_RY_DEF;
 constexpr int SB_TY = (SB_NT / SB_CX) * SB_RY;  // 16 rows per tile
-constexpr int SB_PX = SB_TX + 2, SB_PY = SB_TY + 2, SB_PN = SB_PX * SB_PY;  // 66 x 18 (rows 16-B aligned)
-constexpr int SB_LPT = (SB_PN + SB_NT - 1) / SB_NT;
+constexpr int SB_PY = SB_TY + 2;  // 18 staged rows
 
 template <typename T> struct V2;
 template <> struct V2<double> { using t = double2; };
 template <> struct V2<float> { using t = float2; };
 
-template <typename T>
+// TMA: the plane tile (PX x 18, one-point halo) is one cp.async.bulk.tensor.3d
+// box at (x0-1, y0-1, zp) issued by one thread; the tensor map's out-of-bound
+// fill supplies the zero halo outside the grid (nx, ny); planes zp < 0 or
+// zp >= nz are zero-filled by the CTA's threads instead (no copy issued).  The
+// box's inner extent must be a multiple of 16 B: 66 fp64 (528 B), 68 fp32,
+// and so must its innermost start coordinate (measured on this B200: an
+// origin at x = -1 fp64 traps with an illegal instruction, x = -2 zero-fills;
+// profiles/r01q_tma3d_origin_check.txt).  The TMA tiles are therefore shifted
+// left by SHIFT columns (output columns [64 bx - SHIFT, 64 bx + 64 - SHIFT),
+// staged from 64 bx - SHIFT - 1, a multiple of 16 B), which keeps each
+// thread's 4 staged values one aligned pair of vector loads.
+template <typename T, bool TMA> struct SBL {
+  static constexpr int SHIFT = TMA ? (sizeof(T) == 8 ? 1 : 3) : 0;
+  static constexpr int PX = (TMA && sizeof(T) == 4) ? SB_TX + 4 : SB_TX + 2;  // staged row pitch
+  static constexpr int PN = PX * SB_PY;
+  static constexpr int SLOT = TMA ? ((PN * int(sizeof(T)) + 127) / 128) * 128 / int(sizeof(T)) : PN;
+  static constexpr int LPT = (PN + SB_NT - 1) / SB_NT;
+};
+
+__device__ __forceinline__ void tma_load_3d(void* dst, uint64_t tm, int c0, int c1, int c2, uint64_t* bar) {
+  asm volatile(
+      "cp.async.bulk.tensor.3d.shared::cluster.global.tile.mbarrier::complete_tx::bytes [%0], [%1, {%2, %3, %4}], "
+      "[%5];\n" ::"r"(smem_u32(dst)),
+      "l"(tm), "r"(c0), "r"(c1), "r"(c2), "r"(smem_u32(bar))
+      : "memory");
+}
+
+template <typename T, bool TMA>
 __global__ void __launch_bounds__(SB_NT)
-k_stencil27_box2(StencilArgs a) {
+k_stencil27_box2(StencilArgs a, const __grid_constant__ CUtensorMap tm) {
   using V = typename V2<T>::t;
-  __shared__ __align__(16) T pl[ST_NS][SB_PN];
+  using L = SBL<T, TMA>;
+  constexpr int SB_PX = L::PX, SB_PN = L::PN, SB_LPT = L::LPT;
+  __shared__ __align__(128) T pl[ST_NS][L::SLOT];
+  __shared__ __align__(8) uint64_t bar[ST_NS];
   const T* __restrict__ x = static_cast<const T*>(a.x);
   T* __restrict__ y = static_cast<T*>(a.y);
   const int cx = threadIdx.x % SB_CX, ty = (threadIdx.x / SB_CX) * SB_RY;
   const int64_t nx = a.nx, ny = a.ny, nz = a.nz, nxy = nx * ny;
-  const int64_t x0 = int64_t(blockIdx.x) * SB_TX, y0 = int64_t(blockIdx.y) * SB_TY;
+  const int64_t x0 = int64_t(blockIdx.x) * SB_TX - L::SHIFT, y0 = int64_t(blockIdx.y) * SB_TY;
   const int64_t z0 = int64_t(blockIdx.z) * a.zchunk;
   const int64_t z1 = cmin64(nz, z0 + a.zchunk);
   const int64_t gx = x0 + 2 * cx, gy = y0 + ty;
 
-  int off[SB_LPT];  // in-plane offsets (the host guarantees nx*ny < 2^31); -1 = outside
+  int off[TMA ? 1 : SB_LPT];  // in-plane offsets (the host guarantees nx*ny < 2^31); -1 = outside
+  uint32_t phase = 0;         // TMA: parity bit of each slot's mbarrier
+  // generic address of the __grid_constant__ parameter, taken here: a lambda capturing the parameter
+  // by reference would see a local copy, which the TMA unit cannot read (illegal instruction)
+  const uint64_t tmap = reinterpret_cast<uint64_t>(&tm);
+  if (TMA) {
+    if (threadIdx.x == 0) {
 #pragma unroll
-  for (int u = 0; u < SB_LPT; ++u) {
-    const int e = threadIdx.x + u * SB_NT;
-    off[u] = -1;
-    if (e < SB_PN) {
-      const int64_t X = x0 + (e % SB_PX) - 1, Y = y0 + (e / SB_PX) - 1;
-      if (X >= 0 && X < nx && Y >= 0 && Y < ny) off[u] = int(X + nx * Y);
+      for (int k = 0; k < ST_NS; ++k) mbar_init(&bar[k], 1);
+      asm volatile("fence.mbarrier_init.release.cluster;\n" ::: "memory");
+    }
+  } else {
+#pragma unroll
+    for (int u = 0; u < SB_LPT; ++u) {
+      const int e = threadIdx.x + u * SB_NT;
+      off[u] = -1;
+      if (e < SB_PN) {
+        const int64_t X = x0 + (e % SB_PX) - 1, Y = y0 + (e / SB_PX) - 1;
+        if (X >= 0 && X < nx && Y >= 0 && Y < ny) off[u] = int(X + nx * Y);
+      }
     }
   }
   auto issue = [&](int64_t zp, int slot) {
     const bool zin = zp >= 0 && zp < nz && zp <= z1;
-#pragma unroll
-    for (int u = 0; u < SB_LPT; ++u) {
-      const int e = threadIdx.x + u * SB_NT;
-      if (e < SB_PN) {
-        const bool ok = zin && off[u] >= 0;
-        cp_async_zfill<sizeof(T)>(&pl[slot][e], ok ? x + zp * nxy + off[u] : x, ok ? int(sizeof(T)) : 0);
+    if constexpr (TMA) {
+      if (zp > z1) return;  // never consumed
+      if (zin) {
+        if (threadIdx.x == 0) {
+          asm volatile("fence.proxy.async.shared::cta;\n" ::: "memory");  // after generic zero fills / reads
+          mbar_expect_tx(&bar[slot], uint32_t(SB_PN * sizeof(T)));
+          tma_load_3d(&pl[slot][0], tmap, int(x0 - 1), int(y0 - 1), int(zp), &bar[slot]);
+        }
+      } else {
+        for (int e = threadIdx.x; e < SB_PN; e += SB_NT) pl[slot][e] = T(0);
       }
+    } else {
+#pragma unroll
+      for (int u = 0; u < SB_LPT; ++u) {
+        const int e = threadIdx.x + u * SB_NT;
+        if (e < SB_PN) {
+          const bool ok = zin && off[u] >= 0;
+          cp_async_zfill<sizeof(T)>(&pl[slot][e], ok ? x + zp * nxy + off[u] : x, ok ? int(sizeof(T)) : 0);
+        }
+      }
+      cp_async_commit();
     }
-    cp_async_commit();
   };
   const double alpha = a.alpha, beta = a.beta;
   double acc_m[SB_RY][2], acc_c[SB_RY][2], acc_p[SB_RY][2], cen_m[SB_RY][2];
@@ -308,13 +364,22 @@ k_stencil27_box2(StencilArgs a) {
   for (int r = 0; r < SB_RY; ++r)
 #pragma unroll
     for (int c = 0; c < 2; ++c) acc_m[r][c] = acc_c[r][c] = acc_p[r][c] = cen_m[r][c] = 0.0;
+  if (TMA) __syncthreads();  // barriers initialised before the first copy
 #pragma unroll
   for (int k = 0; k < ST_NS - 1; ++k) issue(z0 - 1 + k, k);
+  if (TMA) __syncthreads();  // zero-filled prologue planes visible
   int cur = 0;
   for (int64_t zp = z0 - 1; zp <= z1; ++zp) {
     issue(zp + ST_NS - 1, (cur + ST_NS - 1) % ST_NS);
-    cp_async_wait<ST_NS - 1>();
-    __syncthreads();
+    if (TMA) {
+      if (zp >= 0 && zp < nz) {  // a copied plane (zero-filled ones were made visible by the last barrier)
+        mbar_wait(&bar[cur], (phase >> cur) & 1u, 7);
+        phase ^= 1u << cur;
+      }
+    } else {
+      cp_async_wait<ST_NS - 1>();
+      __syncthreads();
+    }
     const T* P = pl[cur];
     double rs0[SB_RY + 2], rs1[SB_RY + 2], cc0[SB_RY], cc1[SB_RY];
 #pragma unroll
@@ -343,7 +408,7 @@ k_stencil27_box2(StencilArgs a) {
         if (gy + r >= ny) continue;
 #pragma unroll
         for (int c = 0; c < 2; ++c) {
-          if (gx + c >= nx) continue;
+          if (gx + c >= nx || gx + c < 0) continue;
           const int64_t p = gx + c + nx * (gy + r) + nxy * zo;
           double res = alpha * fma(a.wd, cen_m[r][c], a.wn * acc_m[r][c]);
           if (beta != 0.0) res += beta * double(y[p]);
@@ -365,7 +430,7 @@ k_stencil27_box2(StencilArgs a) {
     __syncthreads();
     cur = (cur + 1) % ST_NS;
   }
-  cp_async_wait<0>();
+  if (!TMA) cp_async_wait<0>();
 }
 
 }  // namespace spmv

@@ -151,3 +151,26 @@ def test_stencil_box_form(env, dims, monkeypatch):
         y2, _, _ = _run(env, dims, x, w=w)
         monkeypatch.delenv("SPMV_STENCIL_BOX")
         check_rows(y2, y_ref, bound, np.float64, f"general {dims}")
+
+
+@pytest.mark.parametrize("dims", [(2, 2, 2), (64, 64, 64), (66, 17, 9), (128, 33, 40), (200, 3, 70), (192, 5, 7)])
+@pytest.mark.parametrize("f32", [False, True])
+@pytest.mark.parametrize("zchunk", [None, "5"])
+def test_stencil_box2_tma_equals_cpasync(env, dims, f32, zchunk, monkeypatch):
+    """The TMA plane tiles of k_stencil27_box2 (default when nx*sizeof(T) is a
+    multiple of 16 B; the tensor map's out-of-bound fill supplies the halo,
+    planes outside the grid are zero-filled by the CTA) stage the same values
+    as the cp.async ring (SPMV_STENCIL_TMA=0): the outputs are bit-identical,
+    and both are within the bound of the oracle.  Ragged x/y tiles, 1-plane
+    grids' neighbours, several z ranges per column."""
+    n = dims[0] * dims[1] * dims[2]
+    x = gen.uniform(n, seed=12)
+    if zchunk:
+        monkeypatch.setenv("SPMV_STENCIL_ZCHUNK", zchunk)
+    y0 = gen.uniform(n, seed=13)
+    y_t, y_ref, bound = _run(env, dims, x, y0=y0, alpha=1.5, beta=-0.5, f32=f32)
+    monkeypatch.setenv("SPMV_STENCIL_TMA", "0")
+    y_c, _, _ = _run(env, dims, x, y0=y0, alpha=1.5, beta=-0.5, f32=f32)
+    monkeypatch.delenv("SPMV_STENCIL_TMA")
+    assert np.array_equal(y_t.view(np.uint64 if not f32 else np.uint32), y_c.view(np.uint64 if not f32 else np.uint32))
+    check_rows(y_t, y_ref, bound, np.float32 if f32 else np.float64, f"tma {dims}")
