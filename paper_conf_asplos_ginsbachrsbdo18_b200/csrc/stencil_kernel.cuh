@@ -278,9 +278,20 @@ template <> struct V2<float> { using t = float2; };
 // left by SHIFT columns (output columns [64 bx - SHIFT, 64 bx + 64 - SHIFT),
 // staged from 64 bx - SHIFT - 1, a multiple of 16 B), which keeps each
 // thread's 4 staged values one aligned pair of vector loads.
+// ST_TMA_SHFL=1 (measured slower, not the default: 256^3 65.5 vs 61.4 us for the
+// shifted tiles, profiles/r01q_stencil_tma_shfl_*): no shift; the box starts HL = 16 B / sizeof(T) columns
+// left of the tile (PX = 64 + 2 HL), each thread loads its aligned pair
+// x[2c], x[2c+1] as one vector and takes x[2c-1], x[2c+2] from its neighbour
+// lanes (warp shuffles; lanes 0 and 31 read the halo column from shared).
+#ifndef ST_TMA_SHFL_DEF
+#define ST_TMA_SHFL_DEF 0
+#endif
+constexpr bool ST_TMA_SHFL = ST_TMA_SHFL_DEF != 0;
 template <typename T, bool TMA> struct SBL {
-  static constexpr int SHIFT = TMA ? (sizeof(T) == 8 ? 1 : 3) : 0;
-  static constexpr int PX = (TMA && sizeof(T) == 4) ? SB_TX + 4 : SB_TX + 2;  // staged row pitch
+  static constexpr bool SHFL = TMA && ST_TMA_SHFL;
+  static constexpr int HL = SHFL ? 16 / int(sizeof(T)) : 1;  // staged columns left of the tile
+  static constexpr int SHIFT = (TMA && !SHFL) ? (sizeof(T) == 8 ? 1 : 3) : 0;
+  static constexpr int PX = SHFL ? SB_TX + 2 * HL : (TMA && sizeof(T) == 4) ? SB_TX + 4 : SB_TX + 2;  // row pitch
   static constexpr int PN = PX * SB_PY;
   static constexpr int SLOT = TMA ? ((PN * int(sizeof(T)) + 127) / 128) * 128 / int(sizeof(T)) : PN;
   static constexpr int LPT = (PN + SB_NT - 1) / SB_NT;
@@ -341,7 +352,7 @@ k_stencil27_box2(StencilArgs a, const __grid_constant__ CUtensorMap tm) {
         if (threadIdx.x == 0) {
           asm volatile("fence.proxy.async.shared::cta;\n" ::: "memory");  // after generic zero fills / reads
           mbar_expect_tx(&bar[slot], uint32_t(SB_PN * sizeof(T)));
-          tma_load_3d(&pl[slot][0], tmap, int(x0 - 1), int(y0 - 1), int(zp), &bar[slot]);
+          tma_load_3d(&pl[slot][0], tmap, int(x0 - L::HL), int(y0 - 1), int(zp), &bar[slot]);
         }
       } else {
         for (int e = threadIdx.x; e < SB_PN; e += SB_NT) pl[slot][e] = T(0);
@@ -384,9 +395,19 @@ k_stencil27_box2(StencilArgs a, const __grid_constant__ CUtensorMap tm) {
     double rs0[SB_RY + 2], rs1[SB_RY + 2], cc0[SB_RY], cc1[SB_RY];
 #pragma unroll
     for (int sy = 0; sy < SB_RY + 2; ++sy) {
-      const V* q = reinterpret_cast<const V*>(P + (ty + sy) * SB_PX + 2 * cx);
-      const V lo = q[0], hi = q[1];  // x[2c-1], x[2c], x[2c+1], x[2c+2] of plane row ty+sy-1
-      const double e0 = double(lo.x), e1 = double(lo.y), e2 = double(hi.x), e3 = double(hi.y);
+      double e0, e1, e2, e3;  // x[2c-1], x[2c], x[2c+1], x[2c+2] of plane row ty+sy-1
+      if constexpr (L::SHFL) {
+        const T* row = P + (ty + sy) * SB_PX + L::HL;  // row[X - x0]
+        const V mid = *reinterpret_cast<const V*>(row + 2 * cx);
+        T l = __shfl_up_sync(0xffffffffu, mid.y, 1), r = __shfl_down_sync(0xffffffffu, mid.x, 1);
+        if (cx == 0) l = row[-1];
+        if (cx == SB_CX - 1) r = row[SB_TX];
+        e0 = double(l); e1 = double(mid.x); e2 = double(mid.y); e3 = double(r);
+      } else {
+        const V* q = reinterpret_cast<const V*>(P + (ty + sy) * SB_PX + 2 * cx);
+        const V lo = q[0], hi = q[1];
+        e0 = double(lo.x); e1 = double(lo.y); e2 = double(hi.x); e3 = double(hi.y);
+      }
       rs0[sy] = (e0 + e1) + e2;
       rs1[sy] = (e1 + e2) + e3;
       if (sy >= 1 && sy <= SB_RY) {
