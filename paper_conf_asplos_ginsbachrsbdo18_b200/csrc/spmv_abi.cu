@@ -1926,6 +1926,8 @@ extern "C" spmv_status stencil27_apply(spmv_dtype dt, int64_t nx, int64_t ny, in
     int tenv = 1;
     env_int("SPMV_STENCIL_TMA", &tenv);
     tma = tenv != 0 && encode_stencil_map(&tm, dt, x, nx, ny, nz);
+    // SPMV_STENCIL_TMA=2 (tests): the TMA form is required, no silent cp.async fallback
+    if (tenv == 2 && !tma) return arg_fail("SPMV_STENCIL_TMA=2 but the grid's tensor map cannot be encoded");
   }
   void (*kfn2)(StencilArgs, const CUtensorMap) = nullptr;
   if (box2)

@@ -174,3 +174,21 @@ def test_stencil_box2_tma_equals_cpasync(env, dims, f32, zchunk, monkeypatch):
     monkeypatch.delenv("SPMV_STENCIL_TMA")
     assert np.array_equal(y_t.view(np.uint64 if not f32 else np.uint32), y_c.view(np.uint64 if not f32 else np.uint32))
     check_rows(y_t, y_ref, bound, np.float32 if f32 else np.float64, f"tma {dims}")
+
+
+def test_stencil_tma_path_is_taken(env, monkeypatch):
+    """SPMV_STENCIL_TMA=2 makes the TMA form mandatory (argument error instead of the
+    cp.async fallback): the 256^3 grid and even fp64 rows take it (so the TMA parity
+    tests above exercise the tensor-map path), odd rows (nx*8 not a multiple of 16 B)
+    cannot."""
+    torch, dev, sp = env
+    monkeypatch.setenv("SPMV_STENCIL_TMA", "2")
+    for dims in [(256, 256, 256), (64, 64, 64), (66, 17, 9), (2, 3, 5)]:
+        n = dims[0] * dims[1] * dims[2]
+        x = torch.rand(n, dtype=torch.float64, device=dev)
+        sp.stencil27_apply(*dims, x, torch.empty_like(x))
+    torch.cuda.synchronize()
+    x = torch.rand(33 * 9 * 17, dtype=torch.float64, device=dev)
+    with pytest.raises(sp.SpmvError) as e:
+        sp.stencil27_apply(33, 9, 17, x, torch.empty_like(x))
+    assert e.value.status == sp.SPMV_ERR_ARG
