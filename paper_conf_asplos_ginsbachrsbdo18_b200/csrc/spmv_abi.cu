@@ -1829,6 +1829,9 @@ extern "C" spmv_status spmv_dist_plan_host(const int32_t* rowptr, const int32_t*
 // plane tiles of k_stencil27_box2: box (SBL::PX, 18, 1), no swizzle, zero fill
 // outside the grid.  The driver entry point is fetched through the runtime
 // (no link against libcuda).  false = not encodable (the caller keeps cp.async).
+#ifndef ST_TMA_L2PROMO
+#define ST_TMA_L2PROMO CU_TENSOR_MAP_L2_PROMOTION_L2_128B
+#endif
 static bool encode_stencil_map(CUtensorMap* tm, spmv_dtype dt, const void* x, int64_t nx, int64_t ny, int64_t nz) {
   using encode_fn = CUresult (*)(CUtensorMap*, CUtensorMapDataType, cuuint32_t, void*, const cuuint64_t*,
                                  const cuuint64_t*, const cuuint32_t*, const cuuint32_t*, CUtensorMapInterleave,
@@ -1857,7 +1860,7 @@ static bool encode_stencil_map(CUtensorMap* tm, spmv_dtype dt, const void* x, in
   const cuuint32_t es[3] = {1u, 1u, 1u};
   const CUresult r = fn(tm, dt == SPMV_F64 ? CU_TENSOR_MAP_DATA_TYPE_FLOAT64 : CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 3,
                         const_cast<void*>(x), dims, strides, box, es, CU_TENSOR_MAP_INTERLEAVE_NONE,
-                        CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_128B,
+                        CU_TENSOR_MAP_SWIZZLE_NONE, ST_TMA_L2PROMO,
                         CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   return r == CUDA_SUCCESS;
 }
