@@ -193,7 +193,18 @@ def stencil27_apply(nx: int, ny: int, nz: int, x, y, alpha: float = 1.0, beta: f
     27 weights indexed (dz+1)*9+(dy+1)*3+(dx+1)).  Asynchronous."""
     import numpy as np
     import torch
+    if y.dtype not in (torch.float64, torch.float32):
+        raise ValueError("y must be float64 or float32")
     dt = SPMV_F64 if y.dtype == torch.float64 else SPMV_F32
+    npts = int(nx) * int(ny) * int(nz)
+    # the C ABI sees raw pointers only: dtype, layout and extent are checked here
+    if not y.is_contiguous() or y.numel() < npts:
+        raise ValueError(f"y must be contiguous with at least nx*ny*nz = {npts} elements")
+    if alpha != 0.0:
+        if x.dtype != y.dtype:
+            raise ValueError(f"x.dtype {x.dtype} != y.dtype {y.dtype}")
+        if not x.is_contiguous() or x.numel() < npts:
+            raise ValueError(f"x must be contiguous with at least nx*ny*nz = {npts} elements")
     w = None if w27 is None else np.ascontiguousarray(w27, dtype=np.float64)
     if w is not None and w.shape != (27,):
         raise ValueError("w27 must hold 27 weights")

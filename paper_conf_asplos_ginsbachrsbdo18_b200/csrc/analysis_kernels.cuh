@@ -8,7 +8,7 @@ namespace spmv {
 
 // Per-CTA partial row statistics: [min, max, sum, sumsq, unsorted_rows].
 // Reduced on the host in CTA order (deterministic on every rank).
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_row_stats(int64_t m, const int* __restrict__ rowptr, const int* __restrict__ colidx,
             int check_sorted, double* __restrict__ part /* 5 * gridDim.x */) {
   __shared__ double red[8];
@@ -50,7 +50,7 @@ k_row_stats(int64_t m, const int* __restrict__ rowptr, const int* __restrict__ c
 
 // validate=1: flags[0] |= 1 if rowptr decreases, flags[0] |= 2 if a column
 // index is outside [0, n).
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_validate(int64_t m, int64_t n, const int* __restrict__ rowptr, const int* __restrict__ colidx,
            int* __restrict__ flags) {
   const int64_t stride = int64_t(gridDim.x) * blockDim.x;
@@ -71,7 +71,7 @@ k_validate(int64_t m, int64_t n, const int* __restrict__ rowptr, const int* __re
 // Device nnz-balanced partition (R20): thread r finds
 //   b_r = min{ i in [0,m] : rowptr[i] - rowptr[0] >= floor(r*nnz/P) }
 // by binary search; b_0 = 0, b_P = m.
-__global__ void k_partition(int64_t m, const int* __restrict__ rowptr, int P,
+static __global__ void k_partition(int64_t m, const int* __restrict__ rowptr, int P,
                             long long* __restrict__ bounds) {
   const int r = blockIdx.x * blockDim.x + threadIdx.x;
   if (r > P) return;
@@ -90,7 +90,7 @@ __global__ void k_partition(int64_t m, const int* __restrict__ rowptr, int P,
 
 // Renumber the columns of a rank's row block into the padded gather layout:
 // column c owned by rank s (bounds[s] <= c < bounds[s+1]) -> s*maxlen + (c - bounds[s]).
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_renumber(int64_t k0, int64_t k1, const int* __restrict__ colidx, const long long* __restrict__ bounds,
            int P, long long maxlen, int* __restrict__ out) {
   extern __shared__ long long sb[];
@@ -114,7 +114,7 @@ k_renumber(int64_t k0, int64_t k1, const int* __restrict__ colidx, const long lo
 // Warp per row over the GLOBAL matrix (every rank computes the whole table,
 // identically: min/max do not depend on the order).  Smem table per CTA,
 // updates only when they change it, then global atomics.
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_halo_bounds(int64_t m, const int* __restrict__ rowptr, const int* __restrict__ colidx,
               const long long* __restrict__ bounds, int P, int* __restrict__ tab) {
   extern __shared__ long long sb[];  // [P+1] bounds, then int [P*P*2]

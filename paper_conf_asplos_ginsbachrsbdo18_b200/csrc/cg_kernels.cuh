@@ -20,7 +20,7 @@ struct CgState {
 };
 
 // z = 0, r = b, p = b, partial r.r
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_cg_init(int64_t n, const double* __restrict__ b, double* __restrict__ z,
           double* __restrict__ r, double* __restrict__ p, double* __restrict__ part_rr) {
   __shared__ double red[8];
@@ -38,7 +38,7 @@ k_cg_init(int64_t n, const double* __restrict__ b, double* __restrict__ z,
 }
 
 // K2.  pq: p.q; rr_old: rho.  If tol_check, iterations stop once done.
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_cg_zr(int64_t n, SumSrc pq, SumSrc rr_old, const double* __restrict__ p,
         const double* __restrict__ q, double* __restrict__ z, double* __restrict__ r,
         double* __restrict__ part_rr_new, int* __restrict__ flags, P2PHook hk) {
@@ -87,7 +87,7 @@ k_cg_zr(int64_t n, SumSrc pq, SumSrc rr_old, const double* __restrict__ p,
 
 // K3.  rr_new: rho', rr_old: rho.  tol > 0: after the update, mark converged
 // once sqrt(rho') <= tol * ||b|| (rr_b: ||b||^2 source), recording `it`+1.
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
        double* __restrict__ p, int* __restrict__ flags, double tol, SumSrc rr_b, int it, P2PHook hk,
        int64_t xoff) {
@@ -163,7 +163,7 @@ k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
 // every CTA computes the same value from the same partials in the same
 // order).  tol > 0: the check sqrt(g) <= tol*||b|| is made on entry, before
 // the update, so the solve stops with the same z_k as the textbook loop.
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_cgcg(int64_t n, int k, SumSrc gam, SumSrc gam_old, SumSrc del, double* __restrict__ alpha2,
        double* __restrict__ p, double* __restrict__ sv, const double* __restrict__ w,
        double* __restrict__ z, double* __restrict__ r, double* __restrict__ part_rr_new,
@@ -286,7 +286,7 @@ k_cg_resid(int64_t n, const double* __restrict__ b, const double* __restrict__ a
 }
 
 // NPB tail: zeta = shift + 1/(x.z); x = z / ||z||; out2 = {zeta, rnorm}.
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_npb_finish(int64_t n, SumSrc res, SumSrc xz, SumSrc zz, const double* __restrict__ z,
              double* __restrict__ x, double shift, double* __restrict__ out2) {
   __shared__ double s0, s1, s2;
@@ -304,14 +304,14 @@ k_npb_finish(int64_t n, SumSrc res, SumSrc xz, SumSrc zz, const double* __restri
 }
 
 // cg_solve tail: rnorm = sqrt(sum).
-__global__ void k_finish_norm(SumSrc res, double* out) {
+static __global__ void k_finish_norm(SumSrc res, double* out) {
   __shared__ double s0;
   const double rr = read_sum(res, &s0);
   if (threadIdx.x == 0) *out = sqrt(rr);
 }
 
 // Per-CTA partials of w.y (used after SpMV kernels without a fused dot).
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_dot_partials(int64_t n, const double* __restrict__ w, const double* __restrict__ y, double* __restrict__ part,
                P2PHook hk) {
   __shared__ double red[8];
@@ -324,7 +324,7 @@ k_dot_partials(int64_t n, const double* __restrict__ w, const double* __restrict
 }
 
 // Distributed mode: sum `count` partials into one value (then all-reduced).
-__global__ void k_finalize(SumSrc s, double* out) {
+static __global__ void k_finalize(SumSrc s, double* out) {
   __shared__ double s0;
   const double v = read_sum(s, &s0);
   if (threadIdx.x == 0) *out = v;

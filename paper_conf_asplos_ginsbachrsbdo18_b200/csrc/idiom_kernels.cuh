@@ -213,7 +213,7 @@ k_hist_global(int64_t n, int nbins, const int32_t* __restrict__ keys, const doub
 }
 
 // Saturating finalize: bins8[b] = min(255, bins8[b] + cnt[b]); cnt re-zeroed.
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_hist_sat_fin(int64_t nbins, unsigned* __restrict__ cnt, uint8_t* __restrict__ bins8) {
   for (int64_t b = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; b < nbins; b += (int64_t)gridDim.x * blockDim.x) {
     const unsigned c = cnt[b];
@@ -247,7 +247,7 @@ constexpr int HB_MAXB = 1024;              // buckets (nbins <= 2^25)
 constexpr int HB_THREADS = 1024;
 constexpr int HB_TILE = 4096;              // keys staged per tile in K3 (16 KB of shared memory)
 
-__global__ void __launch_bounds__(HB_THREADS)
+static __global__ void __launch_bounds__(HB_THREADS)
 k_hb_count(int64_t n, int64_t chunk, int nbins, int nb, const int32_t* __restrict__ keys,
            unsigned* __restrict__ cnt /* [nb][G] */, int vec) {
   __shared__ unsigned sc[HB_MAXB];
@@ -262,7 +262,7 @@ k_hb_count(int64_t n, int64_t chunk, int nbins, int nb, const int32_t* __restric
 }
 
 // grid = nb; block scans the G counts of bucket b (G <= HB_THREADS)
-__global__ void __launch_bounds__(HB_THREADS)
+static __global__ void __launch_bounds__(HB_THREADS)
 k_hb_scan(int G, unsigned* __restrict__ cnt, unsigned* __restrict__ total) {
   __shared__ unsigned ws[32];
   const int b = blockIdx.x, t = threadIdx.x, lane = t & 31, w = t >> 5;
@@ -316,7 +316,7 @@ __device__ __forceinline__ void block_excl_scan(unsigned* a, int nb, unsigned* w
   __syncthreads();
 }
 
-__global__ void __launch_bounds__(HB_THREADS)
+static __global__ void __launch_bounds__(HB_THREADS)
 k_hb_scatter(int64_t n, int64_t chunk, int nbins, int nb, const int32_t* __restrict__ keys,
              const unsigned* __restrict__ off /* [nb][G] exclusive */, const unsigned* __restrict__ total,
              uint16_t* __restrict__ out) {

@@ -1,8 +1,8 @@
-// idioms_abi.cuh -- the C ABI of include/idioms.h (histogram, scalar
-// reduction, NAS EP).  Included at the end of
-// spmv_abi.cu so it shares that file's error/validation helpers; the
+// idioms_abi.cu -- the C ABI of include/idioms.h (histogram, scalar
+// reduction, NAS EP).  Shares the error/validation helpers of
+// abi_common.h; the
 // arithmetic is in idiom_kernels.cuh.  Rn = DESIGN.md reading n.
-#pragma once
+#include "abi_common.h"
 #include "../../include/idioms.h"
 #include "idiom_kernels.cuh"
 
@@ -273,7 +273,7 @@ extern "C" spmv_status ep_npb(int32_t M, int64_t pair_begin, int64_t pair_count,
   const int64_t chunk = std::max<int64_t>(1, cdiv(pair_count, T));
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>(kEpMaxGrid, cdiv(cdiv(pair_count, chunk), kEpThreads)));
   int compact = 1;  // SPMV_EP_COMPACT=0: per-thread tally without the warp queue
-  env_int("SPMV_EP_COMPACT", &compact);
+  tuning_env("SPMV_EP_COMPACT", &compact);
   if (compact)
     k_ep<true><<<(int)grid, kEpThreads, 0, s>>>(pair_begin, pair_count, chunk, out, (unsigned*)workspace,
                                                (double*)((char*)workspace + kWsHeader));

@@ -1,8 +1,8 @@
-// jds_abi.cuh -- the JDS-32 entry points of include/spmv.h (spmv_jds_create,
-// spmv_jds, spmv_jds_destroy; reading R34).  Included at the end of
-// spmv_abi.cu (shares its error/validation helpers); kernels in
+// jds_abi.cu -- the JDS-32 entry points of include/spmv.h (spmv_jds_create,
+// spmv_jds, spmv_jds_destroy; reading R34).  Shares the error/validation
+// helpers of abi_common.h; kernels in
 // jds_kernel.cuh.
-#pragma once
+#include "abi_common.h"
 #include "jds_kernel.cuh"
 
 struct spmv_jds_s {

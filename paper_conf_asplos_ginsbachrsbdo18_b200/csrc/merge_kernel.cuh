@@ -207,7 +207,7 @@ k_merge_fixup(MergeArgs a) {
 // Merge-path splits (reading R21) on the device, bit-exact with the host
 // spmv_csr_merge_splits: thread c finds the split of diagonal floor(c*(m+nnz)/C).
 // With C = ceil((m+nnz)/D) every tile holds at most D items.
-__global__ void k_merge_splits(int64_t m, const int* __restrict__ rowptr, int64_t C,
+static __global__ void k_merge_splits(int64_t m, const int* __restrict__ rowptr, int64_t C,
                                long long* __restrict__ split_row, long long* __restrict__ split_nz) {
   const int64_t c = int64_t(blockIdx.x) * blockDim.x + threadIdx.x;
   if (c > C) return;

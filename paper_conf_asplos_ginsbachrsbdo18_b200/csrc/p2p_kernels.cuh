@@ -24,7 +24,7 @@ namespace spmv {
 
 // All-reduce, push half: sum `in` (fixed order) and push it into slot `slot`
 // of every rank.  One CTA.
-__global__ void k_p2p_push_sum(SumSrc in, int slot, P2PCtx c) {
+static __global__ void k_p2p_push_sum(SumSrc in, int slot, P2PCtx c) {
   __shared__ double s0;
   const double v = read_sum(in, &s0);
   if (threadIdx.x == 0) {
@@ -61,7 +61,7 @@ k_p2p_push_x(int64_t n, int64_t maxlen, P2PCtx c) {
 }
 
 // Block the stream until every peer's x slice of the latest x exchange landed.
-__global__ void k_p2p_wait_x(P2PCtx c) {
+static __global__ void k_p2p_wait_x(P2PCtx c) {
   const unsigned long long* flags = reinterpret_cast<const unsigned long long*>(c.peer[c.me] + c.off_flags);
   p2p_wait_flags(flags, c.me, c.P, c.slot_epoch[P2P_XSLOT]);
 }

@@ -1,0 +1,716 @@
+// plans.cu -- kernel plans of a handle and the local SpMV launch (SURVEY 8(a)
+// a1/a2): the x-stationary XPLAN plan, the zero-copy XSTAT
+// cluster kernel, the SELL-32 plans (5.3a/5.3c), merge-path tiles (5.3b) and
+// run_spmv, which picks among them.  Validation and choice live in
+// spmv_abi.cu; arithmetic in the *_kernel.cuh headers.
+#include <cub/device/device_radix_sort.cuh>
+
+#include "abi_common.h"
+#include "analysis_kernels.cuh"
+#include "cg_kernels.cuh"  // k_dot_partials
+
+// ------------------------------------------------------- kernel dispatch
+template <typename T, int G, bool DOT>
+static void launch_vec_u(int unroll, int64_t grid, cudaStream_t s, const SpmvArgs& a) {
+  switch (unroll) {
+    case 2: k_spmv_vector<T, G, 2, DOT><<<grid, 256, 0, s>>>(a); break;
+    case 8: k_spmv_vector<T, G, 8, DOT><<<grid, 256, 0, s>>>(a); break;
+    default: k_spmv_vector<T, G, 4, DOT><<<grid, 256, 0, s>>>(a); break;
+  }
+}
+
+template <typename T, bool DOT>
+static void launch_vec(int lanes, int unroll, int64_t grid, cudaStream_t s, const SpmvArgs& a) {
+  switch (lanes) {
+    case 1: launch_vec_u<T, 1, DOT>(unroll, grid, s, a); break;
+    case 2: launch_vec_u<T, 2, DOT>(unroll, grid, s, a); break;
+    case 4: launch_vec_u<T, 4, DOT>(unroll, grid, s, a); break;
+    case 8: launch_vec_u<T, 8, DOT>(unroll, grid, s, a); break;
+    case 16: launch_vec_u<T, 16, DOT>(unroll, grid, s, a); break;
+    default: launch_vec_u<T, 32, DOT>(unroll, grid, s, a); break;
+  }
+}
+
+template <typename T, bool DOT, int U>
+static void (*xstat_fn_u(int G))(XstatArgs) {
+  switch (G) {
+    case 4: return k_spmv_xstat<T, 4, U, DOT>;
+    case 16: return k_spmv_xstat<T, 16, U, DOT>;
+    case 32: return k_spmv_xstat<T, 32, U, DOT>;
+    default: return k_spmv_xstat<T, 8, U, DOT>;
+  }
+}
+template <typename T, bool DOT>
+static void (*xstat_fn(int G, int U))(XstatArgs) {
+  return U == 8 ? xstat_fn_u<T, DOT, 8>(G) : xstat_fn_u<T, DOT, 4>(G);
+}
+
+static spmv_status launch_xstat(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
+                                double alpha, double beta, const double* w, double* part, const P2PHook& hook) {
+  XstatArgs a;
+  a.m = h->m_loc;
+  a.nx = h->nx;
+  a.W = h->xW;
+  a.R = h->xR;
+  a.rowptr = h->rp_loc;
+  a.colidx = h->ci_loc;
+  a.vals = vals;
+  a.seg = h->seg;
+  a.crow = h->crow;
+  a.x = x;
+  a.y = y;
+  a.alpha = alpha;
+  a.beta = beta;
+  a.w = w;
+  a.part = part;
+  a.hk = hook;
+  if (h->dt == SPMV_F32) {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+  }
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = dim3((unsigned)(h->nclusters * h->xB), 1, 1);
+  cfg.blockDim = dim3(1024, 1, 1);
+  cfg.dynamicSmemBytes = h->xsmem;
+  cfg.stream = s;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeClusterDimension;
+  at[0].val.clusterDim.x = (unsigned)h->xB;
+  at[0].val.clusterDim.y = 1;
+  at[0].val.clusterDim.z = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  CK(cudaLaunchKernelEx(&cfg, part ? h->xk_dot : h->xk, a));
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+// XSTAT set-up (create): column-block width, cluster size, split points,
+// static nnz-balanced cluster row ranges.  Returns false if not eligible.
+spmv_status xstat_setup(spmv_csr_s* h, bool* ok) {
+  *ok = false;
+  if (!h->sorted || h->m_loc == 0 || h->nx == 0) return SPMV_OK;
+  const size_t budget = 200 * 1024;  // of the 227 KB a CTA may use
+  const size_t pb = 3 * (size_t)h->xR * sizeof(double) + 4 * (size_t)h->xR * sizeof(int) + 16;
+  if (budget <= pb) return SPMV_OK;
+  int B = (int)cdiv((int64_t)h->ts * h->nx, (int64_t)(budget - pb));
+  if (B < 1) B = 1;
+  // cluster sizes that tile the GPCs well: 1, 2, 4, 8
+  B = B <= 1 ? 1 : B <= 2 ? 2 : B <= 4 ? 4 : B <= 8 ? 8 : B;
+  int forced = 0;
+  if (env_int("SPMV_XSTAT_B", &forced) && forced >= B && forced <= 8) B = forced;
+  if (B > 8) return SPMV_OK;
+  int W = (int)cdiv(h->nx, B);
+  W = (W + 3) & ~3;
+  const size_t xbytes = ((size_t)W * h->ts + 15) & ~size_t(15);
+  const size_t smem = xbytes + 3 * (size_t)h->xR * sizeof(double) + 4 * (size_t)h->xR * sizeof(int);
+  const double seg_mean = h->row_mean / B;
+  // lanes x unroll ~ the mean segment length, unroll 8 for memory-level parallelism
+  int G = seg_mean < 48 ? 4 : seg_mean < 96 ? 8 : seg_mean < 192 ? 16 : 32;
+  int U = 8;
+  int g2 = 0;
+  if (env_int("SPMV_XSTAT_G", &g2) && (g2 == 4 || g2 == 8 || g2 == 16 || g2 == 32)) G = g2;
+  if (tuning_env("SPMV_XSTAT_U", &g2) && (g2 == 4 || g2 == 8)) U = g2;
+  void (*fn)(XstatArgs) = h->dt == SPMV_F64 ? xstat_fn<double, false>(G, U) : xstat_fn<float, false>(G, U);
+  void (*fnd)(XstatArgs) = h->dt == SPMV_F64 ? xstat_fn<double, true>(G, U) : nullptr;
+  CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+  if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = dim3((unsigned)B, 1, 1);
+  cfg.blockDim = dim3(1024, 1, 1);
+  cfg.dynamicSmemBytes = smem;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeClusterDimension;
+  at[0].val.clusterDim.x = (unsigned)B;
+  at[0].val.clusterDim.y = 1;
+  at[0].val.clusterDim.z = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  int ncl = 0;
+  cudaError_t e = cudaOccupancyMaxActiveClusters(&ncl, fn, &cfg);
+  if (e != cudaSuccess || ncl < 1) { cudaGetLastError(); return SPMV_OK; }
+  int nc_env = 0;
+  if (env_int("SPMV_XSTAT_CLUSTERS", &nc_env) && nc_env >= 1 && nc_env <= ncl) ncl = nc_env;
+  cudaStream_t s = h->stream;
+  if (B > 1) {
+    CK(cudaMalloc(&h->seg, sizeof(int) * (size_t)(B - 1) * (size_t)h->m_loc));
+    k_xstat_splits<<<std::min<int64_t>(cdiv(h->m_loc, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
+        h->m_loc, h->rp_loc, h->ci_loc, B, W, h->seg);
+    LAUNCHED();
+  }
+  CK(cudaMalloc(&h->crow, sizeof(long long) * (ncl + 1)));
+  k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(h->m_loc, h->rp_loc, ncl, h->crow);
+  LAUNCHED();
+  CK(cudaStreamSynchronize(s));
+  h->xB = B;
+  h->xW = W;
+  h->xG = G;
+  h->xsmem = smem;
+  h->nclusters = ncl;
+  h->xk = fn;
+  h->xk_dot = fnd;
+  *ok = true;
+  return SPMV_OK;
+}
+
+static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha,
+                                double beta, const double* w, double* part, const P2PHook& hook) {
+  XplanArgs a;
+  a.nx = h->nx;
+  a.W = h->xp.W;
+  a.plan = h->xp.plan;
+  a.chunk_off = h->xp.chunk_off;
+  a.chunk_len = h->xp.chunk_len;
+  a.chunk_row = h->xp.chunk_row;
+  a.dbg = dbg() ? 1 : 0;
+  a.prefetch = 0;
+  tuning_env("SPMV_XPLAN_PF", &a.prefetch);
+  a.hk = hook;
+  a.crow = h->xp.crow;
+  a.tile0 = h->xp.tile0;
+  a.x = x;
+  a.y = y;
+  a.alpha = alpha;
+  a.beta = beta;
+  a.w = w;
+  a.part = part;
+  if (h->dt == SPMV_F32) {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+  }
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = dim3((unsigned)(h->xp.ncl * h->xp.B), 1, 1);
+  cfg.blockDim = dim3(XP_THREADS, 1, 1);
+  cfg.dynamicSmemBytes = h->xp.smem;
+  cfg.stream = s;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeClusterDimension;
+  at[0].val.clusterDim.x = (unsigned)h->xp.B;
+  at[0].val.clusterDim.y = 1;
+  at[0].val.clusterDim.z = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  a.tstamp = nullptr;
+  int times = 0;
+  if (tuning_env("SPMV_XPLAN_TIMES", &times) && times) {
+    // diagnostics: per-CTA {start, x ready, streaming done, end} (globaltimer, ns), summarised on stderr
+    const size_t nb = sizeof(unsigned long long) * 4 * cfg.gridDim.x;
+    CK(cudaMalloc(&a.tstamp, nb));
+    CK(cudaMemsetAsync(a.tstamp, 0, nb, s));
+  }
+  const bool side = h->xp.mplan >= 0 && h->xp.mplan < h->m_loc;
+  if (side) {
+    if (!h->side) {
+      CK(cudaStreamCreateWithFlags(&h->side, cudaStreamNonBlocking));
+      CK(cudaEventCreateWithFlags(&h->ev_fork, cudaEventDisableTiming));
+      CK(cudaEventCreateWithFlags(&h->ev_join, cudaEventDisableTiming));
+    }
+    CK(cudaEventRecord(h->ev_fork, s));
+    CK(cudaStreamWaitEvent(h->side, h->ev_fork, 0));
+  }
+  CK(cudaLaunchKernelEx(&cfg, part ? h->xp.kdot : h->xp.k, a));
+  LAUNCHED();
+  if (side) {
+    // rows [mplan, m) in the vector kernel, launched after the clusters so it
+    // takes the SMs they leave idle; its dot partials follow the clusters'
+    const int64_t ms = h->m_loc - h->xp.mplan;
+    SpmvArgs sa;
+    sa.m = ms;
+    sa.rowptr = h->rp_loc + h->xp.mplan;
+    sa.colidx = h->ci_loc;
+    sa.vals = h->vals;
+    sa.x = x;
+    sa.y = (char*)y + h->ts * (size_t)h->xp.mplan;
+    sa.alpha = a.alpha;
+    sa.beta = a.beta;
+    sa.w = w ? (const void*)(w + h->xp.mplan) : nullptr;
+    sa.part = part ? part + cfg.gridDim.x : nullptr;
+    sa.hk = P2PHook();
+    if (h->dt == SPMV_F64) {
+      if (part) launch_vec<double, true>(h->lanes, h->unroll, h->xp.g2, h->side, sa);
+      else launch_vec<double, false>(h->lanes, h->unroll, h->xp.g2, h->side, sa);
+    } else {
+      launch_vec<float, false>(h->lanes, h->unroll, h->xp.g2, h->side, sa);
+    }
+    LAUNCHED();
+    CK(cudaEventRecord(h->ev_join, h->side));
+    CK(cudaStreamWaitEvent(s, h->ev_join, 0));
+  }
+  if (a.tstamp) {
+    std::vector<unsigned long long> t(4 * cfg.gridDim.x);
+    CK(cudaMemcpyAsync(t.data(), a.tstamp, sizeof(unsigned long long) * t.size(), cudaMemcpyDeviceToHost, s));
+    CK(cudaStreamSynchronize(s));
+    cudaFree(a.tstamp);
+    unsigned long long t0 = ~0ull, tend = 0;
+    for (unsigned i = 0; i < cfg.gridDim.x; ++i) { t0 = std::min(t0, t[4 * i]); tend = std::max(tend, t[4 * i + 3]); }
+    fprintf(stderr, "[xplan times] kernel span %.2f us; per CTA (us from first start): start/xready/streamed/end\n",
+            (tend - t0) / 1e3);
+    for (unsigned i = 0; i < cfg.gridDim.x; ++i)
+      fprintf(stderr, "  cta %3u cl %2u  %6.2f %6.2f %6.2f %6.2f\n", i, i / (unsigned)h->xp.B, (t[4 * i] - t0) / 1e3,
+              (t[4 * i + 1] - t0) / 1e3, (t[4 * i + 2] - t0) / 1e3, (t[4 * i + 3] - t0) / 1e3);
+  }
+  return SPMV_OK;
+}
+
+// Pack (or re-pack, values_only) the nonzeros into the plan chunks.
+spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only) {
+  cudaStream_t s = h->stream;
+  auto& P = h->xp;
+  const int64_t g = std::min<int64_t>(cdiv(h->m_loc * 32, 256), 16LL * num_sms(h->device));
+  if (h->dt == SPMV_F64)
+    k_xplan_pack<double><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const double*)vals, P.seg, h->m_loc, P.B, P.W,
+                                          P.crow, P.tile0, P.ncl, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
+                                          values_only, P.mplan);
+  else
+    k_xplan_pack<float><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const float*)vals, P.seg, h->m_loc, P.B, P.W,
+                                         P.crow, P.tile0, P.ncl, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
+                                         values_only, P.mplan);
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+// Build the column-blocked SELL-32 plan (create).  *ok = false if not eligible.
+spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
+  *ok = false;
+  if (!h->sorted || h->m_loc == 0 || h->nx == 0 || h->k1 - h->k0 == 0) return SPMV_OK;
+  const int ts = (int)h->ts;
+  const size_t smem_cap = 227 * 1024 - 1024;  // dynamic smem a CTA may use (static < 1 KB)
+  const size_t recv = (size_t)XP_K * XP_R * 8;
+  if (smem_cap <= recv + 1024) return SPMV_OK;
+  const size_t xbudget = smem_cap - recv - 64;
+  const int64_t Bneed = cdiv((int64_t)(ts * h->nx), (int64_t)xbudget);
+  if (Bneed > 16) return SPMV_OK;  // x does not fit the shared memory of a 16-CTA cluster
+  void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, false> : k_spmv_xplan<float, false>;
+  void (*fnd)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, true> : nullptr;
+  // cluster size: any B >= Bneed that divides the tile height R (rows are
+  // owned in R/B blocks); among those, the one whose resident clusters cover
+  // the most SMs (ties: the smaller B, whose x blocks are larger); clusters of
+  // 16 only when nothing smaller fits.  SPMV_XPLAN_B forces a size.
+  int forced = 0;
+  env_int("SPMV_XPLAN_B", &forced);
+  if (forced < Bneed || forced > 16 || XP_R % std::max(forced, 1)) forced = 0;  // infeasible request: ignored
+  int B = 0, W = 0, ncl = 0;
+  size_t smem = 0;
+  for (int cand = (int)std::max<int64_t>(1, Bneed); cand <= 16; ++cand) {
+    if (XP_R % cand) continue;
+    if (forced && cand != forced) continue;
+    if (cand > 8 && B > 0) break;  // non-portable sizes only as the last resort
+    int Wc = (int)cdiv(h->nx, cand);
+    Wc = (Wc + 7) & ~7;
+    if (Wc > 65534) continue;  // 16-bit column offsets, pad column W
+    const size_t sm = (((size_t)(Wc + 1) * ts + 15) & ~size_t(15)) + recv;
+    if (sm > smem_cap) continue;
+    CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm));
+    if (cand > 8) CK(cudaFuncSetAttribute(fn, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
+    cudaLaunchConfig_t cfg = {};
+    cfg.gridDim = dim3((unsigned)cand, 1, 1);
+    cfg.blockDim = dim3(XP_THREADS, 1, 1);
+    cfg.dynamicSmemBytes = sm;
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeClusterDimension;
+    at[0].val.clusterDim.x = (unsigned)cand;
+    at[0].val.clusterDim.y = 1;
+    at[0].val.clusterDim.z = 1;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    int nc = 0;
+    cudaError_t e = cudaOccupancyMaxActiveClusters(&nc, fn, &cfg);
+    if (e != cudaSuccess || nc < 1) { cudaGetLastError(); continue; }
+    DBG("candidate B=%d W=%d clusters=%d SMs=%d", cand, Wc, nc, nc * cand);
+    if (B == 0 || nc * cand > ncl * B) { B = cand; W = Wc; ncl = nc; smem = sm; }
+  }
+  if (B == 0) return SPMV_OK;
+  CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+  if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+  if (B > 8) {  // clusters of 16 need the non-portable size
+    CK(cudaFuncSetAttribute(fn, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
+    if (fnd) CK(cudaFuncSetAttribute(fnd, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
+  }
+  int nc_env = 0;
+  if (env_int("SPMV_XPLAN_CLUSTERS", &nc_env) && nc_env >= 1 && nc_env <= ncl) ncl = nc_env;
+  cudaStream_t s = h->stream;
+  auto& P = h->xp;
+  auto cleanup = [&]() {
+    void* bufs[] = {P.crow, P.chunk_off, P.tile0, P.chunk_len, P.seg, P.row_slot, P.chunk_row, P.plan};
+    for (void* q : bufs)
+      if (q) cudaFree(q);
+    P = spmv_csr_s::XPlan();
+  };
+  P.B = B; P.W = W; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd;
+  DBG("B=%d W=%d ncl=%d smem=%zu", B, W, ncl, smem);
+  const int64_t m = h->m_loc;
+  // side split: the last SPMV_XPLAN_SIDE per mille of the nonzeros go to the
+  // vector kernel on the idle SMs (single GPU only)
+  P.mplan = m;
+  {
+    int side_pm = 0;
+    tuning_env("SPMV_XPLAN_SIDE", &side_pm);
+    const int idle = num_sms(h->device) - ncl * B;
+    if (side_pm > 0 && side_pm < 500 && !h->dist && idle > 0) {
+      std::vector<int> rph((size_t)m + 1);
+      CK(cudaMemcpyAsync(rph.data(), h->rp_loc, sizeof(int) * (m + 1), cudaMemcpyDeviceToHost, s));
+      CK(cudaStreamSynchronize(s));
+      const long long nz = (long long)rph[m] - rph[0];
+      const long long target = rph[0] + nz - nz * side_pm / 1000;
+      P.mplan = std::lower_bound(rph.begin(), rph.end(), (int)target) - rph.begin();
+      P.mplan = std::min<int64_t>(std::max<int64_t>(P.mplan, 1), m);
+      P.g2 = idle * 8;
+      DBG("side split: plan rows %lld of %lld, side grid %d", (long long)P.mplan, (long long)m, P.g2);
+    }
+  }
+  CK(cudaMalloc(&P.crow, sizeof(long long) * (ncl + 1)));
+  k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(P.mplan, h->rp_loc, ncl, P.crow);
+  LAUNCHED();
+  std::vector<long long> crow(ncl + 1);
+  CK(cudaMemcpyAsync(crow.data(), P.crow, sizeof(long long) * (ncl + 1), cudaMemcpyDeviceToHost, s));
+  CK(cudaStreamSynchronize(s));
+  std::vector<int> tile0(ncl + 1, 0);
+  for (int c = 0; c < ncl; ++c) tile0[c + 1] = tile0[c] + (int)cdiv(crow[c + 1] - crow[c], XP_R);
+  const int ntiles = tile0[ncl];
+  P.ntiles = ntiles;
+  DBG("ntiles=%d", ntiles);
+  CK(cudaMalloc(&P.tile0, sizeof(int) * (ncl + 1)));
+  CK(cudaMemcpyAsync(P.tile0, tile0.data(), sizeof(int) * (ncl + 1), cudaMemcpyHostToDevice, s));
+  if (B > 1) {
+    CK(cudaMalloc(&P.seg, sizeof(int) * (size_t)(B - 1) * (size_t)m));
+    k_xstat_splits<<<std::min<int64_t>(cdiv(m, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
+        m, h->rp_loc, h->ci_loc, B, W, P.seg);
+    LAUNCHED();
+  }
+  DBG("splits done");
+  const int64_t nch = (int64_t)ntiles * B * XP_CPT;
+  P.nchunks = nch;
+  CK(cudaMalloc(&P.chunk_len, sizeof(int) * std::max<int64_t>(nch, 1)));
+  CK(cudaMalloc(&P.chunk_off, sizeof(long long) * std::max<int64_t>(nch, 1)));
+  CK(cudaMalloc(&P.chunk_row, sizeof(uint16_t) * 32 * std::max<int64_t>(nch, 1)));
+  CK(cudaMalloc(&P.row_slot, sizeof(int) * (size_t)B * (size_t)m));
+  if (ntiles > 0) {
+    k_xplan_sell<<<(unsigned)(ntiles * B), XP_THREADS, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, P.tile0, ncl, P.chunk_len,
+                                                          P.chunk_row, P.row_slot);
+    LAUNCHED();
+  }
+  DBG("sell done nch=%lld", (long long)nch);
+  std::vector<int> len(std::max<int64_t>(nch, 1), 0);
+  CK(cudaMemcpyAsync(len.data(), P.chunk_len, sizeof(int) * nch, cudaMemcpyDeviceToHost, s));
+  CK(cudaStreamSynchronize(s));
+  // padding check: SELL must not blow up the stream (skewed segments)
+  long long steps = 0;
+  for (int64_t i = 0; i < nch; ++i) steps += len[i];
+  const long long padded = steps * 32;
+  const long long real = h->k1 - h->k0;
+  double maxpad = 1.5;
+  if (padded > (long long)(maxpad * (double)real) + 64LL * nch) {
+    cleanup();
+    return SPMV_OK;
+  }
+  // chunk offsets in stream order [c][b][t][w]: the chunks of one CTA are contiguous
+  std::vector<long long> off(std::max<int64_t>(nch, 1), 0);
+  long long pos = 0;
+  for (int c = 0; c < ncl; ++c)
+    for (int bb = 0; bb < B; ++bb)
+      for (int t = tile0[c]; t < tile0[c + 1]; ++t)
+        for (int w = 0; w < XP_CPT; ++w) {
+          const size_t id = ((size_t)t * B + bb) * XP_CPT + w;
+          off[id] = pos;
+          pos += (long long)len[id] * 32 * (ts + 2);
+        }
+  P.bytes = pos;
+  CK(cudaMemcpyAsync(P.chunk_off, off.data(), sizeof(long long) * nch, cudaMemcpyHostToDevice, s));
+  CK(cudaMalloc(&P.plan, (size_t)std::max<long long>(pos, 16)));
+  if (nch > 0) {
+    k_xplan_fill<<<(unsigned)std::min<int64_t>(nch, 16LL * num_sms(h->device)), 256, 0, s>>>(
+        P.plan, P.chunk_off, P.chunk_len, nch, ts, (uint16_t)W);
+    LAUNCHED();
+  }
+  DBG("fill done bytes=%lld", (long long)pos);
+  ST(xplan_pack(h, h->vals, 0));
+  DBG("pack done");
+  CK(cudaStreamSynchronize(s));
+  P.built = true;
+  *ok = true;
+  return SPMV_OK;
+}
+
+// ------------------------------------------------------------------ SELL
+spmv_status sell_pack(spmv_csr_s* h, const void* vals, int values_only) {
+  cudaStream_t s = h->stream;
+  const auto& S = h->sl;
+  const int64_t g = std::max<int64_t>(1, std::min<int64_t>(cdiv(h->m_loc - S.nlong, 256), 16LL * num_sms(h->device)));
+  if (h->dt == SPMV_F64)
+    k_sell_pack<double><<<g, 256, 0, s>>>(h->m_loc, h->rp_loc, h->ci_loc, (const double*)vals, S.pair_off, S.perm,
+                                          S.nlong, (double*)S.vals, S.cols, values_only);
+  else
+    k_sell_pack<float><<<g, 256, 0, s>>>(h->m_loc, h->rp_loc, h->ci_loc, (const float*)vals, S.pair_off, S.perm,
+                                         S.nlong, (float*)S.vals, S.cols, values_only);
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+// Build the SELL-32 plan (create).  sorted = 0: chunks of consecutive rows;
+// sorted = 1: rows ordered by length (descending, stable device radix sort),
+// rows longer than SELL_LONG kept in the CSR and processed warp-per-row.
+// Not eligible (*ok = false) when the padding exceeds max_pad x nnz.
+spmv_status sell_build(spmv_csr_s* h, double max_pad, int sorted, bool* ok) {
+  *ok = false;
+  const int64_t m = h->m_loc, nnz = h->k1 - h->k0;
+  if (m == 0 || nnz == 0) return SPMV_OK;
+  if (sorted && m > 2147483647LL) return SPMV_OK;
+  cudaStream_t s = h->stream;
+  auto& S = h->sl;
+  auto cleanup = [&]() {
+    void* bufs[] = {S.pair_off, S.vals, S.cols, S.perm, S.seg, S.seg_part, S.seg_cnt};
+    for (void* q : bufs)
+      if (q) cudaFree(q);
+    S = spmv_csr_s::Sell();
+  };
+  const int sms = num_sms(h->device);
+  if (sorted) {
+    int *keys = nullptr, *keys_out = nullptr, *ids = nullptr;
+    void* tmp = nullptr;
+    size_t tmp_bytes = 0;
+    CK(cudaMalloc(&keys, sizeof(int) * m));
+    CK(cudaMalloc(&keys_out, sizeof(int) * m));
+    CK(cudaMalloc(&ids, sizeof(int) * m));
+    CK(cudaMalloc(&S.perm, sizeof(int) * m));
+    k_row_len_ids<<<(unsigned)std::min<int64_t>(cdiv(m, 256), 8LL * sms), 256, 0, s>>>(m, h->rp_loc, keys, ids);
+    LAUNCHED();
+    CK(cub::DeviceRadixSort::SortPairsDescending(nullptr, tmp_bytes, keys, keys_out, ids, S.perm, (int)m, 0, 32, s));
+    CK(cudaMalloc(&tmp, tmp_bytes));
+    CK(cub::DeviceRadixSort::SortPairsDescending(tmp, tmp_bytes, keys, keys_out, ids, S.perm, (int)m, 0, 32, s));
+    std::vector<int> sk(m);
+    CK(cudaMemcpyAsync(sk.data(), keys_out, sizeof(int) * m, cudaMemcpyDeviceToHost, s));
+    CK(cudaStreamSynchronize(s));
+    cudaFree(tmp);
+    cudaFree(keys);
+    cudaFree(keys_out);
+    cudaFree(ids);
+    // long rows: the prefix with length > SELL_LONG, cut into segments of <= SELL_SEG entries
+    S.nlong = std::lower_bound(sk.begin(), sk.end(), SELL_LONG, std::greater<int>()) - sk.begin();
+    if (S.nlong > 0) {
+      std::vector<int> lp(S.nlong), rp(m + 1);
+      CK(cudaMemcpy(lp.data(), S.perm, sizeof(int) * S.nlong, cudaMemcpyDeviceToHost));
+      CK(cudaMemcpy(rp.data(), h->rp_loc, sizeof(int) * (m + 1), cudaMemcpyDeviceToHost));
+      std::vector<SellSeg> segs;
+      int npart = 0, ncnt = 0;
+      for (int64_t j = 0; j < S.nlong; ++j) {
+        const int i = lp[j], k0 = rp[i], k1 = rp[i + 1];
+        const int ns = (int)cdiv(k1 - k0, SELL_SEG);
+        for (int q = 0; q < ns; ++q) {
+          SellSeg g{};
+          g.row = i;
+          g.k0 = k0 + q * SELL_SEG;
+          g.k1 = std::min(k1, g.k0 + SELL_SEG);
+          g.pbase = ns > 1 ? npart : -1;
+          g.sidx = q;
+          g.nseg = ns;
+          g.cslot = ns > 1 ? ncnt : -1;
+          segs.push_back(g);
+        }
+        if (ns > 1) { npart += ns; ++ncnt; }
+      }
+      S.nseg = (int64_t)segs.size();
+      S.nmulti = ncnt;
+      CK(cudaMalloc(&S.seg, sizeof(SellSeg) * segs.size()));
+      CK(cudaMemcpy(S.seg, segs.data(), sizeof(SellSeg) * segs.size(), cudaMemcpyHostToDevice));
+      CK(cudaMalloc(&S.seg_part, sizeof(double) * std::max(npart, 1)));
+      CK(cudaMalloc(&S.seg_cnt, sizeof(int) * std::max(ncnt, 1)));
+      CK(cudaMemset(S.seg_cnt, 0, sizeof(int) * std::max(ncnt, 1)));
+    }
+  }
+  const int64_t nch = cdiv(m - S.nlong, 32);
+  CK(cudaMalloc(&S.pair_off, sizeof(long long) * (nch + 1)));
+  if (nch > 0) {
+    const unsigned g = (unsigned)std::max<int64_t>(1, std::min<int64_t>(cdiv(nch, 256), 8LL * sms));
+    if (sorted) k_sell_pairs_sorted<<<g, 256, 0, s>>>(m, h->rp_loc, S.perm, S.nlong, nch, S.pair_off);
+    else k_sell_pairs<<<g, 256, 0, s>>>(m, h->rp_loc, nch, S.pair_off);
+    LAUNCHED();
+  }
+  std::vector<long long> off(nch + 1);
+  CK(cudaMemcpyAsync(off.data(), S.pair_off, sizeof(long long) * nch, cudaMemcpyDeviceToHost, s));
+  CK(cudaStreamSynchronize(s));
+  long long pos = 0;
+  for (int64_t c = 0; c < nch; ++c) {
+    const long long np = off[c];
+    off[c] = pos;
+    pos += np;
+  }
+  off[nch] = pos;
+  if ((double)pos * 64.0 > max_pad * (double)nnz + 64.0) {
+    cleanup();
+    return SPMV_OK;
+  }
+  S.nchunks = nch;
+  S.pairs = pos;
+  const size_t slots = (size_t)std::max<long long>(pos, 1) * 64;  // 32 lanes x 2 steps
+  CK(cudaMemcpyAsync(S.pair_off, off.data(), sizeof(long long) * (nch + 1), cudaMemcpyHostToDevice, s));
+  CK(cudaMalloc(&S.vals, slots * h->ts));
+  CK(cudaMalloc(&S.cols, slots * sizeof(int)));
+  CK(cudaMemsetAsync(S.vals, 0, slots * h->ts, s));
+  CK(cudaMemsetAsync(S.cols, 0xff, slots * sizeof(int), s));  // -1: padding
+  ST(sell_pack(h, h->vals, 0));
+  CK(cudaStreamSynchronize(s));
+  // grid: 8 CTAs of SELL_NT per SM, never more warps than work items
+  S.grid = std::max<int64_t>(1, std::min<int64_t>(cdiv(nch + S.nseg, SELL_NT / 32), 8LL * sms));
+  S.sorted = sorted;
+  S.built = true;
+  *ok = true;
+  return SPMV_OK;
+}
+
+static spmv_status launch_sell(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha, double beta,
+                               const double* w, double* part, const P2PHook& hook) {
+  SellArgs a;
+  a.m = h->m_loc;
+  a.nchunks = h->sl.nchunks;
+  a.perm = h->sl.perm;
+  a.nlong = h->sl.nlong;
+  a.nseg = h->sl.nseg;
+  a.seg = h->sl.seg;
+  a.seg_part = h->sl.seg_part;
+  a.seg_cnt = h->sl.seg_cnt;
+  a.colidx = h->ci_loc;
+  a.csr_vals = h->vals;
+  a.vals = h->sl.vals;
+  a.cols = reinterpret_cast<const int2*>(h->sl.cols);
+  a.pair_off = h->sl.pair_off;
+  a.x = x;
+  a.y = y;
+  a.alpha = alpha;
+  a.beta = beta;
+  a.w = w;
+  a.part = part;
+  a.hk = hook;
+  const unsigned g = (unsigned)h->sl.grid;
+  if (h->dt == SPMV_F64) {
+    if (part && h->sl.nmulti > 0) {
+      // multi-segment rows are finished by whichever warp completes them: the dot
+      // runs as a separate pass so its per-CTA partials stay deterministic
+      P2PHook wait_only = hook;
+      wait_only.push_slot = -1;
+      a.hk = wait_only;
+      k_spmv_sell<double, false><<<g, SELL_NT, 0, s>>>(a);
+      LAUNCHED();
+      P2PHook push_only = hook;
+      push_only.wait_x = 0;
+      k_dot_partials<<<(int)h->vgrid, 256, 0, s>>>(h->m_loc, w, (const double*)y, part, push_only);
+    } else if (part) {
+      k_spmv_sell<double, true><<<g, SELL_NT, 0, s>>>(a);
+    } else {
+      k_spmv_sell<double, false><<<g, SELL_NT, 0, s>>>(a);
+    }
+  } else {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+    k_spmv_sell<float, false><<<g, SELL_NT, 0, s>>>(a);
+  }
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+spmv_status merge_setup(spmv_csr_s* h) {
+  const int64_t items = h->m_loc + (h->k1 - h->k0);
+  const int64_t C = std::max<int64_t>(1, cdiv(items, MG_D));
+  if (C > 2147483647LL) return arg_fail("matrix too large for the merge kernel");
+  auto& G = h->mg;
+  G.ntiles = (int)C;
+  CK(cudaMalloc(&G.split_row, sizeof(long long) * (C + 1)));
+  CK(cudaMalloc(&G.split_nz, sizeof(long long) * (C + 1)));
+  CK(cudaMalloc(&G.head, sizeof(double) * C));
+  CK(cudaMalloc(&G.carry, sizeof(double) * C));
+  CK(cudaMalloc(&G.head_flag, sizeof(int) * C));
+  k_merge_splits<<<(unsigned)cdiv(C + 1, 256), 256, 0, h->stream>>>(h->m_loc, h->rp_loc, C, G.split_row, G.split_nz);
+  LAUNCHED();
+  CK(cudaStreamSynchronize(h->stream));
+  return SPMV_OK;
+}
+
+static spmv_status launch_merge(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
+                                double alpha, double beta, const P2PHook& hook) {
+  MergeArgs a;
+  a.m = h->m_loc;
+  a.ntiles = h->mg.ntiles;
+  a.rowptr = h->rp_loc;
+  a.colidx = h->ci_loc;
+  a.vals = vals;
+  a.split_row = h->mg.split_row;
+  a.split_nz = h->mg.split_nz;
+  a.x = x;
+  a.y = y;
+  a.alpha = alpha;
+  a.beta = beta;
+  a.head = h->mg.head;
+  a.carry = h->mg.carry;
+  a.head_flag = h->mg.head_flag;
+  a.hk = hook;
+  if (h->dt == SPMV_F64) {
+    k_spmv_merge<double><<<a.ntiles, MG_NT, 0, s>>>(a);
+    LAUNCHED();
+    k_merge_fixup<double><<<(unsigned)cdiv(a.ntiles, 256), 256, 0, s>>>(a);
+    LAUNCHED();
+  } else {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+    k_spmv_merge<float><<<a.ntiles, MG_NT, 0, s>>>(a);
+    LAUNCHED();
+    k_merge_fixup<float><<<(unsigned)cdiv(a.ntiles, 256), 256, 0, s>>>(a);
+    LAUNCHED();
+  }
+  return SPMV_OK;
+}
+
+spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y, double alpha,
+                     double beta, const double* w, double* part, const P2PHook* hk) {
+  const P2PHook hook = hk ? *hk : P2PHook();
+  if (h->m_loc == 0) {
+    if (part) {
+      CK(cudaMemsetAsync(part, 0, sizeof(double) * h->grid, s));
+    }
+    return SPMV_OK;
+  }
+  if (alpha == 0.0 && !part) {
+    const int64_t g = std::min<int64_t>(cdiv(h->m_loc, 256), 4 * num_sms(h->device));
+    if (h->dt == SPMV_F64) k_scale<double><<<g, 256, 0, s>>>(h->m_loc, (double*)y, beta);
+    else k_scale<float><<<g, 256, 0, s>>>(h->m_loc, (float*)y, (double)(float)beta);
+    LAUNCHED();
+    return SPMV_OK;
+  }
+  if (h->kernel == SPMV_KERNEL_XPLAN && vals == h->vals) return launch_xplan(h, s, x, y, alpha, beta, w, part, hook);
+  const bool sell = h->kernel == SPMV_KERNEL_SELL || h->kernel == SPMV_KERNEL_SELL_SORTED;
+  if (sell && vals == h->vals) return launch_sell(h, s, x, y, alpha, beta, w, part, hook);
+  const int64_t vgrid_spmv = (h->kernel == SPMV_KERNEL_XPLAN || sell) ? h->grid_vec : h->grid;
+  if (h->kernel == SPMV_KERNEL_XSTAT) return launch_xstat(h, s, vals, x, y, alpha, beta, w, part, hook);
+  if (h->kernel == SPMV_KERNEL_MERGE) {
+    P2PHook wait_only = hook;
+    wait_only.push_slot = -1;
+    ST(launch_merge(h, s, vals, x, y, alpha, beta, wait_only));
+    if (part) {  // no fused dot in the merge kernel: one pass over w, y
+      P2PHook push_only = hook;
+      push_only.wait_x = 0;
+      k_dot_partials<<<(int)h->vgrid, 256, 0, s>>>(h->m_loc, w, (const double*)y, part, push_only);
+      LAUNCHED();
+    }
+    return SPMV_OK;
+  }
+  SpmvArgs a;
+  a.m = h->m_loc;
+  a.rowptr = h->rp_loc;
+  a.colidx = h->ci_loc;
+  a.vals = vals;
+  a.x = x;
+  a.y = y;
+  a.alpha = alpha;
+  a.beta = beta;
+  a.w = w;
+  a.part = part;
+  a.hk = hook;
+  if (h->dt == SPMV_F64) {
+    if (part) launch_vec<double, true>(h->lanes, h->unroll, vgrid_spmv, s, a);
+    else launch_vec<double, false>(h->lanes, h->unroll, vgrid_spmv, s, a);
+  } else {
+    a.alpha = (double)(float)alpha;
+    a.beta = (double)(float)beta;
+    launch_vec<float, false>(h->lanes, h->unroll, vgrid_spmv, s, a);
+  }
+  LAUNCHED();
+  return SPMV_OK;
+}

@@ -193,7 +193,7 @@ k_spmv_sell(SellArgs a) {
 
 // ---------------------------------------------------------------- builders
 // pairs[c] = ceil(max row length of chunk c / 2)
-__global__ void k_sell_pairs(int64_t m, const int* __restrict__ rowptr, int64_t nchunks, long long* __restrict__ pairs) {
+static __global__ void k_sell_pairs(int64_t m, const int* __restrict__ rowptr, int64_t nchunks, long long* __restrict__ pairs) {
   for (int64_t c = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; c < nchunks; c += int64_t(gridDim.x) * blockDim.x) {
     int L = 0;
     const int64_t r1 = cmin64(m, c * 32 + 32);
@@ -203,7 +203,7 @@ __global__ void k_sell_pairs(int64_t m, const int* __restrict__ rowptr, int64_t 
 }
 
 // pairs[c] = ceil(longest row of sorted chunk c / 2); rows are perm[nlong + 32c ..]
-__global__ void k_sell_pairs_sorted(int64_t m, const int* __restrict__ rowptr, const int* __restrict__ perm,
+static __global__ void k_sell_pairs_sorted(int64_t m, const int* __restrict__ rowptr, const int* __restrict__ perm,
                                     int64_t nlong, int64_t nchunks, long long* __restrict__ pairs) {
   for (int64_t c = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; c < nchunks; c += int64_t(gridDim.x) * blockDim.x) {
     int L = 0;
@@ -239,7 +239,7 @@ __global__ void k_sell_pack(int64_t m, const int* __restrict__ rowptr, const int
 }
 
 // Row lengths (sort keys) and identity row ids for the sorted variant.
-__global__ void k_row_len_ids(int64_t m, const int* __restrict__ rowptr, int* __restrict__ len, int* __restrict__ ids) {
+static __global__ void k_row_len_ids(int64_t m, const int* __restrict__ rowptr, int* __restrict__ len, int* __restrict__ ids) {
   for (int64_t i = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; i < m; i += int64_t(gridDim.x) * blockDim.x) {
     len[i] = rowptr[i + 1] - rowptr[i];
     ids[i] = int(i);

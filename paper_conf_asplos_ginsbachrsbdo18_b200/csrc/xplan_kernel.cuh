@@ -226,20 +226,11 @@ k_spmv_xplan(XplanArgs a) {
       }
 #pragma unroll
       for (int u = 0; u < XP_U; ++u) {
-#ifdef XP_DBG_NOX  // timing experiment: no x gathers (wrong results)
-        acc += double(v[u].a) * double(cc[u] & 0xffffu) + double(v[u].b);
-#else
         acc += double(v[u].a) * double(xs[cc[u] & 0xffffu]);
         acc += double(v[u].b) * double(xs[cc[u] >> 16]);
-#endif
       }
     }
-#ifdef XP_DBG_NOSYNC  // timing experiment: no partial exchange / tile barriers (wrong results)
-    if (acc == 1.2345) static_cast<T*>(a.y)[0] = T(acc);
-    if (false) {
-#else
     if (row != 0xffff) {
-#endif
       const int q = row / RB, jl = row - q * RB;
       const uint32_t laddr = smem_u32(recv + (t % XP_K) * R + b * RB + jl);
       st_async_f64(mapa_u32(laddr, q), acc, mapa_u32(smem_u32(&tbar[t % XP_K]), q));
@@ -297,12 +288,7 @@ k_spmv_xplan(XplanArgs a) {
   // Buffer reuse: partials of tile t+K (K = 3) are sent only after the sender
   // passed wait(t+1), i.e. after every CTA arrived(t+1), which each does after
   // finalize(t) (reads of recv[t%K] + re-arm of tbar[t%K]).
-#ifdef XP_DBG_NOSYNC
-  for (int t = 0; t < ntiles; ++t) process(t);
-  if (false) {
-#else
   if (ntiles > 0) {
-#endif
     process(0);
     cluster_arrive_relaxed();
     for (int t = 1; t < ntiles; ++t) {
@@ -337,7 +323,7 @@ __device__ __forceinline__ void xp_seg(const int* rowptr, const int* seg, int64_
 // sort the tile's rows by segment length (descending, ties by row: bitonic
 // sort of (len, row) keys), cut into CPT chunks of 32 lanes, record each
 // chunk's even step count and each row's slot (chunk = slot/32, lane = slot%32).
-__global__ void __launch_bounds__(XP_THREADS)
+static __global__ void __launch_bounds__(XP_THREADS)
 k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_t m, int B,
              const long long* __restrict__ crow, const int* __restrict__ tile0, int ncl, int* __restrict__ chunk_len,
              uint16_t* __restrict__ chunk_row, int* __restrict__ row_slot) {
@@ -438,7 +424,7 @@ k_xplan_pack(const int* __restrict__ rowptr, const int* __restrict__ colidx, con
 
 // Padding: value regions 0, column regions the pad column W (x pad 0.0).
 // Chunk c of the plan spans [chunk_off[c], chunk_off[c] + len*32*(ts+2)).
-__global__ void k_xplan_fill(unsigned char* __restrict__ plan, const long long* __restrict__ chunk_off,
+static __global__ void k_xplan_fill(unsigned char* __restrict__ plan, const long long* __restrict__ chunk_off,
                              const int* __restrict__ chunk_len, int64_t nchunks, int ts, uint16_t pad) {
   for (int64_t c = blockIdx.x; c < nchunks; c += gridDim.x) {
     const int len = chunk_len[c];

@@ -266,7 +266,7 @@ k_spmv_xstat(XstatArgs a) {
 // Split points of every row at the column-block boundaries b*W (b = 1..B-1):
 // seg[(b-1)*m + i] = first k in [rowptr[i], rowptr[i+1]) with colidx[k] >= b*W
 // (binary search; needs ascending columns in each row).
-__global__ void __launch_bounds__(256)
+static __global__ void __launch_bounds__(256)
 k_xstat_splits(int64_t m, const int* __restrict__ rowptr, const int* __restrict__ colidx, int B, int W,
                int* __restrict__ seg) {
   for (int64_t i = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; i < m;

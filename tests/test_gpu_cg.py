@@ -117,6 +117,30 @@ def test_npb_host_z_equals_device_z(sp, torch_dev):
             assert torch.equal(od.cpu(), oh)
 
 
+def test_npb_host_graph_replay(sp, torch_dev):
+    """Several host-buffer calls in a row on ONE handle replay the same captured
+    graph (the side-stream z copy waits on the external event of the earlier
+    capture): every call's host z, x and {zeta, rnorm} equal a device-buffer run
+    on a second handle bit for bit."""
+    torch, dev = torch_dev
+    A = gen.makea("S")
+    rp, ci, va = to_dev(A, dev)
+    with sp.CSRMatrix(rp, ci, va, A.n) as Mh, sp.CSRMatrix(rp, ci, va, A.n) as Md:
+        xd = torch.ones(A.n, dtype=torch.float64, device=dev)
+        zd = torch.empty_like(xd)
+        od = torch.zeros(2, dtype=torch.float64, device=dev)
+        xh = torch.ones(A.n, dtype=torch.float64).pin_memory()
+        zh = torch.empty(A.n, dtype=torch.float64).pin_memory()
+        oh = torch.zeros(2, dtype=torch.float64).pin_memory()
+        for it in range(5):
+            zh.fill_(float("nan"))  # a stale or missing copy shows
+            Mh.npb_outer(xh, zh, 25, 10.0, oh)  # synchronous (host buffers)
+            Md.npb_outer(xd, zd, 25, 10.0, od)
+            torch.cuda.synchronize()
+            assert torch.equal(zd.cpu(), zh) and torch.equal(xd.cpu(), xh), it
+            assert torch.equal(od.cpu(), oh), it
+
+
 def _npb(sp, torch, dev, cls, niter=None, host=False):
     na, nonzer, NITER, shift = gen.NPB_CLASSES[cls]
     A = gen.makea(cls)

@@ -192,3 +192,31 @@ def test_stencil_tma_path_is_taken(env, monkeypatch):
     with pytest.raises(sp.SpmvError) as e:
         sp.stencil27_apply(33, 9, 17, x, torch.empty_like(x))
     assert e.value.status == sp.SPMV_ERR_ARG
+
+
+def test_stencil_binding_checks(env):
+    """The binding checks what the raw-pointer ABI cannot: x and y dtypes agree,
+    both are contiguous and hold nx*ny*nz elements."""
+    torch, dev, sp = env
+    n = 8 * 8 * 8
+    x = torch.rand(n, dtype=torch.float64, device=dev)
+    with pytest.raises(ValueError):
+        sp.stencil27_apply(8, 8, 8, x.float(), torch.empty_like(x))
+    with pytest.raises(ValueError):
+        sp.stencil27_apply(8, 8, 8, x, torch.empty(n - 1, dtype=torch.float64, device=dev))
+    with pytest.raises(ValueError):
+        sp.stencil27_apply(8, 8, 8, x[: n - 1], torch.empty_like(x))
+    with pytest.raises(ValueError):
+        sp.stencil27_apply(8, 8, 8, torch.rand(2 * n, dtype=torch.float64, device=dev)[::2], torch.empty_like(x))
+
+
+def test_stencil_tma_mandatory_rejects_general_weights(env, monkeypatch):
+    """SPMV_STENCIL_TMA=2 with general weights (no box2 form) is an argument
+    error, not a silent cp.async run."""
+    torch, dev, sp = env
+    monkeypatch.setenv("SPMV_STENCIL_TMA", "2")
+    x = torch.rand(64 ** 3, dtype=torch.float64, device=dev)
+    w = np.arange(27, dtype=np.float64)
+    with pytest.raises(sp.SpmvError) as e:
+        sp.stencil27_apply(64, 64, 64, x, torch.empty_like(x), w27=w)
+    assert e.value.status == sp.SPMV_ERR_ARG
