@@ -21,7 +21,8 @@ roofline = the SpMV kernel (the dominant kernel, ~97% of the step's bytes),
          timed alone with CUDA events on the launching stream (an L2 flush
          queued ahead of the start event): algorithmic bytes / duration vs
          the measured HBM copy bandwidth of MEASURED_PEAKS.json.
-cpu_baseline = the CPU oracle (oracle/, plain C, 1 thread) on a bounded sample.
+cpu_baseline = the CPU oracle on a bounded sample: its OpenMP copy on all host cores
+         (value) and the plain oracle on 1 thread (single_thread).
 `--impl reference` times the oracle itself as the reference arm.
 """
 from __future__ import annotations
@@ -358,24 +359,46 @@ def run_ours(args):
 
 
 def cpu_baseline(A, shift, budget_s=15.0):
-    """The oracle as it stands (plain C, 1 thread) on a bounded sample: whole NAS
-    outer iterations of the same class-C workload until ~budget_s of CPU work."""
+    """The oracle as it stands on a bounded sample of the same class-C workload:
+    whole NAS outer iterations (after one untimed warm-up iteration, like the
+    reference arm) until ~budget_s/2 of CPU work, (1) oracle/oracle_spmv.c on
+    1 thread and (2) its OpenMP schedule(static) copy oracle/oracle_omp.c on
+    every core of sched_getaffinity.  `value`/`cores`
+    are the all-core run; `single_thread` the plain oracle."""
     import numpy as np
 
     import oracle
-    x = np.ones(A.n)
-    t0 = time.perf_counter()
-    steps = 0
-    while True:
-        oracle.npb_outer(A.rowptr, A.colidx, A.vals, x, 25, shift)
-        steps += 1
-        el = time.perf_counter() - t0
-        if el >= budget_s or steps >= 50:
-            break
-    return {"value": round(25.0 * steps / el, 3), "unit": UNIT, "cores": 1, "kind": "oracle",
-            "sample": f"{steps} NAS CG class {CLS} outer iterations ({25 * steps} CG iterations + "
-                      f"{steps} residual SpMVs) in {el:.1f} s, oracle/oracle_spmv.c -O3 1 thread",
-            "host": _cpu_model()}
+    ncores = len(os.sched_getaffinity(0))
+
+    def timed(fn, budget):
+        x = np.ones(A.n)
+        fn(x)  # warm-up (page faults of the work arrays, caches)
+        x[:] = 1.0
+        t0 = time.perf_counter()
+        steps = 0
+        while True:
+            fn(x)
+            steps += 1
+            el = time.perf_counter() - t0
+            if el >= budget or steps >= 50:
+                return steps, el
+
+    half = budget_s / 2
+    s1, e1 = timed(lambda x: oracle.npb_outer(A.rowptr, A.colidx, A.vals, x, 25, shift), half)
+    used = [1]
+
+    def omp(x):
+        used[0] = oracle.npb_outer_omp(A.rowptr, A.colidx, A.vals, x, 25, shift, nthreads=ncores)[3]
+
+    sN, eN = timed(omp, half)
+    return {"value": round(25.0 * sN / eN, 3), "unit": UNIT, "cores": int(used[0]), "kind": "oracle",
+            "sample": f"{sN} NAS CG class {CLS} outer iterations ({25 * sN} CG iterations + {sN} residual SpMVs) "
+                      f"in {eN:.1f} s after 1 warm-up, oracle/oracle_omp.c (the oracle's loops, OpenMP "
+                      f"schedule(static)) on {used[0]} threads",
+            "single_thread": {"value": round(25.0 * s1 / e1, 3), "cores": 1,
+                              "sample": f"{s1} outer iterations in {e1:.1f} s after 1 warm-up, "
+                                        "oracle/oracle_spmv.c -O3 1 thread"},
+            "affinity_cores": ncores, "host": _cpu_model()}
 
 
 def _cpu_model():

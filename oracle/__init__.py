@@ -273,3 +273,44 @@ def spmv_jds(J, x, y_old=None, alpha=1.0, beta=0.0):
                           _ptr(_c(J.indices, np.int32)), _ptr(_c(J.data, dt)), _ptr(x), _ptr(yo),
                           float(alpha), float(beta), int(f32), _ptr(y_ref), _ptr(bound))
     return y_ref[:J.m], bound[:J.m]
+
+
+# ---------------------------------------------------------------- CPU baseline
+# oracle_omp.c: the textbook-CG loops of oracle_spmv.c with OpenMP
+# schedule(static) row/element loops, for bench.py's all-core CPU baseline
+# (BASELINE.md section 3).  Not pinned, never used for parity.
+_OMP_SRC = os.path.join(_HERE, "oracle_omp.c")
+_OMP_LIB = os.path.join(_HERE, "liboracle_omp.so")
+_omp = None
+
+
+def build_omp(force: bool = False) -> str:
+    if force or not os.path.exists(_OMP_LIB) or os.path.getmtime(_OMP_LIB) < os.path.getmtime(_OMP_SRC):
+        tmp = _OMP_LIB + f".tmp{os.getpid()}"
+        subprocess.check_call(["gcc", "-O3", "-march=native", "-ffp-contract=off", "-std=c11", "-fPIC", "-fopenmp",
+                               "-shared", "-o", tmp, _OMP_SRC, "-lm"])
+        os.replace(tmp, _OMP_LIB)
+    return _OMP_LIB
+
+
+def npb_outer_omp(rowptr, colidx, vals, x, cgitmax, shift, nthreads=0):
+    """oracle_omp.c's NAS outer iteration on nthreads OpenMP threads (0 = all);
+    returns (z, zeta, rnorm, threads_used)."""
+    global _omp
+    if _omp is None:
+        build_omp()
+        _omp = ctypes.CDLL(_OMP_LIB)
+        _omp.omp_npb_outer.argtypes = [_I64, _P, _P, _P, _P, _P, _I32, _D, _P, _P, _I32]
+        _omp.omp_npb_outer.restype = ctypes.c_int
+    assert x.dtype == np.float64 and x.flags.c_contiguous
+    rowptr = _c(rowptr, np.int32)
+    colidx = _c(colidx, np.int32)
+    vals = _c(vals, np.float64)
+    n = rowptr.shape[0] - 1
+    z = np.zeros(n)
+    zeta = ctypes.c_double(0.0)
+    rn = ctypes.c_double(0.0)
+    used = _omp.omp_npb_outer(n, _ptr(rowptr), _ptr(colidx), _ptr(vals), _ptr(x), _ptr(z), int(cgitmax),
+                              float(shift), ctypes.byref(zeta), ctypes.byref(rn), int(nthreads))
+    return z, zeta.value, rn.value, used
+

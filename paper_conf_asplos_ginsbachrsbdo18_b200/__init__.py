@@ -32,7 +32,7 @@ _ST = ctypes.c_int
 SPMV_OK, SPMV_ERR_ARG, SPMV_ERR_INDEX, SPMV_ERR_ALIAS, SPMV_ERR_CUDA = 0, 1, 2, 3, 4
 SPMV_ERR_NCCL, SPMV_ERR_NOMEM, SPMV_ERR_BREAKDOWN, SPMV_ERR_UNSUPPORTED = 5, 6, 7, 8
 SPMV_F64, SPMV_F32 = 0, 1
-KERNELS = {"auto": 0, "scalar": 1, "vector": 2, "merge": 3, "xstat": 4, "xplan": 5, "sell": 6, "sellsort": 7}
+KERNELS = {"auto": 0, "scalar": 1, "vector": 2, "merge": 3, "xstat": 4, "xplan": 5, "sell": 6, "sellsort": 7, "xt": 8}
 KERNEL_NAMES = {v: k for k, v in KERNELS.items()}
 
 
@@ -76,6 +76,7 @@ spmv_dist_get_unique_id_c = _decl("spmv_dist_get_unique_id", [_P])
 spmv_dist_init_c = _decl("spmv_dist_init", [ctypes.POINTER(_P), _I32, _I32, _P, _I32])
 spmv_dist_destroy_c = _decl("spmv_dist_destroy", [_P])
 spmv_dist_init_p2p_c = _decl("spmv_dist_init_p2p", [ctypes.POINTER(_P), _I32, _I32, _I32])
+spmv_dist_init_proxy_c = _decl("spmv_dist_init_proxy", [ctypes.POINTER(_P), _I32, _I32, _I32])
 spmv_csr_p2p_handle_c = _decl("spmv_csr_p2p_handle", [_P, _P])
 spmv_csr_p2p_connect_c = _decl("spmv_csr_p2p_connect", [_P, _P])
 spmv_dist_plan_host_c = _decl("spmv_dist_plan_host", [_P, _P, _I64, _I32, _I32, _P, _P, _P])
@@ -101,7 +102,7 @@ EXPORTS = ["spmv_csr_create", "spmv_csr", "cg_solve", "cg_npb_outer", "spmv_cg_s
            "spmv_csr_destroy", "spmv_csr_partition", "spmv_csr_merge_splits", "spmv_csr_info",
            "spmv_launch_count", "spmv_status_string", "spmv_last_error_string",
            "spmv_dist_get_unique_id", "spmv_dist_init", "spmv_dist_destroy", "spmv_dist_plan_host",
-           "spmv_dist_colidx", "spmv_dist_init_p2p", "spmv_csr_p2p_handle", "spmv_csr_p2p_connect",
+           "spmv_dist_colidx", "spmv_dist_init_p2p", "spmv_dist_init_proxy", "spmv_csr_p2p_handle", "spmv_csr_p2p_connect",
            "spmv_dist_halo_host", "spmv_dist_halo", "stencil27_apply",
            "spmv_jds_create", "spmv_jds", "spmv_jds_destroy"]
 # every symbol include/idioms.h declares
@@ -224,14 +225,21 @@ class Dist:
     transport="p2p": no NCCL; exchanges run in the library's kernels over
     CUDA-IPC peer memory; IPC handles are all-gathered through the torch
     process group when a CSRMatrix is created.
+    transport="proxy": single process, no communication: a handle does rank
+    `rank`'s share of an nranks-way run on one GPU (measurement only,
+    spmv_dist_init_proxy).
     """
 
     def __init__(self, rank: int, nranks: int, device: int, group=None, transport: str = "nccl"):
-        import torch
-        import torch.distributed as dist
         self.group = group
         self.transport = transport
         self.rank, self.nranks, self.device = rank, nranks, device
+        if transport == "proxy":
+            h = _P()
+            _check(spmv_dist_init_proxy_c(ctypes.byref(h), rank, nranks, device), "spmv_dist_init_proxy")
+            self.handle = h
+            return
+        import torch.distributed as dist
         if transport == "p2p":
             h = _P()
             _check(spmv_dist_init_p2p_c(ctypes.byref(h), rank, nranks, device), "spmv_dist_init_p2p")

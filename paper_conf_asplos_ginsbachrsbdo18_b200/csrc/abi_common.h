@@ -31,6 +31,7 @@
 #include "spmv_kernels.cuh"
 #include "xplan_kernel.cuh"
 #include "xstat_kernel.cuh"
+#include "xt_kernel.cuh"
 
 using namespace spmv;
 
@@ -79,6 +80,7 @@ struct spmv_dist_s {
   ncclComm_t comm = nullptr;  // NCCL transport (nullptr for p2p)
   int rank = 0, nranks = 1, device = 0;
   int p2p = 0;                // 1: exchanges over CUDA-IPC peer memory (p2p_kernels.cuh)
+  int proxy = 0;              // 1: measurement proxy: rank r's share on one GPU, exchanges skipped
 };
 
 struct Graph {
@@ -144,6 +146,29 @@ struct spmv_csr_s {
   } xp;
   cudaStream_t side = nullptr;
   cudaEvent_t ev_fork = nullptr, ev_join = nullptr;
+  // XT (TMA-streamed column-parted plan, xt_kernel.cuh)
+  struct XtPlan {
+    bool built = false;
+    int B = 0, Q = 0, NB = 0, NS = 0, ncl = 0, ntiles = 0, xcap = 0;
+    size_t smem = 0;
+    int64_t bytes = 0, nchunks = 0, nstages = 0;
+    unsigned char* plan = nullptr;
+    int *cl_part = nullptr, *cl_tile0 = nullptr, *cta_w = nullptr, *cta_st0 = nullptr, *part_cl0 = nullptr;
+    long long *cl_rows = nullptr, *cta_col0 = nullptr, *st_off = nullptr, *bcol = nullptr, *ck_off = nullptr;
+    uint32_t* st_info = nullptr;
+    uint2* ck_meta = nullptr;
+    int *bseg = nullptr, *ck_len = nullptr, *row_slot = nullptr, *gcnt = nullptr;
+    double* ypart = nullptr;
+    void (*k)(XtArgs) = nullptr;
+    void (*kdot)(XtArgs) = nullptr;
+    void release() {
+      void* bufs[] = {plan, cl_part, cl_tile0, cta_w, cta_st0, part_cl0, cl_rows, cta_col0, st_off, bcol, ck_off,
+                      st_info, ck_meta, bseg, ck_len, row_slot, gcnt, ypart};
+      for (void* q : bufs)
+        if (q) cudaFree(q);
+      *this = XtPlan();
+    }
+  } xt;
   // SELL (SELL-32 device plan, x gathered from global memory)
   struct Sell {
     bool built = false;
@@ -274,6 +299,10 @@ spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only);
 spmv_status sell_build(spmv_csr_s* h, double max_pad, int sorted, bool* ok);
 spmv_status sell_pack(spmv_csr_s* h, const void* vals, int values_only);
 spmv_status merge_setup(spmv_csr_s* h);
+spmv_status xt_build(spmv_csr_s* h, bool* ok);
+spmv_status xt_pack(spmv_csr_s* h, const void* vals, int values_only);
+spmv_status launch_xt(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha, double beta,
+                      const double* w, double* part, const P2PHook& hook);
 // Local SpMV of the handle: y = alpha*A_loc*x + beta*y (+ partial w.y per CTA).
 spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y, double alpha,
                      double beta, const double* w, double* part, const P2PHook* hk = nullptr);

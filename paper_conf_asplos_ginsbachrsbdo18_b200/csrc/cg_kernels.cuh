@@ -125,16 +125,12 @@ k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
     }
   }
   if (hk.enabled) {
-    // all peer stores of the CTA happen-before thread 0's system-scope fence
-    // (bar.sync + cumulative fence), which precedes the ticket; the last CTA
-    // publishes with release stores
+    // the CTA's peer stores happen-before thread 0's acq_rel ticket (bar.sync);
+    // the last CTA fences at system scope and publishes (p2p_signal)
     __syncthreads();
-    if (threadIdx.x == 0) {
-      __threadfence_system();
-      if (atomicAdd(hk.c.ticket, 1) == int(gridDim.x) - 1) {
-        *hk.c.ticket = 0;
-        p2p_signal(hk.c, P2P_XSLOT);
-      }
+    if (threadIdx.x == 0 && ticket_acq_rel_gpu(hk.c.ticket) == int(gridDim.x) - 1) {
+      *hk.c.ticket = 0;
+      p2p_signal(hk.c, P2P_XSLOT);
     }
   }
   if (tol > 0.0) {
@@ -245,12 +241,9 @@ k_cgcg(int64_t n, int k, SumSrc gam, SumSrc gam_old, SumSrc del, double* __restr
     // push above re-arms hk.c.ticket while other CTAs may already be here
     int* tk2 = hk.c.ticket + 2;
     __syncthreads();
-    if (threadIdx.x == 0) {
-      __threadfence_system();
-      if (atomicAdd(tk2, 1) == int(gridDim.x) - 1) {
-        *tk2 = 0;
-        p2p_signal(hk.c, P2P_XSLOT);
-      }
+    if (threadIdx.x == 0 && ticket_acq_rel_gpu(tk2) == int(gridDim.x) - 1) {
+      *tk2 = 0;
+      p2p_signal(hk.c, P2P_XSLOT);
     }
   }
 }

@@ -102,6 +102,18 @@ __device__ __forceinline__ void p2p_wait_flags(const unsigned long long* flags, 
   }
 }
 
+// Last-CTA ticket with acquire-release semantics at GPU scope: the CTA's
+// writes (ordered before thread 0 by the preceding bar.sync) happen-before the
+// increment, and the CTA drawing the last ticket has acquired every other
+// CTA's writes.  Only that CTA then fences at system scope and publishes with
+// st.release.sys (p2p_signal): causality is transitive across the two scopes
+// (PTX memory model), so one system-scope fence per kernel replaces one per CTA.
+__device__ __forceinline__ int ticket_acq_rel_gpu(int* t) {
+  int old;
+  asm volatile("atom.add.acq_rel.gpu.global.s32 %0, [%1], 1;\n" : "=r"(old) : "l"(t) : "memory");
+  return old;
+}
+
 constexpr int P2P_NSLOT = 8;       // scalar slots (same ids as reduce_src slots)
 constexpr int P2P_XSLOT = P2P_NSLOT;  // slot_epoch index of the x exchange
 
@@ -164,12 +176,11 @@ __device__ __forceinline__ void p2p_prologue_wait(const P2PHook& h) {
 __device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const double* part, int count) {
   if (!h.enabled || h.push_slot < 0) return;
   __shared__ int s_last;
-  // part[blockIdx.x] was stored by thread 0: one fence by that thread orders
-  // it before the ticket (threadFenceReduction pattern)
+  // part[blockIdx.x] was stored by thread 0; the acq_rel ticket orders it
+  // before the increment and gives the last CTA every other CTA's partial
   __syncthreads();
   if (threadIdx.x == 0) {
-    __threadfence();
-    const int tk = atomicAdd(h.c.ticket, 1);
+    const int tk = ticket_acq_rel_gpu(h.c.ticket);
     s_last = (tk == int(gridDim.x) - 1);
 #ifdef SPMV_P2P_TRACE
     if (blockIdx.x == 0 || s_last) printf("push_last blk %d ticket %d grid %d slot %d\n", blockIdx.x, tk, gridDim.x, h.push_slot);

@@ -24,6 +24,7 @@ bool use_p2p(const spmv_csr_s* h) { return h->dist && h->dist->p2p; }
 
 // All-gather of this rank's slice (already at xpad + rank*maxlen) and wait.
 spmv_status exchange_x(spmv_csr_s* h, cudaStream_t s) {
+  if (h->dist->proxy) return SPMV_OK;  // measurement proxy: no communication
   if (use_p2p(h)) {
     if (!h->p2p_connected) return arg_fail("p2p handle not connected (spmv_csr_p2p_connect)");
     const P2PCtx c = p2p_ctx(h);
@@ -73,7 +74,7 @@ SumSrc p2p_src(spmv_csr_s* h, int slot) {
 }
 
 spmv_status reduce_src(spmv_csr_s* h, cudaStream_t s, SumSrc in, int slot, SumSrc* out) {
-  if (!h->dist) { *out = in; return SPMV_OK; }
+  if (!h->dist || h->dist->proxy) { *out = in; return SPMV_OK; }  // proxy: this rank's partials only
   if (use_p2p(h)) {
     if (!h->p2p_connected) return arg_fail("p2p handle not connected (spmv_csr_p2p_connect)");
     const P2PCtx c = p2p_ctx(h);
@@ -169,6 +170,19 @@ extern "C" spmv_status spmv_dist_init_p2p(spmv_dist_t* out, int32_t rank, int32_
   d->nranks = nranks;
   d->device = device;
   d->p2p = 1;
+  *out = d;
+  return SPMV_OK;
+}
+
+extern "C" spmv_status spmv_dist_init_proxy(spmv_dist_t* out, int32_t rank, int32_t nranks, int32_t device) {
+  if (!out || nranks < 1 || rank < 0 || rank >= nranks) return arg_fail("bad dist arguments");
+  *out = nullptr;
+  CK(cudaSetDevice(device));
+  spmv_dist_s* d = new spmv_dist_s();
+  d->rank = rank;
+  d->nranks = nranks;
+  d->device = device;
+  d->proxy = 1;
   *out = d;
   return SPMV_OK;
 }

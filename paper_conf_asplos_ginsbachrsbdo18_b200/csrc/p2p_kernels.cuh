@@ -10,7 +10,8 @@
 // plus local (never remote) counters: epoch (this rank's exchange count),
 // slot_epoch[NSLOT+1] (epoch of the latest push of each slot / of x), ticket.
 //
-// A push writes the data into every peer (and itself), fences at system scope,
+// A push writes the data into every peer (and itself); every CTA takes an
+// acq_rel ticket at GPU scope and the last one fences at system scope,
 // increments the local epoch e and stores flags[me] = e into every peer with
 // st.release.sys.  A consumer waits until flags[q] >= e for all q != me with
 // ld.acquire.sys, then reads.  All ranks run the same sequence of pushes, so
@@ -50,13 +51,10 @@ k_p2p_push_x(int64_t n, int64_t maxlen, P2PCtx c) {
     }
   }
   __syncthreads();
-  if (threadIdx.x == 0) {
-    __threadfence_system();  // cumulative: orders the whole CTA's peer stores
-    const int t = atomicAdd(c.ticket, 1);
-    if (t == int(gridDim.x) - 1) {  // last CTA: every slice store is fenced
-      *c.ticket = 0;
-      p2p_signal(c, P2P_XSLOT);
-    }
+  // acq_rel ticket at GPU scope; the last CTA fences at system scope and publishes
+  if (threadIdx.x == 0 && ticket_acq_rel_gpu(c.ticket) == int(gridDim.x) - 1) {
+    *c.ticket = 0;
+    p2p_signal(c, P2P_XSLOT);
   }
 }
 

@@ -674,10 +674,11 @@ spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void
     LAUNCHED();
     return SPMV_OK;
   }
+  if (h->kernel == SPMV_KERNEL_XT && vals == h->vals) return launch_xt(h, s, x, y, alpha, beta, w, part, hook);
   if (h->kernel == SPMV_KERNEL_XPLAN && vals == h->vals) return launch_xplan(h, s, x, y, alpha, beta, w, part, hook);
   const bool sell = h->kernel == SPMV_KERNEL_SELL || h->kernel == SPMV_KERNEL_SELL_SORTED;
   if (sell && vals == h->vals) return launch_sell(h, s, x, y, alpha, beta, w, part, hook);
-  const int64_t vgrid_spmv = (h->kernel == SPMV_KERNEL_XPLAN || sell) ? h->grid_vec : h->grid;
+  const int64_t vgrid_spmv = (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_XT || sell) ? h->grid_vec : h->grid;
   if (h->kernel == SPMV_KERNEL_XSTAT) return launch_xstat(h, s, vals, x, y, alpha, beta, w, part, hook);
   if (h->kernel == SPMV_KERNEL_MERGE) {
     P2PHook wait_only = hook;

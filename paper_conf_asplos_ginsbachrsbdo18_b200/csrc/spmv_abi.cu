@@ -255,7 +255,20 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
   choose_kernel(h, rk, rl);
   int plan = o.plan;
   env_int("SPMV_PLAN", &plan);
-  if (rk == SPMV_KERNEL_XPLAN || (rk == SPMV_KERNEL_AUTO && plan)) {
+  if (rk == SPMV_KERNEL_XT || (rk == SPMV_KERNEL_AUTO && plan)) {
+    // auto + plan: the TMA-streamed column-parted plan whenever x fits 16 parts of
+    // cluster-resident blocks and rows are long enough
+    if (rk == SPMV_KERNEL_XT || h->row_mean >= 16.0) {
+      bool ok = false;
+      spmv_status st = xt_build(h, &ok);
+      if (st != SPMV_OK) return fail(st);
+      if (ok) {
+        h->kernel = SPMV_KERNEL_XT;
+        h->grid = (int64_t)h->xt.ncl * h->xt.B;
+      }
+    }
+  }
+  if (h->kernel != SPMV_KERNEL_XT && (rk == SPMV_KERNEL_XPLAN || (rk == SPMV_KERNEL_AUTO && plan))) {
     // auto + plan: the column-blocked x-stationary plan whenever x fits the
     // shared memory of a cluster and rows are long enough
     if (rk == SPMV_KERNEL_XPLAN || h->row_mean >= 16.0) {
@@ -270,7 +283,7 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
     }
   }
   const bool skewed = (double)h->row_max > 32.0 * std::max(h->row_mean, 1.0);
-  if (h->kernel != SPMV_KERNEL_XPLAN && (rk == SPMV_KERNEL_SELL || rk == SPMV_KERNEL_SELL_SORTED ||
+  if (h->kernel != SPMV_KERNEL_XPLAN && h->kernel != SPMV_KERNEL_XT && (rk == SPMV_KERNEL_SELL || rk == SPMV_KERNEL_SELL_SORTED ||
                                          (rk == SPMV_KERNEL_AUTO && plan))) {
     // auto + plan, x too large for the clusters (or short rows): a SELL-32 plan
     // with global x gathers -- chunks of consecutive rows when they pad by
@@ -285,7 +298,8 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
       h->grid = h->sl.nmulti > 0 ? h->vgrid : h->sl.grid;  // dot partials: k_dot_partials or fused
     }
   }
-  if (h->kernel != SPMV_KERNEL_XPLAN && h->kernel != SPMV_KERNEL_SELL && h->kernel != SPMV_KERNEL_SELL_SORTED &&
+  if (h->kernel != SPMV_KERNEL_XPLAN && h->kernel != SPMV_KERNEL_XT && h->kernel != SPMV_KERNEL_SELL &&
+      h->kernel != SPMV_KERNEL_SELL_SORTED &&
       rk != SPMV_KERNEL_VECTOR && rk != SPMV_KERNEL_SCALAR && rk != SPMV_KERNEL_XSTAT && h->m_loc > 0 &&
       (rk == SPMV_KERNEL_MERGE || skewed)) {
     // skewed rows without a plan (a long row would pin one warp of the vector kernel): merge path
@@ -294,7 +308,8 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
     h->kernel = SPMV_KERNEL_MERGE;
     h->grid = h->vgrid;  // dot partials come from k_dot_partials
   }
-  if (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_MERGE || h->kernel == SPMV_KERNEL_SELL ||
+  if (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_XT || h->kernel == SPMV_KERNEL_MERGE ||
+      h->kernel == SPMV_KERNEL_SELL ||
       h->kernel == SPMV_KERNEL_SELL_SORTED) {
   } else if (rk == SPMV_KERNEL_XSTAT) {
     bool ok = false;
@@ -319,6 +334,7 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   cudaError_t e = h->stream ? cudaStreamSynchronize(h->stream) : cudaDeviceSynchronize();
   if (e != cudaSuccess) st = cuda_fail(e, "pending asynchronous error", __LINE__);
   h->g_npb.reset();
+  h->xt.release();
   for (size_t q = 0; q < h->peers.size(); ++q)
     if (h->peers[q] && h->peers[q] != h->fabric) cudaIpcCloseMemHandle(h->peers[q]);
   if (h->fabric) {
@@ -387,6 +403,7 @@ extern "C" spmv_status spmv_csr_update_values(spmv_csr_t h, const void* vals) {
   ST(need_device(vals, h->device, "vals must be a device pointer", h->nnz == 0));
   h->vals = vals;
   if (h->xp.built) ST(xplan_pack(h, vals, 1));
+  if (h->xt.built) ST(xt_pack(h, vals, 1));
   if (h->sl.built) ST(sell_pack(h, vals, 1));
   h->g_npb.reset();
   return SPMV_OK;
@@ -479,12 +496,16 @@ extern "C" spmv_status spmv_csr_info(spmv_csr_t h, spmv_info_t* info) {
   info->row_end = h->row0 + h->m_loc;
   info->nnz_local = h->k1 - h->k0;
   info->rank = h->dist ? h->dist->rank : 0;
-  info->transport = h->dist ? (h->dist->p2p ? 2 : 1) : 0;
+  info->transport = h->dist ? (h->dist->p2p ? 2 : h->dist->proxy ? 3 : 1) : 0;
   info->nranks = h->dist ? h->dist->nranks : 1;
   info->sorted_cols = h->sorted;
   info->grid = h->grid;
-  info->cluster = h->kernel == SPMV_KERNEL_XPLAN ? h->xp.B : h->kernel == SPMV_KERNEL_XSTAT ? h->xB : 0;
-  info->plan_bytes = h->xp.built ? (int64_t)h->xp.bytes
+  info->cluster = h->kernel == SPMV_KERNEL_XPLAN ? h->xp.B
+                : h->kernel == SPMV_KERNEL_XT    ? h->xt.B
+                : h->kernel == SPMV_KERNEL_XSTAT ? h->xB
+                                                 : 0;
+  info->plan_bytes = h->xt.built ? (int64_t)h->xt.bytes
+                   : h->xp.built ? (int64_t)h->xp.bytes
                    : h->sl.built  ? (int64_t)h->sl.pairs * 64 * (int64_t)(h->ts + 4)
                                   : 0;
   return SPMV_OK;

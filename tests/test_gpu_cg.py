@@ -199,7 +199,7 @@ def test_npb_graph_vs_eager_bitexact(sp, torch_dev, monkeypatch):
     assert np.array_equal(z1, z2) and np.array_equal(r1, r2)
 
 
-@pytest.mark.parametrize("kernel", ["merge", "vector", "xstat", "xplan", "sell", "sellsort"])
+@pytest.mark.parametrize("kernel", ["merge", "vector", "xstat", "xplan", "sell", "sellsort", "xt"])
 def test_npb_s_every_kernel(sp, torch_dev, kernel):
     """NPB class S zeta with every SpMV kernel inside CG (fused or separate dot)."""
     torch, dev = torch_dev

@@ -220,7 +220,7 @@ def test_nas_full_size(sp, torch_dev, cls):
     A = gen.makea(cls)
     x = gen.uniform(A.n, seed=31)
     info = run_case(sp, torch, dev, A, x, what=f"NAS {cls}")
-    assert info["kernel_name"] in ("vector", "merge", "xstat", "xplan", "scalar")
+    assert info["kernel_name"] == "xt", info  # the auto choice for NAS-shaped matrices
 
 
 def test_parboil_full_size_fp32(sp, torch_dev):
@@ -352,13 +352,13 @@ def test_xplan_alpha_beta_update_values(sp, torch_dev):
     x_h = gen.uniform(A.n, seed=19)
     y0 = gen.uniform(A.m, seed=20)
     for a, b in [(2.0, -1.0), (0.0, 3.0), (1.0, 0.0), (-1.5, 1.0)]:
-        info = run_case(sp, torch, dev, A, x_h, alpha=a, beta=b, y0=y0, what=f"xplan a={a} b={b}")
+        info = run_case(sp, torch, dev, A, x_h, alpha=a, beta=b, y0=y0, kernel="xplan", what=f"xplan a={a} b={b}")
         assert info["kernel_name"] == "xplan"
     # in-place value change + update_values (the paper's lazy-copy flag)
     rp, ci, va = to_dev(A, dev)
     x = torch.from_numpy(x_h).to(dev)
     y = torch.empty(A.m, dtype=torch.float64, device=dev)
-    with sp.CSRMatrix(rp, ci, va, A.n) as M:
+    with sp.CSRMatrix(rp, ci, va, A.n, kernel="xplan") as M:
         assert M.info()["kernel_name"] == "xplan"
         v2_h = gen.uniform(A.nnz, seed=23)
         va.copy_(torch.from_numpy(v2_h))
