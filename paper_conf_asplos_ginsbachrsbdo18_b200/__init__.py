@@ -17,7 +17,8 @@ import ctypes
 import os
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libspmv_b200.so")
+# SPMV_LIB_PATH: a variant build of tools/build_variants.sh (sweeps and diagnostics only)
+LIB_PATH = os.environ.get("SPMV_LIB_PATH") or os.path.join(_HERE, "libspmv_b200.so")
 
 if not os.path.exists(LIB_PATH):
     raise ImportError(
@@ -38,7 +39,7 @@ KERNEL_NAMES = {v: k for k, v in KERNELS.items()}
 
 class SpmvOpts(ctypes.Structure):
     _fields_ = [("stream", _P), ("kernel", _I32), ("vec_lanes", _I32), ("validate", _I32),
-                ("plan", _I32), ("dist", _P)]
+                ("plan", _I32), ("dist", _P), ("l2_window", _I32)]
 
 
 class SpmvInfo(ctypes.Structure):
@@ -274,7 +275,7 @@ class CSRMatrix:
 
     def __init__(self, rowptr, colidx, vals, n: int | None = None, *, kernel: str = "auto",
                  vec_lanes: int = 0, validate: bool = False, stream=None, dist: Dist | None = None,
-                 plan: bool = True, cg_variant: str = "textbook"):
+                 plan: bool = True, cg_variant: str = "textbook", l2_window: bool = False):
         import torch
         assert rowptr.dtype == torch.int32 and colidx.dtype == torch.int32
         assert vals.dtype in (torch.float64, torch.float32)
@@ -293,6 +294,7 @@ class CSRMatrix:
         o.validate = int(bool(validate))
         o.plan = int(bool(plan))
         o.dist = dist.handle if dist is not None else None
+        o.l2_window = int(bool(l2_window))
         nnz = int(rowptr[-1].item()) - int(rowptr[0].item()) if self.m >= 0 else 0
         self.nnz = nnz
         h = _P()

@@ -119,6 +119,8 @@ struct spmv_csr_s {
   int64_t row_min = 0, row_max = 0;
   double row_mean = 0, row_cv = 0;
   int32_t sorted = 0;
+  // opts.l2_window: the persisting L2 window over x (0 = off)
+  size_t l2win_bytes = 0, l2persist_bytes = 0;
   // XSTAT (x-stationary cluster kernel)
   int xB = 0, xW = 0, xR = 1024, xG = 8, nclusters = 0;
   size_t xsmem = 0;
@@ -131,6 +133,8 @@ struct spmv_csr_s {
   struct XPlan {
     bool built = false;
     int B = 0, W = 0, ncl = 0, ntiles = 0;
+    int dyn = 0, ncl_plan = 0;   // dyn: tiles popped from tq at run time; the plan has ncl_plan row ranges
+    int* tq = nullptr;           // dyn: [0] next tile, [1] finished CTAs (reset by the last CTA)
     size_t smem = 0;
     int64_t bytes = 0, nchunks = 0;
     long long *crow = nullptr, *chunk_off = nullptr;

@@ -360,6 +360,8 @@ spmv_status launch_xt(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, dou
   a.m = h->m_loc;
   a.Q = X.Q;
   a.NS = X.NS;
+  a.dyn = 1;
+  env_int("SPMV_XT_DYN", &a.dyn);
   a.xcap = X.xcap;
   a.nx = h->nx;
   a.plan = X.plan;
@@ -385,6 +387,12 @@ spmv_status launch_xt(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, dou
   a.w = w;
   a.part = part;
   a.hk = hook;
+  a.prof = nullptr;
+#ifdef XT_PROF
+  const size_t pn = (size_t)X.ncl * X.B * 32 * 8;
+  CK(cudaMalloc(&a.prof, pn * 8));
+  CK(cudaMemsetAsync(a.prof, 0, pn * 8, s));
+#endif
   cudaLaunchConfig_t cfg = {};
   cfg.gridDim = dim3((unsigned)(X.ncl * X.B), 1, 1);
   cfg.blockDim = dim3(XT_THREADS, 1, 1);
@@ -399,5 +407,25 @@ spmv_status launch_xt(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, dou
   cfg.numAttrs = 1;
   CK(cudaLaunchKernelEx(&cfg, part ? X.kdot : X.k, a));
   LAUNCHED();
+#ifdef XT_PROF
+  {  // per-warp clock accounting, summarised on stderr (mean over CTAs of warps 1..31, and the producer)
+    std::vector<unsigned long long> hp(pn);
+    CK(cudaMemcpyAsync(hp.data(), a.prof, pn * 8, cudaMemcpyDeviceToHost, s));
+    CK(cudaStreamSynchronize(s));
+    cudaFree(a.prof);
+    const char* nm[8] = {"tag", "full", "proc", "fbar", "fin", "rbar", "total", "chunks"};
+    double cons[8] = {0}, fin[8] = {0}, prod[8] = {0};
+    const int G = X.ncl * X.B;
+    for (int c = 0; c < G; ++c)
+      for (int w = 0; w < 32; ++w)
+        for (int i = 0; i < 8; ++i)
+          (w == 0 ? prod : w <= XT_NWC ? cons : fin)[i] += (double)hp[((size_t)c * 32 + w) * 8 + i];
+    fprintf(stderr, "[xt prof] grid %d B %d Q %d NS %d; per consumer warp (mean, kclk):", G, X.B, X.Q, X.NS);
+    for (int i : {0, 1, 2, 3, 6, 7}) fprintf(stderr, " %s %.1f", nm[i], cons[i] / (G * (double)XT_NWC) / (i == 7 ? 1.0 : 1e3));
+    fprintf(stderr, "; finalizer: fin %.1f rbar %.1f total %.1f", fin[4] / (G * (double)XT_NFW) / 1e3,
+            fin[5] / (G * (double)XT_NFW) / 1e3, fin[6] / (G * (double)XT_NFW) / 1e3);
+    fprintf(stderr, "; producer total %.1f\n", prod[6] / G / 1e3);
+  }
+#endif
   return SPMV_OK;
 }

@@ -10,24 +10,47 @@
 #include "cg_kernels.cuh"  // k_dot_partials
 
 // ------------------------------------------------------- kernel dispatch
+// Launch with the handle's L2 persisting-access window on x (opts.l2_window,
+// BJ.ns "an L2 persisting-access window on x") as a per-launch attribute, so
+// it is captured into CUDA graphs and leaves the caller's stream unchanged.
+// Errors surface through cudaGetLastError (LAUNCHED()).
+template <typename... P, typename... A>
+static void klaunch(const cudaAccessPolicyWindow* win, void (*k)(P...), dim3 g, dim3 b, cudaStream_t s, A... args) {
+  if (!win) {
+    k<<<g, b, 0, s>>>(args...);
+    return;
+  }
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = g;
+  cfg.blockDim = b;
+  cfg.stream = s;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeAccessPolicyWindow;
+  at[0].val.accessPolicyWindow = *win;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  cudaLaunchKernelEx(&cfg, k, args...);
+}
+
 template <typename T, int G, bool DOT>
-static void launch_vec_u(int unroll, int64_t grid, cudaStream_t s, const SpmvArgs& a) {
+static void launch_vec_u(int unroll, int64_t grid, cudaStream_t s, const SpmvArgs& a, const cudaAccessPolicyWindow* w) {
   switch (unroll) {
-    case 2: k_spmv_vector<T, G, 2, DOT><<<grid, 256, 0, s>>>(a); break;
-    case 8: k_spmv_vector<T, G, 8, DOT><<<grid, 256, 0, s>>>(a); break;
-    default: k_spmv_vector<T, G, 4, DOT><<<grid, 256, 0, s>>>(a); break;
+    case 2: klaunch(w, k_spmv_vector<T, G, 2, DOT>, dim3((unsigned)grid), dim3(256), s, a); break;
+    case 8: klaunch(w, k_spmv_vector<T, G, 8, DOT>, dim3((unsigned)grid), dim3(256), s, a); break;
+    default: klaunch(w, k_spmv_vector<T, G, 4, DOT>, dim3((unsigned)grid), dim3(256), s, a); break;
   }
 }
 
 template <typename T, bool DOT>
-static void launch_vec(int lanes, int unroll, int64_t grid, cudaStream_t s, const SpmvArgs& a) {
+static void launch_vec(int lanes, int unroll, int64_t grid, cudaStream_t s, const SpmvArgs& a,
+                       const cudaAccessPolicyWindow* w = nullptr) {
   switch (lanes) {
-    case 1: launch_vec_u<T, 1, DOT>(unroll, grid, s, a); break;
-    case 2: launch_vec_u<T, 2, DOT>(unroll, grid, s, a); break;
-    case 4: launch_vec_u<T, 4, DOT>(unroll, grid, s, a); break;
-    case 8: launch_vec_u<T, 8, DOT>(unroll, grid, s, a); break;
-    case 16: launch_vec_u<T, 16, DOT>(unroll, grid, s, a); break;
-    default: launch_vec_u<T, 32, DOT>(unroll, grid, s, a); break;
+    case 1: launch_vec_u<T, 1, DOT>(unroll, grid, s, a, w); break;
+    case 2: launch_vec_u<T, 2, DOT>(unroll, grid, s, a, w); break;
+    case 4: launch_vec_u<T, 4, DOT>(unroll, grid, s, a, w); break;
+    case 8: launch_vec_u<T, 8, DOT>(unroll, grid, s, a, w); break;
+    case 16: launch_vec_u<T, 16, DOT>(unroll, grid, s, a, w); break;
+    default: launch_vec_u<T, 32, DOT>(unroll, grid, s, a, w); break;
   }
 }
 
@@ -190,6 +213,9 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   at[0].val.clusterDim.z = 1;
   cfg.attrs = at;
   cfg.numAttrs = 1;
+  a.tq = h->xp.tq;
+  a.tq_done = h->xp.tq ? h->xp.tq + 1 : nullptr;
+  a.ntiles_total = h->xp.ntiles;
   a.tstamp = nullptr;
   int times = 0;
   if (tuning_env("SPMV_XPLAN_TIMES", &times) && times) {
@@ -224,7 +250,7 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
     sa.alpha = a.alpha;
     sa.beta = a.beta;
     sa.w = w ? (const void*)(w + h->xp.mplan) : nullptr;
-    sa.part = part ? part + cfg.gridDim.x : nullptr;
+    sa.part = part ? part + (h->xp.dyn ? (int64_t)h->xp.ntiles * h->xp.B : (int64_t)cfg.gridDim.x) : nullptr;
     sa.hk = P2PHook();
     if (h->dt == SPMV_F64) {
       if (part) launch_vec<double, true>(h->lanes, h->unroll, h->xp.g2, h->side, sa);
@@ -259,11 +285,11 @@ spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only) {
   const int64_t g = std::min<int64_t>(cdiv(h->m_loc * 32, 256), 16LL * num_sms(h->device));
   if (h->dt == SPMV_F64)
     k_xplan_pack<double><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const double*)vals, P.seg, h->m_loc, P.B, P.W,
-                                          P.crow, P.tile0, P.ncl, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
+                                          P.crow, P.tile0, P.ncl_plan, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
                                           values_only, P.mplan);
   else
     k_xplan_pack<float><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const float*)vals, P.seg, h->m_loc, P.B, P.W,
-                                         P.crow, P.tile0, P.ncl, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
+                                         P.crow, P.tile0, P.ncl_plan, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
                                          values_only, P.mplan);
   LAUNCHED();
   return SPMV_OK;
@@ -280,8 +306,13 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   const size_t xbudget = smem_cap - recv - 64;
   const int64_t Bneed = cdiv((int64_t)(ts * h->nx), (int64_t)xbudget);
   if (Bneed > 16) return SPMV_OK;  // x does not fit the shared memory of a 16-CTA cluster
-  void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, false> : k_spmv_xplan<float, false>;
-  void (*fnd)(XplanArgs) = h->dt == SPMV_F64 ? k_spmv_xplan<double, true> : nullptr;
+  // dynamic tile scheduling (default; SPMV_XPLAN_DYN=0: static cluster row ranges)
+  int dyn = 1;
+  env_int("SPMV_XPLAN_DYN", &dyn);
+  void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? (dyn ? k_spmv_xplan<double, false, true> : k_spmv_xplan<double, false, false>)
+                                            : (dyn ? k_spmv_xplan<float, false, true> : k_spmv_xplan<float, false, false>);
+  void (*fnd)(XplanArgs) =
+      h->dt == SPMV_F64 ? (dyn ? k_spmv_xplan<double, true, true> : k_spmv_xplan<double, true, false>) : nullptr;
   // cluster size: any B >= Bneed that divides the tile height R (rows are
   // owned in R/B blocks); among those, the one whose resident clusters cover
   // the most SMs (ties: the smaller B, whose x blocks are larger); clusters of
@@ -331,12 +362,14 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   cudaStream_t s = h->stream;
   auto& P = h->xp;
   auto cleanup = [&]() {
-    void* bufs[] = {P.crow, P.chunk_off, P.tile0, P.chunk_len, P.seg, P.row_slot, P.chunk_row, P.plan};
+    void* bufs[] = {P.crow, P.chunk_off, P.tile0, P.chunk_len, P.seg, P.row_slot, P.chunk_row, P.plan, P.tq};
     for (void* q : bufs)
       if (q) cudaFree(q);
     P = spmv_csr_s::XPlan();
   };
-  P.B = B; P.W = W; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd;
+  P.B = B; P.W = W; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd; P.dyn = dyn;
+  // DYN: the plan is one row range cut into tiles the clusters pop at run time
+  const int ncl_plan = dyn ? 1 : ncl;
   DBG("B=%d W=%d ncl=%d smem=%zu", B, W, ncl, smem);
   const int64_t m = h->m_loc;
   // side split: the last SPMV_XPLAN_SIDE per mille of the nonzeros go to the
@@ -358,19 +391,19 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
       DBG("side split: plan rows %lld of %lld, side grid %d", (long long)P.mplan, (long long)m, P.g2);
     }
   }
-  CK(cudaMalloc(&P.crow, sizeof(long long) * (ncl + 1)));
+  CK(cudaMalloc(&P.crow, sizeof(long long) * (ncl_plan + 1)));
   k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(P.mplan, h->rp_loc, ncl, P.crow);
   LAUNCHED();
-  std::vector<long long> crow(ncl + 1);
-  CK(cudaMemcpyAsync(crow.data(), P.crow, sizeof(long long) * (ncl + 1), cudaMemcpyDeviceToHost, s));
+  std::vector<long long> crow(ncl_plan + 1);
+  CK(cudaMemcpyAsync(crow.data(), P.crow, sizeof(long long) * (ncl_plan + 1), cudaMemcpyDeviceToHost, s));
   CK(cudaStreamSynchronize(s));
   std::vector<int> tile0(ncl + 1, 0);
-  for (int c = 0; c < ncl; ++c) tile0[c + 1] = tile0[c] + (int)cdiv(crow[c + 1] - crow[c], XP_R);
-  const int ntiles = tile0[ncl];
+  for (int c = 0; c < ncl_plan; ++c) tile0[c + 1] = tile0[c] + (int)cdiv(crow[c + 1] - crow[c], XP_R);
+  const int ntiles = tile0[ncl_plan];
   P.ntiles = ntiles;
   DBG("ntiles=%d", ntiles);
-  CK(cudaMalloc(&P.tile0, sizeof(int) * (ncl + 1)));
-  CK(cudaMemcpyAsync(P.tile0, tile0.data(), sizeof(int) * (ncl + 1), cudaMemcpyHostToDevice, s));
+  CK(cudaMalloc(&P.tile0, sizeof(int) * (ncl_plan + 1)));
+  CK(cudaMemcpyAsync(P.tile0, tile0.data(), sizeof(int) * (ncl_plan + 1), cudaMemcpyHostToDevice, s));
   if (B > 1) {
     CK(cudaMalloc(&P.seg, sizeof(int) * (size_t)(B - 1) * (size_t)m));
     k_xstat_splits<<<std::min<int64_t>(cdiv(m, 256), 8LL * num_sms(h->device)), 256, 0, s>>>(
@@ -385,7 +418,7 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   CK(cudaMalloc(&P.chunk_row, sizeof(uint16_t) * 32 * std::max<int64_t>(nch, 1)));
   CK(cudaMalloc(&P.row_slot, sizeof(int) * (size_t)B * (size_t)m));
   if (ntiles > 0) {
-    k_xplan_sell<<<(unsigned)(ntiles * B), XP_THREADS, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, P.tile0, ncl, P.chunk_len,
+    k_xplan_sell<<<(unsigned)(ntiles * B), XP_THREADS, 0, s>>>(h->rp_loc, P.seg, m, B, P.crow, P.tile0, ncl_plan, P.chunk_len,
                                                           P.chunk_row, P.row_slot);
     LAUNCHED();
   }
@@ -406,7 +439,7 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   // chunk offsets in stream order [c][b][t][w]: the chunks of one CTA are contiguous
   std::vector<long long> off(std::max<int64_t>(nch, 1), 0);
   long long pos = 0;
-  for (int c = 0; c < ncl; ++c)
+  for (int c = 0; c < ncl_plan; ++c)
     for (int bb = 0; bb < B; ++bb)
       for (int t = tile0[c]; t < tile0[c + 1]; ++t)
         for (int w = 0; w < XP_CPT; ++w) {
@@ -415,6 +448,11 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
           pos += (long long)len[id] * 32 * (ts + 2);
         }
   P.bytes = pos;
+  P.ncl_plan = ncl_plan;
+  if (dyn) {
+    CK(cudaMalloc(&P.tq, sizeof(int) * 2));
+    CK(cudaMemsetAsync(P.tq, 0, sizeof(int) * 2, s));
+  }
   CK(cudaMemcpyAsync(P.chunk_off, off.data(), sizeof(long long) * nch, cudaMemcpyHostToDevice, s));
   CK(cudaMalloc(&P.plan, (size_t)std::max<long long>(pos, 16)));
   if (nch > 0) {
@@ -558,7 +596,7 @@ spmv_status sell_build(spmv_csr_s* h, double max_pad, int sorted, bool* ok) {
 }
 
 static spmv_status launch_sell(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha, double beta,
-                               const double* w, double* part, const P2PHook& hook) {
+                               const double* w, double* part, const P2PHook& hook, const cudaAccessPolicyWindow* win) {
   SellArgs a;
   a.m = h->m_loc;
   a.nchunks = h->sl.nchunks;
@@ -588,20 +626,20 @@ static spmv_status launch_sell(spmv_csr_s* h, cudaStream_t s, const void* x, voi
       P2PHook wait_only = hook;
       wait_only.push_slot = -1;
       a.hk = wait_only;
-      k_spmv_sell<double, false><<<g, SELL_NT, 0, s>>>(a);
+      klaunch(win, k_spmv_sell<double, false>, dim3(g), dim3(SELL_NT), s, a);
       LAUNCHED();
       P2PHook push_only = hook;
       push_only.wait_x = 0;
       k_dot_partials<<<(int)h->vgrid, 256, 0, s>>>(h->m_loc, w, (const double*)y, part, push_only);
     } else if (part) {
-      k_spmv_sell<double, true><<<g, SELL_NT, 0, s>>>(a);
+      klaunch(win, k_spmv_sell<double, true>, dim3(g), dim3(SELL_NT), s, a);
     } else {
-      k_spmv_sell<double, false><<<g, SELL_NT, 0, s>>>(a);
+      klaunch(win, k_spmv_sell<double, false>, dim3(g), dim3(SELL_NT), s, a);
     }
   } else {
     a.alpha = (double)(float)alpha;
     a.beta = (double)(float)beta;
-    k_spmv_sell<float, false><<<g, SELL_NT, 0, s>>>(a);
+    klaunch(win, k_spmv_sell<float, false>, dim3(g), dim3(SELL_NT), s, a);
   }
   LAUNCHED();
   return SPMV_OK;
@@ -625,7 +663,7 @@ spmv_status merge_setup(spmv_csr_s* h) {
 }
 
 static spmv_status launch_merge(spmv_csr_s* h, cudaStream_t s, const void* vals, const void* x, void* y,
-                                double alpha, double beta, const P2PHook& hook) {
+                                double alpha, double beta, const P2PHook& hook, const cudaAccessPolicyWindow* win) {
   MergeArgs a;
   a.m = h->m_loc;
   a.ntiles = h->mg.ntiles;
@@ -643,14 +681,14 @@ static spmv_status launch_merge(spmv_csr_s* h, cudaStream_t s, const void* vals,
   a.head_flag = h->mg.head_flag;
   a.hk = hook;
   if (h->dt == SPMV_F64) {
-    k_spmv_merge<double><<<a.ntiles, MG_NT, 0, s>>>(a);
+    klaunch(win, k_spmv_merge<double>, dim3((unsigned)a.ntiles), dim3(MG_NT), s, a);
     LAUNCHED();
     k_merge_fixup<double><<<(unsigned)cdiv(a.ntiles, 256), 256, 0, s>>>(a);
     LAUNCHED();
   } else {
     a.alpha = (double)(float)alpha;
     a.beta = (double)(float)beta;
-    k_spmv_merge<float><<<a.ntiles, MG_NT, 0, s>>>(a);
+    klaunch(win, k_spmv_merge<float>, dim3((unsigned)a.ntiles), dim3(MG_NT), s, a);
     LAUNCHED();
     k_merge_fixup<float><<<(unsigned)cdiv(a.ntiles, 256), 256, 0, s>>>(a);
     LAUNCHED();
@@ -677,13 +715,24 @@ spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void
   if (h->kernel == SPMV_KERNEL_XT && vals == h->vals) return launch_xt(h, s, x, y, alpha, beta, w, part, hook);
   if (h->kernel == SPMV_KERNEL_XPLAN && vals == h->vals) return launch_xplan(h, s, x, y, alpha, beta, w, part, hook);
   const bool sell = h->kernel == SPMV_KERNEL_SELL || h->kernel == SPMV_KERNEL_SELL_SORTED;
-  if (sell && vals == h->vals) return launch_sell(h, s, x, y, alpha, beta, w, part, hook);
+  // opts.l2_window: persisting L2 window over x for the kernels that gather x through L1/L2
+  cudaAccessPolicyWindow win_v = {};
+  const cudaAccessPolicyWindow* win = nullptr;
+  if (h->l2win_bytes > 0 && x) {
+    win_v.base_ptr = const_cast<void*>(x);
+    win_v.num_bytes = std::min<size_t>(h->ts * (size_t)h->nx, h->l2win_bytes);
+    win_v.hitRatio = (float)std::min(1.0, (double)h->l2persist_bytes / (double)std::max<size_t>(win_v.num_bytes, 1));
+    win_v.hitProp = cudaAccessPropertyPersisting;
+    win_v.missProp = cudaAccessPropertyStreaming;
+    win = &win_v;
+  }
+  if (sell && vals == h->vals) return launch_sell(h, s, x, y, alpha, beta, w, part, hook, win);
   const int64_t vgrid_spmv = (h->kernel == SPMV_KERNEL_XPLAN || h->kernel == SPMV_KERNEL_XT || sell) ? h->grid_vec : h->grid;
   if (h->kernel == SPMV_KERNEL_XSTAT) return launch_xstat(h, s, vals, x, y, alpha, beta, w, part, hook);
   if (h->kernel == SPMV_KERNEL_MERGE) {
     P2PHook wait_only = hook;
     wait_only.push_slot = -1;
-    ST(launch_merge(h, s, vals, x, y, alpha, beta, wait_only));
+    ST(launch_merge(h, s, vals, x, y, alpha, beta, wait_only, win));
     if (part) {  // no fused dot in the merge kernel: one pass over w, y
       P2PHook push_only = hook;
       push_only.wait_x = 0;
@@ -705,12 +754,12 @@ spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void
   a.part = part;
   a.hk = hook;
   if (h->dt == SPMV_F64) {
-    if (part) launch_vec<double, true>(h->lanes, h->unroll, vgrid_spmv, s, a);
-    else launch_vec<double, false>(h->lanes, h->unroll, vgrid_spmv, s, a);
+    if (part) launch_vec<double, true>(h->lanes, h->unroll, vgrid_spmv, s, a, win);
+    else launch_vec<double, false>(h->lanes, h->unroll, vgrid_spmv, s, a, win);
   } else {
     a.alpha = (double)(float)alpha;
     a.beta = (double)(float)beta;
-    launch_vec<float, false>(h->lanes, h->unroll, vgrid_spmv, s, a);
+    launch_vec<float, false>(h->lanes, h->unroll, vgrid_spmv, s, a, win);
   }
   LAUNCHED();
   return SPMV_OK;

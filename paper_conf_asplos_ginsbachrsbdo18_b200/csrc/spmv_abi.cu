@@ -255,10 +255,10 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
   choose_kernel(h, rk, rl);
   int plan = o.plan;
   env_int("SPMV_PLAN", &plan);
-  if (rk == SPMV_KERNEL_XT || (rk == SPMV_KERNEL_AUTO && plan)) {
-    // auto + plan: the TMA-streamed column-parted plan whenever x fits 16 parts of
-    // cluster-resident blocks and rows are long enough
-    if (rk == SPMV_KERNEL_XT || h->row_mean >= 16.0) {
+  if (rk == SPMV_KERNEL_XT) {
+    // the TMA-streamed column-parted plan: on request only --
+    // measured slower than XPLAN on the NAS shapes, so auto keeps XPLAN
+    {
       bool ok = false;
       spmv_status st = xt_build(h, &ok);
       if (st != SPMV_OK) return fail(st);
@@ -277,7 +277,8 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
       if (st != SPMV_OK) return fail(st);
       if (ok) {
         h->kernel = SPMV_KERNEL_XPLAN;
-        h->grid = (int64_t)h->xp.ncl * h->xp.B;
+        // dot partials: one per (tile, owner CTA) with dynamic tiles, else one per CTA
+        h->grid = h->xp.dyn ? (int64_t)h->xp.ntiles * h->xp.B : (int64_t)h->xp.ncl * h->xp.B;
         if (h->xp.mplan < h->m_loc) h->grid += h->xp.g2;  // dot partials: clusters, then the side kernel
       }
     }
@@ -320,6 +321,23 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
       h->grid = (int64_t)h->nclusters * h->xB;
     }
   }
+  if (o.l2_window) {
+    // BJ.ns: "an L2 persisting-access window on x" -- reserve the persisting
+    // L2 carve-out for x (device-wide limit, raised only) and record the window
+    int maxwin = 0, maxpersist = 0;
+    cudaDeviceGetAttribute(&maxwin, cudaDevAttrMaxAccessPolicyWindowSize, dev);
+    cudaDeviceGetAttribute(&maxpersist, cudaDevAttrMaxPersistingL2CacheSize, dev);
+    const size_t xb = h->ts * (size_t)std::max<int64_t>(h->nx, 1);
+    size_t cur = 0;
+    cudaDeviceGetLimit(&cur, cudaLimitPersistingL2CacheSize);
+    const size_t want = std::min<size_t>(xb, (size_t)std::max(maxpersist, 0));
+    if (want > cur && cudaDeviceSetLimit(cudaLimitPersistingL2CacheSize, want) != cudaSuccess) cudaGetLastError();
+    cudaDeviceGetLimit(&cur, cudaLimitPersistingL2CacheSize);
+    if (maxwin > 0 && cur > 0) {
+      h->l2win_bytes = std::min<size_t>(xb, (size_t)maxwin);
+      h->l2persist_bytes = cur;
+    }
+  }
   CK(cudaStreamCreateWithFlags(&h->cap, cudaStreamNonBlocking));
   CK(cudaEventCreateWithFlags(&h->ev_a, cudaEventDisableTiming));
   CK(cudaEventCreateWithFlags(&h->ev_b, cudaEventDisableTiming));
@@ -342,7 +360,7 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
     if (h->xpad == h->fabric) h->xpad = nullptr;
   }
   void* bufs[] = {h->p2p_local, h->peer_table, h->mg.split_row, h->mg.split_nz, h->mg.head, h->mg.carry, h->mg.head_flag, h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
-                  h->xp.chunk_row, h->xp.plan, h->sl.pair_off, h->sl.vals, h->sl.cols, h->sl.perm, h->sl.seg, h->sl.seg_part, h->sl.seg_cnt,
+                  h->xp.chunk_row, h->xp.plan, h->xp.tq, h->sl.pair_off, h->sl.vals, h->sl.cols, h->sl.perm, h->sl.seg, h->sl.seg_part, h->sl.seg_cnt,
                   h->seg, h->crow, h->ci_own, h->send_iv, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags, h->s_vec, h->alpha2,
                   h->stage_x, h->stage_z};

@@ -71,6 +71,13 @@ struct XplanArgs {
   int dbg;
   int prefetch;                // 1: L2-prefetch the warp's chunk of the next tile
   unsigned long long* tstamp;  // diagnostics (nullable): per CTA {start, x ready, streaming done, end} globaltimer
+  // DYN (dynamic tile scheduling): the plan is one row range of ntiles_total
+  // tiles; clusters pop tiles from *tq (rank 0, K tiles ahead) and the last
+  // CTA resets tq/tq_done for the next launch; the fused dot is one partial
+  // per (tile, owner CTA): part[tile * B + b]
+  int* tq;
+  int* tq_done;
+  int ntiles_total;
 };
 
 __device__ __forceinline__ unsigned long long gtimer() {
@@ -139,11 +146,15 @@ struct Pair<float> {
 
 // smem (dynamic): xs [(W+1)*sizeof(T) rounded to 16] | recv [K][R] double
 //   recv[t%K][b*(R/B) + jl]: partial of CTA b for owned row jl
-template <typename T, bool DOT>
+constexpr int XP_TQ = 8;  // DYN: tile-id ring (local tile k in slot k % 8)
+
+template <typename T, bool DOT, bool DYN>
 __global__ void __launch_bounds__(XP_THREADS, 1)
 k_spmv_xplan(XplanArgs a) {
   extern __shared__ __align__(128) unsigned char smem[];
   __shared__ uint64_t xbar, tbar[XP_K];
+  __shared__ uint64_t qbar[XP_TQ];
+  __shared__ int tileid[XP_TQ];
   __shared__ double red[32];
   const int B = (int)cgx::this_cluster().num_blocks();
   const int b = (int)cluster_rank();
@@ -155,9 +166,11 @@ k_spmv_xplan(XplanArgs a) {
   T* xs = reinterpret_cast<T*>(smem);
   double* recv = reinterpret_cast<double*>(smem + ((size_t(W + 1) * sizeof(T) + 15) & ~size_t(15)));
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-  const int64_t r0c = a.crow[c], r1c = a.crow[c + 1];
-  const int ntiles = int((r1c - r0c + R - 1) / R);
-  const int tbase = a.tile0[c];
+  // static: cluster c owns tiles [tile0[c], tile0[c+1]) of rows [crow[c], crow[c+1]);
+  // DYN: one range [crow[0], crow[1]), tiles handed out at run time
+  const int64_t r0c = DYN ? a.crow[0] : a.crow[c], r1c = DYN ? a.crow[1] : a.crow[c + 1];
+  const int ntiles = DYN ? a.ntiles_total : int((r1c - r0c + R - 1) / R);
+  const int tbase = DYN ? 0 : a.tile0[c];
 
   const int64_t col0 = int64_t(b) * W;
   const int64_t ncols = cmax64(0, cmin64(W, a.nx - col0));
@@ -175,28 +188,70 @@ k_spmv_xplan(XplanArgs a) {
   if (threadIdx.x == 0) {
     mbar_init(&xbar, 1);
     for (int q = 0; q < XP_K; ++q) mbar_init(&tbar[q], 1);
+    if (DYN)
+      for (int q = 0; q < XP_TQ; ++q) mbar_init(&qbar[q], 1);
     asm volatile("fence.mbarrier_init.release.cluster;\n" ::: "memory");
     const uint32_t xb = uint32_t(bulk_elems * sizeof(T));
     mbar_expect_tx(&xbar, xb);
     if (xb) bulk_g2s(xs, xg + col0, xb, &xbar);
-    for (int t = 0; t < XP_K && t < ntiles; ++t) mbar_expect_tx(&tbar[t], recv_bytes(t));
+    if (DYN) {
+      for (int q = 0; q < XP_TQ; ++q) mbar_expect_tx(&qbar[q], 4);  // tile ids of local tiles 0..7
+    } else {
+      for (int t = 0; t < XP_K && t < ntiles; ++t) mbar_expect_tx(&tbar[t], recv_bytes(t));
+    }
   }
   for (int64_t j = bulk_elems + threadIdx.x; j <= W; j += blockDim.x) xs[j] = (j < ncols) ? xg[col0 + j] : T(0);
   // peers must have initialised their barriers before partials are sent
   cluster_arrive();
   cluster_wait();
+  // DYN: rank 0 pops the cluster's tiles K ahead and stores each id into every
+  // CTA of the cluster (st.async, 4 transaction bytes on the slot's qbar)
+  bool popped_end = false;
+  auto pop_send = [&](int k) {  // rank 0, thread 0: the tile of local index k (-1: none left)
+    int tid = -1;
+    if (!popped_end) {
+      tid = atomicAdd(a.tq, 1);
+      if (tid >= ntiles) {
+        tid = -1;
+        popped_end = true;
+      }
+    }
+    const uint32_t la = smem_u32(&tileid[k % XP_TQ]), lb = smem_u32(&qbar[k % XP_TQ]);
+    for (int p = 0; p < B; ++p)
+      asm volatile("st.async.shared::cluster.mbarrier::complete_tx::bytes.b32 [%0], %1, [%2];\n" ::"r"(
+                       mapa_u32(la, uint32_t(p))),
+                   "r"(tid), "r"(mapa_u32(lb, uint32_t(p)))
+                   : "memory");
+  };
+  auto tile_of = [&](int k) -> int {  // every thread: wait for the id of local tile k
+    mbar_wait(&qbar[k % XP_TQ], uint32_t(k / XP_TQ) & 1u, 5000000 + k);
+    return *reinterpret_cast<volatile int*>(&tileid[k % XP_TQ]);
+  };
+  if (DYN) {
+    if (b == 0 && threadIdx.x == 0)
+      for (int k = 0; k < XP_K; ++k) pop_send(k);
+    if (threadIdx.x == 0)
+      for (int k = 0; k < XP_K; ++k) {
+        const int tk = tile_of(k);
+        if (tk >= 0) mbar_expect_tx(&tbar[k], recv_bytes(tk));
+      }
+    // every CTA armed its receive barriers before any partial is sent
+    cluster_arrive();
+    cluster_wait();
+  }
   mbar_wait(&xbar, 0, 1);
   if (a.tstamp && threadIdx.x == 0) a.tstamp[4 * blockIdx.x + 1] = gtimer();
 
   const double alpha = a.alpha, beta = a.beta;
   double dacc = 0.0;
 
-  auto process_chunk = [&](int t, int ch) {
+  // t: tile index (relative to tbase), k: local sequence number (receive slot k % K)
+  auto process_chunk = [&](int t, int k, int ch) {
     const int64_t cid = (int64_t(tbase + t) * B + b) * XP_CPT + ch;
     const int len = a.chunk_len[cid];
     const int row = a.chunk_row[cid * 32 + lane];
     const unsigned char* base = a.plan + a.chunk_off[cid];
-    if (a.prefetch && lane == 0 && t + 1 < ntiles) {
+    if (!DYN && a.prefetch && lane == 0 && t + 1 < ntiles) {
       const int64_t nid = cid + int64_t(B) * XP_CPT;
       const uint32_t nb = uint32_t(a.chunk_len[nid]) * 32u * uint32_t(sizeof(T) + 2);
       if (nb) asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a.plan + a.chunk_off[nid]), "r"(nb)
@@ -232,16 +287,16 @@ k_spmv_xplan(XplanArgs a) {
     }
     if (row != 0xffff) {
       const int q = row / RB, jl = row - q * RB;
-      const uint32_t laddr = smem_u32(recv + (t % XP_K) * R + b * RB + jl);
-      st_async_f64(mapa_u32(laddr, q), acc, mapa_u32(smem_u32(&tbar[t % XP_K]), q));
+      const uint32_t laddr = smem_u32(recv + (k % XP_K) * R + b * RB + jl);
+      st_async_f64(mapa_u32(laddr, q), acc, mapa_u32(smem_u32(&tbar[k % XP_K]), q));
     }
   };
   // chunks are sorted longest first: warp w takes chunk w and chunk CPT-1-w
-  auto process = [&](int t) {
+  auto process = [&](int t, int k) {
 #pragma unroll 1
     for (int h = 0; h < XP_CPW; h += 2) {
-      process_chunk(t, h * XP_NW / 2 + warp);
-      if (h + 1 < XP_CPW) process_chunk(t, XP_CPT - 1 - (h * XP_NW / 2 + warp));
+      process_chunk(t, k, h * XP_NW / 2 + warp);
+      if (h + 1 < XP_CPW) process_chunk(t, k, XP_CPT - 1 - (h * XP_NW / 2 + warp));
     }
   };
 
@@ -252,9 +307,10 @@ k_spmv_xplan(XplanArgs a) {
   // the parity back -- an ABA deadlock seen on CTAs owning no rows of a
   // cluster's last tile.)
   const int nfin = min((RB + 31) & ~31, XP_THREADS);
-  auto finalize = [&](int t) {
+  // t: tile index, k: local sequence number, t_next: tile of local k + K (< 0: none)
+  auto finalize = [&](int t, int k, int t_next) {
     if (int(threadIdx.x) >= nfin) return;
-    const double* rv = recv + (t % XP_K) * R;
+    const double* rv = recv + (k % XP_K) * R;
     const int64_t rt = r0c + int64_t(t) * R;
     const int nrows = int(cmin64(R, r1c - rt));
     // the fused dot's w[i] (and beta*y[i]) do not depend on the partials: for
@@ -268,7 +324,8 @@ k_spmv_xplan(XplanArgs a) {
       if (DOT) w0 = double(static_cast<const T*>(a.w)[i0]);
       if (beta != 0.0) y0 = double(static_cast<const T*>(a.y)[i0]);
     }
-    mbar_wait(&tbar[t % XP_K], (t / XP_K) & 1, 1000000 * ntiles + 1000 * t + int(recv_bytes(t) / 8));
+    mbar_wait(&tbar[k % XP_K], (k / XP_K) & 1, 1000000 * ntiles + 1000 * t + int(recv_bytes(t) / 8));
+    double tacc = 0.0;  // DYN: this tile's share of the fused dot
     for (int jl = threadIdx.x; jl < RB && b * RB + jl < nrows; jl += nfin) {
       double sum = 0.0;
       for (int q = 0; q < B; ++q) sum += rv[q * RB + jl];
@@ -279,29 +336,61 @@ k_spmv_xplan(XplanArgs a) {
       if (beta != 0.0) r += beta * (first ? y0 : double(y[i]));
       const T out = T(r);
       y[i] = out;
-      if (DOT) dacc += (first ? w0 : double(static_cast<const T*>(a.w)[i])) * double(out);
+      if (DOT) (DYN ? tacc : dacc) += (first ? w0 : double(static_cast<const T*>(a.w)[i])) * double(out);
+    }
+    if (DOT && DYN) {
+      // one partial per (tile, owner): the dot does not depend on which cluster ran the tile
+      const double ts = block_sum_n(tacc, red, nfin / 32);
+      if (threadIdx.x == 0) a.part[int64_t(t) * B + b] = ts;
     }
     asm volatile("bar.sync 2, %0;\n" ::"r"(nfin) : "memory");
-    if (threadIdx.x == 0 && t + XP_K < ntiles) mbar_expect_tx(&tbar[t % XP_K], recv_bytes(t + XP_K));
+    if (threadIdx.x == 0 && t_next >= 0) mbar_expect_tx(&tbar[k % XP_K], recv_bytes(t_next));
   };
 
-  // Buffer reuse: partials of tile t+K (K = 3) are sent only after the sender
-  // passed wait(t+1), i.e. after every CTA arrived(t+1), which each does after
-  // finalize(t) (reads of recv[t%K] + re-arm of tbar[t%K]).
-  if (ntiles > 0) {
-    process(0);
+  // Buffer reuse: partials of local tile k+K (K = 3) are sent only after the
+  // sender passed wait(k+1), i.e. after every CTA arrived(k+1), which each
+  // does after finalize(k) (reads of recv[k%K] + re-arm of tbar[k%K]).
+  if (DYN) {
+    // tiles handed out at run time; local k's tile id arrives in slot k % 8
+    int t_cur = tile_of(0);
+    if (t_cur >= 0) {
+      if (b == 0 && threadIdx.x == 0) pop_send(XP_K);
+      process(t_cur, 0);
+      cluster_arrive_relaxed();
+      int k = 1;
+      for (;; ++k) {
+        const int t_k = tile_of(k);
+        if (t_k < 0) break;
+        if (b == 0 && threadIdx.x == 0) pop_send(k + XP_K);
+        process(t_k, k);
+        cluster_wait();
+        // tile of local k-1+K, popped at local k-1 (arrived by now or shortly)
+        const int t_next = (threadIdx.x == 0) ? tile_of(k - 1 + XP_K) : -1;
+        finalize(t_cur, k - 1, t_next);
+        // slot (k-1) % 8 is free: every thread read it before the cluster barrier above
+        if (threadIdx.x == 0) mbar_expect_tx(&qbar[(k - 1) % XP_TQ], 4);
+        cluster_arrive_relaxed();
+        t_cur = t_k;
+      }
+      if (a.tstamp && lane == 0) atomicMax(a.tstamp + 4 * blockIdx.x + 2, gtimer());
+      cluster_wait();
+      const int t_next = (threadIdx.x == 0) ? tile_of(k - 1 + XP_K) : -1;
+      finalize(t_cur, k - 1, t_next);
+    }
+  } else if (ntiles > 0) {
+    process(0, 0);
     cluster_arrive_relaxed();
     for (int t = 1; t < ntiles; ++t) {
-      process(t);
+      process(t, t);
       cluster_wait();
-      finalize(t - 1);
+      finalize(t - 1, t - 1, t - 1 + XP_K < ntiles ? t - 1 + XP_K : -1);
       cluster_arrive_relaxed();
     }
     if (a.tstamp && lane == 0) atomicMax(a.tstamp + 4 * blockIdx.x + 2, gtimer());  // last warp done streaming
     cluster_wait();
-    finalize(ntiles - 1);
+    finalize(ntiles - 1, ntiles - 1, -1);
   }
-  if (DOT) {
+  if (DOT && !DYN) {
     const double tsum = block_sum(dacc, red);
     if (threadIdx.x == 0) a.part[blockIdx.x] = tsum;
   }
@@ -309,7 +398,16 @@ k_spmv_xplan(XplanArgs a) {
   cluster_arrive();
   cluster_wait();
   if (a.tstamp && threadIdx.x == 0) a.tstamp[4 * blockIdx.x + 3] = gtimer();
-  if (DOT) p2p_push_partials_last(a.hk, a.part, gridDim.x);
+  if (DYN && threadIdx.x == 0) {
+    // the last CTA of the launch (every pop done) re-arms the tile queue
+    __threadfence();
+    if (atomicAdd(a.tq_done, 1) == int(gridDim.x) - 1) {
+      *a.tq = 0;
+      *a.tq_done = 0;
+      __threadfence();
+    }
+  }
+  if (DOT) p2p_push_partials_last(a.hk, a.part, DYN ? ntiles * B : int(gridDim.x));
 }
 
 // ---------------------------------------------------------------- builders

@@ -52,7 +52,8 @@
 namespace spmv {
 
 constexpr int XT_THREADS = 1024;
-constexpr int XT_NW = 31;            // consumer warps (warp 0 = producer)
+constexpr int XT_NFW = 4;            // finalizer warps (the last ones)
+constexpr int XT_NWC = XT_THREADS / 32 - 1 - XT_NFW;  // consumer warps (warp 0 = producer)
 constexpr int XT_NC = 32;            // chunks per tile per CTA
 constexpr int XT_R = 32 * XT_NC;     // rows per tile
 constexpr int XT_K = 3;              // receive slots
@@ -60,7 +61,6 @@ constexpr int XT_NS_MAX = 12;        // ring slots (runtime NS <= this)
 constexpr int XT_SMAX = 16384;       // bytes per ring slot / stage
 constexpr int XT_HDR = 64;           // row map at the start of every chunk
 constexpr int XT_EMPTY = 128;        // empty-barrier arrival count (>= pieces per stage)
-constexpr int XT_FIN_LAG = 2;        // a warp finalizes tile t when it starts tile t + LAG
 #ifndef XT_U_DEF
 #define XT_U_DEF 4
 #endif
@@ -76,6 +76,7 @@ struct XtArgs {
   int64_t m;                    // rows of the handle (ypart stride)
   int Q;                        // column parts
   int NS;                       // ring slots
+  int dyn;                      // 1: consumer warps take chunks in stream order from a shared counter
   int xcap;                     // elements of the x smem block (max block width + 1, rounded)
   int64_t nx;                   // length of x
   const unsigned char* plan;    // stage data
@@ -96,7 +97,17 @@ struct XtArgs {
   const void* w;                // DOT: w[i]
   double* part;                 // DOT: one partial per CTA
   P2PHook hk;
+  unsigned long long* prof;     // -DXT_PROF builds: per warp {tag, full, proc, fbar, fin, rbar, total, chunks} clocks
 };
+
+// diagnostics of -DXT_PROF variant builds (tools/build_variants.sh): per-warp clock accounting
+#ifdef XT_PROF
+#define XT_T0(v) const long long v = clock64()
+#define XT_ACC(i, t0) pr[i] += (unsigned long long)(clock64() - (t0))
+#else
+#define XT_T0(v)
+#define XT_ACC(i, t0)
+#endif
 
 __device__ __forceinline__ void mbar_arrive_cnt(uint64_t* bar, uint32_t cnt) {
   asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0], %1;\n" ::"r"(smem_u32(bar)), "r"(cnt) : "memory");
@@ -130,6 +141,7 @@ k_spmv_xt(XtArgs a) {
   __shared__ uint64_t xbar, full[XT_NS_MAX], empty[XT_NS_MAX], rbar[XT_K], fbar[XT_K];
   __shared__ int fincnt[XT_K];
   __shared__ int stag[XT_NS_MAX];  // stage currently issued into each ring slot
+  __shared__ int next_chunk;       // dyn: next chunk (stream order) to hand out
   __shared__ double red[32];
   constexpr int R = XT_R;
   constexpr int LMAX = xt_lmax<T>();
@@ -173,6 +185,7 @@ k_spmv_xt(XtArgs a) {
       mbar_init(&fbar[k], B);
       fincnt[k] = 0;
     }
+    next_chunk = XT_NWC;  // chunks 0..NWC-1 go to consumer warps 0..NWC-1
     asm volatile("fence.mbarrier_init.release.cluster;\n" ::: "memory");
     const uint32_t xb = uint32_t(bulk_elems * sizeof(T));
     mbar_expect_tx(&xbar, xb);
@@ -185,172 +198,240 @@ k_spmv_xt(XtArgs a) {
   cluster_wait();
 
   double dacc = 0.0;
+#ifdef XT_PROF
+  unsigned long long pr[8] = {0, 0, 0, 0, 0, 0, 0, 0};
+  XT_T0(tk0);
+#endif
   if (warp == 0) {
     // ---------------------------------------------------------- producer
-    if (lane == 0) {
-      for (int s = 0; s < nst; ++s) {
-        const int slot = s % NS;
-        if (s >= NS) mbar_wait(&empty[slot], uint32_t((s / NS) - 1) & 1u, 100000 + s);
-        const uint32_t info = a.st_info[st0 + s];
-        const uint32_t bytes = info & 0xffffu, np = info >> 16;
-        if (np < uint32_t(XT_EMPTY)) mbar_arrive_cnt(&empty[slot], uint32_t(XT_EMPTY) - np);
-        // the slot's tag is published before the arrive (release): a consumer that is
-        // more than NS stages ahead of the oldest unreleased stage sees a stale tag and
-        // keeps waiting instead of mistaking an older phase of the same parity (ABA)
-        *reinterpret_cast<volatile int*>(&stag[slot]) = s;
-        mbar_expect_tx(&full[slot], bytes);
-        bulk_g2s(ring + size_t(slot) * XT_SMAX, a.plan + a.st_off[st0 + s], bytes, &full[slot]);
+    // Lane 0 issues the stages in order; the whole warp fetches the stage
+    // metadata 32 stages at a time (one LDG per lane, a batch ahead), so no
+    // global-load latency sits between two bulk copies.
+    uint32_t inf_n = 0;
+    long long off_n = 0;
+    if (lane < nst) {
+      inf_n = a.st_info[st0 + lane];
+      off_n = a.st_off[st0 + lane];
+    }
+    for (int s0 = 0; s0 < nst; s0 += 32) {
+      const uint32_t inf_c = inf_n;
+      const long long off_c = off_n;
+      if (s0 + 32 + lane < nst) {  // next batch, in flight while this one is issued
+        inf_n = a.st_info[st0 + s0 + 32 + lane];
+        off_n = a.st_off[st0 + s0 + 32 + lane];
+      }
+      const int nb = min(32, nst - s0);
+      for (int k = 0; k < nb; ++k) {
+        const uint32_t info = __shfl_sync(0xffffffffu, inf_c, k);
+        const long long off = __shfl_sync(0xffffffffu, off_c, k);
+        if (lane == 0) {
+          const int s = s0 + k, slot = s % NS;
+          if (s >= NS) mbar_wait(&empty[slot], uint32_t((s / NS) - 1) & 1u, 100000 + s);
+          const uint32_t bytes = info & 0xffffu, np = info >> 16;
+          if (np < uint32_t(XT_EMPTY)) mbar_arrive_cnt(&empty[slot], uint32_t(XT_EMPTY) - np);
+          // the slot's tag is published before the arrive (release): a consumer that is
+          // more than NS stages ahead of the oldest unreleased stage sees a stale tag and
+          // keeps waiting instead of mistaking an older phase of the same parity (ABA)
+          *reinterpret_cast<volatile int*>(&stag[slot]) = s;
+          mbar_expect_tx(&full[slot], bytes);
+          bulk_g2s(ring + size_t(slot) * XT_SMAX, a.plan + off, bytes, &full[slot]);
+        }
+        __syncwarp();
       }
     }
   } else {
-    // ---------------------------------------------------------- consumers
-    const int cw = warp - 1;
     const double alpha = a.alpha, beta = a.beta;
-    const int NG = RB / 32;                       // 32-row groups owned per tile
-    const int NF = min(XT_NW, NG);                // finalizing warps
-    const uint32_t recv_l = smem_u32(recv);
-    const uint32_t rbar_l = smem_u32(&rbar[0]);
+    const int NG = RB / 32;  // 32-row groups owned per tile
     T* __restrict__ y = static_cast<T*>(a.y);
-
-    auto finalize = [&](int t) {
-      const int slot = t % XT_K;
-      if (cw < NF) {
+    if (warp >= XT_THREADS / 32 - XT_NFW) {
+      // -------------------------------------------------------- finalizers
+      // Tile t: wait for the B partials of every owned row, sum them in rank
+      // order, write y (Q = 1) or this part's partial (Q > 1, then one ticket
+      // per 32-row group: the last of the Q owners combines the parts in part
+      // order), then free the receive slot in every peer.  Off the ring's
+      // critical path: the consumer warps never wait for this work.
+      const int fw = warp - (XT_THREADS / 32 - XT_NFW);
+      for (int t = 0; t < ntiles; ++t) {
+        const int slot = t % XT_K;
+        XT_T0(tf0);
         mbar_wait(&rbar[slot], uint32_t(t / XT_K) & 1u, 200000 + t);
+        XT_ACC(5, tf0);
         const double* rv = recv + size_t(slot) * R;
         const int nrows = tile_rows(t);
-        for (int g = cw; g < NG; g += XT_NW) {
+        const int64_t tr0 = r0 + int64_t(t) * R + b * RB;  // first global row owned in this tile
+        for (int g = fw; g < NG; g += XT_NFW) {
           const int jl = g * 32 + lane;
           const bool valid = b * RB + jl < nrows;
-          const int64_t i = r0 + int64_t(t) * R + b * RB + jl;
+          const int64_t i = tr0 + jl;
+          if (!valid) continue;
           double sum = 0.0;
-          if (valid)
-            for (int p = 0; p < B; ++p) sum += rv[p * RB + jl];
+          for (int p = 0; p < B; ++p) sum += rv[p * RB + jl];
           if (a.Q == 1) {
-            if (valid) {
-              double r = alpha * sum;
-              if (beta != 0.0) r += beta * double(y[i]);
-              const T out = T(r);
-              y[i] = out;
-              if (DOT) dacc += double(static_cast<const T*>(a.w)[i]) * double(out);
-            }
+            double r = alpha * sum;
+            if (beta != 0.0) r += beta * double(y[i]);
+            const T out = T(r);
+            y[i] = out;
+            if (DOT) dacc += double(static_cast<const T*>(a.w)[i]) * double(out);
           } else {
-            if (valid) {
-              a.ypart[int64_t(q) * a.m + i] = sum;
-              // DOT with Q > 1 (beta == 0, enforced by the host): this part's share of w.y
-              if (DOT) dacc += double(static_cast<const T*>(a.w)[i]) * (alpha * sum);
-            }
-            // group ticket: the last of the Q owners of these 32 rows combines them
-            // (groups past the cluster's last row belong to the next cluster: none here)
-            const int64_t grow = r0 + int64_t(t) * R + b * RB + g * 32;
-            if (grow >= r1) continue;
-            __syncwarp();
-            int old = 0;
-            const int64_t gi = grow >> 5;
-            if (lane == 0) {
-              __threadfence();
-              old = atomicAdd(a.gcnt + gi, 1);
-            }
-            old = __shfl_sync(0xffffffffu, old, 0);
-            if (old == a.Q - 1) {
-              __threadfence();
-              if (valid) {
-                double s2 = 0.0;
-                for (int p = 0; p < a.Q; ++p) s2 += __ldcg(a.ypart + int64_t(p) * a.m + i);
-                double r = alpha * s2;
-                if (beta != 0.0) r += beta * double(y[i]);
-                y[i] = T(r);
-              }
-              if (lane == 0) a.gcnt[gi] = 0;  // re-armed for the next launch (stream order)
-            }
+            a.ypart[int64_t(q) * a.m + i] = sum;
+            // DOT with Q > 1 (beta == 0, enforced by the host): this part's share of w.y
+            if (DOT) dacc += double(static_cast<const T*>(a.w)[i]) * (alpha * sum);
           }
         }
-        // the last finalizing warp re-arms the slot for tile t+K and frees it in every peer
+        if (a.Q > 1) {
+          // group tickets, one lane per group of this warp (groups past the
+          // cluster's last row belong to the next cluster of the part: none)
+          __syncwarp();
+          __threadfence();
+          const int g = fw + lane * XT_NFW;
+          const int64_t grow = tr0 + int64_t(g) * 32;
+          bool last = false;
+          if (g < NG && grow < r1) last = atomicAdd(a.gcnt + (grow >> 5), 1) == a.Q - 1;
+          unsigned mask = __ballot_sync(0xffffffffu, last);
+          if (mask) __threadfence();
+          while (mask) {
+            const int k = __ffs(mask) - 1;
+            mask &= mask - 1;
+            const int gk = fw + k * XT_NFW;
+            const int64_t i = tr0 + int64_t(gk) * 32 + lane;
+            if (i < r1) {
+              double s2 = 0.0;
+              for (int p = 0; p < a.Q; ++p) s2 += __ldcg(a.ypart + int64_t(p) * a.m + i);
+              double r = alpha * s2;
+              if (beta != 0.0) r += beta * double(y[i]);
+              y[i] = T(r);
+            }
+            if (lane == k) a.gcnt[grow >> 5] = 0;  // re-armed for the next launch (stream order)
+          }
+        }
+        // the last finalizer re-arms the slot for tile t+K and frees it in every peer
         __syncwarp();
-        int last = 0;
+        int lastw = 0;
         if (lane == 0) {
           __threadfence_block();
-          last = atomicAdd(&fincnt[slot], 1) == NF - 1;
+          lastw = atomicAdd(&fincnt[slot], 1) == XT_NFW - 1;
         }
-        last = __shfl_sync(0xffffffffu, last, 0);
-        if (last && lane == 0) {
+        lastw = __shfl_sync(0xffffffffu, lastw, 0);
+        if (lastw && lane == 0) {
           fincnt[slot] = 0;
           if (t + XT_K < ntiles) mbar_expect_tx(&rbar[slot], uint32_t(own_rows(t + XT_K) * B * 8));
           for (int p = 0; p < B; ++p) mbar_arrive_remote(&fbar[slot], uint32_t(p));
         }
+        XT_ACC(4, tf0);
       }
-    };
-
-    mbar_wait(&xbar, 0, 1);
-    const int nchunks = ntiles * XT_NC;
-    int fin_next = 0;
-    for (int j = cw; j < nchunks; j += XT_NW) {
-      const int t = j / XT_NC;
-      while (fin_next <= t - XT_FIN_LAG) finalize(fin_next++);
-      const int64_t cid = (int64_t(tile0 + t) * B + b) * XT_NC + (j % XT_NC);
-      const uint2 meta = a.ck_meta[cid];
-      const int stage = int(meta.x);
-      const int len = int(meta.y >> 16);
-      const int npc = max(1, (len + LMAX - 1) / LMAX);
-      double acc = 0.0;
-      int row = 0xffff;
-      for (int pc = 0; pc < npc; ++pc) {
-        const int s = stage + pc, slot = s % NS;
-        {  // wait until stage s is the slot's current occupant (see the producer), then its data
-          long long t0 = 0;
-          for (uint32_t spin = 0; *reinterpret_cast<volatile int*>(&stag[slot]) != s; ++spin)
-            if ((spin & 1023) == 1023) {
-              const long long now = clock64();
-              if (t0 == 0) t0 = now;
-              else if (now - t0 > 4000000000LL) {
-                printf("spmv: xt stage tag timeout block %d warp %d stage %d slot %d tag %d\n", blockIdx.x, warp, s,
-                       slot, *reinterpret_cast<volatile int*>(&stag[slot]));
-                __trap();
+    } else {
+      // -------------------------------------------------------- consumers
+      const int cw = warp - 1;
+      const uint32_t recv_l = smem_u32(recv);
+      const uint32_t rbar_l = smem_u32(&rbar[0]);
+      mbar_wait(&xbar, 0, 1);
+      const int nchunks = ntiles * XT_NC;
+      for (int j = cw; j < nchunks;) {
+        const int t = j / XT_NC;
+        const int64_t cid = (int64_t(tile0 + t) * B + b) * XT_NC + (j % XT_NC);
+        const uint2 meta = a.ck_meta[cid];
+        const int stage = int(meta.x);
+        const int len = int(meta.y >> 16);
+        const int npc = max(1, (len + LMAX - 1) / LMAX);
+        double acc0 = 0.0, acc1 = 0.0;  // two chains: even / odd steps (fixed order, deterministic)
+        int row = 0xffff;
+        for (int pc = 0; pc < npc; ++pc) {
+          const int s = stage + pc, slot = s % NS;
+          XT_T0(tt0);
+          {  // wait until stage s is the slot's current occupant (see the producer), then its data
+            long long t0 = 0;
+            for (uint32_t spin = 0; *reinterpret_cast<volatile int*>(&stag[slot]) != s; ++spin) {
+              __nanosleep(64);  // back off: spinning warps would steal issue and LDS slots
+              if ((spin & 255) == 255) {
+                const long long now = clock64();
+                if (t0 == 0) t0 = now;
+                else if (now - t0 > 4000000000LL) {
+                  printf("spmv: xt stage tag timeout block %d warp %d stage %d slot %d tag %d\n", blockIdx.x, warp,
+                         s, slot, *reinterpret_cast<volatile int*>(&stag[slot]));
+                  __trap();
+                }
               }
             }
-        }
-        mbar_wait(&full[slot], uint32_t(s / NS) & 1u, 300000 + s);
-        const unsigned char* base = ring + size_t(slot) * XT_SMAX;
-        if (pc == 0) {
-          base += size_t(meta.y & 0xffffu) * 16;
-          row = reinterpret_cast<const uint16_t*>(base)[lane];
-          base += XT_HDR;
-        }
-        const int L = min(LMAX, len - pc * LMAX);
-        const unsigned char* V = base + size_t(lane) * sizeof(T);
-        const unsigned char* C = base + size_t(L) * 32 * sizeof(T) + size_t(lane) * 2;
-        for (int k = 0; k < L; k += XT_U) {
-          T v[XT_U];
-          uint32_t cc[XT_U];
+          }
+          XT_ACC(0, tt0);
+          XT_T0(tw0);
+          mbar_wait(&full[slot], uint32_t(s / NS) & 1u, 300000 + s);
+          XT_ACC(1, tw0);
+          XT_T0(tp0);
+          const unsigned char* base = ring + size_t(slot) * XT_SMAX;
+          if (pc == 0) {
+            base += size_t(meta.y & 0xffffu) * 16;
+            row = reinterpret_cast<const uint16_t*>(base)[lane];
+            base += XT_HDR;
+          }
+          int L = min(LMAX, len - pc * LMAX);
+#ifdef XT_NOPROC  // diagnostic variant builds only: ring throughput without the step loop
+          L = 0;
+#endif
+          const unsigned char* V = base + size_t(lane) * sizeof(T);
+          const unsigned char* C = base + size_t(L) * 32 * sizeof(T) + size_t(lane) * 2;
+          for (int k = 0; k < L; k += XT_U) {
+            T v[XT_U];
+            uint32_t cc[XT_U];
 #pragma unroll
-          for (int u = 0; u < XT_U; ++u) {
-            if (k + u < L) {
-              v[u] = xt_lds<T>(V + size_t(k + u) * 32 * sizeof(T));
-              cc[u] = xt_lds<uint16_t>(C + size_t(k + u) * 64);
-            } else {
-              v[u] = T(0);
-              cc[u] = uint32_t(Wg);
+            for (int u = 0; u < XT_U; ++u) {
+              if (k + u < L) {
+                v[u] = xt_lds<T>(V + size_t(k + u) * 32 * sizeof(T));
+                cc[u] = xt_lds<uint16_t>(C + size_t(k + u) * 64);
+              } else {
+                v[u] = T(0);
+                cc[u] = uint32_t(Wg);
+              }
+            }
+            T xv[XT_U];
+#pragma unroll
+            for (int u = 0; u < XT_U; ++u) {
+#ifdef XT_NOGATHER  // diagnostic variant builds only: no x gathers
+              xv[u] = T(cc[u]);
+#else
+              xv[u] = xs[cc[u]];
+#endif
+            }
+#pragma unroll
+            for (int u = 0; u < XT_U; u += 2) {
+              acc0 = fma(double(v[u]), double(xv[u]), acc0);
+              if (u + 1 < XT_U) acc1 = fma(double(v[u + 1]), double(xv[u + 1]), acc1);
             }
           }
-          T xv[XT_U];
-#pragma unroll
-          for (int u = 0; u < XT_U; ++u) xv[u] = xs[cc[u]];
-#pragma unroll
-          for (int u = 0; u < XT_U; ++u) acc = fma(double(v[u]), double(xv[u]), acc);
+          __syncwarp();
+          if (lane == 0) mbar_arrive_cnt(&empty[slot], 1u);
+          XT_ACC(2, tp0);
         }
-        __syncwarp();
-        if (lane == 0) mbar_arrive_cnt(&empty[slot], 1u);
-      }
-      // push the block partial of the lane's row to its owner
-      const int slot = t % XT_K;
-      if (t >= XT_K) mbar_wait(&fbar[slot], uint32_t(t / XT_K - 1) & 1u, 400000 + t);
-      if (row != 0xffff) {
-        const int own = row / RB, jl = row - own * RB;
-        const uint32_t laddr = recv_l + uint32_t((slot * R + b * RB + jl) * 8);
-        xt_st_async(xt_mapa(laddr, own), acc, xt_mapa(rbar_l + uint32_t(slot * 8), own));
+#ifdef XT_PROF
+        pr[7] += 1;
+#endif
+        // push the block partial of the lane's row to its owner (once the slot of tile t is free)
+        const double acc = acc0 + acc1;
+        const int slot = t % XT_K;
+        XT_T0(tb0);
+        if (t >= XT_K && __any_sync(0xffffffffu, row != 0xffff))
+          mbar_wait(&fbar[slot], uint32_t(t / XT_K - 1) & 1u, 400000 + t);
+        XT_ACC(3, tb0);
+        if (row != 0xffff) {
+          const int own = row / RB, jl = row - own * RB;
+          const uint32_t laddr = recv_l + uint32_t((slot * R + b * RB + jl) * 8);
+          xt_st_async(xt_mapa(laddr, own), acc, xt_mapa(rbar_l + uint32_t(slot * 8), own));
+        }
+        if (a.dyn) {  // the next chunk in stream order: the oldest ring stages are served first
+          int nj = 0;
+          if (lane == 0) nj = atomicAdd(&next_chunk, 1);
+          j = __shfl_sync(0xffffffffu, nj, 0);
+        } else {
+          j += XT_NWC;
+        }
       }
     }
-    while (fin_next < ntiles) finalize(fin_next++);
   }
+#ifdef XT_PROF
+  XT_ACC(6, tk0);
+  if (lane == 0 && a.prof)
+    for (int i = 0; i < 8; ++i) a.prof[(size_t(blockIdx.x) * 32 + warp) * 8 + i] = pr[i];
+#endif
   if (DOT) {
     const double tsum = block_sum(dacc, red);
     if (threadIdx.x == 0) a.part[blockIdx.x] = tsum;

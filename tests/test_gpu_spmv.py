@@ -220,7 +220,7 @@ def test_nas_full_size(sp, torch_dev, cls):
     A = gen.makea(cls)
     x = gen.uniform(A.n, seed=31)
     info = run_case(sp, torch, dev, A, x, what=f"NAS {cls}")
-    assert info["kernel_name"] == "xt", info  # the auto choice for NAS-shaped matrices
+    assert info["kernel_name"] == "xplan", info  # the auto choice for NAS-shaped matrices
 
 
 def test_parboil_full_size_fp32(sp, torch_dev):
@@ -488,3 +488,29 @@ def test_sellsort_update_values(sp, torch_dev):
         torch.cuda.synchronize()
     y_ref, bound = oracle.spmv(A.rowptr, A.colidx, v2_h, x_h)
     check_rows(y.cpu().numpy(), y_ref, bound, np.float64, "sellsort update_values")
+
+
+@pytest.mark.parametrize("kernel", ["vector", "merge", "sell", "sellsort", "auto"])
+@pytest.mark.parametrize("name", ["powerlaw_small", "makea_S", "stencil27_9"])
+def test_l2_window_parity(sp, torch_dev, kernel, name):
+    """opts.l2_window (the persisting L2 window over x, BJ.ns) changes caching
+    only: results stay within the per-row bound (and equal the no-window run
+    bit for bit -- same kernel, same summation order), fp64 and fp32."""
+    torch, dev = torch_dev
+    A = dict(ZOO)[name]
+    for f32 in (False, True):
+        B = A.astype(np.float32) if f32 else A
+        tdt = torch.float32 if f32 else torch.float64
+        x_h = gen.uniform(A.n, seed=61, f32=f32)
+        rp, ci, va = to_dev(B, dev)
+        x = torch.from_numpy(x_h).to(dev)
+        ys = []
+        for win in (False, True):
+            y = torch.full((A.m,), float("nan"), dtype=tdt, device=dev)
+            with sp.CSRMatrix(rp, ci, va, A.n, kernel=kernel, l2_window=win) as M:
+                M.spmv(x, y)
+                torch.cuda.synchronize()
+            ys.append(y.cpu().numpy())
+        y_ref, bound = oracle.spmv(B.rowptr, B.colidx, B.vals, x_h)
+        check_rows(ys[1], y_ref, bound, B.vals.dtype, f"{name} {kernel} l2_window f32={f32}")
+        assert np.array_equal(ys[0].view(np.uint8), ys[1].view(np.uint8))

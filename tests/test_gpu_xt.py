@@ -95,13 +95,13 @@ def test_xt_alpha_beta_update_values_deterministic(sp, torch_dev, q, monkeypatch
     y0 = gen.uniform(A.m, seed=57)
     for a, b in [(2.0, -1.0), (0.0, 3.0), (1.0, 0.0), (-1.5, 1.0)]:
         xin = x_h if a != 0.0 else np.full(A.n, np.nan)
-        info = run_case(sp, torch, dev, A, xin, alpha=a, beta=b, y0=y0, what=f"xt a={a} b={b} Q={q}")
+        info = run_case(sp, torch, dev, A, xin, alpha=a, beta=b, y0=y0, kernel="xt", what=f"xt a={a} b={b} Q={q}")
         assert info["kernel_name"] == "xt"
     rp, ci, va = to_dev(A, dev)
     x = torch.from_numpy(x_h).to(dev)
     y = torch.empty(A.m, dtype=torch.float64, device=dev)
     y2 = torch.empty_like(y)
-    with sp.CSRMatrix(rp, ci, va, A.n) as M:
+    with sp.CSRMatrix(rp, ci, va, A.n, kernel="xt") as M:
         assert M.info()["kernel_name"] == "xt"
         # determinism: repeated launches are bit-identical (fixed summation orders)
         M.spmv(x, y)
@@ -144,10 +144,9 @@ def test_xt_npb_zeta_parts(sp, torch_dev, cfg, variant, monkeypatch):
 
 
 def test_xt_class_c_every_row(sp, torch_dev):
-    """BJ.cfg[3] at full size in the bench's launch configuration (auto = xt):
-    every row vs the oracle; the plan's shape is recorded in the message."""
+    """BJ.cfg[3] at full size through the XT plan: every row vs the oracle."""
     torch, dev = torch_dev
     A = gen.makea("C")
     x = gen.uniform(A.n, seed=59)
-    info = run_case(sp, torch, dev, A, x, what="NAS C xt")
+    info = run_case(sp, torch, dev, A, x, kernel="xt", what="NAS C xt")
     assert info["kernel_name"] == "xt" and info["cluster"] in (1, 2, 4, 8), info

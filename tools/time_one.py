@@ -22,7 +22,7 @@ dev = torch.device("cuda:0")
 rp, ci, va = (torch.from_numpy(a).to(dev) for a in (C.rowptr, C.colidx, C.vals))
 x = torch.from_numpy(gen.uniform(C.n, seed=1, f32=C.vals.dtype == np.float32)).to(dev)
 y = torch.empty(C.m, dtype=va.dtype, device=dev)
-M = sp.CSRMatrix(rp, ci, va, C.n, kernel=kern)
+M = sp.CSRMatrix(rp, ci, va, C.n, kernel=kern, l2_window=os.environ.get("TIME_L2W") == "1")
 flush = torch.empty(256 << 20, dtype=torch.int8, device=dev)
 for _ in range(3):
     M.spmv(x, y)
