@@ -213,7 +213,8 @@ struct spmv_csr_s {
   // CG workspace (lazy)
   double *z = nullptr, *r = nullptr, *q = nullptr, *p_single = nullptr;
   double *s_vec = nullptr, *alpha2 = nullptr;  // single-reduction CG (NEXT-1): s = A p, alpha_{k-1}
-  int cg_variant = 0;                          // 0 textbook (NPB conj_grad), 1 Chronopoulos-Gear
+  int cg_variant = 0;                          // 0 textbook (NPB conj_grad), 1 Chronopoulos-Gear, 2 persistent C-G
+  unsigned int* gbar = nullptr;                // persistent CG: grid barrier counter
   double *part_pq = nullptr, *part_rr = nullptr, *part_res = nullptr, *part_xz = nullptr,
          *part_zz = nullptr, *scal = nullptr, *out2 = nullptr;
   int* flags = nullptr;
@@ -304,6 +305,10 @@ spmv_status sell_build(spmv_csr_s* h, double max_pad, int sorted, bool* ok);
 spmv_status sell_pack(spmv_csr_s* h, const void* vals, int values_only);
 spmv_status merge_setup(spmv_csr_s* h);
 spmv_status xt_build(spmv_csr_s* h, bool* ok);
+bool persist_eligible(const spmv_csr_s* h);
+spmv_status launch_cg_persist(spmv_csr_s* h, cudaStream_t s, const void* x_input, double* r, double* p, double* sv,
+                              double* w, double* z, double* part_d, double* part_g, int64_t pstride,
+                              const double* gam0, int gam0_count, int iters);
 spmv_status xt_pack(spmv_csr_s* h, const void* vals, int values_only);
 spmv_status launch_xt(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha, double beta,
                       const double* w, double* part, const P2PHook& hook);

@@ -53,7 +53,7 @@ static spmv_status cg_enqueue_init(spmv_csr_s* h, cudaStream_t s, const double* 
   double* prb = h->part_rr + 2 * std::max(std::max(h->grid, h->grid_vec), h->vgrid);
   // textbook: r = h->r, p = the SpMV input (cg_p); single-reduction: the SpMV
   // input is r (cg_p) and h->r holds p (overwritten before it is read)
-  if (h->cg_variant == 1) k_cg_init<<<vg, 256, 0, s>>>(h->m_loc, b, z, cg_p(h), h->r, prb);
+  if (h->cg_variant >= 1) k_cg_init<<<vg, 256, 0, s>>>(h->m_loc, b, z, cg_p(h), h->r, prb);
   else k_cg_init<<<vg, 256, 0, s>>>(h->m_loc, b, z, h->r, cg_p(h), prb);
   LAUNCHED();
   ST(reduce_src(h, s, SumSrc{prb, vg}, 0, &run->rr_b));
@@ -79,8 +79,18 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
     base.c = p2p_ctx(h);
     base.enabled = 1;
   }
-  if (h->cg_variant == 1) {
+  if (h->cg_variant == 2 && tol == 0.0 && iters > 0 && persist_eligible(h)) {
+    // NEXT-1: the persistent single-reduction CG -- all `iters` iterations in ONE
+    // launch (persist_kernel.cuh); the scalars of the last iteration stay in
+    // the kernel, so the run's sources are not used afterwards
+    ST(launch_cg_persist(h, s, xg, p, h->r, h->s_vec, h->q, z, h->part_pq, h->part_rr + 3 * pstride, pstride,
+                         run->rr_b.p, run->rr_b.count, iters));
+    run->it += iters;
+    return SPMV_OK;
+  }
+  if (h->cg_variant >= 1) {
     // single-reduction CG (cg_kernels.cuh k_cgcg): SpMV w = A r with w.r fused, then one update
+    // (variant 2 when the persistent kernel is not eligible: tol > 0, a non-XPLAN kernel, >1 GPU)
     double* rv = p;  // the SpMV input slice holds r
     static const int kGamSlot[3] = {2, 3, 7};
     for (int c = 0; c < iters; ++c) {
@@ -328,7 +338,8 @@ extern "C" spmv_status cg_npb_outer(spmv_csr_t h, void* x, void* z, int32_t cgit
 
 extern "C" spmv_status spmv_csr_set_cg_variant(spmv_csr_t h, int32_t variant) {
   if (!h) return arg_fail("handle is NULL");
-  if (variant != 0 && variant != 1) return arg_fail("variant must be 0 (textbook) or 1 (single reduction)");
+  if (variant < 0 || variant > 2)
+    return arg_fail("variant must be 0 (textbook), 1 (single reduction) or 2 (persistent single reduction)");
   if (h->cg_variant != variant) {
     h->cg_variant = variant;
     h->g_npb.reset();  // the captured NPB graph belongs to the other variant

@@ -134,9 +134,12 @@ __device__ __forceinline__ bool p2p_sends(const P2PCtx& c, int q, int64_t j) {
   return j >= iv.x && j < iv.y;
 }
 
-// Publish: bump the local epoch, record it for `slot`, flag every peer.
+// Publish: bump the local epoch, record it for `slot`, flag every peer.  The
+// flag stores are releases at system scope: they order every write this
+// thread made or acquired (the other CTAs' stores, through their acq_rel GPU
+// tickets) before the flag -- no separate fence; with one rank nothing is
+// stored and nothing is fenced.
 __device__ __forceinline__ void p2p_signal(const P2PCtx& c, int slot) {
-  __threadfence_system();
   const unsigned long long e = *c.epoch + 1;
   *c.epoch = e;
   c.slot_epoch[slot] = e;

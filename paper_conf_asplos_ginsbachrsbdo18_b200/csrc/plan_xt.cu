@@ -81,7 +81,7 @@ spmv_status xt_build(spmv_csr_s* h, bool* ok) {
   env_int("SPMV_XT_B", &forcedB);
   env_int("SPMV_XT_Q", &forcedQ);
   XtShape best;
-  for (int B : {2, 4, 8, 1}) {
+  for (int B : {2, 4, 8}) {  // >= 2: st.async / remote arrives need a real cluster
     if (forcedB && B != forcedB) continue;
     int nc = 0;
     ST(xt_clusters(fn, B, smem_cap, &nc));

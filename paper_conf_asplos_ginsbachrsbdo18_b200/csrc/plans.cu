@@ -8,6 +8,7 @@
 #include "abi_common.h"
 #include "analysis_kernels.cuh"
 #include "cg_kernels.cuh"  // k_dot_partials
+#include "persist_kernel.cuh"
 
 // ------------------------------------------------------- kernel dispatch
 // Launch with the handle's L2 persisting-access window on x (opts.l2_window,
@@ -176,8 +177,8 @@ spmv_status xstat_setup(spmv_csr_s* h, bool* ok) {
   return SPMV_OK;
 }
 
-static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha,
-                                double beta, const double* w, double* part, const P2PHook& hook) {
+static XplanArgs xplan_args(spmv_csr_s* h, const void* x, void* y, double alpha, double beta, const double* w,
+                            double* part, const P2PHook& hook) {
   XplanArgs a;
   a.nx = h->nx;
   a.W = h->xp.W;
@@ -201,6 +202,16 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
     a.alpha = (double)(float)alpha;
     a.beta = (double)(float)beta;
   }
+  a.tq = h->xp.tq;
+  a.tq_done = h->xp.tq ? h->xp.tq + 1 : nullptr;
+  a.ntiles_total = h->xp.ntiles;
+  a.tstamp = nullptr;
+  return a;
+}
+
+static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, void* y, double alpha,
+                                double beta, const double* w, double* part, const P2PHook& hook) {
+  XplanArgs a = xplan_args(h, x, y, alpha, beta, w, part, hook);
   cudaLaunchConfig_t cfg = {};
   cfg.gridDim = dim3((unsigned)(h->xp.ncl * h->xp.B), 1, 1);
   cfg.blockDim = dim3(XP_THREADS, 1, 1);
@@ -213,10 +224,6 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   at[0].val.clusterDim.z = 1;
   cfg.attrs = at;
   cfg.numAttrs = 1;
-  a.tq = h->xp.tq;
-  a.tq_done = h->xp.tq ? h->xp.tq + 1 : nullptr;
-  a.ntiles_total = h->xp.ntiles;
-  a.tstamp = nullptr;
   int times = 0;
   if (tuning_env("SPMV_XPLAN_TIMES", &times) && times) {
     // diagnostics: per-CTA {start, x ready, streaming done, end} (globaltimer, ns), summarised on stderr
@@ -306,8 +313,9 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   const size_t xbudget = smem_cap - recv - 64;
   const int64_t Bneed = cdiv((int64_t)(ts * h->nx), (int64_t)xbudget);
   if (Bneed > 16) return SPMV_OK;  // x does not fit the shared memory of a 16-CTA cluster
-  // dynamic tile scheduling (default; SPMV_XPLAN_DYN=0: static cluster row ranges)
-  int dyn = 1;
+  // dynamic tile scheduling (SPMV_XPLAN_DYN=1; measured slower: 85.3 vs 79.9 us on class C,
+  // 55.3 vs 45.1 us on B) -- static nnz-balanced cluster row ranges by default
+  int dyn = 0;
   env_int("SPMV_XPLAN_DYN", &dyn);
   void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? (dyn ? k_spmv_xplan<double, false, true> : k_spmv_xplan<double, false, false>)
                                             : (dyn ? k_spmv_xplan<float, false, true> : k_spmv_xplan<float, false, false>);
@@ -319,10 +327,12 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   // 16 only when nothing smaller fits.  SPMV_XPLAN_B forces a size.
   int forced = 0;
   env_int("SPMV_XPLAN_B", &forced);
-  if (forced < Bneed || forced > 16 || XP_R % std::max(forced, 1)) forced = 0;  // infeasible request: ignored
+  if (forced < Bneed || forced < 2 || forced > 16 || XP_R % std::max(forced, 1)) forced = 0;  // infeasible request: ignored
   int B = 0, W = 0, ncl = 0;
   size_t smem = 0;
-  for (int cand = (int)std::max<int64_t>(1, Bneed); cand <= 16; ++cand) {
+  // clusters of >= 2 CTAs: st.async / remote mbarrier completion need a real
+  // cluster (compute-sanitizer memcheck rejects them in a 1-CTA "cluster")
+  for (int cand = (int)std::max<int64_t>(2, Bneed); cand <= 16; ++cand) {
     if (XP_R % cand) continue;
     if (forced && cand != forced) continue;
     if (cand > 8 && B > 0) break;  // non-portable sizes only as the last resort
@@ -392,12 +402,12 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
     }
   }
   CK(cudaMalloc(&P.crow, sizeof(long long) * (ncl_plan + 1)));
-  k_partition<<<cdiv(ncl + 1, 128), 128, 0, s>>>(P.mplan, h->rp_loc, ncl, P.crow);
+  k_partition<<<cdiv(ncl_plan + 1, 128), 128, 0, s>>>(P.mplan, h->rp_loc, ncl_plan, P.crow);
   LAUNCHED();
   std::vector<long long> crow(ncl_plan + 1);
   CK(cudaMemcpyAsync(crow.data(), P.crow, sizeof(long long) * (ncl_plan + 1), cudaMemcpyDeviceToHost, s));
   CK(cudaStreamSynchronize(s));
-  std::vector<int> tile0(ncl + 1, 0);
+  std::vector<int> tile0(ncl_plan + 1, 0);
   for (int c = 0; c < ncl_plan; ++c) tile0[c + 1] = tile0[c] + (int)cdiv(crow[c + 1] - crow[c], XP_R);
   const int ntiles = tile0[ncl_plan];
   P.ntiles = ntiles;
@@ -761,6 +771,60 @@ spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void
     a.beta = (double)(float)beta;
     launch_vec<float, false>(h->lanes, h->unroll, vgrid_spmv, s, a, win);
   }
+  LAUNCHED();
+  return SPMV_OK;
+}
+
+// ------------------------------------------------------------- NEXT-1
+// Persistent single-reduction CG over the XPLAN plan (persist_kernel.cuh):
+// eligible with the static XPLAN plan whose co-resident clusters fit the grid.
+bool persist_eligible(const spmv_csr_s* h) {
+  if (h->kernel != SPMV_KERNEL_XPLAN || !h->xp.built || h->xp.dyn || h->dt != SPMV_F64) return false;
+  if (h->xp.mplan >= 0 && h->xp.mplan < h->m_loc) return false;  // side split
+  if (h->dist && !h->dist->proxy && h->dist->nranks > 1) return false;  // no cross-GPU grid barrier
+  return true;
+}
+
+spmv_status launch_cg_persist(spmv_csr_s* h, cudaStream_t s, const void* x_input, double* r, double* p, double* sv,
+                              double* w, double* z, double* part_d, double* part_g, int64_t pstride,
+                              const double* gam0, int gam0_count, int iters) {
+  static std::atomic<size_t> attr_smem{0};  // largest dynamic smem requested so far
+  if (h->xp.smem > attr_smem.load()) {
+    CK(cudaFuncSetAttribute(k_cg_persist, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)h->xp.smem));
+    attr_smem.store(h->xp.smem);
+  }
+  if (!h->gbar) CK(cudaMalloc(&h->gbar, sizeof(unsigned int)));
+  CK(cudaMemsetAsync(h->gbar, 0, sizeof(unsigned int), s));
+  PersistArgs pa;
+  pa.sp = xplan_args(h, x_input, w, 1.0, 0.0, r, part_d, P2PHook());
+  pa.n = h->m_loc;
+  pa.iters = iters;
+  pa.r = r;
+  pa.p = p;
+  pa.s = sv;
+  pa.w = w;
+  pa.z = z;
+  pa.part_d = part_d;
+  pa.part_g = part_g;
+  pa.pstride = pstride;
+  pa.gam0 = gam0;
+  pa.gam0_count = gam0_count;
+  pa.alpha2 = h->alpha2;
+  pa.flags = h->flags;
+  pa.gbar = h->gbar;
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = dim3((unsigned)(h->xp.ncl * h->xp.B), 1, 1);
+  cfg.blockDim = dim3(XP_THREADS, 1, 1);
+  cfg.dynamicSmemBytes = h->xp.smem;
+  cfg.stream = s;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeClusterDimension;
+  at[0].val.clusterDim.x = (unsigned)h->xp.B;
+  at[0].val.clusterDim.y = 1;
+  at[0].val.clusterDim.z = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = 1;
+  CK(cudaLaunchKernelEx(&cfg, k_cg_persist, pa));
   LAUNCHED();
   return SPMV_OK;
 }

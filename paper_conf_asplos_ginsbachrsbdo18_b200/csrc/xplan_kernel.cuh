@@ -14,10 +14,11 @@
 //   in shared memory; cluster c owns rows [crow[c], crow[c+1]) (nnz-balanced),
 //   cut into tiles of R = 32*NW rows; inside a tile the rows are sorted by the
 //   length of their segment in block b (SELL-C-sigma with C = 32, sigma = R)
-//   and cut into NW chunks of 32 rows.  Chunk (tile, b, w) stores len (even)
+//   and cut into NW chunks of 32 rows.  Chunk (tile, b, w) stores len
 //   steps column-major: vals as [len/2][32 lanes][2] (2 values per lane per
-//   step pair) then columns as [len/2][32][2] uint16 offsets inside the
-//   block; padding entries have value 0 and column W (x pad 0.0).
+//   step pair; an odd last step as one [32] row) then columns as
+//   [len/2][32][2] uint16 offsets inside the block (odd last step [32]);
+//   padding entries have value 0 and column W (x pad 0.0).
 //
 // Kernel (one CTA of NW warps per SM, clusters of B): per tile, warp w streams
 // chunk w with coalesced 16-B loads, 4 step pairs in flight, lane = row, so no
@@ -58,7 +59,7 @@ struct XplanArgs {
   int W;                       // column block width (pad column = W)
   const unsigned char* plan;   // chunk data
   const long long* chunk_off;  // [tile][b][chunk] byte offset of chunk data
-  const int* chunk_len;        // [tile][b][chunk] steps (even)
+  const int* chunk_len;        // [tile][b][chunk] steps (the chunk's longest segment)
   const uint16_t* chunk_row;   // [tile][b][chunk][32] tile-local row of each lane (0xffff = none)
   const long long* crow;       // [ncl+1] cluster row ranges
   const int* tile0;            // [ncl+1] first global tile of each cluster
@@ -78,6 +79,26 @@ struct XplanArgs {
   int* tq;
   int* tq_done;
   int ntiles_total;
+};
+
+// Arguments of the persistent CG kernel (persist_kernel.cuh, NEXT-1).
+struct PersistArgs {
+  XplanArgs sp;                 // the plan; sp.x = the SpMV input (r, or the padded buffer holding r)
+  int64_t n;                    // local vector length (rows)
+  int iters;
+  double* r;                    // the SpMV input slice (cg_p): r
+  double* p;                    // p
+  double* s;                    // s = A p (recurrence)
+  double* w;                    // w = A r (the SpMV output)
+  double* z;                    // solution
+  double* part_d;               // [grid] delta partials
+  double* part_g;               // [3][pstride] gamma partials (rotating)
+  int64_t pstride;
+  const double* gam0;           // k_cg_init's r.r partials
+  int gam0_count;
+  double* alpha2;               // [2] alpha of the last two iterations (for the host-side status)
+  int* flags;                   // [0] breakdown, [2] iterations done
+  unsigned int* gbar;           // grid barrier counter (zeroed before the launch)
 };
 
 __device__ __forceinline__ unsigned long long gtimer() {
@@ -143,6 +164,49 @@ struct Pair<float> {
     return {__uint_as_float(r.x), __uint_as_float(r.y)};
   }
 };
+
+// The block partial of one chunk for the calling lane: len steps in the
+// chunk's layout -- vals [len/2][32 lanes][2] then, for odd len, the last step
+// [32]; cols likewise ([len/2][32][2] u16, then [32] u16), starting at
+// base + len*32*sizeof(T).  XP_U step pairs of 16-B loads in flight per lane
+// (the tail batch predicated: masked pairs add 0 * x[W] = 0); the odd last
+// step is loaded with the first batch and added last (the chunk's step order).
+template <typename T>
+__device__ __forceinline__ double xplan_chunk_dot(const unsigned char* base, int len, int lane, const T* xs, int W) {
+  const unsigned char* V = base + size_t(lane) * 2 * sizeof(T);
+  const unsigned char* C = base + size_t(len) * 32 * sizeof(T) + size_t(lane) * 4;
+  constexpr size_t VS = 32 * 2 * sizeof(T);  // bytes per step pair (vals)
+  const int np = len >> 1;                   // step pairs
+  T vt = T(0);
+  uint32_t ct = uint32_t(W);
+  if (len & 1) {  // the odd last step, issued ahead of the pairs
+    vt = *reinterpret_cast<const T*>(base + size_t(np) * VS + size_t(lane) * sizeof(T));
+    ct = *reinterpret_cast<const uint16_t*>(base + size_t(len) * 32 * sizeof(T) + size_t(np) * 128 + size_t(lane) * 2);
+  }
+  double acc = 0.0;
+  const uint32_t padcc = uint32_t(W) | (uint32_t(W) << 16);  // both steps -> x pad 0.0
+  for (int p = 0; p < np; p += XP_U) {
+    Pair<T> v[XP_U];
+    uint32_t cc[XP_U];
+#pragma unroll
+    for (int u = 0; u < XP_U; ++u) {
+      if (p + u < np) {
+        v[u] = Pair<T>::load(V + size_t(p + u) * VS);
+        cc[u] = ldg_stream4(C + size_t(p + u) * 128);
+      } else {
+        v[u] = Pair<T>{T(0), T(0)};
+        cc[u] = padcc;
+      }
+    }
+#pragma unroll
+    for (int u = 0; u < XP_U; ++u) {
+      acc += double(v[u].a) * double(xs[cc[u] & 0xffffu]);
+      acc += double(v[u].b) * double(xs[cc[u] >> 16]);
+    }
+  }
+  if (len & 1) acc += double(vt) * double(xs[ct]);
+  return acc;
+}
 
 // smem (dynamic): xs [(W+1)*sizeof(T) rounded to 16] | recv [K][R] double
 //   recv[t%K][b*(R/B) + jl]: partial of CTA b for owned row jl
@@ -257,34 +321,7 @@ k_spmv_xplan(XplanArgs a) {
       if (nb) asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a.plan + a.chunk_off[nid]), "r"(nb)
                            : "memory");
     }
-    const unsigned char* V = base + size_t(lane) * 2 * sizeof(T);
-    const unsigned char* C = base + size_t(len) * 32 * sizeof(T) + size_t(lane) * 4;
-    constexpr size_t VS = 32 * 2 * sizeof(T);  // bytes per step pair (vals)
-    double acc = 0.0;
-    const int np = len >> 1;  // step pairs
-    const uint32_t padcc = uint32_t(W) | (uint32_t(W) << 16);  // both steps -> x pad 0.0
-    // every batch issues up to XP_U independent 16-B loads (the tail batch is
-    // predicated: masked pairs contribute 0 * x[W] = 0), so a chunk costs
-    // ceil(np / XP_U) memory round trips
-    for (int p = 0; p < np; p += XP_U) {
-      Pair<T> v[XP_U];
-      uint32_t cc[XP_U];
-#pragma unroll
-      for (int u = 0; u < XP_U; ++u) {
-        if (p + u < np) {
-          v[u] = Pair<T>::load(V + size_t(p + u) * VS);
-          cc[u] = ldg_stream4(C + size_t(p + u) * 128);
-        } else {
-          v[u] = Pair<T>{T(0), T(0)};
-          cc[u] = padcc;
-        }
-      }
-#pragma unroll
-      for (int u = 0; u < XP_U; ++u) {
-        acc += double(v[u].a) * double(xs[cc[u] & 0xffffu]);
-        acc += double(v[u].b) * double(xs[cc[u] >> 16]);
-      }
-    }
+    const double acc = xplan_chunk_dot<T>(base, len, lane, xs, W);
     if (row != 0xffff) {
       const int q = row / RB, jl = row - q * RB;
       const uint32_t laddr = smem_u32(recv + (k % XP_K) * R + b * RB + jl);
@@ -420,7 +457,7 @@ __device__ __forceinline__ void xp_seg(const int* rowptr, const int* seg, int64_
 // One CTA (XP_THREADS threads, R/XP_THREADS rows each) per (global tile, b):
 // sort the tile's rows by segment length (descending, ties by row: bitonic
 // sort of (len, row) keys), cut into CPT chunks of 32 lanes, record each
-// chunk's even step count and each row's slot (chunk = slot/32, lane = slot%32).
+// chunk's step count and each row's slot (chunk = slot/32, lane = slot%32).
 static __global__ void __launch_bounds__(XP_THREADS)
 k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_t m, int B,
              const long long* __restrict__ crow, const int* __restrict__ tile0, int ncl, int* __restrict__ chunk_len,
@@ -478,8 +515,8 @@ k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_
     const int64_t cid = (int64_t(tg) * B + b) * XP_CPT + w;
     chunk_row[cid * 32 + ln] = (Ls >= 0) ? uint16_t(row) : uint16_t(0xffff);
     if (Ls >= 0) row_slot[int64_t(b) * m + rt + row] = j;
-    // chunk length = the first (longest) lane's length, rounded up to even
-    if (ln == 0) chunk_len[cid] = (max(Ls, 0) + 1) & ~1;
+    // chunk length = the first (longest) lane's length
+    if (ln == 0) chunk_len[cid] = max(Ls, 0);  // the longest segment (odd lengths: a single last step)
   }
 }
 
@@ -510,11 +547,15 @@ k_xplan_pack(const int* __restrict__ rowptr, const int* __restrict__ colidx, con
       const int ln = slot % 32, len = chunk_len[cid];
       const int s = k - s0;  // step
       unsigned char* base = plan + chunk_off[cid];
-      T* v = reinterpret_cast<T*>(base + (size_t(s >> 1) * 32 + ln) * 2 * sizeof(T));
-      v[s & 1] = vals[k];
+      unsigned char* cbase = base + size_t(len) * 32 * sizeof(T);
+      const bool tail = (len & 1) && s == len - 1;  // odd last step: its own [32] row of vals and cols
+      T* v = tail ? reinterpret_cast<T*>(base + size_t(s >> 1) * 64 * sizeof(T) + size_t(ln) * sizeof(T))
+                  : reinterpret_cast<T*>(base + (size_t(s >> 1) * 32 + ln) * 2 * sizeof(T)) + (s & 1);
+      *v = vals[k];
       if (!values_only) {
-        uint16_t* cc = reinterpret_cast<uint16_t*>(base + size_t(len) * 32 * sizeof(T) + (size_t(s >> 1) * 32 + ln) * 4);
-        cc[s & 1] = uint16_t(col - bb * W);
+        uint16_t* cc = tail ? reinterpret_cast<uint16_t*>(cbase + size_t(s >> 1) * 128 + size_t(ln) * 2)
+                            : reinterpret_cast<uint16_t*>(cbase + (size_t(s >> 1) * 32 + ln) * 4) + (s & 1);
+        *cc = uint16_t(col - bb * W);
       }
     }
   }

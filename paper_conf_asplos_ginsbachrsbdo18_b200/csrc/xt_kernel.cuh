@@ -232,7 +232,7 @@ k_spmv_xt(XtArgs a) {
           // the slot's tag is published before the arrive (release): a consumer that is
           // more than NS stages ahead of the oldest unreleased stage sees a stale tag and
           // keeps waiting instead of mistaking an older phase of the same parity (ABA)
-          *reinterpret_cast<volatile int*>(&stag[slot]) = s;
+          atomicExch(&stag[slot], s);  // atomic: the tag is a flag read concurrently by consumers
           mbar_expect_tx(&full[slot], bytes);
           bulk_g2s(ring + size_t(slot) * XT_SMAX, a.plan + off, bytes, &full[slot]);
         }
@@ -340,14 +340,14 @@ k_spmv_xt(XtArgs a) {
           XT_T0(tt0);
           {  // wait until stage s is the slot's current occupant (see the producer), then its data
             long long t0 = 0;
-            for (uint32_t spin = 0; *reinterpret_cast<volatile int*>(&stag[slot]) != s; ++spin) {
+            for (uint32_t spin = 0; atomicOr(&stag[slot], 0) != s; ++spin) {
               __nanosleep(64);  // back off: spinning warps would steal issue and LDS slots
               if ((spin & 255) == 255) {
                 const long long now = clock64();
                 if (t0 == 0) t0 = now;
                 else if (now - t0 > 4000000000LL) {
                   printf("spmv: xt stage tag timeout block %d warp %d stage %d slot %d tag %d\n", blockIdx.x, warp,
-                         s, slot, *reinterpret_cast<volatile int*>(&stag[slot]));
+                         s, slot, atomicOr(&stag[slot], 0));
                   __trap();
                 }
               }

@@ -199,13 +199,16 @@ def test_npb_graph_vs_eager_bitexact(sp, torch_dev, monkeypatch):
     assert np.array_equal(z1, z2) and np.array_equal(r1, r2)
 
 
-@pytest.mark.parametrize("kernel", ["merge", "vector", "xstat", "xplan", "sell", "sellsort", "xt"])
-def test_npb_s_every_kernel(sp, torch_dev, kernel):
+@pytest.mark.parametrize("kernel", ["merge", "vector", "xstat", "xplan", "sell", "sellsort", "xt", "xplan_dyn"])
+def test_npb_s_every_kernel(sp, torch_dev, kernel, monkeypatch):
     """NPB class S zeta with every SpMV kernel inside CG (fused or separate dot)."""
     torch, dev = torch_dev
     na, nonzer, niter, shift = gen.NPB_CLASSES["S"]
     A = gen.makea("S")
     rp, ci, va = to_dev(A, dev)
+    if kernel == "xplan_dyn":  # XPLAN with dynamic tile scheduling (per-tile dot partials)
+        monkeypatch.setenv("SPMV_XPLAN_DYN", "1")
+        kernel = "xplan"
     with sp.CSRMatrix(rp, ci, va, A.n, kernel=kernel) as M:
         assert M.info()["kernel_name"] == kernel
         x = torch.ones(A.n, dtype=torch.float64, device=dev)

@@ -325,7 +325,8 @@ def test_xstat_alpha_beta_and_offset(sp, torch_dev):
 
 
 @pytest.mark.parametrize("cfg", [{}, {"SPMV_XPLAN_B": "2"}, {"SPMV_XPLAN_B": "4"}, {"SPMV_XPLAN_B": "8"},
-                                 {"SPMV_XPLAN_CLUSTERS": "1"}, {"SPMV_XPLAN_CLUSTERS": "3", "SPMV_XPLAN_B": "2"}])
+                                 {"SPMV_XPLAN_CLUSTERS": "1"}, {"SPMV_XPLAN_CLUSTERS": "3", "SPMV_XPLAN_B": "2"},
+                                 {"SPMV_XPLAN_DYN": "1"}, {"SPMV_XPLAN_DYN": "1", "SPMV_XPLAN_CLUSTERS": "2"}])
 @pytest.mark.parametrize("name,A", ZOO, ids=[c[0] for c in ZOO])
 def test_zoo_xplan(sp, torch_dev, name, A, cfg, monkeypatch):
     """x-stationary kernel over the column-blocked SELL-32 plan (clusters,

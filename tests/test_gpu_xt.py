@@ -40,7 +40,7 @@ def _sorted_cols(A):
 
 
 CFGS = [{}, {"SPMV_XT_B": "2", "SPMV_XT_Q": "3"}, {"SPMV_XT_B": "4", "SPMV_XT_Q": "2"},
-        {"SPMV_XT_B": "8"}, {"SPMV_XT_B": "1", "SPMV_XT_Q": "5"}, {"SPMV_XT_NS": "3", "SPMV_XT_Q": "2"},
+        {"SPMV_XT_B": "8"}, {"SPMV_XT_B": "2", "SPMV_XT_Q": "5"}, {"SPMV_XT_NS": "3", "SPMV_XT_Q": "2"},
         {"SPMV_XT_B": "2", "SPMV_XT_Q": "16"}]
 
 
