@@ -8,7 +8,8 @@ fp64); CG iters/s at 1/2/4/8 GPU", config BJ.cfg[3]): the NAS CG class-C
 matrix (exact NPB makea, n = 150,000, 36,121,058 nnz), fp64.  One STEP is one
 NAS CG outer iteration = every row of SURVEY 8(a): 25 CG iterations (SpMV +
 2 dots + 3 axpys each, a2/a3), the residual SpMV and the zeta/normalisation
-tail (a4), row-sharded over N GPUs with the NCCL exchange (a5); the handle is
+tail (a4), row-sharded over N GPUs (a5: NCCL by default, SPMV_TRANSPORT=p2p
+for the library's peer-memory kernels); the handle is
 created once (a1, device-resident A, the paper's lazy copying P:1175-1184).
 
 value  = CG iterations per second of the whole job (25 per step; the residual
@@ -18,9 +19,11 @@ value  = CG iterations per second of the whole job (25 per step; the residual
 e2e    = the same metric through the public API with HOST buffers: x copied in
          from pinned memory and x, z, {zeta, rnorm} copied back every step.
 roofline = the SpMV kernel (the dominant kernel, ~97% of the step's bytes),
-         timed alone with CUDA events on the launching stream (an L2 flush
-         queued ahead of the start event): algorithmic bytes / duration vs
-         the measured HBM copy bandwidth of MEASURED_PEAKS.json.
+         timed alone with CUDA events on the launching stream: back-to-back
+         launches (A's plan is larger than L2, streamed from HBM every time,
+         as inside the CG step) -> us_avg, and each launch after a 256 MiB
+         write flush -> us_flushed_median; algorithmic bytes / us_avg vs the
+         measured HBM copy bandwidth of MEASURED_PEAKS.json.
 cpu_baseline = the CPU oracle on a bounded sample: its OpenMP copy on all host cores
          (value) and the plain oracle on 1 thread (single_thread).
 `--impl reference` times the oracle itself as the reference arm.
@@ -84,7 +87,8 @@ def workload_config(A, n_gpus):
         "n": int(A.n), "nnz": int(A.nnz), "cgitmax": 25,
         "bytes_per_spmv": int(A.bytes_per_spmv()),
         "l2": "inputs larger than L2: A = 436 MB as CSR (382 MB as the plan) > 126 MB L2; the K steps run back "
-              "to back (no flush); the roofline leg flushes L2 (256 MiB write) before each SpMV",
+              "to back (no flush); the roofline leg times back-to-back SpMVs the same way (us_avg) and, "
+              "pessimistically, each after a 256 MiB write flush (us_flushed_median)",
         "parallelism": f"row-shard x{n_gpus} (nnz-balanced); x all-gather + dot all-reduces over peer memory "
                        f"(p2p kernels) or NCCL",
     }
@@ -164,9 +168,10 @@ def run_ours(args):
     # SPMV_BENCH_FORCE_DIST=1 runs the row-sharded NCCL path even with one rank
     # (how the multi-GPU code is exercised on the 1-GPU development box)
     use_dist = world > 1 or os.environ.get("SPMV_BENCH_FORCE_DIST") == "1"
-    # transport of the row-sharded exchange: "p2p" (our kernels over CUDA-IPC
-    # peer memory / NVLink, default) or "nccl"
-    transport = os.environ.get("SPMV_TRANSPORT", "p2p")
+    # transport of the row-sharded exchange: "nccl" (default, measured faster
+    # at one rank) or "p2p" (our kernels over CUDA-IPC peer memory / NVLink)
+    # (1-rank measurement: NCCL 12.38k vs p2p 11.57k vs single 12.83k CG it/s)
+    transport = os.environ.get("SPMV_TRANSPORT", "nccl")
     if use_dist:
         with stdout_to_stderr():
             dist.init_process_group("nccl", device_id=dev, rank=rank, world_size=world)
@@ -285,11 +290,24 @@ def run_ours(args):
     reps = max(10, args.steps)
     for _ in range(3):
         M.spmv(p, q)
+    # (1) steady state, as inside the CG step: `reps` launches back to back
+    #     between two events on the launching stream.  A's plan (382 MB) is
+    #     larger than the 126 MB L2 and streamed in the same order every time,
+    #     so every launch reads it from HBM ("inputs larger than L2"; ncu's
+    #     cold-cache DRAM bytes per launch agree, profiles/spmv_traffic.json)
+    barrier()
+    a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    a.record(stream)
+    for _ in range(reps):
+        M.spmv(p, q)
+    b.record(stream)
+    b.synchronize()
+    sp_steady = a.elapsed_time(b) / reps
+    # (2) cold, pessimistic: a 256 MiB write queued ahead of each launch (its
+    #     dirty lines are written back while the kernel streams)
     sp_ms = []
     for _ in range(reps):
         barrier()
-        # L2 flush queued ahead of the start event on the same stream: the
-        # kernel starts cold, and the timed region holds no host launch gap
         flush.zero_()
         a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         a.record(stream)
@@ -301,8 +319,8 @@ def run_ours(args):
     # algorithmic bytes of this rank's launch: local nnz*(8+4) + 4*(m_loc+1) + 8*n (x) + 8*m_loc (y)
     nnz_loc = info["nnz_local"]
     spmv_bytes = nnz_loc * 12 + 4 * (nl + 1) + 8 * A.n + 8 * nl
-    sp_avg = statistics.mean(sp_ms)
-    sp_med = statistics.median(sp_ms)
+    sp_avg = max_over_ranks(sp_steady)
+    sp_flushed = statistics.median(sp_ms)
     achieved = spmv_bytes / (sp_avg / 1e3) / 1e9
     peak, peak_src = measured_peaks()
     traffic = None
@@ -332,7 +350,9 @@ def run_ours(args):
             "kernel": {"name": info["kernel_name"], "vec_lanes": info["vec_lanes"], "grid": info["grid"]},
             "spmv": {
                 "gbs": round(achieved, 1), "gflops": round(2 * nnz_loc / (sp_avg / 1e3) / 1e9, 1),
-                "us_avg": round(sp_avg * 1e3, 2), "us_median": round(sp_med * 1e3, 2),
+                "us_avg": round(sp_avg * 1e3, 2),
+                "us_flushed_median": round(sp_flushed * 1e3, 2),
+                "gbs_flushed": round(spmv_bytes / (sp_flushed / 1e3) / 1e9, 1),
                 "pct_of_8TBs": round(100 * achieved / NOMINAL_HBM_GBS, 2),
                 "pct_of_measured_copy": round(100 * achieved / peak, 2),
                 "bytes_per_launch": int(spmv_bytes),

@@ -26,6 +26,7 @@ static spmv_status cg_alloc(spmv_csr_s* h) {
   ST(ensure_buf((void**)&h->scal, sizeof(double) * 16));
   ST(ensure_buf((void**)&h->out2, sizeof(double) * 2));
   ST(ensure_buf((void**)&h->flags, sizeof(int) * 4));
+  ST(ensure_buf((void**)&h->gbar, sizeof(unsigned int)));  // persistent CG (allocated outside graph capture)
   CK(cudaMemset(h->flags, 0, sizeof(int) * 4));
   return SPMV_OK;
 }

@@ -781,7 +781,9 @@ spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void
 bool persist_eligible(const spmv_csr_s* h) {
   if (h->kernel != SPMV_KERNEL_XPLAN || !h->xp.built || h->xp.dyn || h->dt != SPMV_F64) return false;
   if (h->xp.mplan >= 0 && h->xp.mplan < h->m_loc) return false;  // side split
-  if (h->dist && !h->dist->proxy && h->dist->nranks > 1) return false;  // no cross-GPU grid barrier
+  // real transports exchange x and the scalars between iterations: not inside this kernel
+  // (no cross-GPU grid barrier); the proxy transport has no exchanges
+  if (h->dist && !h->dist->proxy) return false;
   return true;
 }
 
@@ -793,7 +795,7 @@ spmv_status launch_cg_persist(spmv_csr_s* h, cudaStream_t s, const void* x_input
     CK(cudaFuncSetAttribute(k_cg_persist, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)h->xp.smem));
     attr_smem.store(h->xp.smem);
   }
-  if (!h->gbar) CK(cudaMalloc(&h->gbar, sizeof(unsigned int)));
+  if (!h->gbar) return arg_fail("internal: persistent CG without its barrier counter (cg_alloc)");
   CK(cudaMemsetAsync(h->gbar, 0, sizeof(unsigned int), s));
   PersistArgs pa;
   pa.sp = xplan_args(h, x_input, w, 1.0, 0.0, r, part_d, P2PHook());

@@ -53,6 +53,9 @@ constexpr int XP_K = 3;              // receive buffers
 #define XP_U_DEF 9
 #endif
 constexpr int XP_U = XP_U_DEF;       // step pairs (16-B loads) in flight per lane
+#ifndef XP_ODD
+#define XP_ODD 0  // 1: odd chunk lengths (no even-rounding padding: measured 87.0 vs 78.9 us on C); 0: even
+#endif
 
 struct XplanArgs {
   int64_t nx;                  // length of x
@@ -179,7 +182,7 @@ __device__ __forceinline__ double xplan_chunk_dot(const unsigned char* base, int
   const int np = len >> 1;                   // step pairs
   T vt = T(0);
   uint32_t ct = uint32_t(W);
-  if (len & 1) {  // the odd last step, issued ahead of the pairs
+  if (XP_ODD && (len & 1)) {  // the odd last step, issued ahead of the pairs
     vt = *reinterpret_cast<const T*>(base + size_t(np) * VS + size_t(lane) * sizeof(T));
     ct = *reinterpret_cast<const uint16_t*>(base + size_t(len) * 32 * sizeof(T) + size_t(np) * 128 + size_t(lane) * 2);
   }
@@ -204,7 +207,7 @@ __device__ __forceinline__ double xplan_chunk_dot(const unsigned char* base, int
       acc += double(v[u].b) * double(xs[cc[u] >> 16]);
     }
   }
-  if (len & 1) acc += double(vt) * double(xs[ct]);
+  if (XP_ODD && (len & 1)) acc += double(vt) * double(xs[ct]);
   return acc;
 }
 
@@ -516,7 +519,7 @@ k_xplan_sell(const int* __restrict__ rowptr, const int* __restrict__ seg, int64_
     chunk_row[cid * 32 + ln] = (Ls >= 0) ? uint16_t(row) : uint16_t(0xffff);
     if (Ls >= 0) row_slot[int64_t(b) * m + rt + row] = j;
     // chunk length = the first (longest) lane's length
-    if (ln == 0) chunk_len[cid] = max(Ls, 0);  // the longest segment (odd lengths: a single last step)
+    if (ln == 0) chunk_len[cid] = XP_ODD ? max(Ls, 0) : (max(Ls, 0) + 1) & ~1;  // the longest segment
   }
 }
 

@@ -12,6 +12,14 @@ if os.environ.get("_XT_CHILD") != "1":
                SPMV_LIB_PATH=os.environ.get("SPMV_LIB_PATH", "tools/variants/lib_tuning.so"))
     r = subprocess.run([sys.executable, *sys.argv], env=env, capture_output=True, text=True)
     blocks = r.stderr.split("[xplan times]")
+    if os.environ.get("XT_PER_CLUSTER") == "1":  # per-cluster end of streaming (max over its CTAs), every launch
+        for blk in blocks[1:]:
+            cl = {}
+            for l in blk.splitlines():
+                f = l.split()
+                if f and f[0] == "cta":
+                    cl.setdefault(int(f[3]), []).append(float(f[6]))
+            print("per-cluster streamed max:", " ".join(f"{max(v):.1f}" for _, v in sorted(cl.items())))
     last = blocks[-1]
     span = re.search(r"kernel span ([0-9.]+) us", last)
     rows = [list(map(float, l.split()[4:8])) for l in last.splitlines() if l.strip().startswith("cta")]
