@@ -135,6 +135,7 @@ struct spmv_csr_s {
     int B = 0, W = 0, ncl = 0, ntiles = 0;
     int dyn = 0, ncl_plan = 0;   // dyn: tiles popped from tq at run time; the plan has ncl_plan row ranges
     int* tq = nullptr;           // dyn: [0] next tile, [1] finished CTAs (reset by the last CTA)
+    long long* cta_range = nullptr;  // small plans: [grid][2] chunk byte range per CTA (whole-range L2 prefetch)
     size_t smem = 0;
     int64_t bytes = 0, nchunks = 0;
     long long *crow = nullptr, *chunk_off = nullptr;

@@ -116,6 +116,12 @@ k_cg_persist(PersistArgs pa) {
 
   for (int k = 0; k < pa.iters; ++k) {
     // ---------------------------------------------------------- (A) w = A r
+    if (a.cta_range && warp == 1) {  // small plan: the CTA's chunk range into L2 (see k_spmv_xplan)
+      const long long q0 = a.cta_range[2 * blockIdx.x], q1 = a.cta_range[2 * blockIdx.x + 1];
+      for (long long o = q0 + int64_t(lane) * 65536; o < q1; o += 32 * 65536)
+        asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a.plan + o), "r"(uint32_t(cmin64(65536, q1 - o)))
+                     : "memory");
+    }
     if (threadIdx.x == 0) {
       const uint32_t xb = uint32_t(bulk_elems * sizeof(T));
       mbar_expect_tx(&xbar, xb);

@@ -189,6 +189,7 @@ static XplanArgs xplan_args(spmv_csr_s* h, const void* x, void* y, double alpha,
   a.dbg = dbg() ? 1 : 0;
   a.prefetch = 0;
   tuning_env("SPMV_XPLAN_PF", &a.prefetch);
+  a.cta_range = h->xp.cta_range;  // set at build for small plans (whole-range L2 prefetch)
   a.hk = hook;
   a.crow = h->xp.crow;
   a.tile0 = h->xp.tile0;
@@ -358,7 +359,13 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
     cudaError_t e = cudaOccupancyMaxActiveClusters(&nc, fn, &cfg);
     if (e != cudaSuccess || nc < 1) { cudaGetLastError(); continue; }
     DBG("candidate B=%d W=%d clusters=%d SMs=%d", cand, Wc, nc, nc * cand);
-    if (B == 0 || nc * cand > ncl * B) { B = cand; W = Wc; ncl = nc; smem = sm; }
+    // prefer >= 2 tiles per cluster (the split tile barrier then overlaps one tile's exchange with
+    // the next tile's streaming: class B 35.6 us with B = 8 / 2.4 tiles vs 37.2 us with B = 4 /
+    // 1.1 tiles, steady state), then the most SMs
+    const bool two = h->m_loc >= 2LL * XP_R * nc, two_best = B > 0 && h->m_loc >= 2LL * XP_R * ncl;
+    if (B == 0 || (two && !two_best) || (two == two_best && nc * cand > ncl * B)) {
+      B = cand; W = Wc; ncl = nc; smem = sm;
+    }
   }
   if (B == 0) return SPMV_OK;
   CK(cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
@@ -372,7 +379,8 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   cudaStream_t s = h->stream;
   auto& P = h->xp;
   auto cleanup = [&]() {
-    void* bufs[] = {P.crow, P.chunk_off, P.tile0, P.chunk_len, P.seg, P.row_slot, P.chunk_row, P.plan, P.tq};
+    void* bufs[] = {P.crow, P.chunk_off, P.tile0, P.chunk_len, P.seg, P.row_slot, P.chunk_row, P.plan, P.tq,
+                    P.cta_range};
     for (void* q : bufs)
       if (q) cudaFree(q);
     P = spmv_csr_s::XPlan();
@@ -459,6 +467,32 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
         }
   P.bytes = pos;
   P.ncl_plan = ncl_plan;
+  // small plans: each CTA prefetches its whole contiguous chunk range into L2 at
+  // kernel start; SPMV_XPLAN_L2PF=0/1 forces it off/on
+  {
+    // plans that stay L2-resident across CG iterations (<= 96 MB of the 126 MB L2; measured on the
+    // class-C rank blocks: P = 4 (94 MB) 38.1 -> 32.2 us, P = 8 (47 MB) 24.4 -> 21.4 us per CG
+    // iteration; P = 2 (188 MB) and the whole matrix lose: the prefetch thrashes L2)
+    int pf = (!dyn && pos <= (long long)(96) << 20) ? 1 : 0;
+    env_int("SPMV_XPLAN_L2PF", &pf);
+    if (pf && !dyn) {
+      std::vector<long long> rng(2 * (size_t)ncl * B, 0);
+      for (int c = 0; c < ncl; ++c)
+        for (int bb = 0; bb < B; ++bb) {
+          long long lo = 0, hi = 0;
+          if (tile0[c + 1] > tile0[c]) {
+            const size_t first = ((size_t)tile0[c] * B + bb) * XP_CPT;
+            const size_t last = ((size_t)(tile0[c + 1] - 1) * B + bb) * XP_CPT + XP_CPT - 1;
+            lo = off[first];
+            hi = off[last] + (long long)len[last] * 32 * (ts + 2);
+          }
+          rng[2 * ((size_t)c * B + bb)] = lo;
+          rng[2 * ((size_t)c * B + bb) + 1] = hi;
+        }
+      CK(cudaMalloc(&P.cta_range, sizeof(long long) * rng.size()));
+      CK(cudaMemcpyAsync(P.cta_range, rng.data(), sizeof(long long) * rng.size(), cudaMemcpyHostToDevice, s));
+    }
+  }
   if (dyn) {
     CK(cudaMalloc(&P.tq, sizeof(int) * 2));
     CK(cudaMemsetAsync(P.tq, 0, sizeof(int) * 2, s));
@@ -790,9 +824,10 @@ bool persist_eligible(const spmv_csr_s* h) {
 spmv_status launch_cg_persist(spmv_csr_s* h, cudaStream_t s, const void* x_input, double* r, double* p, double* sv,
                               double* w, double* z, double* part_d, double* part_g, int64_t pstride,
                               const double* gam0, int gam0_count, int iters) {
+  void (*kfn)(PersistArgs) = k_cg_persist;
   static std::atomic<size_t> attr_smem{0};  // largest dynamic smem requested so far
   if (h->xp.smem > attr_smem.load()) {
-    CK(cudaFuncSetAttribute(k_cg_persist, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)h->xp.smem));
+    CK(cudaFuncSetAttribute(kfn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)h->xp.smem));
     attr_smem.store(h->xp.smem);
   }
   if (!h->gbar) return arg_fail("internal: persistent CG without its barrier counter (cg_alloc)");
@@ -826,7 +861,7 @@ spmv_status launch_cg_persist(spmv_csr_s* h, cudaStream_t s, const void* x_input
   at[0].val.clusterDim.z = 1;
   cfg.attrs = at;
   cfg.numAttrs = 1;
-  CK(cudaLaunchKernelEx(&cfg, k_cg_persist, pa));
+  CK(cudaLaunchKernelEx(&cfg, kfn, pa));
   LAUNCHED();
   return SPMV_OK;
 }

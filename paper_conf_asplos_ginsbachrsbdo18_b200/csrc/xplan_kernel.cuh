@@ -74,6 +74,8 @@ struct XplanArgs {
   P2PHook hk;                  // p2p transport: wait for x / push the dot
   int dbg;
   int prefetch;                // 1: L2-prefetch the warp's chunk of the next tile
+  const long long* cta_range;  // small plans (nullable): [grid][2] byte range of each CTA's chunks, prefetched
+                               // into L2 whole at kernel start
   unsigned long long* tstamp;  // diagnostics (nullable): per CTA {start, x ready, streaming done, end} globaltimer
   // DYN (dynamic tile scheduling): the plan is one row range of ntiles_total
   // tiles; clusters pop tiles from *tq (rank 0, K tiles ahead) and the last
@@ -246,6 +248,16 @@ k_spmv_xplan(XplanArgs a) {
   const int64_t bulk_elems = x_aligned ? ((ncols * int64_t(sizeof(T))) & ~int64_t(15)) / int64_t(sizeof(T)) : 0;
 
   if (a.tstamp && threadIdx.x == 0) a.tstamp[4 * blockIdx.x] = gtimer();
+  if (a.cta_range && warp == 1) {
+    // small plan (a few tiles per cluster, latency-bound): ask the TMA unit to
+    // stream the CTA's whole chunk range into L2 now, so the warps' dependent
+    // load batches hit L2 instead of waiting on HBM one round trip at a time
+    const long long r0 = a.cta_range[2 * blockIdx.x], r1 = a.cta_range[2 * blockIdx.x + 1];
+    for (long long o = r0 + int64_t(lane) * 65536; o < r1; o += 32 * 65536) {
+      const uint32_t nb = uint32_t(cmin64(65536, r1 - o));
+      asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a.plan + o), "r"(nb) : "memory");
+    }
+  }
   p2p_prologue_wait(a.hk);  // x slices of the peers (p2p transport)
   auto recv_bytes = [&](int t) -> uint32_t {
     const int nrows = int(cmin64(R, r1c - (r0c + int64_t(t) * R)));

@@ -21,7 +21,7 @@ __device__ __forceinline__ void wait_par(uint64_t* b, uint32_t ph) {
 
 // mode: 0 = release at once, 1 = read every byte of the chunk (LDS.64 per lane), 2 = mode 1 + 8-B gathers
 __global__ void __launch_bounds__(1024, 1) k_ring(const char* __restrict__ g, int nst, int NS, int S, int CPS,
-                                                  int mode, int dyn, unsigned long long* sink) {
+                                                  int mode, int dyn, unsigned long long* sink, int ncons) {
   extern __shared__ __align__(128) char sm[];
   __shared__ uint64_t full[16], empty[16];
   __shared__ int tag[16];
@@ -33,7 +33,7 @@ __global__ void __launch_bounds__(1024, 1) k_ring(const char* __restrict__ g, in
       asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(&empty[s])), "r"(CPS));
       tag[s] = -1;
     }
-    next = 31;
+    next = ncons;
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
   }
   __syncthreads();
@@ -54,7 +54,7 @@ __global__ void __launch_bounds__(1024, 1) k_ring(const char* __restrict__ g, in
             "l"(base + size_t(s) * S), "r"(S), "r"(smem_u32(&full[slot]))
             : "memory");
       }
-  } else {
+  } else if (warp <= ncons) {
     const int nch = nst * CPS, C = S / CPS;
     for (int c = warp - 1; c < nch;) {
       const int s = c / CPS, slot = s % NS;
@@ -74,7 +74,7 @@ __global__ void __launch_bounds__(1024, 1) k_ring(const char* __restrict__ g, in
         if (lane == 0) n = atomicAdd(&next, 1);
         c = __shfl_sync(0xffffffffu, n, 0);
       } else {
-        c += 31;
+        c += ncons;
       }
     }
   }
@@ -91,11 +91,13 @@ int main() {
   char* flush;
   cudaMalloc(&flush, 256 << 20);
   cudaFuncSetAttribute(k_ring, cudaFuncAttributeMaxDynamicSharedMemorySize, 220 * 1024);
-  struct Cfg { int grid, NS, S, CPS, mode, dyn; };
-  const Cfg cfgs[] = {{148, 7, 12288, 2, 0, 1}, {148, 7, 16384, 2, 0, 1}, {148, 4, 16384, 2, 0, 1},
-                      {148, 8, 16384, 2, 0, 1}, {148, 7, 12288, 2, 0, 0}, {148, 7, 12288, 2, 1, 1},
-                      {148, 7, 12288, 2, 2, 1}, {120, 7, 16384, 2, 0, 1}, {148, 7, 16384, 1, 0, 1},
-                      {148, 12, 8192, 1, 0, 1}, {148, 10, 12288, 3, 1, 1}};
+  struct Cfg { int grid, NS, S, CPS, mode, dyn, ncons, threads; };
+  const Cfg cfgs[] = {{148, 7, 16384, 2, 0, 1, 31, 1024}, {148, 7, 16384, 2, 0, 1, 15, 1024},
+                      {148, 7, 16384, 2, 0, 1, 7, 1024},  {148, 7, 16384, 2, 0, 1, 3, 1024},
+                      {148, 7, 16384, 2, 0, 1, 1, 1024},  {148, 7, 16384, 2, 0, 1, 3, 128},
+                      {148, 8, 16384, 1, 0, 1, 3, 128},   {148, 8, 16384, 1, 0, 1, 31, 1024},
+                      {148, 7, 16384, 2, 1, 1, 7, 1024},  {148, 7, 16384, 2, 2, 1, 7, 1024},
+                      {148, 7, 16384, 2, 2, 1, 31, 1024}};
   for (const Cfg& c : cfgs) {
     const int smem = c.NS * c.S + 32768;
     const int nst = int(gbytes / size_t(c.grid) / size_t(c.S));
@@ -106,15 +108,15 @@ int main() {
       cudaEventCreate(&a);
       cudaEventCreate(&b);
       cudaEventRecord(a);
-      k_ring<<<c.grid, 1024, smem>>>(g, nst, c.NS, c.S, c.CPS, c.mode, c.dyn, sink);
+      k_ring<<<c.grid, c.threads, smem>>>(g, nst, c.NS, c.S, c.CPS, c.mode, c.dyn, sink, c.ncons);
       cudaEventRecord(b);
       cudaEventSynchronize(b);
       float ms;
       cudaEventElapsedTime(&ms, a, b);
       best = ms < best ? ms : best;
     }
-    printf("grid %3d NS %2d S %5d CPS %d mode %d dyn %d: %7.1f GB/s  %7.1f us  %s\n", c.grid, c.NS, c.S, c.CPS,
-           c.mode, c.dyn, double(c.grid) * nst * c.S / best / 1e6, best * 1e3, cudaGetErrorString(cudaGetLastError()));
+    printf("grid %3d thr %4d consumers %2d NS %2d S %5d CPS %d mode %d dyn %d: %7.1f GB/s  %7.1f us  %s\n", c.grid,
+           c.threads, c.ncons, c.NS, c.S, c.CPS, c.mode, c.dyn, double(c.grid) * nst * c.S / best / 1e6, best * 1e3, cudaGetErrorString(cudaGetLastError()));
   }
   return 0;
 }
