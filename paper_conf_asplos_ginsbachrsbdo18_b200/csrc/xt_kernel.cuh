@@ -4,9 +4,10 @@
 // bottleneck of the NAS CG benchmark".
 //
 // Why a second x-stationary kernel (measured on this GPU, DESIGN.md 5.1/5.2):
-//   * the SpMV is HBM-bound; LDG streaming of the plan tops out at ~5.9 TB/s
-//     whatever the access pattern, TMA bulk copies of >= 16 KB with >= 64 KB
-//     in flight per SM reach 6.7-7.2 TB/s;
+//   * the SpMV is HBM-bound; LDG streaming measured ~5.9 TB/s and TMA bulk
+//     copies of >= 16 KB with >= 64 KB in flight per SM 6.7-7.2 TB/s (both
+//     re-measured in round 2 without a write flush: LDG 6.4-6.8, the XT ring
+//     alone 6.6-6.8 TB/s -- DESIGN.md 5.2b/5.2c);
 //   * random 8-B gathers of x run at ~5/clk/SM from local shared memory, ~1
 //     through L1 and ~0.35 through DSMEM, so x must sit in each CTA's own
 //     shared memory;
