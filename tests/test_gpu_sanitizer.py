@@ -4,7 +4,8 @@ racecheck and synccheck over small invocations of every kernel family
 st.async / mbarrier / cluster-barrier protocols, the TMA rings, SELL, merge,
 vector, stencil, JDS, histogram / reduction / EP, CG).  The paper's admitted
 weak spot is the soundness of sparse accesses (section 6.3); a
-report fails the test.  The logs of the round's runs are kept in
+report fails the test.  Also covered: the persistent CG kernel (grid barriers)
+and the two ranks of the p2p transport, each under its own sanitizer.  The logs of the round's runs are kept in
 profiles/r02_sanitizer_*.log."""
 import os
 import re
@@ -30,17 +31,45 @@ def _run(tool, cases, timeout=900):
     assert r.returncode == 0 and clean and "sanitize cases OK" in out, out[-4000:]
 
 
-@pytest.mark.parametrize("cases", [["xplan", "xt", "cg"], ["sell", "sellsort", "merge", "vector", "xstat"],
+@pytest.mark.parametrize("cases", [["xplan", "xt", "cg", "persist"], ["sell", "sellsort", "merge", "vector", "xstat"],
                                    ["stencil", "jds", "idioms"]])
 def test_memcheck(cases):
     _run("memcheck", cases)
 
 
-@pytest.mark.parametrize("cases", [["xplan"], ["xt"], ["stencil", "idioms"]])
+@pytest.mark.parametrize("cases", [["xplan"], ["xt"], ["persist"], ["stencil", "idioms"]])
 def test_racecheck(cases):
     _run("racecheck", cases, timeout=1500)
 
 
-@pytest.mark.parametrize("cases", [["xplan", "xt"], ["stencil", "sell", "merge", "idioms"]])
+@pytest.mark.parametrize("cases", [["xplan", "xt", "persist"], ["stencil", "sell", "merge", "idioms"]])
 def test_synccheck(cases):
     _run("synccheck", cases)
+
+
+@pytest.mark.parametrize("tool", ["memcheck", "racecheck"])
+def test_p2p_two_ranks(tool):
+    """The p2p transport's two ranks (two processes on the one GPU, CUDA IPC peer
+    stores and system-scope epoch flags), each rank a top-level process under
+    its own compute-sanitizer, so both are instrumented."""
+    import socket
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    cmd = lambda r: [SAN, "--tool", tool, "--error-exitcode", "9", "--print-limit", "20", sys.executable, CASES,  # noqa: E731
+                     "p2prank", str(r), str(port)]
+    ps = [subprocess.Popen(cmd(r), stdout=subprocess.PIPE, stderr=subprocess.STDOUT, text=True, cwd=ROOT) for r in (0, 1)]
+    outs = []
+    for p in ps:
+        try:
+            out, _ = p.communicate(timeout=900)
+        except subprocess.TimeoutExpired:
+            for q in ps:
+                q.kill()
+            raise
+        outs.append((p.returncode, out))
+    for rc, out in outs:
+        clean = re.search(r"ERROR SUMMARY: 0 errors", out) or \
+            re.search(r"RACECHECK SUMMARY: 0 hazards displayed \(0 errors, 0 warnings\)", out)
+        assert rc == 0 and clean and "sanitize cases OK" in out, out[-4000:]

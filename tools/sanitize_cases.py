@@ -65,6 +65,75 @@ def cg_case(kernel, variant, env=None):
     assert abs(float(out[0]) - zeta) <= 1e-10 * abs(zeta)
 
 
+def _p2p_worker(rank, world, port, q):
+    import torch.distributed as dist
+    try:
+        dist.init_process_group("gloo", init_method=f"tcp://127.0.0.1:{port}", rank=rank, world_size=world)
+        torch.cuda.set_device(dev)
+        d = sp.Dist(rank, world, 0, transport="p2p")
+        A = gen.makea("S")
+        t = lambda v: torch.from_numpy(np.ascontiguousarray(v)).to(dev)  # noqa: E731
+        with sp.CSRMatrix(t(A.rowptr), t(A.colidx), t(A.vals), A.n, dist=d) as M:
+            b0, b1 = M.row_range
+            x_h = gen.uniform(A.n, seed=9)
+            y = torch.empty(b1 - b0, dtype=torch.float64, device=dev)
+            M.spmv(t(x_h[b0:b1]), y)
+            torch.cuda.synchronize()
+            y_ref, bound = oracle.spmv(A.rowptr, A.colidx, A.vals, x_h)
+            assert np.all(np.abs(y.cpu().numpy() - y_ref[b0:b1]) <= 1e-12 * bound[b0:b1])
+            zeta = {}
+            for variant in ("textbook", "cgcg"):
+                M.set_cg_variant(variant)
+                xs = torch.ones(b1 - b0, dtype=torch.float64, device=dev)
+                z = torch.empty_like(xs)
+                o2 = torch.zeros(2, dtype=torch.float64, device=dev)
+                M.npb_outer(xs, z, 25, 10.0, o2)
+                torch.cuda.synchronize()
+                zeta[variant] = float(o2[0])
+            _, zr, _ = oracle.npb_outer(A.rowptr, A.colidx, A.vals, np.ones(A.n), 25, 10.0, variant=0)
+            assert abs(zeta["textbook"] - zr) <= 1e-10 * abs(zr), zeta
+        S = gen.stencil27(12)
+        with sp.CSRMatrix(t(S.rowptr), t(S.colidx), t(S.vals), S.n, dist=d) as M:
+            b0, b1 = M.row_range
+            x_h = gen.uniform(S.n, seed=10)
+            y = torch.empty(b1 - b0, dtype=torch.float64, device=dev)
+            for _ in range(2):
+                M.spmv(t(x_h[b0:b1]), y)
+            torch.cuda.synchronize()
+            y_ref, bound = oracle.spmv(S.rowptr, S.colidx, S.vals, x_h)
+            assert np.all(np.abs(y.cpu().numpy() - y_ref[b0:b1]) <= 1e-12 * bound[b0:b1])
+        dist.barrier()
+        d.close()
+        dist.destroy_process_group()
+        # under compute-sanitizer --target-processes all the tool is injected into this child too
+        q.put((rank, "ok", os.environ.get("CUDA_INJECTION64_PATH", "")))
+    except Exception as e:  # pragma: no cover
+        import traceback
+        q.put((rank, "".join(traceback.format_exception(e)), ""))
+
+
+def p2p_case():
+    """Two ranks of the p2p transport as two processes on the one GPU (CUDA IPC
+    peer stores, epoch flags, last-CTA publication), as tests/test_gpu_p2p_mp.py."""
+    import socket
+    import torch.multiprocessing as mp
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    ps = [ctx.Process(target=_p2p_worker, args=(r, 2, port, q)) for r in range(2)]
+    for p in ps:
+        p.start()
+    res = [q.get(timeout=900) for _ in ps]
+    for p in ps:
+        p.join(timeout=60)
+    for r, msg, inj in res:
+        assert msg == "ok", f"rank {r}: {msg}"
+        print(f"p2p rank {r} ok; sanitizer injection: {inj or 'none'}", flush=True)
+
+
 def stencil_case(env=None):
     env = env or {}
     os.environ.update(env)
@@ -118,12 +187,30 @@ CASES = {
     "vector": lambda: spmv_case(gen.makea("S"), "vector"),
     "xstat": lambda: spmv_case(gen.makea("S"), "xstat"),
     "cg": lambda: [cg_case("xplan", "cgcg"), cg_case("xplan", "textbook"), cg_case("sell", "cgcg")],
+    "persist": lambda: cg_case("xplan", "persist"),
+    "p2p": p2p_case,
     "stencil": lambda: [stencil_case(), stencil_case({"SPMV_STENCIL_TMA": "0"}), stencil_case({"SPMV_STENCIL_BOX": "0"})],
     "jds": jds_case,
     "idioms": idioms_case,
 }
 
+def p2p_rank_main(rank, port):
+    """One rank of the p2p case as its own top-level process, so that a
+    compute-sanitizer wrapping this command certainly instruments it:
+    tests/test_gpu_sanitizer.py starts two of these, each under the tool."""
+    import queue
+    q = queue.Queue()
+    _p2p_worker(rank, 2, port, q)
+    r, msg, _ = q.get()
+    assert msg == "ok", f"rank {r}: {msg}"
+    print(f"p2p rank {r} OK", flush=True)
+
+
 if __name__ == "__main__":
+    if sys.argv[1:2] == ["p2prank"]:
+        p2p_rank_main(int(sys.argv[2]), int(sys.argv[3]))
+        print("sanitize cases OK")
+        sys.exit(0)
     names = sys.argv[1:] or list(CASES)
     for nm in names:
         CASES[nm]()
