@@ -193,6 +193,7 @@ __device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const d
   if (!s_last) return;
   if (threadIdx.x < 32) {
     double a = 0.0;
+#pragma unroll 4
     for (int i = threadIdx.x; i < count; i += 32) a += __ldcg(part + i);  // L2: other CTAs' stores
     a = warp_sum(a);
     if (threadIdx.x == 0) {

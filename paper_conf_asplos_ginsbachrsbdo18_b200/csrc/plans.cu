@@ -276,12 +276,13 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
     CK(cudaStreamSynchronize(s));
     cudaFree(a.tstamp);
     unsigned long long t0 = ~0ull, tend = 0;
-    for (unsigned i = 0; i < cfg.gridDim.x; ++i) { t0 = std::min(t0, t[4 * i]); tend = std::max(tend, t[4 * i + 3]); }
+    for (unsigned i = 0; i < cfg.gridDim.x; ++i) { t0 = std::min(t0, t[4 * i] & ~0xffull); tend = std::max(tend, t[4 * i + 3]); }
     fprintf(stderr, "[xplan times] kernel span %.2f us; per CTA (us from first start): start/xready/streamed/end\n",
             (tend - t0) / 1e3);
     for (unsigned i = 0; i < cfg.gridDim.x; ++i)
-      fprintf(stderr, "  cta %3u cl %2u  %6.2f %6.2f %6.2f %6.2f\n", i, i / (unsigned)h->xp.B, (t[4 * i] - t0) / 1e3,
-              (t[4 * i + 1] - t0) / 1e3, (t[4 * i + 2] - t0) / 1e3, (t[4 * i + 3] - t0) / 1e3);
+      fprintf(stderr, "  cta %3u cl %2u  %6.2f %6.2f %6.2f %6.2f sm %3u\n", i, i / (unsigned)h->xp.B,
+              ((t[4 * i] & ~0xffull) - t0) / 1e3, (t[4 * i + 1] - t0) / 1e3, (t[4 * i + 2] - t0) / 1e3,
+              (t[4 * i + 3] - t0) / 1e3, unsigned(t[4 * i] & 0xff));
   }
   return SPMV_OK;
 }

@@ -247,7 +247,11 @@ k_spmv_xplan(XplanArgs a) {
   const bool x_aligned = (reinterpret_cast<uintptr_t>(xg + col0) & 15) == 0;
   const int64_t bulk_elems = x_aligned ? ((ncols * int64_t(sizeof(T))) & ~int64_t(15)) / int64_t(sizeof(T)) : 0;
 
-  if (a.tstamp && threadIdx.x == 0) a.tstamp[4 * blockIdx.x] = gtimer();
+  if (a.tstamp && threadIdx.x == 0) {
+    uint32_t smid;
+    asm volatile("mov.u32 %0, %%smid;" : "=r"(smid));
+    a.tstamp[4 * blockIdx.x] = (gtimer() & ~0xffull) | smid;  // low byte: the SM (diagnostics)
+  }
   if (a.cta_range && warp == 1) {
     // small plan (a few tiles per cluster, latency-bound): ask the TMA unit to
     // stream the CTA's whole chunk range into L2 now, so the warps' dependent

@@ -21,6 +21,9 @@ if os.environ.get("_XT_CHILD") != "1":
                     cl.setdefault(int(f[3]), []).append(float(f[6]))
             print("per-cluster streamed max:", " ".join(f"{max(v):.1f}" for _, v in sorted(cl.items())))
     last = blocks[-1]
+    if os.environ.get("XT_DUMP"):  # the last launch's per-CTA lines
+        with open(os.environ["XT_DUMP"], "a") as f:
+            f.write(last)
     span = re.search(r"kernel span ([0-9.]+) us", last)
     rows = [list(map(float, l.split()[4:8])) for l in last.splitlines() if l.strip().startswith("cta")]
     import statistics as st
@@ -47,7 +50,8 @@ nl = info["row_end"] - info["row_begin"]
 x = torch.ones(nl, dtype=torch.float64, device=dev)
 y = torch.empty(nl, dtype=torch.float64, device=dev)
 flush = torch.empty(256 << 20, dtype=torch.int8, device=dev)
-for _ in range(3):
-    flush.zero_()
+for _ in range(int(os.environ.get("XT_REPS", "3"))):
+    if os.environ.get("XT_NOFLUSH") != "1":  # XT_NOFLUSH=1: back-to-back launches (steady state)
+        flush.zero_()
     M.spmv(x, y)
 torch.cuda.synchronize()
