@@ -321,11 +321,15 @@ def run_ours(args):
                 M.spmv(p, q)
         g.replay()
         barrier()
-        a.record(stream)
-        g.replay()
-        b.record(stream)
-        b.synchronize()
-        sp_steady, us_method = a.elapsed_time(b) / reps, "CUDA-graph replay of back-to-back launches"
+        per = []
+        for _ in range(5):  # median of 5 replays of `reps` launches each
+            a.record(stream)
+            g.replay()
+            b.record(stream)
+            b.synchronize()
+            per.append(a.elapsed_time(b) / reps)
+        sp_steady = statistics.median(per)
+        us_method = f"CUDA-graph replay of {reps} back-to-back launches, median of 5 replays"
     except Exception as e:  # capture unsupported on this path: keep the eager number, say so
         log(f"[rank {rank}] roofline graph capture failed ({e}); using eager launches")
     # (2) cold, pessimistic: a 256 MiB write queued ahead of each launch (its
