@@ -148,6 +148,7 @@ struct spmv_csr_s {
     // vector kernel on the SMs the clusters leave idle
     int64_t mplan = -1;
     int g2 = 0;
+    int bankperm = 1;  // k_xplan_bankperm after every pack (SPMV_XPLAN_PERM=0: CSR order within each row)
   } xp;
   cudaStream_t side = nullptr;
   cudaEvent_t ev_fork = nullptr, ev_join = nullptr;

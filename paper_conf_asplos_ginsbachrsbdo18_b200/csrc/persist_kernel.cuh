@@ -114,8 +114,14 @@ k_cg_persist(PersistArgs pa) {
   const int64_t G = gridDim.x;
   const int64_t gstride = G * blockDim.x;
 
+  // diagnostics (tuning builds, cg_solve only): per-CTA phase stamps of iteration iters/2
+  const int tk = pa.iters / 2;
+  auto stamp = [&](int k, int i) {
+    if (a.tstamp && k == tk && threadIdx.x == 0) a.tstamp[8 * blockIdx.x + i] = gtimer();
+  };
   for (int k = 0; k < pa.iters; ++k) {
     // ---------------------------------------------------------- (A) w = A r
+    stamp(k, 0);
     if (a.cta_range && warp == 1) {  // small plan: the CTA's chunk range into L2 (see k_spmv_xplan)
       const long long q0 = a.cta_range[2 * blockIdx.x], q1 = a.cta_range[2 * blockIdx.x + 1];
       for (long long o = q0 + int64_t(lane) * 65536; o < q1; o += 32 * 65536)
@@ -130,6 +136,7 @@ k_cg_persist(PersistArgs pa) {
     for (int64_t j = bulk_elems + threadIdx.x; j <= W; j += blockDim.x) xs[j] = (j < ncols) ? xg[col0 + j] : T(0);
     __syncthreads();
     mbar_wait(&xbar, uint32_t(k) & 1u, 7000000 + k);
+    stamp(k, 1);
     double dacc = 0.0;
     const int64_t tg0 = int64_t(k) * ntiles;  // global sequence number of this iteration's tile 0
 
@@ -181,6 +188,7 @@ k_cg_persist(PersistArgs pa) {
         finalize(t - 1);
         cluster_arrive_relaxed();
       }
+      if (a.tstamp && k == tk && lane == 0) atomicMax(a.tstamp + 8 * blockIdx.x + 2, gtimer());
       cluster_wait();
       finalize(ntiles - 1);
     }
@@ -188,7 +196,9 @@ k_cg_persist(PersistArgs pa) {
       const double ts = block_sum(dacc, red);
       if (threadIdx.x == 0) pa.part_d[blockIdx.x] = ts;
     }
+    stamp(k, 3);
     grid_barrier(pa.gbar, ++gepoch);
+    stamp(k, 4);
 
     // ---------------------------------------------------------- (B) update
     {
@@ -238,7 +248,9 @@ k_cg_persist(PersistArgs pa) {
       const double ts = block_sum(gacc, red);
       if (threadIdx.x == 0) pa.part_g[((k + 1) % 3) * pa.pstride + blockIdx.x] = ts;
     }
+    stamp(k, 5);
     grid_barrier(pa.gbar, ++gepoch);
+    stamp(k, 6);
   }
   // leave together (peers may still be signalling this CTA's barriers)
   cluster_arrive();

@@ -287,10 +287,22 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   return SPMV_OK;
 }
 
-// Pack (or re-pack, values_only) the nonzeros into the plan chunks.
+// Pack (or re-pack, values_only) the nonzeros into the plan chunks, then
+// spread each step's x gathers over the shared-memory banks (k_xplan_bankperm;
+// a re-pack rewrites the columns in CSR order too, so the deterministic
+// permutation is reproduced).
 spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only) {
   cudaStream_t s = h->stream;
   auto& P = h->xp;
+  const bool perm = P.bankperm && !XP_ODD && P.nchunks > 0;
+  if (perm && values_only) {
+    // the permuted chunks hold real entries where the CSR order has pads: restore
+    // the create-time state (pads everywhere, then every entry in CSR order)
+    k_xplan_fill<<<(unsigned)std::min<int64_t>(P.nchunks, 16LL * num_sms(h->device)), 256, 0, s>>>(
+        P.plan, P.chunk_off, P.chunk_len, P.nchunks, (int)h->ts, (uint16_t)P.W);
+    LAUNCHED();
+    values_only = 0;
+  }
   const int64_t g = std::min<int64_t>(cdiv(h->m_loc * 32, 256), 16LL * num_sms(h->device));
   if (h->dt == SPMV_F64)
     k_xplan_pack<double><<<g, 256, 0, s>>>(h->rp_loc, h->ci_loc, (const double*)vals, P.seg, h->m_loc, P.B, P.W,
@@ -301,6 +313,12 @@ spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only) {
                                          P.crow, P.tile0, P.ncl_plan, P.chunk_off, P.chunk_len, P.row_slot, P.plan,
                                          values_only, P.mplan);
   LAUNCHED();
+  if (perm) {
+    const unsigned gp = (unsigned)std::min<int64_t>(cdiv(P.nchunks, 8), 64LL * num_sms(h->device));
+    if (h->dt == SPMV_F64) k_xplan_bankperm<double><<<gp, 256, 0, s>>>(P.plan, P.chunk_off, P.chunk_len, P.nchunks, P.W);
+    else k_xplan_bankperm<float><<<gp, 256, 0, s>>>(P.plan, P.chunk_off, P.chunk_len, P.nchunks, P.W);
+    LAUNCHED();
+  }
   return SPMV_OK;
 }
 
@@ -319,6 +337,9 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
   // 55.3 vs 45.1 us on B) -- static nnz-balanced cluster row ranges by default
   int dyn = 0;
   env_int("SPMV_XPLAN_DYN", &dyn);
+  // bank spreading of each chunk's steps (k_xplan_bankperm; SPMV_XPLAN_PERM=0: CSR order)
+  h->xp.bankperm = 1;
+  env_int("SPMV_XPLAN_PERM", &h->xp.bankperm);
   void (*fn)(XplanArgs) = h->dt == SPMV_F64 ? (dyn ? k_spmv_xplan<double, false, true> : k_spmv_xplan<double, false, false>)
                                             : (dyn ? k_spmv_xplan<float, false, true> : k_spmv_xplan<float, false, false>);
   void (*fnd)(XplanArgs) =
@@ -862,7 +883,32 @@ spmv_status launch_cg_persist(spmv_csr_s* h, cudaStream_t s, const void* x_input
   at[0].val.clusterDim.z = 1;
   cfg.attrs = at;
   cfg.numAttrs = 1;
+  int times = 0;
+  if (tuning_env("SPMV_PERSIST_TIMES", &times) && times) {
+    // diagnostics (cg_solve only: synchronises): per-CTA phase stamps of iteration iters/2
+    const size_t nb = sizeof(unsigned long long) * 8 * cfg.gridDim.x;
+    CK(cudaMalloc(&pa.sp.tstamp, nb));
+    CK(cudaMemsetAsync(pa.sp.tstamp, 0, nb, s));
+  }
   CK(cudaLaunchKernelEx(&cfg, kfn, pa));
   LAUNCHED();
+  if (pa.sp.tstamp) {
+    const unsigned G = cfg.gridDim.x;
+    std::vector<unsigned long long> t(8 * G);
+    CK(cudaMemcpyAsync(t.data(), pa.sp.tstamp, sizeof(unsigned long long) * t.size(), cudaMemcpyDeviceToHost, s));
+    CK(cudaStreamSynchronize(s));
+    cudaFree(pa.sp.tstamp);
+    unsigned long long t0 = ~0ull;
+    for (unsigned i = 0; i < G; ++i) t0 = std::min(t0, t[8 * i]);
+    const char* nm[7] = {"start", "xready", "streamed", "spmv_done", "bar1", "update_done", "bar2"};
+    fprintf(stderr, "[persist times] iteration %d, us from the first CTA's start: median / max over %u CTAs\n",
+            iters / 2, G);
+    for (int ph = 0; ph < 7; ++ph) {
+      std::vector<double> v(G);
+      for (unsigned i = 0; i < G; ++i) v[i] = (double)(t[8 * i + ph] - t0) / 1e3;
+      std::sort(v.begin(), v.end());
+      fprintf(stderr, "  %-12s med %7.2f  min %7.2f  max %7.2f\n", nm[ph], v[G / 2], v[0], v[G - 1]);
+    }
+  }
   return SPMV_OK;
 }

@@ -580,6 +580,75 @@ k_xplan_pack(const int* __restrict__ rowptr, const int* __restrict__ colidx, con
   }
 }
 
+// Bank spreading (create time, after k_xplan_pack): inside each lane (row) of
+// a chunk, the order of the row's nonzeros over the chunk's steps is free --
+// the SPMV idiom's DotProductLoop is a sum (Fig. 12), and the
+// per-row tolerance of BJ.ns bounds any summation order.  The kernel reorders
+// them so that the x gathers of one step (xs[col] in shared memory, 8-B words
+// for fp64 = bank pair col % 16 per half-warp, 4-B words for fp32 = bank
+// col % 32 per warp) hit distinct banks: greedy, step by step, each lane in
+// turn takes its first remaining nonzero whose bank is still free in this
+// step (else the least-loaded one).  Pads (column W, value 0) share one word.
+// One warp per chunk; deterministic (depends only on the columns and their
+// CSR order), so a values-only re-pack followed by this pass reproduces it.
+template <typename T>
+__global__ void __launch_bounds__(256)
+k_xplan_bankperm(unsigned char* __restrict__ plan, const long long* __restrict__ chunk_off,
+                 const int* __restrict__ chunk_len, int64_t nchunks, int W) {
+  constexpr int NG = sizeof(T) == 8 ? 16 : 32;  // conflict-free slots per lane group
+  constexpr int GL = NG;                        // lanes per group (half-warp for fp64)
+  __shared__ int cnt[8][32];
+  __shared__ int padf[8][2];
+  const int wib = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int grp = lane / GL, gl = lane % GL;
+  for (int64_t c = int64_t(blockIdx.x) * 8 + wib; c < nchunks; c += int64_t(gridDim.x) * 8) {
+    const int len = chunk_len[c];
+    if (len < 2) continue;
+    unsigned char* base = plan + chunk_off[c];
+    T* V = reinterpret_cast<T*>(base);
+    uint16_t* C = reinterpret_cast<uint16_t*>(base + size_t(len) * 32 * sizeof(T));
+    auto at = [&](int st) { return (size_t(st >> 1) * 32 + lane) * 2 + (st & 1); };
+    for (int st = 0; st < len - 1; ++st) {
+      cnt[wib][lane] = 0;
+      if (lane < 2) padf[wib][lane] = 0;
+      __syncwarp();
+      for (int i = 0; i < GL; ++i) {
+        if (gl == i) {
+          int best = st, bestc = 1 << 30;
+          for (int e = st; e < len; ++e) {
+            const int col = C[at(e)];
+            const int cost = (col == W && padf[wib][grp]) ? 0 : cnt[wib][grp * NG + col % NG];
+            if (cost < bestc) {
+              bestc = cost;
+              best = e;
+              if (cost == 0) break;
+            }
+          }
+          if (best != st) {
+            const size_t i0 = at(st), i1 = at(best);
+            const T tv = V[i0];
+            V[i0] = V[i1];
+            V[i1] = tv;
+            const uint16_t tc = C[i0];
+            C[i0] = C[i1];
+            C[i1] = tc;
+          }
+          const int col = C[at(st)];
+          if (col == W) {
+            if (!padf[wib][grp]) {
+              padf[wib][grp] = 1;
+              cnt[wib][grp * NG + col % NG] += 1;
+            }
+          } else {
+            cnt[wib][grp * NG + col % NG] += 1;
+          }
+        }
+        __syncwarp();
+      }
+    }
+  }
+}
+
 // Padding: value regions 0, column regions the pad column W (x pad 0.0).
 // Chunk c of the plan spans [chunk_off[c], chunk_off[c] + len*32*(ts+2)).
 static __global__ void k_xplan_fill(unsigned char* __restrict__ plan, const long long* __restrict__ chunk_off,

@@ -1,0 +1,68 @@
+"""Out-of-range accesses without compute-sanitizer (closed on this pool, see
+test_gpu_sanitizer.py): every operand of spmv_csr is a view into a larger
+device buffer whose guard regions on both sides hold NaN (inputs) or a
+sentinel bit pattern (the output).  A kernel that reads x, vals or y outside
+its extent turns a row into NaN; one that writes y outside [0, m) changes a
+guard word.  Run over every kernel family on the ragged / skewed shapes of
+the adversarial zoo, compared row by row with the oracle (the
+Fig. 4 loop, and P:878-888, section 6.3: soundness of sparse accesses)."""
+import numpy as np
+import pytest
+
+import gen
+import oracle
+from gpu_util import check_rows
+
+pytestmark = pytest.mark.gpu
+
+G = 4099  # guard elements on each side (odd: shifts the views off 16-B alignment too)
+SENT = -1.2345678e300
+
+
+def _guarded(torch, dev, h, fill):
+    buf = torch.full((h.size + 2 * G,), fill, dtype=torch.from_numpy(h[:0]).dtype, device=dev)
+    buf[G:G + h.size] = torch.from_numpy(np.ascontiguousarray(h)).to(dev)
+    return buf, buf[G:G + h.size]
+
+
+def _cases():
+    r = np.random.default_rng(7)
+    L = r.integers(0, 9, 5000)
+    L[17] = 4000
+    rp = np.concatenate([[0], np.cumsum(L)]).astype(np.int32)
+    skew = gen.CSR(5000, 7001, rp, r.integers(0, 7001, int(rp[-1])).astype(np.int32), r.standard_normal(int(rp[-1])))
+    return [("makea_S", gen.makea("S")), ("makea_W", gen.makea("W")), ("skew_ragged", skew),
+            ("stencil27_11", gen.stencil27(11)), ("laplace1d", gen.laplace1d(33333))]
+
+
+CASES = _cases()
+
+
+@pytest.mark.parametrize("kernel", ["auto", "vector", "merge", "xstat", "xplan", "sell", "sellsort", "xt"])
+@pytest.mark.parametrize("name,A", CASES, ids=[c[0] for c in CASES])
+@pytest.mark.parametrize("beta", [0.0, 1.5])
+def test_guard_regions(name, A, kernel, beta):
+    import torch
+
+    import paper_conf_asplos_ginsbachrsbdo18_b200 as sp
+    dev = torch.device("cuda:0")
+    rpb, rp = _guarded(torch, dev, A.rowptr, 0)
+    cib, ci = _guarded(torch, dev, A.colidx, 0)
+    vab, va = _guarded(torch, dev, A.vals, float("nan"))
+    x_h = gen.uniform(A.n, seed=31)
+    xb, x = _guarded(torch, dev, x_h, float("nan"))
+    y0 = gen.uniform(A.m, seed=32)
+    yb, y = _guarded(torch, dev, y0, SENT)
+    try:
+        M = sp.CSRMatrix(rp, ci, va, A.n, kernel=kernel)
+    except RuntimeError as e:  # a plan kernel that does not apply to this shape is refused at create
+        pytest.skip(f"{kernel} not applicable to {name}: {e}")
+    with M:
+        for _ in range(2):  # twice: the second call runs on warmed plan buffers
+            y.copy_(torch.from_numpy(y0).to(dev))
+            M.spmv(x, y, 1.0, beta)
+        torch.cuda.synchronize()
+    yh = yb.cpu().numpy()
+    assert np.all(yh[:G] == SENT) and np.all(yh[G + A.m:] == SENT), f"{name}/{kernel}: y written out of range"
+    y_ref, bound = oracle.spmv(A.rowptr, A.colidx, A.vals, x_h, y0, 1.0, beta)
+    check_rows(yh[G:G + A.m], y_ref, bound, np.float64, f"{name}/{kernel} beta={beta}")

@@ -6,7 +6,13 @@ vector, stencil, JDS, histogram / reduction / EP, CG).  The paper's admitted
 weak spot is the soundness of sparse accesses (section 6.3); a
 report fails the test.  Also covered: the persistent CG kernel (grid barriers)
 and the two ranks of the p2p transport, each under its own sanitizer.  The logs of the round's runs are kept in
-profiles/r02_sanitizer_*.log."""
+profiles/r02_sanitizer_*.log.
+
+Opt-in (SPMV_SANITIZE=1): compute-sanitizer was closed on this GPU pool late in
+round 2 ("runs under it have left GPUs needing a reset"), so the default GPU
+suite skips the tier; the committed logs are the round's evidence and
+tests/test_gpu_bounds.py covers out-of-range accesses with the library's own
+device-side checks (SPMV_DEBUG validation pass) instead."""
 import os
 import re
 import shutil
@@ -15,7 +21,9 @@ import sys
 
 import pytest
 
-pytestmark = pytest.mark.gpu
+pytestmark = [pytest.mark.gpu,
+              pytest.mark.skipif(os.environ.get("SPMV_SANITIZE") != "1",
+                                 reason="compute-sanitizer tier is opt-in (SPMV_SANITIZE=1): closed on this pool")]
 
 ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
 SAN = shutil.which("compute-sanitizer") or "/usr/local/cuda/bin/compute-sanitizer"
@@ -26,6 +34,8 @@ def _run(tool, cases, timeout=900):
     cmd = [SAN, "--tool", tool, "--error-exitcode", "9", "--print-limit", "20", sys.executable, CASES, *cases]
     r = subprocess.run(cmd, capture_output=True, text=True, timeout=timeout, cwd=ROOT)
     out = r.stdout + r.stderr
+    if "closed on this pool" in out:
+        pytest.skip("compute-sanitizer closed on this pool")
     # memcheck / synccheck: "ERROR SUMMARY: 0 errors"; racecheck: "RACECHECK SUMMARY: 0 hazards displayed (0 errors, 0 warnings)"
     clean = re.search(r"ERROR SUMMARY: 0 errors", out) or re.search(r"RACECHECK SUMMARY: 0 hazards displayed \(0 errors, 0 warnings\)", out)
     assert r.returncode == 0 and clean and "sanitize cases OK" in out, out[-4000:]
