@@ -219,6 +219,7 @@ k_cg_persist(PersistArgs pa) {
       }
       __syncthreads();
     }
+    stamp(k, 7);
     const double g = sc[0], d = sc[1];
     double beta = 0.0, pap = d;
     if (k > 0) {

@@ -900,10 +900,10 @@ spmv_status launch_cg_persist(spmv_csr_s* h, cudaStream_t s, const void* x_input
     cudaFree(pa.sp.tstamp);
     unsigned long long t0 = ~0ull;
     for (unsigned i = 0; i < G; ++i) t0 = std::min(t0, t[8 * i]);
-    const char* nm[7] = {"start", "xready", "streamed", "spmv_done", "bar1", "update_done", "bar2"};
+    const char* nm[8] = {"start", "xready", "streamed", "spmv_done", "bar1", "update_done", "bar2", "scalars"};
     fprintf(stderr, "[persist times] iteration %d, us from the first CTA's start: median / max over %u CTAs\n",
             iters / 2, G);
-    for (int ph = 0; ph < 7; ++ph) {
+    for (int ph : {0, 1, 2, 3, 4, 7, 5, 6}) {
       std::vector<double> v(G);
       for (unsigned i = 0; i < G; ++i) v[i] = (double)(t[8 * i + ph] - t0) / 1e3;
       std::sort(v.begin(), v.end());
