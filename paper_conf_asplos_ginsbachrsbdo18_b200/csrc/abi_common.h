@@ -216,6 +216,7 @@ struct spmv_csr_s {
   double *z = nullptr, *r = nullptr, *q = nullptr, *p_single = nullptr;
   double *s_vec = nullptr, *alpha2 = nullptr;  // single-reduction CG (NEXT-1): s = A p, alpha_{k-1}
   int cg_variant = 0;                          // 0 textbook (NPB conj_grad), 1 Chronopoulos-Gear, 2 persistent C-G
+  int pdl = 1;                                 // programmatic dependent launch of the SpMV / k_cgcg chain (SPMV_PDL=0: off)
   unsigned int* gbar = nullptr;                // persistent CG: grid barrier counter
   double *part_pq = nullptr, *part_rr = nullptr, *part_res = nullptr, *part_xz = nullptr,
          *part_zz = nullptr, *scal = nullptr, *out2 = nullptr;
@@ -245,6 +246,25 @@ inline bool tuning_env(const char* name, int* v) {
   (void)v;
   return false;
 #endif
+}
+
+// Launch with programmatic stream serialization (PDL) when `pdl`: the kernel may
+// start while its stream predecessor runs and synchronises with pdl_wait()
+// (common.cuh).  Without it, an ordinary launch.
+template <typename... KArgs, typename... Args>
+inline cudaError_t launch_maybe_pdl(void (*k)(KArgs...), dim3 grid, dim3 block, size_t smem, cudaStream_t s, bool pdl,
+                                    Args&&... args) {
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = grid;
+  cfg.blockDim = block;
+  cfg.dynamicSmemBytes = smem;
+  cfg.stream = s;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+  at[0].val.programmaticStreamSerializationAllowed = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = pdl ? 1 : 0;
+  return cudaLaunchKernelEx(&cfg, k, std::forward<Args>(args)...);
 }
 
 inline int num_sms(int dev) {

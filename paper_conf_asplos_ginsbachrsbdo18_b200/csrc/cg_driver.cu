@@ -113,8 +113,9 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
       P2PHook hz = base;
       hz.push_slot = p2p ? gslot : -1;
       const int64_t xoff = h->dist ? (int64_t)h->dist->rank * h->maxlen : 0;
-      k_cgcg<<<vg, 256, 0, s>>>(n, k, run->rr_old, run->rr_prev, del, h->alpha2, h->r, h->s_vec, h->q, z, rv,
-                                gnew, h->flags, tol, run->rr_b, hz, xoff);
+      CK(launch_maybe_pdl(k_cgcg, dim3(vg), dim3(256), 0, s, h->pdl && !p2p, n, k, run->rr_old, run->rr_prev, del,
+                          h->alpha2, h->r, h->s_vec, (const double*)h->q, z, rv, gnew, h->flags, tol, run->rr_b, hz,
+                          xoff));
       LAUNCHED();
       SumSrc g1;
       if (p2p) g1 = p2p_src(h, gslot);

@@ -170,19 +170,31 @@ k_cgcg(int64_t n, int k, SumSrc gam, SumSrc gam_old, SumSrc del, double* __restr
   const int64_t stride = int64_t(gridDim.x) * blockDim.x;
   const int64_t jstart = int64_t(blockIdx.x) * blockDim.x + threadIdx.x;
   double pr[CG_U], pw[CG_U], pp[CG_U], ps[CG_U], pz[CG_U];
-  auto load = [&](int64_t j0) {
+  auto load_own = [&](int64_t j0) {  // r, z, p, s: written only by the previous update
 #pragma unroll
     for (int u = 0; u < CG_U; ++u) {
       const int64_t j = j0 + u * stride;
       if (j < n) {
-        pr[u] = r[j]; pw[u] = w[j]; pz[u] = z[j];
+        pr[u] = r[j]; pz[u] = z[j];
         if (k > 0) { pp[u] = p[j]; ps[u] = sv[j]; }
       }
     }
   };
+  auto load_w = [&](int64_t j0) {  // w: the SpMV's output
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) pw[u] = w[j];
+    }
+  };
   // the first batch of vector loads does not depend on the scalars: issue it,
-  // then read the (up to four) scalar sources concurrently, one warp each
-  if (jstart < n) load(jstart);
+  // then read the (up to four) scalar sources concurrently, one warp each.
+  // Under PDL the SpMV may still be running: r, z, p, s (complete since the
+  // SpMV passed its own pdl_wait) are loaded before pdl_wait, w after it.
+  if (jstart < n) load_own(jstart);
+  pdl_wait();
+  pdl_trigger();
+  if (jstart < n) load_w(jstart);
   {
     const int wid = threadIdx.x >> 5, lane = threadIdx.x & 31;
     double v = 0.0;
@@ -214,7 +226,10 @@ k_cgcg(int64_t n, int k, SumSrc gam, SumSrc gam_old, SumSrc del, double* __restr
   }
   double acc = 0.0;
   for (int64_t j0 = jstart; j0 < n; j0 += CG_U * stride) {
-    if (j0 != jstart) load(j0);
+    if (j0 != jstart) {
+      load_own(j0);
+      load_w(j0);
+    }
 #pragma unroll
     for (int u = 0; u < CG_U; ++u) {
       const int64_t j = j0 + u * stride;

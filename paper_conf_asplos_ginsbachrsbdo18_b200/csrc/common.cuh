@@ -164,6 +164,16 @@ struct P2PHook {
   int push_slot = -1;
 };
 
+// Programmatic dependent launch (PDL): a kernel launched with
+// cudaLaunchAttributeProgrammaticStreamSerialization may start while its
+// predecessor in the stream is still running; pdl_wait() blocks until the
+// predecessor grid has completed and its memory is visible (a no-op when the
+// kernel was launched without the attribute).  pdl_trigger() lets the NEXT
+// kernel start launching; called only after pdl_wait(), so a kernel's
+// successor can never overlap its predecessor.
+__device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;\n" ::: "memory"); }
+__device__ __forceinline__ void pdl_trigger() { asm volatile("griddepcontrol.launch_dependents;\n" ::: "memory"); }
+
 __device__ __forceinline__ void p2p_prologue_wait(const P2PHook& h) {
   if (h.enabled && h.wait_x) {
     if (threadIdx.x == 0) {

@@ -218,13 +218,17 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   cfg.blockDim = dim3(XP_THREADS, 1, 1);
   cfg.dynamicSmemBytes = h->xp.smem;
   cfg.stream = s;
-  cudaLaunchAttribute at[1];
+  cudaLaunchAttribute at[2];
   at[0].id = cudaLaunchAttributeClusterDimension;
   at[0].val.clusterDim.x = (unsigned)h->xp.B;
   at[0].val.clusterDim.y = 1;
   at[0].val.clusterDim.z = 1;
+  // PDL (programmatic dependent launch): the barrier set-up overlaps the previous
+  // kernel's tail; off with the p2p hooks (their flag protocol is validated without it)
+  at[1].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+  at[1].val.programmaticStreamSerializationAllowed = 1;
   cfg.attrs = at;
-  cfg.numAttrs = 1;
+  cfg.numAttrs = (h->pdl && !hook.enabled && !h->xp.dyn) ? 2 : 1;
   int times = 0;
   if (tuning_env("SPMV_XPLAN_TIMES", &times) && times) {
     // diagnostics: per-CTA {start, x ready, streaming done, end} (globaltimer, ns), summarised on stderr

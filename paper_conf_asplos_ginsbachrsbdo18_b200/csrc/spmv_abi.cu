@@ -248,6 +248,8 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
     h->ci_loc = h->ci_own - h->k0;  // absolute k addressing
   }
 
+  h->pdl = 1;
+  env_int("SPMV_PDL", &h->pdl);  // programmatic dependent launch of the SpMV / k_cgcg chain (A/B: 0 = off)
   int rk = 0, rl = 0;
   if (!env_int("SPMV_KERNEL", &rk)) rk = o.kernel;
   if (!env_int("SPMV_LANES", &rl)) rl = o.vec_lanes;

@@ -262,26 +262,32 @@ k_spmv_xplan(XplanArgs a) {
       asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a.plan + o), "r"(nb) : "memory");
     }
   }
-  p2p_prologue_wait(a.hk);  // x slices of the peers (p2p transport)
   auto recv_bytes = [&](int t) -> uint32_t {
     const int nrows = int(cmin64(R, r1c - (r0c + int64_t(t) * R)));
     const int own = max(0, min((b + 1) * RB, nrows) - b * RB);
     return uint32_t(own * B * 8);
   };
+  // barrier set-up reads nothing a predecessor writes: it runs before pdl_wait
+  // (overlapping the previous kernel's tail under PDL)
   if (threadIdx.x == 0) {
     mbar_init(&xbar, 1);
     for (int q = 0; q < XP_K; ++q) mbar_init(&tbar[q], 1);
     if (DYN)
       for (int q = 0; q < XP_TQ; ++q) mbar_init(&qbar[q], 1);
     asm volatile("fence.mbarrier_init.release.cluster;\n" ::: "memory");
-    const uint32_t xb = uint32_t(bulk_elems * sizeof(T));
-    mbar_expect_tx(&xbar, xb);
-    if (xb) bulk_g2s(xs, xg + col0, xb, &xbar);
     if (DYN) {
       for (int q = 0; q < XP_TQ; ++q) mbar_expect_tx(&qbar[q], 4);  // tile ids of local tiles 0..7
     } else {
       for (int t = 0; t < XP_K && t < ntiles; ++t) mbar_expect_tx(&tbar[t], recv_bytes(t));
     }
+  }
+  pdl_wait();               // x (and w, y) of the predecessor kernel
+  pdl_trigger();
+  p2p_prologue_wait(a.hk);  // x slices of the peers (p2p transport)
+  if (threadIdx.x == 0) {
+    const uint32_t xb = uint32_t(bulk_elems * sizeof(T));
+    mbar_expect_tx(&xbar, xb);
+    if (xb) bulk_g2s(xs, xg + col0, xb, &xbar);
   }
   for (int64_t j = bulk_elems + threadIdx.x; j <= W; j += blockDim.x) xs[j] = (j < ncols) ? xg[col0 + j] : T(0);
   // peers must have initialised their barriers before partials are sent
