@@ -145,14 +145,16 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
     const int rslot = 2 + ((it + 1) & 1);
     P2PHook hz = base;
     hz.push_slot = p2p ? rslot : -1;
-    k_cg_zr<<<vg, 256, 0, s>>>(n, pq, run->rr_old, p, h->q, z, h->r, pnew, h->flags, hz);
+    CK(launch_maybe_pdl(k_cg_zr, dim3(vg), dim3(256), 0, s, h->pdl && !p2p, n, pq, run->rr_old, (const double*)p,
+                        (const double*)h->q, z, h->r, pnew, h->flags, hz));
     LAUNCHED();
     SumSrc rr_new;
     if (p2p) rr_new = p2p_src(h, rslot);
     else ST(reduce_src(h, s, SumSrc{pnew, vg}, rslot, &rr_new));
     // p2p: the p update stores its slice into every peer's x buffer and publishes it
     const int64_t xoff = h->dist ? (int64_t)h->dist->rank * h->maxlen : 0;
-    k_cg_p<<<vg, 256, 0, s>>>(n, rr_new, run->rr_old, h->r, p, h->flags, tol, run->rr_b, it, base, xoff);
+    CK(launch_maybe_pdl(k_cg_p, dim3(vg), dim3(256), 0, s, h->pdl && !p2p, n, rr_new, run->rr_old,
+                        (const double*)h->r, p, h->flags, tol, run->rr_b, it, base, xoff));
     LAUNCHED();
     run->rr_old = rr_new;
   }

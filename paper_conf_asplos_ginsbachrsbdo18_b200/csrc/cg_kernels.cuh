@@ -45,6 +45,27 @@ k_cg_zr(int64_t n, SumSrc pq, SumSrc rr_old, const double* __restrict__ p,
   __shared__ double red[8];
   __shared__ double sc[2];
   if (flags[1]) return;  // converged (tol mode): no-op
+  const int64_t stride = int64_t(gridDim.x) * blockDim.x;
+  const int64_t jstart = int64_t(blockIdx.x) * blockDim.x + threadIdx.x;
+  double pz[CG_U], pp[CG_U], pr[CG_U], pq_[CG_U];
+  auto load_own = [&](int64_t j0) {  // z, p, r: complete before the SpMV passed its pdl_wait
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) { pz[u] = z[j]; pp[u] = p[j]; pr[u] = r[j]; }
+    }
+  };
+  auto load_q = [&](int64_t j0) {  // q = A p: the SpMV's output
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) pq_[u] = q[j];
+    }
+  };
+  if (jstart < n) load_own(jstart);
+  pdl_wait();
+  pdl_trigger();
+  if (jstart < n) load_q(jstart);
   {  // both scalar sources at once, one warp each (bit-identical to read_sum)
     const int wid = threadIdx.x >> 5;
     double v = 0.0;
@@ -60,13 +81,10 @@ k_cg_zr(int64_t n, SumSrc pq, SumSrc rr_old, const double* __restrict__ p,
   const double alpha = rho / d;
   double acc = 0.0;
   // CG_U consecutive-stride elements per thread with all loads issued first
-  const int64_t stride = int64_t(gridDim.x) * blockDim.x;
-  for (int64_t j0 = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j0 < n; j0 += CG_U * stride) {
-    double pz[CG_U], pp[CG_U], pr[CG_U], pq_[CG_U];
-#pragma unroll
-    for (int u = 0; u < CG_U; ++u) {
-      const int64_t j = j0 + u * stride;
-      if (j < n) { pz[u] = z[j]; pp[u] = p[j]; pr[u] = r[j]; pq_[u] = q[j]; }
+  for (int64_t j0 = jstart; j0 < n; j0 += CG_U * stride) {
+    if (j0 != jstart) {
+      load_own(j0);
+      load_q(j0);
     }
 #pragma unroll
     for (int u = 0; u < CG_U; ++u) {
@@ -94,6 +112,27 @@ k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
   __shared__ double s_b;
   __shared__ double sc[2];
   if (flags[1]) return;
+  const int64_t stride = int64_t(gridDim.x) * blockDim.x;
+  const int64_t jstart = int64_t(blockIdx.x) * blockDim.x + threadIdx.x;
+  double pr[CG_U], pp[CG_U];
+  auto load_p = [&](int64_t j0) {  // p: last written by the previous k_cg_p
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) pp[u] = p[j];
+    }
+  };
+  auto load_r = [&](int64_t j0) {  // r: k_cg_zr's output
+#pragma unroll
+    for (int u = 0; u < CG_U; ++u) {
+      const int64_t j = j0 + u * stride;
+      if (j < n) pr[u] = r[j];
+    }
+  };
+  if (jstart < n) load_p(jstart);
+  pdl_wait();
+  pdl_trigger();
+  if (jstart < n) load_r(jstart);
   {  // both scalar sources at once, one warp each (bit-identical to read_sum)
     const int wid = threadIdx.x >> 5;
     double v = 0.0;
@@ -104,13 +143,10 @@ k_cg_p(int64_t n, SumSrc rr_new, SumSrc rr_old, const double* __restrict__ r,
   }
   const double rho1 = sc[0], rho0 = sc[1];
   const double beta = rho1 / rho0;
-  const int64_t stride = int64_t(gridDim.x) * blockDim.x;
-  for (int64_t j0 = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j0 < n; j0 += CG_U * stride) {
-    double pr[CG_U], pp[CG_U];
-#pragma unroll
-    for (int u = 0; u < CG_U; ++u) {
-      const int64_t j = j0 + u * stride;
-      if (j < n) { pr[u] = r[j]; pp[u] = p[j]; }
+  for (int64_t j0 = jstart; j0 < n; j0 += CG_U * stride) {
+    if (j0 != jstart) {
+      load_p(j0);
+      load_r(j0);
     }
 #pragma unroll
     for (int u = 0; u < CG_U; ++u) {
