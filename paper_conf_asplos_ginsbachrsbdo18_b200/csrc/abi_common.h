@@ -149,6 +149,9 @@ struct spmv_csr_s {
     int64_t mplan = -1;
     int g2 = 0;
     int bankperm = 1;  // k_xplan_bankperm after every pack (SPMV_XPLAN_PERM=0: CSR order within each row)
+    // persisting-L2 access window over the plan (SPMV_XPLAN_PLANWIN=1; small plans that stay L2-resident)
+    size_t win_bytes = 0;
+    float win_ratio = 0.f;
   } xp;
   cudaStream_t side = nullptr;
   cudaEvent_t ev_fork = nullptr, ev_join = nullptr;

@@ -218,7 +218,7 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   cfg.blockDim = dim3(XP_THREADS, 1, 1);
   cfg.dynamicSmemBytes = h->xp.smem;
   cfg.stream = s;
-  cudaLaunchAttribute at[2];
+  cudaLaunchAttribute at[3];
   at[0].id = cudaLaunchAttributeClusterDimension;
   at[0].val.clusterDim.x = (unsigned)h->xp.B;
   at[0].val.clusterDim.y = 1;
@@ -229,6 +229,15 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   at[1].val.programmaticStreamSerializationAllowed = 1;
   cfg.attrs = at;
   cfg.numAttrs = (h->pdl && !hook.enabled && !h->xp.dyn) ? 2 : 1;
+  if (h->xp.win_bytes) {
+    at[cfg.numAttrs].id = cudaLaunchAttributeAccessPolicyWindow;
+    at[cfg.numAttrs].val.accessPolicyWindow.base_ptr = h->xp.plan;
+    at[cfg.numAttrs].val.accessPolicyWindow.num_bytes = h->xp.win_bytes;
+    at[cfg.numAttrs].val.accessPolicyWindow.hitRatio = h->xp.win_ratio;
+    at[cfg.numAttrs].val.accessPolicyWindow.hitProp = cudaAccessPropertyPersisting;
+    at[cfg.numAttrs].val.accessPolicyWindow.missProp = cudaAccessPropertyStreaming;
+    ++cfg.numAttrs;
+  }
   int times = 0;
   if (tuning_env("SPMV_XPLAN_TIMES", &times) && times) {
     // diagnostics: per-CTA {start, x ready, streaming done, end} (globaltimer, ns), summarised on stderr
@@ -499,7 +508,31 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
     // plans that stay L2-resident across CG iterations (<= 96 MB of the 126 MB L2; measured on the
     // class-C rank blocks: P = 4 (94 MB) 38.1 -> 32.2 us, P = 8 (47 MB) 24.4 -> 21.4 us per CG
     // iteration; P = 2 (188 MB) and the whole matrix lose: the prefetch thrashes L2)
-    int pf = (!dyn && pos <= (long long)(96) << 20) ? 1 : 0;
+    // plans that fit the device's persisting-L2 carve-out (B200: 79 MB; the P = 8 rank block's 47 MB)
+    // are pinned there instead: a persisting access window over the plan on every launch
+    // (SPMV_XPLAN_PLANWIN=0/1 forces it).  Measured, class-C P = 8 block (profiles/r02u_*): CG
+    // iteration 16.67 vs 16.86 us (graph path), 17.15 vs 17.48 us (persistent), SpMV back to back
+    // 0.664 vs 0.585 of the copy peak; the P = 4 block (94 MB) only fits partly and keeps the prefetch
+    // (31.7 us with the window vs 25.7 us with the prefetch).
+    {
+      int maxwin = 0, maxpersist = 0;
+      cudaDeviceGetAttribute(&maxwin, cudaDevAttrMaxAccessPolicyWindowSize, h->device);
+      cudaDeviceGetAttribute(&maxpersist, cudaDevAttrMaxPersistingL2CacheSize, h->device);
+      int pw = (!dyn && maxwin > 0 && maxpersist > 0 && pos <= (long long)maxpersist && pos <= (long long)maxwin) ? 1 : 0;
+      env_int("SPMV_XPLAN_PLANWIN", &pw);
+      if (pw && maxwin > 0 && maxpersist > 0) {
+        size_t cur = 0;
+        cudaDeviceGetLimit(&cur, cudaLimitPersistingL2CacheSize);
+        const size_t want = std::min<size_t>((size_t)pos, (size_t)maxpersist);
+        if (want > cur && cudaDeviceSetLimit(cudaLimitPersistingL2CacheSize, want) != cudaSuccess) cudaGetLastError();
+        cudaDeviceGetLimit(&cur, cudaLimitPersistingL2CacheSize);
+        if (cur > 0) {
+          P.win_bytes = std::min<size_t>((size_t)pos, (size_t)maxwin);
+          P.win_ratio = (float)std::min(1.0, (double)cur / (double)P.win_bytes);
+        }
+      }
+    }
+    int pf = (!dyn && !P.win_bytes && pos <= (long long)(96) << 20) ? 1 : 0;
     env_int("SPMV_XPLAN_L2PF", &pf);
     if (pf && !dyn) {
       std::vector<long long> rng(2 * (size_t)ncl * B, 0);
@@ -880,13 +913,22 @@ spmv_status launch_cg_persist(spmv_csr_s* h, cudaStream_t s, const void* x_input
   cfg.blockDim = dim3(XP_THREADS, 1, 1);
   cfg.dynamicSmemBytes = h->xp.smem;
   cfg.stream = s;
-  cudaLaunchAttribute at[1];
+  cudaLaunchAttribute at[2];
   at[0].id = cudaLaunchAttributeClusterDimension;
   at[0].val.clusterDim.x = (unsigned)h->xp.B;
   at[0].val.clusterDim.y = 1;
   at[0].val.clusterDim.z = 1;
   cfg.attrs = at;
   cfg.numAttrs = 1;
+  if (h->xp.win_bytes) {  // the plan pinned in the persisting L2 carve-out (see xplan_build)
+    at[1].id = cudaLaunchAttributeAccessPolicyWindow;
+    at[1].val.accessPolicyWindow.base_ptr = h->xp.plan;
+    at[1].val.accessPolicyWindow.num_bytes = h->xp.win_bytes;
+    at[1].val.accessPolicyWindow.hitRatio = h->xp.win_ratio;
+    at[1].val.accessPolicyWindow.hitProp = cudaAccessPropertyPersisting;
+    at[1].val.accessPolicyWindow.missProp = cudaAccessPropertyStreaming;
+    cfg.numAttrs = 2;
+  }
   int times = 0;
   if (tuning_env("SPMV_PERSIST_TIMES", &times) && times) {
     // diagnostics (cg_solve only: synchronises): per-CTA phase stamps of iteration iters/2

@@ -366,6 +366,9 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
                   h->seg, h->crow, h->ci_own, h->send_iv, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
                   h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags, h->s_vec, h->alpha2,
                   h->stage_x, h->stage_z, h->gbar};
+  // lines pinned by a persisting window over the plan go back to normal (device-wide; other
+  // handles' windows re-pin theirs on their next launch)
+  if (h->xp.win_bytes) cudaCtxResetPersistingL2Cache();
   for (void* b : bufs)
     if (b) cudaFree(b);
   if (h->cap) cudaStreamDestroy(h->cap);

@@ -49,6 +49,7 @@ def main():
     ap.add_argument("--cls", default="C")
     ap.add_argument("--ranks", default="first,last")
     ap.add_argument("--variant", default="cgcg")
+    ap.add_argument("--ps", default="1,2,4,8", help="rank counts P to run")
     args = ap.parse_args()
     dev = torch.device("cuda:0")
     na, nonzer, niter, shift = gen.NPB_CLASSES[args.cls]
@@ -58,7 +59,7 @@ def main():
     stream = torch.cuda.Stream(dev)  # non-default: the graph-timed leg captures on it
     torch.cuda.set_stream(stream)  # every handle launches on the stream current at its creation
     t1 = None
-    for P in (1, 2, 4, 8):
+    for P in [int(v) for v in args.ps.split(",")]:
         ranks = sorted({0 if s == "first" else P - 1 for s in args.ranks.split(",")})
         for r in ranks:
             d = sp.Dist(r, P, 0, transport="proxy")
