@@ -113,7 +113,7 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
       P2PHook hz = base;
       hz.push_slot = p2p ? gslot : -1;
       const int64_t xoff = h->dist ? (int64_t)h->dist->rank * h->maxlen : 0;
-      CK(launch_maybe_pdl(k_cgcg, dim3(vg), dim3(256), 0, s, h->pdl && !p2p, n, k, run->rr_old, run->rr_prev, del,
+      CK(launch_maybe_pdl(k_cgcg, dim3(vg), dim3(256), 0, s, h->pdl, n, k, run->rr_old, run->rr_prev, del,
                           h->alpha2, h->r, h->s_vec, (const double*)h->q, z, rv, gnew, h->flags, tol, run->rr_b, hz,
                           xoff));
       LAUNCHED();
@@ -145,7 +145,7 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
     const int rslot = 2 + ((it + 1) & 1);
     P2PHook hz = base;
     hz.push_slot = p2p ? rslot : -1;
-    CK(launch_maybe_pdl(k_cg_zr, dim3(vg), dim3(256), 0, s, h->pdl && !p2p, n, pq, run->rr_old, (const double*)p,
+    CK(launch_maybe_pdl(k_cg_zr, dim3(vg), dim3(256), 0, s, h->pdl, n, pq, run->rr_old, (const double*)p,
                         (const double*)h->q, z, h->r, pnew, h->flags, hz));
     LAUNCHED();
     SumSrc rr_new;
@@ -153,7 +153,7 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
     else ST(reduce_src(h, s, SumSrc{pnew, vg}, rslot, &rr_new));
     // p2p: the p update stores its slice into every peer's x buffer and publishes it
     const int64_t xoff = h->dist ? (int64_t)h->dist->rank * h->maxlen : 0;
-    CK(launch_maybe_pdl(k_cg_p, dim3(vg), dim3(256), 0, s, h->pdl && !p2p, n, rr_new, run->rr_old,
+    CK(launch_maybe_pdl(k_cg_p, dim3(vg), dim3(256), 0, s, h->pdl, n, rr_new, run->rr_old,
                         (const double*)h->r, p, h->flags, tol, run->rr_b, it, base, xoff));
     LAUNCHED();
     run->rr_old = rr_new;

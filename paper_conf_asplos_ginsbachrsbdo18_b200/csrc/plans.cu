@@ -224,11 +224,11 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   at[0].val.clusterDim.y = 1;
   at[0].val.clusterDim.z = 1;
   // PDL (programmatic dependent launch): the barrier set-up overlaps the previous
-  // kernel's tail; off with the p2p hooks (their flag protocol is validated without it)
+  // kernel's tail (the p2p hooks wait on their peers' flags after pdl_wait)
   at[1].id = cudaLaunchAttributeProgrammaticStreamSerialization;
   at[1].val.programmaticStreamSerializationAllowed = 1;
   cfg.attrs = at;
-  cfg.numAttrs = (h->pdl && !hook.enabled && !h->xp.dyn) ? 2 : 1;
+  cfg.numAttrs = (h->pdl && !h->xp.dyn) ? 2 : 1;
   if (h->xp.win_bytes) {
     at[cfg.numAttrs].id = cudaLaunchAttributeAccessPolicyWindow;
     at[cfg.numAttrs].val.accessPolicyWindow.base_ptr = h->xp.plan;
