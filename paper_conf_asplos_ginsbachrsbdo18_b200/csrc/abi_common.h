@@ -343,6 +343,8 @@ spmv_status run_spmv(spmv_csr_s* h, cudaStream_t s, const void* vals, const void
 // dist.cu
 bool use_p2p(const spmv_csr_s* h);
 P2PCtx p2p_ctx(spmv_csr_s* h);
-SumSrc p2p_src(spmv_csr_s* h, int slot);
+SumSrc p2p_src(spmv_csr_s* h, int slot, int per);  // per: partials pushed per rank (1: one value)
+int p2p_push_per(const spmv_csr_s* h, int64_t grid);  // per-CTA pushes for a producer of `grid` CTAs, else 0
+int p2p_spmv_push_per(const spmv_csr_s* h);           // ... for the SpMV's fused dot
 spmv_status exchange_x(spmv_csr_s* h, cudaStream_t s);
 spmv_status reduce_src(spmv_csr_s* h, cudaStream_t s, SumSrc in, int slot, SumSrc* out);

@@ -101,8 +101,9 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
         P2PHook hs = base;
         hs.wait_x = 1;
         hs.push_slot = 1;
+        hs.push_per = p2p_spmv_push_per(h);
         ST(run_spmv(h, s, h->vals, xg, h->q, 1.0, 0.0, rv, h->part_pq, &hs));
-        del = p2p_src(h, 1);
+        del = p2p_src(h, 1, std::max(hs.push_per, 1));
       } else {
         ST(gather_p(h, s));
         ST(run_spmv(h, s, h->vals, xg, h->q, 1.0, 0.0, rv, h->part_pq));
@@ -112,13 +113,14 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
       const int gslot = kGamSlot[(k + 1) % 3];
       P2PHook hz = base;
       hz.push_slot = p2p ? gslot : -1;
+      hz.push_per = p2p_push_per(h, vg);
       const int64_t xoff = h->dist ? (int64_t)h->dist->rank * h->maxlen : 0;
       CK(launch_maybe_pdl(k_cgcg, dim3(vg), dim3(256), 0, s, h->pdl, n, k, run->rr_old, run->rr_prev, del,
                           h->alpha2, h->r, h->s_vec, (const double*)h->q, z, rv, gnew, h->flags, tol, run->rr_b, hz,
                           xoff));
       LAUNCHED();
       SumSrc g1;
-      if (p2p) g1 = p2p_src(h, gslot);
+      if (p2p) g1 = p2p_src(h, gslot, std::max(hz.push_per, 1));
       else ST(reduce_src(h, s, SumSrc{gnew, vg}, gslot, &g1));
       run->rr_prev = run->rr_old;
       run->rr_old = g1;
@@ -134,8 +136,9 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
       P2PHook hs = base;
       hs.wait_x = 1;
       hs.push_slot = 1;
+      hs.push_per = p2p_spmv_push_per(h);
       ST(run_spmv(h, s, h->vals, xg, h->q, 1.0, 0.0, p, h->part_pq, &hs));
-      pq = p2p_src(h, 1);
+      pq = p2p_src(h, 1, std::max(hs.push_per, 1));
     } else {
       ST(gather_p(h, s));
       ST(run_spmv(h, s, h->vals, xg, h->q, 1.0, 0.0, p, h->part_pq));
@@ -145,11 +148,12 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
     const int rslot = 2 + ((it + 1) & 1);
     P2PHook hz = base;
     hz.push_slot = p2p ? rslot : -1;
+    hz.push_per = p2p_push_per(h, vg);
     CK(launch_maybe_pdl(k_cg_zr, dim3(vg), dim3(256), 0, s, h->pdl, n, pq, run->rr_old, (const double*)p,
                         (const double*)h->q, z, h->r, pnew, h->flags, hz));
     LAUNCHED();
     SumSrc rr_new;
-    if (p2p) rr_new = p2p_src(h, rslot);
+    if (p2p) rr_new = p2p_src(h, rslot, std::max(hz.push_per, 1));
     else ST(reduce_src(h, s, SumSrc{pnew, vg}, rslot, &rr_new));
     // p2p: the p update stores its slice into every peer's x buffer and publishes it
     const int64_t xoff = h->dist ? (int64_t)h->dist->rank * h->maxlen : 0;

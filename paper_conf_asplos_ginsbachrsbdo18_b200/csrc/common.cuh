@@ -116,6 +116,7 @@ __device__ __forceinline__ int ticket_acq_rel_gpu(int* t) {
 
 constexpr int P2P_NSLOT = 8;       // scalar slots (same ids as reduce_src slots)
 constexpr int P2P_XSLOT = P2P_NSLOT;  // slot_epoch index of the x exchange
+constexpr int P2P_PMAX = 1024;     // partials per rank per slot: exch is [NSLOT][P][PMAX] doubles
 
 struct P2PCtx {
   unsigned char* const* peer;      // device array [P]: fabric base of every rank (own included)
@@ -154,14 +155,18 @@ __device__ __forceinline__ void p2p_signal(const P2PCtx& c, int slot) {
 // zero / disabled otherwise):
 //   wait_x    -- the kernel reads x from xpad: thread 0 of every CTA first
 //                waits until every peer published the latest x exchange;
-//   push_slot -- the kernel writes one dot partial per CTA into part[]: the
-//                last CTA to finish sums them (read_sum order) and pushes the
-//                value into `push_slot` of every rank (fused all-reduce half).
+//   push_slot -- the kernel writes one dot partial per CTA into part[]:
+//                push_per == gridDim.x (round 2): every CTA stores its partial
+//                into entry blockIdx.x of this rank's row of `push_slot` in
+//                every rank, the last CTA only publishes (consumers sum the
+//                P x push_per values); push_per == 0: the last CTA to finish
+//                sums them (read_sum order) and pushes the one value.
 struct P2PHook {
   P2PCtx c;
   int enabled = 0;
   int wait_x = 0;
   int push_slot = -1;
+  int push_per = 0;
 };
 
 // Programmatic dependent launch (PDL): a kernel launched with
@@ -189,31 +194,42 @@ __device__ __forceinline__ void p2p_prologue_wait(const P2PHook& h) {
 __device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const double* part, int count) {
   if (!h.enabled || h.push_slot < 0) return;
   __shared__ int s_last;
+  const bool per_cta = h.push_per == int(gridDim.x) && count == int(gridDim.x);
+  if (per_cta && threadIdx.x == 0) {
+    // this CTA's partial straight into every rank (plain stores, ordered before
+    // the ticket below and, through the last CTA's release, before the flag)
+    const double v = part[blockIdx.x];
+    for (int q = 0; q < h.c.P; ++q) {
+      double* ex = reinterpret_cast<double*>(h.c.peer[q] + h.c.off_exch);
+      ex[(size_t(h.push_slot) * h.c.P + h.c.me) * P2P_PMAX + blockIdx.x] = v;
+    }
+  }
   // part[blockIdx.x] was stored by thread 0; the acq_rel ticket orders it
   // before the increment and gives the last CTA every other CTA's partial
   __syncthreads();
   if (threadIdx.x == 0) {
     const int tk = ticket_acq_rel_gpu(h.c.ticket);
     s_last = (tk == int(gridDim.x) - 1);
-#ifdef SPMV_P2P_TRACE
-    if (blockIdx.x == 0 || s_last) printf("push_last blk %d ticket %d grid %d slot %d\n", blockIdx.x, tk, gridDim.x, h.push_slot);
-#endif
   }
   __syncthreads();
   if (!s_last) return;
+  if (per_cta) {
+    if (threadIdx.x == 0) {
+      *h.c.ticket = 0;
+      p2p_signal(h.c, h.push_slot);
+    }
+    return;
+  }
   if (threadIdx.x < 32) {
     double a = 0.0;
 #pragma unroll 4
     for (int i = threadIdx.x; i < count; i += 32) a += __ldcg(part + i);  // L2: other CTAs' stores
     a = warp_sum(a);
     if (threadIdx.x == 0) {
-#ifdef SPMV_P2P_TRACE
-      printf("push value %g count %d\n", a, count);
-#endif
       *h.c.ticket = 0;
       for (int q = 0; q < h.c.P; ++q) {
         double* ex = reinterpret_cast<double*>(h.c.peer[q] + h.c.off_exch);
-        ex[h.push_slot * h.c.P + h.c.me] = a;
+        ex[(size_t(h.push_slot) * h.c.P + h.c.me) * P2P_PMAX] = a;
       }
       p2p_signal(h.c, h.push_slot);
     }
@@ -223,30 +239,43 @@ __device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const d
 // A scalar source for the CG kernels: either `count` > 0 per-block partials to
 // be summed (single GPU: every consuming block sums them in the same fixed
 // order, so all blocks see bit-identical scalars), count == 1 pointing at a
-// finalized (NCCL-all-reduced) value, or count == -P: the P values pushed by
-// the ranks over peer memory (p2p_kernels.cuh), read once flags[q] >= *epoch
-// for every other rank q and summed in rank order (identical on all ranks).
+// finalized (NCCL-all-reduced) value, or count == -P: the values pushed by
+// the ranks over peer memory (p2p_kernels.cuh), `per` per rank at stride
+// P2P_PMAX, read once flags[q] >= *epoch for every other rank q and summed
+// rank by rank (per == 1: one value each, in rank order; per > 1: lane-strided
+// within each rank, then the warp tree) -- identical on all ranks.
 struct SumSrc {
   const double* p;
   int count;
   const unsigned long long* flags = nullptr;
   const unsigned long long* epoch = nullptr;
   int me = 0;
+  int per = 1;
 };
+
+// Warp-wide sum of the pushed values of a p2p source (after its flags).
+__device__ __forceinline__ double pushed_sum(const SumSrc& s, int P) {
+  const int lane = threadIdx.x & 31;
+  double a = 0.0;
+  if (s.per <= 1) {
+    if (lane == 0)
+      for (int q = 0; q < P; ++q) a += s.p[size_t(q) * P2P_PMAX];  // rank order
+    return __shfl_sync(0xffffffffu, a, 0);
+  }
+  for (int q = 0; q < P; ++q)
+    for (int i = lane; i < s.per; i += 32) a += s.p[size_t(q) * P2P_PMAX + i];
+  return warp_sum(a);
+}
 
 // Sum of a SumSrc by warp 0 of the block; returns the value in every thread.
 __device__ __forceinline__ double read_sum(SumSrc s, double* slot) {
   if (threadIdx.x < 32) {
     int n = s.count;
-    if (n < 0) {
-      n = -n;
-      if (threadIdx.x == 0) p2p_wait_flags(s.flags, s.me, n, *s.epoch);
-      __syncwarp();
-    }
     double a = 0.0;
-    if (s.count < 0) {
-      if (threadIdx.x == 0)
-        for (int i = 0; i < n; ++i) a += s.p[i];  // rank order
+    if (n < 0) {
+      if (threadIdx.x == 0) p2p_wait_flags(s.flags, s.me, -n, *s.epoch);
+      __syncwarp();
+      a = pushed_sum(s, -n);
     } else {
 #pragma unroll 4
       for (int i = threadIdx.x; i < n; i += 32) a += s.p[i];
@@ -267,12 +296,9 @@ __device__ __forceinline__ double warp_read_sum(SumSrc s) {
   int n = s.count;
   double a = 0.0;
   if (n < 0) {
-    n = -n;
-    if (lane == 0) {
-      p2p_wait_flags(s.flags, s.me, n, *s.epoch);
-      for (int i = 0; i < n; ++i) a += s.p[i];  // rank order
-    }
-    return __shfl_sync(0xffffffffu, a, 0);
+    if (lane == 0) p2p_wait_flags(s.flags, s.me, -n, *s.epoch);
+    __syncwarp();
+    return pushed_sum(s, -n);
   }
 #pragma unroll 4
   for (int i = lane; i < n; i += 32) a += s.p[i];

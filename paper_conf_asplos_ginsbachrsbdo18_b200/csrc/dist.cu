@@ -22,6 +22,17 @@ P2PCtx p2p_ctx(spmv_csr_s* h) {
 
 bool use_p2p(const spmv_csr_s* h) { return h->dist && h->dist->p2p; }
 
+int p2p_push_per(const spmv_csr_s* h, int64_t grid) { return (grid >= 1 && grid <= P2P_PMAX) ? (int)grid : 0; }
+
+// Partials per rank the SpMV's fused dot pushes: one per CTA for the static
+// XPLAN grid (its partial count is its launch grid), else the last-CTA sum.
+static int spmv_push_per(const spmv_csr_s* h) {
+  const bool side = h->xp.mplan >= 0 && h->xp.mplan < h->m_loc;
+  if (h->kernel != SPMV_KERNEL_XPLAN || !h->xp.built || h->xp.dyn || side) return 0;
+  return p2p_push_per(h, (int64_t)h->xp.ncl * h->xp.B);
+}
+int p2p_spmv_push_per(const spmv_csr_s* h) { return spmv_push_per(h); }
+
 // All-gather of this rank's slice (already at xpad + rank*maxlen) and wait.
 spmv_status exchange_x(spmv_csr_s* h, cudaStream_t s) {
   if (h->dist->proxy) return SPMV_OK;  // measurement proxy: no communication
@@ -62,11 +73,12 @@ spmv_status exchange_x(spmv_csr_s* h, cudaStream_t s) {
 // In distributed mode a SumSrc of per-CTA partials is finalized into scal[slot]
 // and all-reduced over the ranks; single GPU returns the partials unchanged.
 // The exchange-mode scalar source of `slot` (values pushed by every rank).
-SumSrc p2p_src(spmv_csr_s* h, int slot) {
+SumSrc p2p_src(spmv_csr_s* h, int slot, int per) {
   const P2PCtx c = p2p_ctx(h);
   SumSrc o;
-  o.p = reinterpret_cast<const double*>(h->fabric + h->off_exch) + slot * c.P;
+  o.p = reinterpret_cast<const double*>(h->fabric + h->off_exch) + (size_t)slot * c.P * P2P_PMAX;
   o.count = -c.P;
+  o.per = per;
   o.flags = reinterpret_cast<const unsigned long long*>(h->fabric + h->off_flags);
   o.epoch = c.slot_epoch + slot;
   o.me = c.me;
@@ -80,7 +92,7 @@ spmv_status reduce_src(spmv_csr_s* h, cudaStream_t s, SumSrc in, int slot, SumSr
     const P2PCtx c = p2p_ctx(h);
     k_p2p_push_sum<<<1, 32, 0, s>>>(in, slot, c);
     LAUNCHED();
-    *out = p2p_src(h, slot);
+    *out = p2p_src(h, slot, 1);
     return SPMV_OK;
   }
   double* dst = h->scal + slot;

@@ -5,7 +5,8 @@
 //
 // Fabric of a rank (one cudaMalloc, IPC-exported):
 //   xpad  [P * maxlen] T       gathered x / p (slice q written by rank q)
-//   exch  [NSLOT][P]  double   pushed scalars (slot s, value of rank q)
+//   exch  [NSLOT][P][PMAX] double  pushed partials (slot s, rank q: one
+//                                  value, or one per producing CTA)
 //   flags [P]         u64      flags[q] = latest exchange epoch rank q completed
 // plus local (never remote) counters: epoch (this rank's exchange count),
 // slot_epoch[NSLOT+1] (epoch of the latest push of each slot / of x), ticket.
@@ -31,7 +32,7 @@ static __global__ void k_p2p_push_sum(SumSrc in, int slot, P2PCtx c) {
   if (threadIdx.x == 0) {
     for (int q = 0; q < c.P; ++q) {
       double* ex = reinterpret_cast<double*>(c.peer[q] + c.off_exch);
-      ex[slot * c.P + c.me] = v;
+      ex[(size_t(slot) * c.P + c.me) * P2P_PMAX] = v;
     }
     p2p_signal(c, slot);
   }

@@ -175,10 +175,10 @@ extern "C" spmv_status spmv_csr_create(spmv_csr_t* out, spmv_dtype dt, int64_t m
       okm = cudaMalloc(&h->xpad, h->ts * (size_t)(maxlen * P)) == cudaSuccess;
       if (okm) cudaMemsetAsync(h->xpad, 0, h->ts * (size_t)(maxlen * P), s);
     } else if (okm) {
-      // fabric: xpad | exch [NSLOT][P] double | flags [P] u64, one IPC-exportable allocation
+      // fabric: xpad | exch [NSLOT][P][PMAX] double | flags [P] u64, one IPC-exportable allocation
       const size_t xb = (h->ts * (size_t)(maxlen * P) + 255) & ~size_t(255);
       h->off_exch = xb;
-      h->off_flags = xb + ((sizeof(double) * P2P_NSLOT * P + 255) & ~size_t(255));
+      h->off_flags = xb + ((sizeof(double) * P2P_NSLOT * P * P2P_PMAX + 255) & ~size_t(255));
       h->fab_bytes = h->off_flags + ((sizeof(unsigned long long) * P + 255) & ~size_t(255));
       okm = cudaMalloc(&h->fabric, h->fab_bytes) == cudaSuccess &&
             cudaMalloc(&h->p2p_local, sizeof(unsigned long long) * (P2P_NSLOT + 4)) == cudaSuccess &&
