@@ -592,22 +592,25 @@ k_xplan_pack(const int* __restrict__ rowptr, const int* __restrict__ colidx, con
 // per-row tolerance of BJ.ns bounds any summation order.  The kernel reorders
 // them so that the x gathers of one step (xs[col] in shared memory, 8-B words
 // for fp64 = bank pair col % 16 per half-warp, 4-B words for fp32 = bank
-// col % 32 per warp) hit distinct banks: greedy, step by step, each lane in
-// turn takes its first remaining nonzero whose bank is still free in this
-// step (else the least-loaded one).  Pads (column W, value 0) share one word.
-// One warp per chunk; deterministic (depends only on the columns and their
-// CSR order), so a values-only re-pack followed by this pass reproduces it.
+// col % 32 per warp) hit distinct banks.  Step by step, in up to BP_ROUNDS
+// rounds, every unplaced lane proposes its first remaining nonzero whose bank
+// is still free in this step; lanes proposing the same bank are resolved in
+// favour of the lowest lane (the others retry against the grown set of taken
+// banks); lanes left over keep their next entry.  Pads (column W, value 0)
+// share one word.  One warp per chunk; deterministic (it depends only on the
+// columns and their CSR order), so a values-only re-pack followed by this pass
+// reproduces it.
+constexpr int BP_ROUNDS = 4;
 template <typename T>
 __global__ void __launch_bounds__(256)
 k_xplan_bankperm(unsigned char* __restrict__ plan, const long long* __restrict__ chunk_off,
                  const int* __restrict__ chunk_len, int64_t nchunks, int W) {
-  constexpr int NG = sizeof(T) == 8 ? 16 : 32;  // conflict-free slots per lane group
-  constexpr int GL = NG;                        // lanes per group (half-warp for fp64)
-  __shared__ int cnt[8][32];
-  __shared__ int padf[8][2];
-  const int wib = threadIdx.x >> 5, lane = threadIdx.x & 31;
-  const int grp = lane / GL, gl = lane % GL;
-  for (int64_t c = int64_t(blockIdx.x) * 8 + wib; c < nchunks; c += int64_t(gridDim.x) * 8) {
+  constexpr int NG = sizeof(T) == 8 ? 16 : 32;  // conflict-free slots per lane group (half-warp for fp64)
+  const int lane = threadIdx.x & 31;
+  const int grp = lane / NG;
+  const uint32_t gshift = uint32_t(grp * NG);   // this group's bits in a warp-wide 32-bit mask
+  const int64_t warps = int64_t(gridDim.x) * (blockDim.x >> 5);
+  for (int64_t c = int64_t(blockIdx.x) * (blockDim.x >> 5) + (threadIdx.x >> 5); c < nchunks; c += warps) {
     const int len = chunk_len[c];
     if (len < 2) continue;
     unsigned char* base = plan + chunk_off[c];
@@ -615,23 +618,35 @@ k_xplan_bankperm(unsigned char* __restrict__ plan, const long long* __restrict__
     uint16_t* C = reinterpret_cast<uint16_t*>(base + size_t(len) * 32 * sizeof(T));
     auto at = [&](int st) { return (size_t(st >> 1) * 32 + lane) * 2 + (st & 1); };
     for (int st = 0; st < len - 1; ++st) {
-      cnt[wib][lane] = 0;
-      if (lane < 2) padf[wib][lane] = 0;
-      __syncwarp();
-      for (int i = 0; i < GL; ++i) {
-        if (gl == i) {
-          int best = st, bestc = 1 << 30;
+      uint32_t taken = 0;  // warp-wide: bit (grp*NG + slot)
+      uint32_t padded = 0;  // warp-wide: bit grp*NG set once a pad holds the group's pad slot
+      bool placed = false;
+#pragma unroll 1
+      for (int r = 0; r < BP_ROUNDS; ++r) {
+        int cand = -1, slot = 0;
+        bool pad = false;
+        if (!placed) {
           for (int e = st; e < len; ++e) {
             const int col = C[at(e)];
-            const int cost = (col == W && padf[wib][grp]) ? 0 : cnt[wib][grp * NG + col % NG];
-            if (cost < bestc) {
-              bestc = cost;
-              best = e;
-              if (cost == 0) break;
+            const int sl = col % NG;
+            const bool isp = col == W;
+            const bool free_ = !(taken & (1u << (gshift + sl))) || (isp && (padded & (1u << gshift)));
+            if (free_) {
+              cand = e;
+              slot = sl;
+              pad = isp;
+              break;
             }
           }
-          if (best != st) {
-            const size_t i0 = at(st), i1 = at(best);
+        }
+        // lowest lane per (group, slot) wins; pads of a group all win together
+        const bool want = cand >= 0;
+        const uint32_t key = want ? (pad ? 0x10000u + uint32_t(grp) : uint32_t(grp * 64 + slot)) : 0xffffffffu;
+        const uint32_t peers = __match_any_sync(0xffffffffu, key);
+        const bool win = want && (pad || (__ffs(peers) - 1) == lane);
+        if (win) {
+          if (cand != st) {
+            const size_t i0 = at(st), i1 = at(cand);
             const T tv = V[i0];
             V[i0] = V[i1];
             V[i1] = tv;
@@ -639,17 +654,11 @@ k_xplan_bankperm(unsigned char* __restrict__ plan, const long long* __restrict__
             C[i0] = C[i1];
             C[i1] = tc;
           }
-          const int col = C[at(st)];
-          if (col == W) {
-            if (!padf[wib][grp]) {
-              padf[wib][grp] = 1;
-              cnt[wib][grp * NG + col % NG] += 1;
-            }
-          } else {
-            cnt[wib][grp * NG + col % NG] += 1;
-          }
+          placed = true;
         }
-        __syncwarp();
+        taken |= __reduce_or_sync(0xffffffffu, win ? (1u << (gshift + slot)) : 0u);
+        padded |= __reduce_or_sync(0xffffffffu, (win && pad) ? (1u << gshift) : 0u);
+        if (__all_sync(0xffffffffu, placed)) break;
       }
     }
   }
