@@ -1,6 +1,6 @@
 # round-2 (second session) regression: GPU suite, smoke, bench x2, launch list, ncu captures, idiom rows
 cd $GRAFT_REPO_ROOT
-O=gpurun_out/r02z2; mkdir -p $O
+O=gpurun_out/${OUT:-r02z3}; mkdir -p $O
 timeout 3000 python -m pytest tests -m gpu -q > $O/pytest_gpu.log 2>&1; echo "rc=$?" >> $O/pytest_gpu.log
 timeout 600 python -c "import __graft_entry__ as g; g.smoke()" > $O/smoke.log 2>&1; echo "rc=$?" >> $O/smoke.log
 timeout 900 python bench.py --steps 20 --warmup 5 > $O/bench1.json 2> $O/bench1.err
