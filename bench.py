@@ -392,6 +392,10 @@ def run_ours(args):
             "cg_gbs_effective": round(value * (spmv_bytes + 10 * 8 * nl) / 1e9 * world, 1),
             "roofline": {"bound": "hbm", "achieved": round(achieved, 1), "peak": peak, "unit": "GB/s",
                          "frac": round(achieved / peak, 4), "traffic": traffic,
+                         # the kernel's own DRAM rate: ncu bytes per launch (the plan is smaller than
+                         # the CSR arrays) over the same launch time
+                         "achieved_dram": (round(traffic / (sp_avg / 1e3) / 1e9, 1) if traffic else None),
+                         "frac_dram": (round(traffic / (sp_avg / 1e3) / 1e9 / peak, 4) if traffic else None),
                          "peak_source": peak_src, "kernel": f"k_spmv_{info['kernel_name']}<double>",
                          "traffic_source": "profiles/spmv_traffic.json (ncu --set full, dram__bytes_read+write per launch)"},
             "e2e": {"value": round(e2e_val, 2), "unit": UNIT, "h2d_bytes_per_step": 8 * nl,
