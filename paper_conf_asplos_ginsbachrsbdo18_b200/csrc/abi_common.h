@@ -218,6 +218,12 @@ struct spmv_csr_s {
   // CG workspace (lazy)
   double *z = nullptr, *r = nullptr, *q = nullptr, *p_single = nullptr;
   double *s_vec = nullptr, *alpha2 = nullptr;  // single-reduction CG (NEXT-1): s = A p, alpha_{k-1}
+  // z, r, q, p_single, s_vec live in ONE allocation (cg_alloc), so one persisting-L2 window can keep
+  // the CG vectors resident while the plan streams through L2 (SPMV_CG_L2WIN)
+  unsigned char* cgws = nullptr;
+  size_t cgws_bytes = 0;
+  size_t cgwin_bytes = 0;
+  float cgwin_ratio = 0.f;
   int cg_variant = 0;                          // 0 textbook (NPB conj_grad), 1 Chronopoulos-Gear, 2 persistent C-G
   int pdl = 1;                                 // programmatic dependent launch of the SpMV / k_cgcg chain (SPMV_PDL=0: off)
   unsigned int* gbar = nullptr;                // persistent CG: grid barrier counter
@@ -254,20 +260,40 @@ inline bool tuning_env(const char* name, int* v) {
 // Launch with programmatic stream serialization (PDL) when `pdl`: the kernel may
 // start while its stream predecessor runs and synchronises with pdl_wait()
 // (common.cuh).  Without it, an ordinary launch.
+// `win` (nullable): a persisting access window carried by the launch.
 template <typename... KArgs, typename... Args>
 inline cudaError_t launch_maybe_pdl(void (*k)(KArgs...), dim3 grid, dim3 block, size_t smem, cudaStream_t s, bool pdl,
-                                    Args&&... args) {
+                                    const cudaAccessPolicyWindow* win, Args&&... args) {
   cudaLaunchConfig_t cfg = {};
   cfg.gridDim = grid;
   cfg.blockDim = block;
   cfg.dynamicSmemBytes = smem;
   cfg.stream = s;
-  cudaLaunchAttribute at[1];
-  at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
-  at[0].val.programmaticStreamSerializationAllowed = 1;
+  cudaLaunchAttribute at[2];
   cfg.attrs = at;
-  cfg.numAttrs = pdl ? 1 : 0;
+  cfg.numAttrs = 0;
+  if (pdl) {
+    at[cfg.numAttrs].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    at[cfg.numAttrs].val.programmaticStreamSerializationAllowed = 1;
+    ++cfg.numAttrs;
+  }
+  if (win) {
+    at[cfg.numAttrs].id = cudaLaunchAttributeAccessPolicyWindow;
+    at[cfg.numAttrs].val.accessPolicyWindow = *win;
+    ++cfg.numAttrs;
+  }
   return cudaLaunchKernelEx(&cfg, k, std::forward<Args>(args)...);
+}
+
+// The CG-vector window of a handle (nullptr when off).
+inline const cudaAccessPolicyWindow* cg_window(const spmv_csr_s* h, cudaAccessPolicyWindow* w) {
+  if (!h->cgwin_bytes) return nullptr;
+  w->base_ptr = h->cgws;
+  w->num_bytes = h->cgwin_bytes;
+  w->hitRatio = h->cgwin_ratio;
+  w->hitProp = cudaAccessPropertyPersisting;
+  w->missProp = cudaAccessPropertyStreaming;
+  return w;
 }
 
 inline int num_sms(int dev) {

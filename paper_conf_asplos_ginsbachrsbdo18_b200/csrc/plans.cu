@@ -229,6 +229,13 @@ static spmv_status launch_xplan(spmv_csr_s* h, cudaStream_t s, const void* x, vo
   at[1].val.programmaticStreamSerializationAllowed = 1;
   cfg.attrs = at;
   cfg.numAttrs = (h->pdl && !h->xp.dyn) ? 2 : 1;
+  cudaAccessPolicyWindow cwv;
+  if (!h->xp.win_bytes && cg_window(h, &cwv) && (y == h->q || x == (const void*)h->p_single || x == (const void*)h->r)) {
+    // a CG SpMV on a plan without its own window: the CG vectors' window (SPMV_CG_L2WIN)
+    at[cfg.numAttrs].id = cudaLaunchAttributeAccessPolicyWindow;
+    at[cfg.numAttrs].val.accessPolicyWindow = cwv;
+    ++cfg.numAttrs;
+  }
   if (h->xp.win_bytes) {
     at[cfg.numAttrs].id = cudaLaunchAttributeAccessPolicyWindow;
     at[cfg.numAttrs].val.accessPolicyWindow.base_ptr = h->xp.plan;
@@ -928,6 +935,13 @@ spmv_status launch_cg_persist(spmv_csr_s* h, cudaStream_t s, const void* x_input
     at[1].val.accessPolicyWindow.hitProp = cudaAccessPropertyPersisting;
     at[1].val.accessPolicyWindow.missProp = cudaAccessPropertyStreaming;
     cfg.numAttrs = 2;
+  } else {
+    cudaAccessPolicyWindow cwv;  // no plan window: the CG vectors' (see cg_alloc)
+    if (cg_window(h, &cwv)) {
+      at[1].id = cudaLaunchAttributeAccessPolicyWindow;
+      at[1].val.accessPolicyWindow = cwv;
+      cfg.numAttrs = 2;
+    }
   }
   int times = 0;
   if (tuning_env("SPMV_PERSIST_TIMES", &times) && times) {

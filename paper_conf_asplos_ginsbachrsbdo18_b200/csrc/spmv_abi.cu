@@ -363,12 +363,12 @@ extern "C" spmv_status spmv_csr_destroy(spmv_csr_t h) {
   }
   void* bufs[] = {h->p2p_local, h->peer_table, h->mg.split_row, h->mg.split_nz, h->mg.head, h->mg.carry, h->mg.head_flag, h->xp.crow, h->xp.chunk_off, h->xp.tile0, h->xp.chunk_len, h->xp.seg, h->xp.row_slot,
                   h->xp.chunk_row, h->xp.plan, h->xp.tq, h->xp.cta_range, h->sl.pair_off, h->sl.vals, h->sl.cols, h->sl.perm, h->sl.seg, h->sl.seg_part, h->sl.seg_cnt,
-                  h->seg, h->crow, h->ci_own, h->send_iv, h->xpad, h->z, h->r, h->q, h->p_single, h->part_pq, h->part_rr,
-                  h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags, h->s_vec, h->alpha2,
+                  h->seg, h->crow, h->ci_own, h->send_iv, h->xpad, h->cgws, h->part_pq, h->part_rr,
+                  h->part_res, h->part_xz, h->part_zz, h->scal, h->out2, h->flags, h->alpha2,
                   h->stage_x, h->stage_z, h->gbar};
   // lines pinned by a persisting window over the plan go back to normal (device-wide; other
   // handles' windows re-pin theirs on their next launch)
-  if (h->xp.win_bytes) cudaCtxResetPersistingL2Cache();
+  if (h->xp.win_bytes || h->cgwin_bytes) cudaCtxResetPersistingL2Cache();
   for (void* b : bufs)
     if (b) cudaFree(b);
   if (h->cap) cudaStreamDestroy(h->cap);
