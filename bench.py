@@ -249,9 +249,9 @@ def run_ours(args):
     zeta_last = float(out2[0].item())
     value = 25.0 * args.steps / (t_ms / 1e3)
 
-    # the other CG variants (NEXT-1: single reduction, persistent, fused), same protocol, reported beside the headline
+    # the other CG variants (NEXT-1: single reduction, persistent), same protocol, reported beside the headline
     variants = {args.cg_variant: round(value, 2)}
-    for other in [v for v in ("textbook", "cgcg", "persist", "fused") if v != args.cg_variant]:
+    for other in [v for v in ("textbook", "cgcg", "persist") if v != args.cg_variant]:
         M.set_cg_variant(other)
         x.fill_(1.0)
         for _ in range(args.warmup):
@@ -513,11 +513,10 @@ def main():
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
     ap.add_argument("--no-cpu", action="store_true", help="skip the cpu_baseline leg")
     ap.add_argument("--cpu-budget", type=float, default=15.0)
-    ap.add_argument("--cg-variant", choices=["textbook", "cgcg", "persist", "fused"],
+    ap.add_argument("--cg-variant", choices=["textbook", "cgcg", "persist"],
                     default=os.environ.get("SPMV_CG_VARIANT", "cgcg"),
-                    help="CG inside the NAS step: textbook (NPB conj_grad), cgcg (single reduction), "
-                         "persist (single reduction, one persistent kernel per CG solve) or fused "
-                         "(single reduction, the update folded into the next SpMV)")
+                    help="CG inside the NAS step: textbook (NPB conj_grad), cgcg (single reduction) or "
+                         "persist (single reduction, one persistent kernel per CG solve)")
     args = ap.parse_args()
     if args.warmup < 3:
         log("warmup < 3 is not allowed by the timing rules; using 3")

@@ -325,12 +325,11 @@ class CSRMatrix:
         if cg_variant != "textbook":
             self.set_cg_variant(cg_variant)
 
-    CG_VARIANTS = {"textbook": 0, "cgcg": 1, "persist": 2, "fused": 3}
+    CG_VARIANTS = {"textbook": 0, "cgcg": 1, "persist": 2}
 
     def set_cg_variant(self, variant: str):
-        """'textbook' (NPB conj_grad), 'cgcg' (single-reduction Chronopoulos-Gear), 'persist'
-        (the single-reduction CG as one persistent kernel per solve, NEXT-1) or 'fused' (the
-        update folded into the next SpMV: one kernel per iteration)."""
+        """'textbook' (NPB conj_grad), 'cgcg' (single-reduction Chronopoulos-Gear) or 'persist'
+        (the single-reduction CG as one persistent kernel per solve, NEXT-1)."""
         _check(spmv_csr_set_cg_variant_c(self.handle, self.CG_VARIANTS[variant]), "spmv_csr_set_cg_variant")
         self.cg_variant = variant
 

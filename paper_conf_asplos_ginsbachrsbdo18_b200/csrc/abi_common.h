@@ -144,7 +144,6 @@ struct spmv_csr_s {
     unsigned char* plan = nullptr;
     void (*k)(XplanArgs) = nullptr;
     void (*kdot)(XplanArgs) = nullptr;
-    void (*kfused)(XplanArgs) = nullptr;  // cg variant 3 (FUSED instantiation; fp64, static tiles)
     // side split (SPMV_XPLAN_SIDE): rows [mplan, m) run concurrently in the
     // vector kernel on the SMs the clusters leave idle
     int64_t mplan = -1;
@@ -221,8 +220,6 @@ struct spmv_csr_s {
   double *s_vec = nullptr, *alpha2 = nullptr;  // single-reduction CG (NEXT-1): s = A p, alpha_{k-1}
   // z, r, q, p_single, s_vec live in ONE allocation (cg_alloc), so one persisting-L2 window can keep
   // the CG vectors resident while the plan streams through L2 (SPMV_CG_L2WIN)
-  double *r2 = nullptr, *s2 = nullptr, *w2 = nullptr;  // cg variant 3: the second buffers of r, s, w
-  double* part_fu = nullptr;                          // cg variant 3: delta [2][pb], gamma [3][pb] partials
   unsigned char* cgws = nullptr;
   size_t cgws_bytes = 0;
   size_t cgwin_bytes = 0;
@@ -355,11 +352,6 @@ inline spmv_status ensure_buf(void** p, size_t bytes) {
 spmv_status xstat_setup(spmv_csr_s* h, bool* ok);
 spmv_status xplan_build(spmv_csr_s* h, bool* ok);
 spmv_status xplan_pack(spmv_csr_s* h, const void* vals, int values_only);
-namespace spmv { struct FusedArgs; }
-spmv_status launch_xplan_fused(spmv_csr_s* h, cudaStream_t s, const spmv::FusedArgs& fu, double* w_out,
-                               double* part_del);
-spmv_status launch_cg_fused_tail(spmv_csr_s* h, cudaStream_t s, const spmv::FusedArgs& fu);
-bool fused_eligible(const spmv_csr_s* h);
 spmv_status sell_build(spmv_csr_s* h, double max_pad, int sorted, bool* ok);
 spmv_status sell_pack(spmv_csr_s* h, const void* vals, int values_only);
 spmv_status merge_setup(spmv_csr_s* h);

@@ -5,7 +5,6 @@
 // dist.cu.
 #include "abi_common.h"
 #include "cg_kernels.cuh"
-#include "xplan_kernel.cuh"  // FusedArgs (cg variant 3)
 
 // ------------------------------------------------------------------ CG
 static spmv_status cg_alloc(spmv_csr_s* h) {
@@ -15,18 +14,13 @@ static spmv_status cg_alloc(spmv_csr_s* h) {
   {
     // z | r | q | s | p_single: one allocation (see cgws in abi_common.h)
     const size_t nba = (nb + 255) & ~size_t(255);
-    h->cgws_bytes = nba * (h->dist ? 4 : 8);
+    h->cgws_bytes = nba * (h->dist ? 4 : 5);
     CK(cudaMalloc(&h->cgws, h->cgws_bytes));
     h->z = reinterpret_cast<double*>(h->cgws);
     h->r = reinterpret_cast<double*>(h->cgws + nba);
     h->q = reinterpret_cast<double*>(h->cgws + 2 * nba);
     h->s_vec = reinterpret_cast<double*>(h->cgws + 3 * nba);
-    if (!h->dist) {
-      h->p_single = reinterpret_cast<double*>(h->cgws + 4 * nba);
-      h->r2 = reinterpret_cast<double*>(h->cgws + 5 * nba);
-      h->s2 = reinterpret_cast<double*>(h->cgws + 6 * nba);
-      h->w2 = reinterpret_cast<double*>(h->cgws + 7 * nba);
-    }
+    if (!h->dist) h->p_single = reinterpret_cast<double*>(h->cgws + 4 * nba);
     // a persisting-L2 window over the CG vectors on every CG launch, so the plan's stream (larger
     // than L2) does not evict them between the update and the SpMV (SPMV_CG_L2WIN=0: off).
     // Measured, class C (profiles/r02ae_*): 12,956 / 12,961 -> 13,055 / 13,048 CG it/s
@@ -48,7 +42,6 @@ static spmv_status cg_alloc(spmv_csr_s* h) {
     }
   }
   ST(ensure_buf((void**)&h->part_pq, pb));
-  if (!h->dist) ST(ensure_buf((void**)&h->part_fu, 5 * pb));
   // [0],[1]: parity slots; [2]: ||b||^2 (init); [3..5]: rotating r.r of the single-reduction CG
   ST(ensure_buf((void**)&h->part_rr, 6 * pb));
   ST(ensure_buf((void**)&h->alpha2, sizeof(double) * 2));
@@ -111,42 +104,6 @@ static spmv_status cg_enqueue_iters(spmv_csr_s* h, cudaStream_t s, double* z, in
   if (p2p) {
     base.c = p2p_ctx(h);
     base.enabled = 1;
-  }
-  if (h->cg_variant == 3 && tol == 0.0 && iters > 0 && run->it == 0 && fused_eligible(h)) {
-    // cg variant 3: iteration 0 is the plain fused-dot SpMV w_0 = A r_0;
-    // iteration k >= 1 is ONE kernel (k_spmv_xplan<FUSED>) that applies the update of k-1
-    // while it builds its x block and finalizes its rows; a tail kernel applies the last one
-    const int64_t G = (int64_t)h->xp.ncl * h->xp.B;
-    double* R[2] = {cg_p(h), h->r2};  // r_0 = b (k_cg_init)
-    double* S[2] = {h->s_vec, h->s2};
-    double* Wv[2] = {h->q, h->w2};
-    double* P = h->r;                  // k_cg_init's p (unused at k = 0)
-    double* pd[2] = {h->part_fu, h->part_fu + pstride};
-    double* pg[3] = {h->part_fu + 2 * pstride, h->part_fu + 3 * pstride, h->part_fu + 4 * pstride};
-    ST(run_spmv(h, s, h->vals, R[0], Wv[0], 1.0, 0.0, R[0], pd[0]));
-    auto gam_src = [&](int j) { return j == 0 ? run->rr_b : SumSrc{pg[j % 3], (int)G}; };  // gamma_j
-    FusedArgs fu;
-    fu.flags = h->flags;
-    for (int k = 1; k <= iters; ++k) {
-      fu.k = k;
-      fu.r_prev = R[(k - 1) & 1];
-      fu.w_prev = Wv[(k - 1) & 1];
-      fu.s_prev2 = S[k & 1];
-      fu.r_out = R[k & 1];
-      fu.s_out = S[(k - 1) & 1];
-      fu.p = P;
-      fu.z = z;
-      fu.gam = gam_src(k - 1);
-      fu.del = SumSrc{pd[(k - 1) & 1], (int)G};
-      fu.gam_old = k >= 2 ? gam_src(k - 2) : gam_src(0);
-      fu.alpha_old = h->alpha2 + ((k - 2) & 1);
-      fu.alpha_store = h->alpha2 + ((k - 1) & 1);
-      fu.part_gam = pg[k % 3];
-      if (k < iters) ST(launch_xplan_fused(h, s, fu, Wv[k & 1], pd[k & 1]));
-      else ST(launch_cg_fused_tail(h, s, fu));
-    }
-    run->it += iters;
-    return SPMV_OK;
   }
   if (h->cg_variant == 2 && tol == 0.0 && iters > 0 && persist_eligible(h)) {
     // NEXT-1: the persistent single-reduction CG -- all `iters` iterations in ONE
@@ -416,8 +373,8 @@ extern "C" spmv_status cg_npb_outer(spmv_csr_t h, void* x, void* z, int32_t cgit
 
 extern "C" spmv_status spmv_csr_set_cg_variant(spmv_csr_t h, int32_t variant) {
   if (!h) return arg_fail("handle is NULL");
-  if (variant < 0 || variant > 3)
-    return arg_fail("variant must be 0 (textbook), 1 (single reduction), 2 (persistent single reduction) or 3 (fused single reduction)");
+  if (variant < 0 || variant > 2)
+    return arg_fail("variant must be 0 (textbook), 1 (single reduction) or 2 (persistent single reduction)");
   if (h->cg_variant != variant) {
     h->cg_variant = variant;
     h->g_npb.reset();  // the captured NPB graph belongs to the other variant

@@ -428,11 +428,6 @@ spmv_status xplan_build(spmv_csr_s* h, bool* ok) {
     P = spmv_csr_s::XPlan();
   };
   P.B = B; P.W = W; P.ncl = ncl; P.smem = smem; P.k = fn; P.kdot = fnd; P.dyn = dyn;
-  if (h->dt == SPMV_F64 && !dyn) {
-    P.kfused = k_spmv_xplan<double, true, false, true>;
-    CK(cudaFuncSetAttribute(P.kfused, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
-    if (B > 8) CK(cudaFuncSetAttribute(P.kfused, cudaFuncAttributeNonPortableClusterSizeAllowed, 1));
-  }
   // DYN: the plan is one row range cut into tiles the clusters pop at run time
   const int ncl_plan = dyn ? 1 : ncl;
   DBG("B=%d W=%d ncl=%d smem=%zu", B, W, ncl, smem);
@@ -975,58 +970,5 @@ spmv_status launch_cg_persist(spmv_csr_s* h, cudaStream_t s, const void* x_input
       fprintf(stderr, "  %-12s med %7.2f  min %7.2f  max %7.2f\n", nm[ph], v[G / 2], v[0], v[G - 1]);
     }
   }
-  return SPMV_OK;
-}
-
-// ------------------------------------------------------------ cg variant 3
-bool fused_eligible(const spmv_csr_s* h) {
-  if (h->kernel != SPMV_KERNEL_XPLAN || !h->xp.built || !h->xp.kfused || h->xp.dyn || h->dt != SPMV_F64) return false;
-  if (h->xp.mplan >= 0 && h->xp.mplan < h->m_loc) return false;  // side split
-  return !h->dist;  // the x block is the whole local r: one GPU
-}
-
-spmv_status launch_xplan_fused(spmv_csr_s* h, cudaStream_t s, const FusedArgs& fu, double* w_out, double* part_del) {
-  XplanArgs a = xplan_args(h, fu.r_prev, w_out, 1.0, 0.0, nullptr, part_del, P2PHook());
-  a.fu = fu;
-  cudaLaunchConfig_t cfg = {};
-  cfg.gridDim = dim3((unsigned)(h->xp.ncl * h->xp.B), 1, 1);
-  cfg.blockDim = dim3(XP_THREADS, 1, 1);
-  cfg.dynamicSmemBytes = h->xp.smem;
-  cfg.stream = s;
-  cudaLaunchAttribute at[3];
-  at[0].id = cudaLaunchAttributeClusterDimension;
-  at[0].val.clusterDim.x = (unsigned)h->xp.B;
-  at[0].val.clusterDim.y = 1;
-  at[0].val.clusterDim.z = 1;
-  cfg.attrs = at;
-  cfg.numAttrs = 1;
-  if (h->pdl) {
-    at[cfg.numAttrs].id = cudaLaunchAttributeProgrammaticStreamSerialization;
-    at[cfg.numAttrs].val.programmaticStreamSerializationAllowed = 1;
-    ++cfg.numAttrs;
-  }
-  cudaAccessPolicyWindow w = {};
-  if (h->xp.win_bytes) {
-    w.base_ptr = h->xp.plan;
-    w.num_bytes = h->xp.win_bytes;
-    w.hitRatio = h->xp.win_ratio;
-    w.hitProp = cudaAccessPropertyPersisting;
-    w.missProp = cudaAccessPropertyStreaming;
-  }
-  if (h->xp.win_bytes || cg_window(h, &w)) {
-    at[cfg.numAttrs].id = cudaLaunchAttributeAccessPolicyWindow;
-    at[cfg.numAttrs].val.accessPolicyWindow = w;
-    ++cfg.numAttrs;
-  }
-  CK(cudaLaunchKernelEx(&cfg, h->xp.kfused, a));
-  LAUNCHED();
-  return SPMV_OK;
-}
-
-spmv_status launch_cg_fused_tail(spmv_csr_s* h, cudaStream_t s, const FusedArgs& fu) {
-  cudaAccessPolicyWindow cwv;
-  CK(launch_maybe_pdl(k_cg_fused_tail, dim3((unsigned)h->vgrid), dim3(256), 0, s, h->pdl != 0, cg_window(h, &cwv),
-                      h->m_loc, fu));
-  LAUNCHED();
   return SPMV_OK;
 }

@@ -57,48 +57,6 @@ constexpr int XP_U = XP_U_DEF;       // step pairs (16-B loads) in flight per la
 #define XP_ODD 0  // 1: odd chunk lengths (no even-rounding padding: measured 87.0 vs 78.9 us on C); 0: even
 #endif
 
-// FUSED (cg variant 3): the single-reduction CG update of
-// iteration k-1 folded into the SpMV of iteration k.  Every CTA derives
-// alpha_{k-1}, beta_{k-1} from the previous launch's partials, builds its x
-// block r_k = r_{k-1} - alpha s_{k-1}, s_{k-1} = w_{k-1} + beta s_{k-2} on the
-// fly, and the owners of the rows write r_k, s_{k-1}, p_{k-1}, z and w_k = A r_k
-// and take the partials of delta_k = w_k.r_k and gamma_k = r_k.r_k.
-struct FusedArgs {
-  int k = 0;                        // iteration (>= 1)
-  const double* r_prev = nullptr;   // r_{k-1}
-  const double* w_prev = nullptr;   // w_{k-1} = A r_{k-1}
-  const double* s_prev2 = nullptr;  // s_{k-2}
-  double* r_out = nullptr;          // r_k
-  double* s_out = nullptr;          // s_{k-1}
-  double* p = nullptr;              // p_{k-2} -> p_{k-1} (owned rows)
-  double* z = nullptr;              // z += alpha_{k-1} p_{k-1}
-  SumSrc gam, del, gam_old;         // gamma_{k-1}, delta_{k-1}, gamma_{k-2}
-  const double* alpha_old = nullptr;  // alpha_{k-2} (k >= 2)
-  double* alpha_store = nullptr;    // alpha_{k-1} (written by CTA 0)
-  int* flags = nullptr;             // [0] breakdown, [2] iterations done
-  double* part_gam = nullptr;       // gamma_k partial per CTA
-};
-
-// alpha_{k-1}, beta_{k-1} of the single-reduction CG (the k_cgcg formulas).
-__device__ __forceinline__ void fused_scalars(int k, double g, double d, double g_old, double a_old, double* alpha,
-                                              double* beta, double* pap) {
-  double b = 0.0, pp = d;
-  if (k - 1 > 0) {
-    b = g / g_old;
-    pp = d - b * g / a_old;
-  }
-  *beta = b;
-  *pap = pp;
-  *alpha = g / pp;
-}
-// s_{k-1} and r_k of one row: the same instructions wherever they are evaluated
-// (the x block of every cluster and the row's owner agree bit for bit).
-__device__ __forceinline__ void fused_rs(bool first, double alpha, double beta, double r, double w, double s2,
-                                         double* s1, double* rk) {
-  *s1 = first ? w : __fma_rn(beta, s2, w);
-  *rk = __fma_rn(-alpha, *s1, r);
-}
-
 struct XplanArgs {
   int64_t nx;                  // length of x
   int W;                       // column block width (pad column = W)
@@ -126,7 +84,6 @@ struct XplanArgs {
   int* tq;
   int* tq_done;
   int ntiles_total;
-  FusedArgs fu;                // FUSED instantiation only
 };
 
 // Arguments of the persistent CG kernel (persist_kernel.cuh, NEXT-1).
@@ -260,10 +217,9 @@ __device__ __forceinline__ double xplan_chunk_dot(const unsigned char* base, int
 //   recv[t%K][b*(R/B) + jl]: partial of CTA b for owned row jl
 constexpr int XP_TQ = 8;  // DYN: tile-id ring (local tile k in slot k % 8)
 
-template <typename T, bool DOT, bool DYN, bool FUSED = false>
+template <typename T, bool DOT, bool DYN>
 __global__ void __launch_bounds__(XP_THREADS, 1)
 k_spmv_xplan(XplanArgs a) {
-  static_assert(!FUSED || (DOT && !DYN && sizeof(T) == 8), "FUSED: fp64, fused dot, static tiles");
   extern __shared__ __align__(128) unsigned char smem[];
   __shared__ uint64_t xbar, tbar[XP_K];
   __shared__ uint64_t qbar[XP_TQ];
@@ -328,47 +284,12 @@ k_spmv_xplan(XplanArgs a) {
   pdl_wait();               // x (and w, y) of the predecessor kernel
   pdl_trigger();
   p2p_prologue_wait(a.hk);  // x slices of the peers (p2p transport)
-  double f_alpha = 0.0, f_beta = 0.0;  // FUSED: alpha_{k-1}, beta_{k-1}
-  if constexpr (FUSED) {
-    __shared__ double fsc[4];
-    {
-      const int wid = threadIdx.x >> 5;
-      double v = 0.0;
-      if (wid == 0) v = warp_read_sum(a.fu.gam);
-      else if (wid == 1) v = warp_read_sum(a.fu.del);
-      else if (wid == 2 && a.fu.k >= 2) v = warp_read_sum(a.fu.gam_old);
-      else if (wid == 3 && a.fu.k >= 2) v = __ldcg(a.fu.alpha_old);
-      if (wid < 4 && lane == 0) fsc[wid] = v;
-      __syncthreads();
-    }
-    double pap;
-    fused_scalars(a.fu.k, fsc[0], fsc[1], fsc[2], fsc[3], &f_alpha, &f_beta, &pap);
-    if (blockIdx.x == 0 && threadIdx.x == 0) {
-      if (pap == 0.0 || !isfinite(pap)) a.fu.flags[0] = 1;
-      *a.fu.alpha_store = f_alpha;
-      a.fu.flags[2] = a.fu.k;
-    }
-    // the x block r_k[col0 .. col0 + ncols), computed from r_{k-1}, w_{k-1}, s_{k-2}
-    if (threadIdx.x == 0) mbar_expect_tx(&xbar, 0);
-    const bool first = a.fu.k == 1;
-    for (int64_t j = threadIdx.x; j <= W; j += blockDim.x) {
-      double v = 0.0;
-      if (j < ncols) {
-        const int64_t gi = col0 + j;
-        double s1;
-        fused_rs(first, f_alpha, f_beta, __ldcg(a.fu.r_prev + gi), __ldcg(a.fu.w_prev + gi),
-                 first ? 0.0 : __ldcg(a.fu.s_prev2 + gi), &s1, &v);
-      }
-      xs[j] = T(v);
-    }
-  } else {
-    if (threadIdx.x == 0) {
-      const uint32_t xb = uint32_t(bulk_elems * sizeof(T));
-      mbar_expect_tx(&xbar, xb);
-      if (xb) bulk_g2s(xs, xg + col0, xb, &xbar);
-    }
-    for (int64_t j = bulk_elems + threadIdx.x; j <= W; j += blockDim.x) xs[j] = (j < ncols) ? xg[col0 + j] : T(0);
+  if (threadIdx.x == 0) {
+    const uint32_t xb = uint32_t(bulk_elems * sizeof(T));
+    mbar_expect_tx(&xbar, xb);
+    if (xb) bulk_g2s(xs, xg + col0, xb, &xbar);
   }
+  for (int64_t j = bulk_elems + threadIdx.x; j <= W; j += blockDim.x) xs[j] = (j < ncols) ? xg[col0 + j] : T(0);
   // peers must have initialised their barriers before partials are sent
   cluster_arrive();
   cluster_wait();
@@ -412,7 +333,6 @@ k_spmv_xplan(XplanArgs a) {
 
   const double alpha = a.alpha, beta = a.beta;
   double dacc = 0.0;
-  double gacc = 0.0;  // FUSED: gamma_k partial
 
   // t: tile index (relative to tbase), k: local sequence number (receive slot k % K)
   auto process_chunk = [&](int t, int k, int ch) {
@@ -461,29 +381,10 @@ k_spmv_xplan(XplanArgs a) {
     const int jl0 = threadIdx.x;
     const bool has0 = jl0 < RB && b * RB + jl0 < nrows;
     double w0 = 0.0, y0 = 0.0;
-    if (has0 && !FUSED) {
+    if (has0) {
       const int64_t i0 = rt + b * RB + jl0;
       if (DOT) w0 = double(static_cast<const T*>(a.w)[i0]);
       if (beta != 0.0) y0 = double(static_cast<const T*>(a.y)[i0]);
-    }
-    if constexpr (FUSED) {
-      // the CG update of the owned rows does not depend on this tile's partials:
-      // done before the wait (its loads overlap the cluster's streaming)
-      const bool first = a.fu.k == 1;
-      for (int jl = threadIdx.x; jl < RB && b * RB + jl < nrows; jl += nfin) {
-        const int64_t i = rt + b * RB + jl;
-        const double r1 = __ldcg(a.fu.r_prev + i), w1 = __ldcg(a.fu.w_prev + i);
-        const double s2 = first ? 0.0 : __ldcg(a.fu.s_prev2 + i), p2 = first ? 0.0 : a.fu.p[i];
-        const double z1 = a.fu.z[i];
-        double s1, rk;
-        fused_rs(first, f_alpha, f_beta, r1, w1, s2, &s1, &rk);
-        const double p1 = first ? r1 : __fma_rn(f_beta, p2, r1);
-        a.fu.s_out[i] = s1;
-        a.fu.r_out[i] = rk;
-        a.fu.p[i] = p1;
-        a.fu.z[i] = __fma_rn(f_alpha, p1, z1);
-        gacc = __fma_rn(rk, rk, gacc);
-      }
     }
     mbar_wait(&tbar[k % XP_K], (k / XP_K) & 1, 1000000 * ntiles + 1000 * t + int(recv_bytes(t) / 8));
     double tacc = 0.0;  // DYN: this tile's share of the fused dot
@@ -492,12 +393,6 @@ k_spmv_xplan(XplanArgs a) {
       for (int q = 0; q < B; ++q) sum += rv[q * RB + jl];
       const int64_t i = rt + b * RB + jl;
       T* y = static_cast<T*>(a.y);
-      if constexpr (FUSED) {
-        // w_k = A r_k (alpha 1, beta 0) and delta_k = w_k.r_k with the r_k just written by this thread
-        y[i] = T(sum);
-        dacc += sum * a.fu.r_out[i];
-        continue;
-      }
       const bool first = jl == jl0;
       double r = alpha * sum;
       if (beta != 0.0) r += beta * (first ? y0 : double(y[i]));
@@ -561,10 +456,6 @@ k_spmv_xplan(XplanArgs a) {
     const double tsum = block_sum(dacc, red);
     if (threadIdx.x == 0) a.part[blockIdx.x] = tsum;
   }
-  if constexpr (FUSED) {
-    const double gsum = block_sum(gacc, red);
-    if (threadIdx.x == 0) a.fu.part_gam[blockIdx.x] = gsum;
-  }
   // leave together (peers may still be sending to / reading this CTA)
   cluster_arrive();
   cluster_wait();
@@ -579,39 +470,6 @@ k_spmv_xplan(XplanArgs a) {
     }
   }
   if (DOT) p2p_push_partials_last(a.hk, a.part, DYN ? ntiles * B : int(gridDim.x));
-}
-
-// The last update of a fused solve (cg variant 3): alpha_{K-1}, beta_{K-1}
-// from the last launch's partials, p_{K-1} = r_{K-1} + beta p_{K-2}, z += alpha p.
-static __global__ void __launch_bounds__(256)
-k_cg_fused_tail(int64_t n, FusedArgs fu) {
-  __shared__ double sc[4];
-  pdl_wait();
-  pdl_trigger();
-  {
-    const int wid = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    double v = 0.0;
-    if (wid == 0) v = warp_read_sum(fu.gam);
-    else if (wid == 1) v = warp_read_sum(fu.del);
-    else if (wid == 2 && fu.k >= 2) v = warp_read_sum(fu.gam_old);
-    else if (wid == 3 && fu.k >= 2) v = __ldcg(fu.alpha_old);
-    if (wid < 4 && lane == 0) sc[wid] = v;
-    __syncthreads();
-  }
-  double alpha, beta, pap;
-  fused_scalars(fu.k, sc[0], sc[1], sc[2], sc[3], &alpha, &beta, &pap);
-  if (blockIdx.x == 0 && threadIdx.x == 0) {
-    if (pap == 0.0 || !isfinite(pap)) fu.flags[0] = 1;
-    *fu.alpha_store = alpha;
-    fu.flags[2] = fu.k;
-  }
-  const bool first = fu.k == 1;
-  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n; j += int64_t(gridDim.x) * blockDim.x) {
-    const double r1 = fu.r_prev[j];
-    const double p1 = first ? r1 : __fma_rn(beta, fu.p[j], r1);
-    fu.p[j] = p1;
-    fu.z[j] = __fma_rn(alpha, p1, fu.z[j]);
-  }
 }
 
 // ---------------------------------------------------------------- builders
