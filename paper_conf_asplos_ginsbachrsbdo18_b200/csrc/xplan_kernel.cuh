@@ -601,6 +601,7 @@ k_xplan_pack(const int* __restrict__ rowptr, const int* __restrict__ colidx, con
 // columns and their CSR order), so a values-only re-pack followed by this pass
 // reproduces it.
 constexpr int BP_ROUNDS = 4;
+constexpr int BP_MAXLEN = 512;  // longer chunks keep CSR order (the pass is quadratic in the chunk length)
 template <typename T>
 __global__ void __launch_bounds__(256)
 k_xplan_bankperm(unsigned char* __restrict__ plan, const long long* __restrict__ chunk_off,
@@ -612,7 +613,7 @@ k_xplan_bankperm(unsigned char* __restrict__ plan, const long long* __restrict__
   const int64_t warps = int64_t(gridDim.x) * (blockDim.x >> 5);
   for (int64_t c = int64_t(blockIdx.x) * (blockDim.x >> 5) + (threadIdx.x >> 5); c < nchunks; c += warps) {
     const int len = chunk_len[c];
-    if (len < 2) continue;
+    if (len < 2 || len > BP_MAXLEN) continue;
     unsigned char* base = plan + chunk_off[c];
     T* V = reinterpret_cast<T*>(base);
     uint16_t* C = reinterpret_cast<uint16_t*>(base + size_t(len) * 32 * sizeof(T));
