@@ -286,10 +286,12 @@ k_cgcg(int64_t n, int k, SumSrc gam, SumSrc gam_old, SumSrc del, double* __restr
   }
   const double t = block_sum(acc, red);
   if (threadIdx.x == 0) part_rr_new[blockIdx.x] = t;
-  p2p_push_partials_last(hk, part_rr_new, gridDim.x);
-  if (hk.enabled) {
-    // publication of x uses its own ticket (the next u64 slot): the partials
-    // push above re-arms hk.c.ticket while other CTAs may already be here
+  if (hk.enabled && hk.push_slot >= 0) {
+    // one ticket publishes both the r.r partials and this rank's x slice (the
+    // peer stores above precede every CTA's ticket like the partials do)
+    p2p_push_partials_last(hk, part_rr_new, gridDim.x, P2P_XSLOT);
+  } else if (hk.enabled) {
+    // x only: its own ticket (the next u64 slot)
     int* tk2 = hk.c.ticket + 2;
     __syncthreads();
     if (threadIdx.x == 0 && ticket_acq_rel_gpu(tk2) == int(gridDim.x) - 1) {

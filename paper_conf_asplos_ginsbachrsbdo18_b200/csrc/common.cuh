@@ -140,10 +140,11 @@ __device__ __forceinline__ bool p2p_sends(const P2PCtx& c, int q, int64_t j) {
 // thread made or acquired (the other CTAs' stores, through their acq_rel GPU
 // tickets) before the flag -- no separate fence; with one rank nothing is
 // stored and nothing is fenced.
-__device__ __forceinline__ void p2p_signal(const P2PCtx& c, int slot) {
-  const unsigned long long e = *c.epoch + 1;
-  *c.epoch = e;
+__device__ __forceinline__ void p2p_signal(const P2PCtx& c, int slot, int slot2 = -1) {
+  unsigned long long e = *c.epoch + 1;
   c.slot_epoch[slot] = e;
+  if (slot2 >= 0) c.slot_epoch[slot2] = ++e;  // a second slot in the same publication
+  *c.epoch = e;
   for (int q = 0; q < c.P; ++q) {
     if (q == c.me) continue;
     unsigned long long* f = reinterpret_cast<unsigned long long*>(c.peer[q] + c.off_flags);
@@ -191,7 +192,10 @@ __device__ __forceinline__ void p2p_prologue_wait(const P2PHook& h) {
 }
 
 // Call from every thread of every CTA after part[blockIdx.x] was written.
-__device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const double* part, int count) {
+// also_slot >= 0: the last CTA publishes that slot too (its data written before
+// every CTA's ticket), with one flag store per peer.
+__device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const double* part, int count,
+                                                       int also_slot = -1) {
   if (!h.enabled || h.push_slot < 0) return;
   __shared__ int s_last;
   const bool per_cta = h.push_per == int(gridDim.x) && count == int(gridDim.x);
@@ -216,7 +220,7 @@ __device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const d
   if (per_cta) {
     if (threadIdx.x == 0) {
       *h.c.ticket = 0;
-      p2p_signal(h.c, h.push_slot);
+      p2p_signal(h.c, h.push_slot, also_slot);
     }
     return;
   }
@@ -231,7 +235,7 @@ __device__ __forceinline__ void p2p_push_partials_last(const P2PHook& h, const d
         double* ex = reinterpret_cast<double*>(h.c.peer[q] + h.c.off_exch);
         ex[(size_t(h.push_slot) * h.c.P + h.c.me) * P2P_PMAX] = a;
       }
-      p2p_signal(h.c, h.push_slot);
+      p2p_signal(h.c, h.push_slot, also_slot);
     }
   }
 }
