@@ -277,19 +277,32 @@ static spmv_status npb_enqueue(spmv_csr_s* h, cudaStream_t s, double* x, double*
   CgRun run;
   ST(cg_enqueue_init(h, s, x, z, &run));
   ST(cg_enqueue_iters(h, s, z, cgitmax, 0.0, &run));
-  // z is final here: an external event lets the host copy of z overlap the residual
+  // z is final here: an external event lets the host copy of z overlap the rest
   cudaStreamCaptureStatus cst = cudaStreamCaptureStatusNone;
   CK(cudaStreamIsCapturing(s, &cst));
-  if (cst == cudaStreamCaptureStatusActive) CK(cudaEventRecordWithFlags(h->ev_a, s, cudaEventRecordExternal));
-  else CK(cudaEventRecord(h->ev_a, s));
-  ST(cg_resid<true>(h, s, x, z));
-  SumSrc res, xz, zz;
+  auto mark = [&](cudaEvent_t ev) -> spmv_status {
+    if (cst == cudaStreamCaptureStatusActive) CK(cudaEventRecordWithFlags(ev, s, cudaEventRecordExternal));
+    else CK(cudaEventRecord(ev, s));
+    return SPMV_OK;
+  };
+  ST(mark(h->ev_a));
+  // zeta and x_new = z/||z|| first (they do not need the residual), x_new into a free CG
+  // vector (s), so its host copy overlaps the residual SpMV, which still reads the old x
   const int vg = (int)h->vgrid;
-  ST(reduce_src(h, s, SumSrc{h->part_res, vg}, 4, &res));
+  k_npb_xz<<<vg, 256, 0, s>>>(h->m_loc, x, z, h->part_xz, h->part_zz);
+  LAUNCHED();
+  SumSrc res, xz, zz;
   ST(reduce_src(h, s, SumSrc{h->part_xz, vg}, 5, &xz));
   ST(reduce_src(h, s, SumSrc{h->part_zz, vg}, 6, &zz));
-  k_npb_finish<<<vg, 256, 0, s>>>(h->m_loc, res, xz, zz, z, x, shift, out2);
+  double* xn = h->s_vec;
+  k_npb_xnew<<<vg, 256, 0, s>>>(h->m_loc, xz, zz, z, xn, shift, out2);
   LAUNCHED();
+  ST(mark(h->ev_b));
+  ST(cg_resid<false>(h, s, x, z));
+  ST(reduce_src(h, s, SumSrc{h->part_res, vg}, 4, &res));
+  k_finish_norm<<<1, 32, 0, s>>>(res, out2 + 1);
+  LAUNCHED();
+  if (h->m_loc > 0) CK(cudaMemcpyAsync(x, xn, sizeof(double) * h->m_loc, cudaMemcpyDeviceToDevice, s));
   return SPMV_OK;
 }
 
@@ -342,17 +355,21 @@ extern "C" spmv_status cg_npb_outer(spmv_csr_t h, void* x, void* z, int32_t cgit
   }
   bool sync = false;
   if (ok == 1) CK(cudaMemcpyAsync(out2, o2, sizeof(double) * 2, cudaMemcpyDeviceToDevice, s));
-  if (xd != x && h->m_loc > 0) {
-    CK(cudaMemcpyAsync(x, xd, sizeof(double) * h->m_loc, cudaMemcpyDeviceToHost, s));
-    sync = true;
-  }
   bool copy_used = false;
+  if ((zd != z || xd != x) && h->m_loc > 0 && !h->copy)
+    CK(cudaStreamCreateWithFlags(&h->copy, cudaStreamNonBlocking));
   if (zd != z && h->m_loc > 0) {
     // z (host) is copied on a side stream as soon as the CG loop wrote it,
-    // overlapping the residual SpMV and the finishing kernel
-    if (!h->copy) CK(cudaStreamCreateWithFlags(&h->copy, cudaStreamNonBlocking));
+    // overlapping the residual SpMV and the finishing kernels
     CK(cudaStreamWaitEvent(h->copy, h->ev_a, 0));
     CK(cudaMemcpyAsync(z, zd, sizeof(double) * h->m_loc, cudaMemcpyDeviceToHost, h->copy));
+    copy_used = true;
+    sync = true;
+  }
+  if (xd != x && h->m_loc > 0) {
+    // x_new (host) likewise, from the buffer it is computed into before the residual
+    CK(cudaStreamWaitEvent(h->copy, h->ev_b, 0));
+    CK(cudaMemcpyAsync(x, h->s_vec, sizeof(double) * h->m_loc, cudaMemcpyDeviceToHost, h->copy));
     copy_used = true;
     sync = true;
   }

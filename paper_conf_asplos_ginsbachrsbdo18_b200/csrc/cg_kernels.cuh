@@ -331,22 +331,36 @@ k_cg_resid(int64_t n, const double* __restrict__ b, const double* __restrict__ a
   }
 }
 
-// NPB tail: zeta = shift + 1/(x.z); x = z / ||z||; out2 = {zeta, rnorm}.
+// NAS outer iteration, split so the new x exists before the residual SpMV
+// (its host copy then overlaps the residual): partials of x.z and z.z (the
+// same accumulation and block sums as k_cg_resid<true>), then zeta and
+// x_new = z / ||z|| into a separate buffer (the residual still reads the old x).
 static __global__ void __launch_bounds__(256)
-k_npb_finish(int64_t n, SumSrc res, SumSrc xz, SumSrc zz, const double* __restrict__ z,
-             double* __restrict__ x, double shift, double* __restrict__ out2) {
-  __shared__ double s0, s1, s2;
-  const double rr = read_sum(res, &s0);
+k_npb_xz(int64_t n, const double* __restrict__ x, const double* __restrict__ z, double* __restrict__ part_xz,
+         double* __restrict__ part_zz) {
+  __shared__ double red[8];
+  double a1 = 0.0, a2 = 0.0;
+  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n; j += int64_t(gridDim.x) * blockDim.x) {
+    const double zj = z[j];
+    a1 += x[j] * zj;
+    a2 += zj * zj;
+  }
+  double t = block_sum(a1, red);
+  if (threadIdx.x == 0) part_xz[blockIdx.x] = t;
+  t = block_sum(a2, red);
+  if (threadIdx.x == 0) part_zz[blockIdx.x] = t;
+}
+
+static __global__ void __launch_bounds__(256)
+k_npb_xnew(int64_t n, SumSrc xz, SumSrc zz, const double* __restrict__ z, double* __restrict__ xn, double shift,
+           double* __restrict__ out2) {
+  __shared__ double s1, s2;
   const double nt1 = read_sum(xz, &s1);
   double nt2 = read_sum(zz, &s2);
   nt2 = 1.0 / sqrt(nt2);
-  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n;
-       j += int64_t(gridDim.x) * blockDim.x)
-    x[j] = nt2 * z[j];
-  if (blockIdx.x == 0 && threadIdx.x == 0) {
-    out2[0] = shift + 1.0 / nt1;
-    out2[1] = sqrt(rr);
-  }
+  for (int64_t j = int64_t(blockIdx.x) * blockDim.x + threadIdx.x; j < n; j += int64_t(gridDim.x) * blockDim.x)
+    xn[j] = nt2 * z[j];
+  if (blockIdx.x == 0 && threadIdx.x == 0) out2[0] = shift + 1.0 / nt1;
 }
 
 // cg_solve tail: rnorm = sqrt(sum).
